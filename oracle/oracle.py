@@ -106,7 +106,7 @@ _SIZES = ('extern "C" void oracle_sizes(size_t* out, int* np) '
 
 def entry_name(src: str) -> str:
     """The oracle is told nothing but the text: the user function is the last
-    top-level function definition in it (boundary convention, include/skel.h)."""
+    top-level function definition in it (the convention stated in DESIGN.md §1)."""
     names = re.findall(r"([A-Za-z_]\w*)\s*\([^;{}]*\)\s*\{", src)
     names = [n for n in names if n not in ("if", "for", "while", "switch", "return")]
     if not names:

@@ -1,0 +1,127 @@
+// internal.h -- private declarations of libskel (not part of the C-ABI).
+#pragma once
+
+#include <cuda_runtime.h>
+#include <nccl.h>
+
+#include <cstddef>
+#include <cstdint>
+#include <map>
+#include <memory>
+#include <set>
+#include <string>
+#include <vector>
+
+#include "skel.h"
+
+namespace skelrt {
+
+// ---------------------------------------------------------------------------
+// errors: every CUDA/NCCL/NVRTC failure becomes a status + message
+// ---------------------------------------------------------------------------
+struct Error {
+    int status;
+    std::string msg;
+};
+
+// ---------------------------------------------------------------------------
+// JIT modules (NVRTC injection + kernel cache)
+// ---------------------------------------------------------------------------
+enum class Kind { Map = 0, Zip = 1, Red = 2 };
+
+struct Module {
+    Kind kind;
+    std::string key;
+    cudaLibrary_t lib = nullptr;
+    cudaKernel_t k_main = nullptr;  // skel_ew_kernel | skel_reduce_kernel
+    cudaKernel_t k_scan = nullptr;
+    cudaKernel_t k_fold = nullptr;
+    cudaKernel_t k_seed = nullptr;
+    uint64_t sig[16 + 4 * 32] = {0};
+    std::set<int> attr_set_on;  // devices on which smem attributes were set
+};
+
+// signature accessors (layout documented in map.cuh / red.cuh)
+struct ArgSlot {
+    uint64_t size, align, isptr, off;
+};
+
+// ---------------------------------------------------------------------------
+// devices
+// ---------------------------------------------------------------------------
+struct Slot {
+    int d = 0;      // logical device index (0..D-1)
+    int dev = 0;    // CUDA device ordinal
+    int sms = 148;  // multiprocessor count
+    cudaStream_t stream = nullptr;
+    cudaEvent_t ev = nullptr;  // join event
+    // grow-only workspace for reduce/scan partials, look-back status, seeds
+    char *ws = nullptr;
+    size_t ws_cap = 0;
+    unsigned *counters = nullptr;  // [0] scan ticket, [1] scan done, [2] reduce done, [3] pad
+    // look-back status words (only ever hold status words; zeroed at allocation)
+    unsigned long long *st64 = nullptr;
+    size_t st64_cap = 0;  // entries
+    unsigned *fl32 = nullptr;
+    size_t fl32_cap = 0;  // entries
+    // scratch for rank-mode downloads
+    char *scratch = nullptr;
+    size_t scratch_cap = 0;
+};
+
+struct Buf {  // one logical device's storage of a vector
+    char *base = nullptr;
+    size_t cap = 0;    // bytes allocated at base
+    size_t off = 0;    // element offset of the live data inside base
+    size_t count = 0;  // live elements
+    char *ptr(size_t es) const { return base ? base + off * es : nullptr; }
+};
+
+}  // namespace skelrt
+
+struct skel_vec_s;
+
+struct skel_ctx_s {
+    int D = 1;                   // logical devices
+    bool rank_mode = false;      // one process per GPU, NCCL exchanges
+    int rank = 0;                // rank mode: this process's logical device
+    std::vector<skelrt::Slot> slots;  // local logical devices
+    ncclComm_t comm = nullptr;
+    int block_size = 0;
+    std::string cache_dir;
+    bool disk_cache = true;
+    bool fmad = false;
+    skel_stats stats{};
+    std::string last_error;
+    std::map<std::string, std::unique_ptr<skelrt::Module>> modules;
+    std::set<skel_vec_s *> vecs;
+    unsigned scan_epoch = 0;
+};
+
+struct skel_vec_s {
+    skel_ctx_s *ctx = nullptr;
+    size_t n = 0, es = 0;
+    skel_dist dist = SKEL_SINGLE;
+    skel_dtype dt = SKEL_DT_OPAQUE;
+    char *host = nullptr;   // pinned mirror (lazily allocated)
+    bool host_valid = false;
+    bool dev_valid = true;  // created zero-filled on the devices
+    bool diverged = false;  // copy distribution after mark_device_modified
+    std::vector<skelrt::Buf> bufs;  // indexed like ctx->slots
+};
+
+namespace skelrt {
+// jit.cpp
+int get_module(skel_ctx_s *ctx, Kind kind, const char *src, Module **out);
+std::string entry_name(const std::string &src, std::string *err);
+// NVRTC compile without any device (used by skel_compile_check)
+int compile_only(Kind kind, const char *src, int block, bool fmad, std::string *log, std::vector<char> *cubin);
+
+// builtin.cu (nvcc-compiled helper kernels)
+cudaError_t launch_fill(void *dst, size_t n, const void *elem, size_t es, cudaStream_t s);
+// dst[i] = op(srcs[0][i], ..., srcs[nsrc-1][i]) for i < count; dst may alias srcs[j]
+cudaError_t launch_combine(void *dst, const void *const *srcs, int nsrc, size_t count, skel_dtype dt,
+                           skel_combine op, cudaStream_t s);
+// dst[j*bytes ...] = srcs[j][0 .. bytes) for j < nsrc
+cudaError_t launch_gather(void *dst, const void *const *srcs, int nsrc, size_t bytes, cudaStream_t s);
+}  // namespace skelrt

@@ -1,0 +1,1473 @@
+// runtime.cpp -- the host side of libskel: contexts, the Vector coherence
+// tracker, the distribution planner/executor and the skeleton launchers,
+// exported through the C-ABI of include/skel.h.
+//
+// Paper passages implemented here:
+//  * Vector + lazy coherence (§III-A): a vector has a (pinned)
+//    host mirror and per-device storage; each side carries a valid bit; a
+//    transfer happens only when the destination is stale;
+//    skeleton outputs stay on the devices.
+//  * Distributions (§III-D; Listing 4): single /
+//    block / copy placement over D logical devices, redistribution with data
+//    exchange, copy -> block with element-wise combine.
+//  * Skeleton execution on several devices: block parts run on
+//    their own device; Reduce/Scan add one exchange of D partial results and an
+//    ordered fold (cross-device combination in device order).
+#include <cuda.h>
+#include <cudaTypedefs.h>
+
+#include <algorithm>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <mutex>
+
+#include "internal.h"
+
+using namespace skelrt;
+
+namespace {
+
+thread_local std::string g_last_error;  // failures without a context
+
+int fail(skel_ctx_s *ctx, int st, const std::string &msg) {
+    if (ctx) ctx->last_error = msg;
+    else g_last_error = msg;
+    if (getenv("SKEL_LOG")) fprintf(stderr, "[skel] error %d: %s\n", st, msg.c_str());
+    return st;
+}
+
+#define CK(ctx, call)                                                                                      \
+    do {                                                                                                   \
+        cudaError_t _e = (call);                                                                           \
+        if (_e != cudaSuccess)                                                                             \
+            return fail((ctx), SKEL_ERR_CUDA, std::string(#call) + ": " + cudaGetErrorString(_e));         \
+    } while (0)
+#define NK(ctx, call)                                                                                      \
+    do {                                                                                                   \
+        ncclResult_t _r = (call);                                                                          \
+        if (_r != ncclSuccess)                                                                             \
+            return fail((ctx), SKEL_ERR_NCCL, std::string(#call) + ": " + ncclGetErrorString(_r));         \
+    } while (0)
+#define TRY(expr)                          \
+    do {                                   \
+        int _s = (expr);                   \
+        if (_s != SKEL_OK) return _s;      \
+    } while (0)
+
+inline size_t part_size(size_t n, int D) { return D > 0 ? (n + D - 1) / D : 0; }
+inline void part_range(size_t n, int D, int k, size_t *lo, size_t *hi) {
+    const size_t s = part_size(n, D);
+    *lo = std::min(n, (size_t)k * s);
+    *hi = std::min(n, (size_t)(k + 1) * s);
+}
+inline size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
+inline bool al16(const void *p) { return (reinterpret_cast<uintptr_t>(p) & 15) == 0; }
+
+size_t want_count(const skel_vec_s *v, skel_dist dist, int d) {
+    size_t lo, hi;
+    switch (dist) {
+        case SKEL_SINGLE: return d == 0 ? v->n : 0;
+        case SKEL_COPY: return v->n;
+        default: part_range(v->n, v->ctx->D, d, &lo, &hi); return hi - lo;
+    }
+}
+size_t part_lo(const skel_vec_s *v, int d) {
+    size_t lo, hi;
+    part_range(v->n, v->ctx->D, d, &lo, &hi);
+    return lo;
+}
+// bytes of a "full" per-device buffer: D parts of ceil(n/D) elements (NCCL
+// collectives need equal part sizes; the padding is never read as data)
+size_t full_bytes(const skel_vec_s *v) {
+    return std::max<size_t>(part_size(v->n, v->ctx->D) * v->ctx->D * v->es, 16);
+}
+
+struct DevGuard {
+    explicit DevGuard(int dev) { cudaSetDevice(dev); }
+};
+
+// ---- device memory -----------------------------------------------------------
+int dev_alloc(skel_ctx_s *ctx, Slot &s, size_t bytes, char **out) {
+    DevGuard g(s.dev);
+    void *p = nullptr;
+    cudaError_t e = cudaMalloc(&p, std::max<size_t>(bytes, 256));
+    if (e != cudaSuccess) {
+        cudaGetLastError();
+        return fail(ctx, SKEL_ERR_OOM, std::string("cudaMalloc(") + std::to_string(bytes) + "): " +
+                                           cudaGetErrorString(e));
+    }
+    *out = static_cast<char *>(p);
+    return SKEL_OK;
+}
+int dev_free(skel_ctx_s *ctx, Slot &s, char *p) {
+    if (!p) return SKEL_OK;
+    DevGuard g(s.dev);
+    CK(ctx, cudaStreamSynchronize(s.stream));
+    CK(ctx, cudaFree(p));
+    return SKEL_OK;
+}
+// make b hold at least `bytes`; the first `keep` bytes at element offset
+// b.off move to byte offset new_off_bytes of the new allocation
+int buf_grow(skel_ctx_s *ctx, Slot &s, Buf &b, size_t bytes, size_t es, size_t keep, size_t new_off_elems) {
+    if (b.cap >= bytes && (keep == 0 || b.off == new_off_elems)) {
+        b.off = new_off_elems;
+        return SKEL_OK;
+    }
+    if (b.cap >= bytes && keep) {  // same buffer, move data
+        DevGuard g(s.dev);
+        CK(ctx, cudaMemcpyAsync(b.base + new_off_elems * es, b.base + b.off * es, keep, cudaMemcpyDeviceToDevice,
+                                s.stream));
+        b.off = new_off_elems;
+        return SKEL_OK;
+    }
+    char *nb = nullptr;
+    TRY(dev_alloc(ctx, s, bytes, &nb));
+    DevGuard g(s.dev);
+    if (keep) CK(ctx, cudaMemcpyAsync(nb + new_off_elems * es, b.base + b.off * es, keep, cudaMemcpyDeviceToDevice,
+                                      s.stream));
+    TRY(dev_free(ctx, s, b.base));
+    b.base = nb;
+    b.cap = bytes;
+    b.off = new_off_elems;
+    return SKEL_OK;
+}
+
+// Place the (uninitialised) storage of v for `dist` on every local device.
+// Block parts sit at offset lo when the buffer is a full one (so that NCCL's
+// in-place all-gather / reduce-scatter layout holds), else at 0.
+int place(skel_vec_s *v, skel_dist dist) {
+    skel_ctx_s *ctx = v->ctx;
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        Buf &b = v->bufs[li];
+        const size_t cnt = want_count(v, dist, s.d);
+        size_t need, off = 0;
+        if (dist == SKEL_COPY) {
+            need = full_bytes(v);
+        } else if (dist == SKEL_BLOCK) {
+            const size_t fb = full_bytes(v);
+            if (b.cap >= fb) {
+                need = fb;
+                off = part_lo(v, s.d);
+            } else {
+                need = std::max<size_t>(part_size(v->n, ctx->D) * v->es, 16);
+            }
+        } else {
+            need = std::max<size_t>(cnt * v->es, 16);
+        }
+        if (b.cap < need) TRY(buf_grow(ctx, s, b, need, v->es, 0, 0));
+        b.off = off;
+        b.count = cnt;
+    }
+    return SKEL_OK;
+}
+
+// every local stream waits for all others (exchanges between logical devices)
+int join(skel_ctx_s *ctx) {
+    if (ctx->slots.size() < 2) return SKEL_OK;
+    for (auto &s : ctx->slots) {
+        DevGuard g(s.dev);
+        CK(ctx, cudaEventRecord(s.ev, s.stream));
+    }
+    for (auto &s : ctx->slots) {
+        DevGuard g(s.dev);
+        for (auto &o : ctx->slots)
+            if (&o != &s) CK(ctx, cudaStreamWaitEvent(s.stream, o.ev, 0));
+    }
+    return SKEL_OK;
+}
+
+int host_mirror(skel_vec_s *v) {
+    if (v->host) return SKEL_OK;
+    void *p = nullptr;
+    cudaError_t e = cudaHostAlloc(&p, std::max<size_t>(v->n * v->es, 16), cudaHostAllocPortable);
+    if (e != cudaSuccess) {
+        cudaGetLastError();
+        return fail(v->ctx, SKEL_ERR_OOM, std::string("cudaHostAlloc: ") + cudaGetErrorString(e));
+    }
+    v->host = static_cast<char *>(p);
+    return SKEL_OK;
+}
+
+// lazy H2D: make the devices hold v's data
+int ensure_device(skel_vec_s *v) {
+    if (v->dev_valid) return SKEL_OK;
+    skel_ctx_s *ctx = v->ctx;
+    if (!v->host_valid || !v->host) return fail(ctx, SKEL_ERR_STATE, "vector has no valid copy");
+    TRY(place(v, v->dist));
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        Buf &b = v->bufs[li];
+        if (!b.count) continue;
+        const size_t lo = (v->dist == SKEL_BLOCK) ? part_lo(v, s.d) : 0;
+        DevGuard g(s.dev);
+        CK(ctx, cudaMemcpyAsync(b.ptr(v->es), v->host + lo * v->es, b.count * v->es, cudaMemcpyHostToDevice,
+                                s.stream));
+        ctx->stats.h2d_bytes += b.count * v->es;
+        ctx->stats.h2d_copies++;
+    }
+    v->dev_valid = true;
+    v->diverged = false;
+    return SKEL_OK;
+}
+
+int sync_all(skel_ctx_s *ctx) {
+    for (auto &s : ctx->slots) {
+        DevGuard g(s.dev);
+        CK(ctx, cudaStreamSynchronize(s.stream));
+    }
+    if (ctx->comm) {
+        ncclResult_t ae = ncclSuccess;
+        NK(ctx, ncclCommGetAsyncError(ctx->comm, &ae));
+        if (ae != ncclSuccess) return fail(ctx, SKEL_ERR_NCCL, std::string("NCCL async: ") + ncclGetErrorString(ae));
+    }
+    return SKEL_OK;
+}
+
+int scratch(skel_ctx_s *ctx, Slot &s, size_t bytes) {
+    if (s.scratch_cap >= bytes) return SKEL_OK;
+    TRY(dev_free(ctx, s, s.scratch));
+    s.scratch = nullptr;
+    s.scratch_cap = 0;
+    TRY(dev_alloc(ctx, s, bytes, &s.scratch));
+    s.scratch_cap = bytes;
+    return SKEL_OK;
+}
+
+// lazy D2H into the host mirror
+int ensure_host(skel_vec_s *v) {
+    if (v->host_valid) return SKEL_OK;
+    skel_ctx_s *ctx = v->ctx;
+    TRY(host_mirror(v));
+    const size_t es = v->es;
+    if (!ctx->rank_mode) {
+        for (size_t li = 0; li < ctx->slots.size(); ++li) {
+            Slot &s = ctx->slots[li];
+            Buf &b = v->bufs[li];
+            if (!b.count) continue;
+            if (v->dist == SKEL_COPY && s.d != 0) continue;  // read device 0's copy (reading R6)
+            const size_t lo = (v->dist == SKEL_BLOCK) ? part_lo(v, s.d) : 0;
+            DevGuard g(s.dev);
+            CK(ctx, cudaMemcpyAsync(v->host + lo * es, b.ptr(es), b.count * es, cudaMemcpyDeviceToHost, s.stream));
+            ctx->stats.d2h_bytes += b.count * es;
+            ctx->stats.d2h_copies++;
+        }
+    } else {
+        Slot &s = ctx->slots[0];
+        Buf &b = v->bufs[0];
+        DevGuard g(s.dev);
+        const char *src = b.ptr(es);
+        if (ctx->D > 1 && v->dist != SKEL_COPY) {
+            const size_t ps = part_size(v->n, ctx->D);
+            TRY(scratch(ctx, s, std::max<size_t>(ps * ctx->D * es, 16)));
+            if (v->dist == SKEL_BLOCK) {
+                NK(ctx, ncclAllGather(b.ptr(es), s.scratch, ps * es, ncclUint8, ctx->comm, s.stream));
+            } else {  // SINGLE: rank 0 broadcasts
+                NK(ctx, ncclBroadcast(s.d == 0 ? b.ptr(es) : s.scratch, s.scratch, v->n * es, ncclUint8, 0, ctx->comm,
+                                      s.stream));
+            }
+            ctx->stats.nccl_bytes += ps * ctx->D * es;
+            src = s.scratch;
+        } else if (ctx->D > 1 && v->diverged) {
+            TRY(scratch(ctx, s, std::max<size_t>(v->n * es, 16)));
+            NK(ctx, ncclBroadcast(b.ptr(es), s.scratch, v->n * es, ncclUint8, 0, ctx->comm, s.stream));
+            ctx->stats.nccl_bytes += v->n * es;
+            src = s.scratch;
+        }
+        if (v->n) {
+            CK(ctx, cudaMemcpyAsync(v->host, src, v->n * es, cudaMemcpyDeviceToHost, s.stream));
+            ctx->stats.d2h_bytes += v->n * es;
+            ctx->stats.d2h_copies++;
+        }
+    }
+    TRY(sync_all(ctx));
+    v->host_valid = true;
+    return SKEL_OK;
+}
+
+ncclDataType_t nccl_type(skel_dtype dt) {
+    switch (dt) {
+        case SKEL_DT_F32: return ncclFloat32;
+        case SKEL_DT_F64: return ncclFloat64;
+        case SKEL_DT_I32: return ncclInt32;
+        case SKEL_DT_U32: return ncclUint32;
+        case SKEL_DT_I64: return ncclInt64;
+        case SKEL_DT_U64: return ncclUint64;
+        default: return ncclUint8;
+    }
+}
+ncclRedOp_t nccl_op(skel_combine c) {
+    switch (c) {
+        case SKEL_COMBINE_MIN: return ncclMin;
+        case SKEL_COMBINE_MAX: return ncclMax;
+        case SKEL_COMBINE_PROD: return ncclProd;
+        default: return ncclSum;
+    }
+}
+
+int plan_exchange(skel_dist from, skel_dist to, skel_combine combine) {
+    if (combine != SKEL_COMBINE_NONE) {
+        if (from != SKEL_COPY) return -1;
+        if (to == SKEL_BLOCK) return SKEL_XCHG_REDUCE_SCATTER;
+        if (to == SKEL_SINGLE) return SKEL_XCHG_REDUCE;
+        return SKEL_XCHG_ALLREDUCE;
+    }
+    if (from == to) return SKEL_XCHG_NONE;
+    if (from == SKEL_SINGLE) return to == SKEL_BLOCK ? SKEL_XCHG_SCATTER : SKEL_XCHG_BROADCAST;
+    if (from == SKEL_BLOCK) return to == SKEL_SINGLE ? SKEL_XCHG_GATHER : SKEL_XCHG_ALLGATHER;
+    return to == SKEL_BLOCK ? SKEL_XCHG_LOCAL_SLICE : SKEL_XCHG_KEEP_ROOT;
+}
+
+// ---- the exchanges (DESIGN.md §5 table T1) -----------------------------------
+// Local mode: every logical device is in this process; data moves with
+// cudaMemcpyAsync (peer or same GPU) and the combine kernel.
+int xchg_local(skel_vec_s *v, int x, skel_combine combine) {
+    skel_ctx_s *ctx = v->ctx;
+    const int D = ctx->D;
+    const size_t es = v->es, n = v->n;
+    auto &S = ctx->slots;
+    auto &B = v->bufs;
+    TRY(join(ctx));
+    switch (x) {
+        case SKEL_XCHG_SCATTER: {
+            for (int d = 1; d < D; ++d) {
+                const size_t cnt = want_count(v, SKEL_BLOCK, d);
+                if (B[d].cap < std::max<size_t>(part_size(n, D) * es, 16))
+                    TRY(buf_grow(ctx, S[d], B[d], std::max<size_t>(part_size(n, D) * es, 16), es, 0, 0));
+                B[d].off = 0;
+                B[d].count = cnt;
+                if (cnt) {
+                    DevGuard g(S[d].dev);
+                    CK(ctx, cudaMemcpyAsync(B[d].ptr(es), B[0].ptr(es) + part_lo(v, d) * es, cnt * es,
+                                            cudaMemcpyDefault, S[d].stream));
+                    ctx->stats.d2d_bytes += cnt * es;
+                }
+            }
+            B[0].count = want_count(v, SKEL_BLOCK, 0);
+            break;
+        }
+        case SKEL_XCHG_BROADCAST: {
+            TRY(buf_grow(ctx, S[0], B[0], full_bytes(v), es, n * es, 0));
+            for (int d = 1; d < D; ++d) {
+                if (B[d].cap < full_bytes(v)) TRY(buf_grow(ctx, S[d], B[d], full_bytes(v), es, 0, 0));
+                B[d].off = 0;
+                B[d].count = n;
+                if (n) {
+                    DevGuard g(S[d].dev);
+                    CK(ctx, cudaMemcpyAsync(B[d].base, B[0].ptr(es), n * es, cudaMemcpyDefault, S[d].stream));
+                    ctx->stats.d2d_bytes += n * es;
+                }
+            }
+            B[0].count = n;
+            break;
+        }
+        case SKEL_XCHG_GATHER: {
+            TRY(buf_grow(ctx, S[0], B[0], std::max<size_t>(n * es, 16), es, B[0].count * es, 0));
+            TRY(join(ctx));
+            for (int d = 1; d < D; ++d) {
+                if (B[d].count) {
+                    DevGuard g(S[0].dev);
+                    CK(ctx, cudaMemcpyAsync(B[0].base + part_lo(v, d) * es, B[d].ptr(es), B[d].count * es,
+                                            cudaMemcpyDefault, S[0].stream));
+                    ctx->stats.d2d_bytes += B[d].count * es;
+                }
+                B[d].count = 0;
+            }
+            B[0].off = 0;
+            B[0].count = n;
+            break;
+        }
+        case SKEL_XCHG_ALLGATHER:
+        case SKEL_XCHG_ALLREDUCE: {
+            if (x == SKEL_XCHG_ALLREDUCE) {
+                TRY(xchg_local(v, SKEL_XCHG_REDUCE_SCATTER, combine));
+                TRY(join(ctx));
+            }
+            for (int d = 0; d < D; ++d) TRY(buf_grow(ctx, S[d], B[d], full_bytes(v), es, B[d].count * es, part_lo(v, d)));
+            TRY(join(ctx));
+            for (int d = 0; d < D; ++d) {
+                DevGuard g(S[d].dev);
+                for (int j = 0; j < D; ++j) {
+                    if (j == d) continue;
+                    const size_t cnt = want_count(v, SKEL_BLOCK, j);
+                    if (!cnt) continue;
+                    const size_t lo = part_lo(v, j);
+                    CK(ctx, cudaMemcpyAsync(B[d].base + lo * es, B[j].base + lo * es, cnt * es, cudaMemcpyDefault,
+                                            S[d].stream));
+                    ctx->stats.d2d_bytes += cnt * es;
+                }
+                B[d].off = 0;
+                B[d].count = n;
+            }
+            break;
+        }
+        case SKEL_XCHG_LOCAL_SLICE: {
+            for (int d = 0; d < D; ++d) {
+                B[d].off = part_lo(v, d);
+                B[d].count = want_count(v, SKEL_BLOCK, d);
+            }
+            break;
+        }
+        case SKEL_XCHG_REDUCE_SCATTER: {
+            for (int d = 0; d < D; ++d) {
+                const size_t lo = part_lo(v, d), cnt = want_count(v, SKEL_BLOCK, d);
+                B[d].off = lo;
+                B[d].count = cnt;
+                if (!cnt) continue;
+                std::vector<const void *> src(D);
+                for (int j = 0; j < D; ++j) src[j] = B[j].base + lo * es;
+                DevGuard g(S[d].dev);
+                CK(ctx, launch_combine(B[d].base + lo * es, src.data(), D, cnt, v->dt, combine, S[d].stream));
+                ctx->stats.kernel_launches++;
+                ctx->stats.d2d_bytes += (D - 1) * cnt * es;
+            }
+            break;
+        }
+        case SKEL_XCHG_KEEP_ROOT: {
+            for (int d = 1; d < D; ++d) B[d].count = 0;
+            break;
+        }
+        case SKEL_XCHG_REDUCE: {
+            std::vector<const void *> src(D);
+            for (int j = 0; j < D; ++j) src[j] = B[j].base;
+            DevGuard g(S[0].dev);
+            CK(ctx, launch_combine(B[0].base, src.data(), D, n, v->dt, combine, S[0].stream));
+            ctx->stats.kernel_launches++;
+            ctx->stats.d2d_bytes += (D - 1) * n * es;
+            for (int d = 1; d < D; ++d) B[d].count = 0;
+            B[0].off = 0;
+            B[0].count = n;
+            break;
+        }
+        default: break;
+    }
+    return join(ctx);
+}
+
+// Rank mode: this process holds logical device `rank`; NCCL moves the data,
+// in place wherever NCCL allows it (part k at offset k*ceil(n/D) of a full
+// buffer).
+int xchg_rank(skel_vec_s *v, int x, skel_combine combine) {
+    skel_ctx_s *ctx = v->ctx;
+    const int D = ctx->D, r = ctx->rank;
+    const size_t es = v->es, n = v->n, ps = part_size(n, D);
+    Slot &s = ctx->slots[0];
+    Buf &b = v->bufs[0];
+    ncclComm_t c = ctx->comm;
+    DevGuard g(s.dev);
+    switch (x) {
+        case SKEL_XCHG_SCATTER: {
+            if (r == 0) TRY(buf_grow(ctx, s, b, full_bytes(v), es, n * es, 0));
+            else if (b.cap < std::max<size_t>(ps * es, 16)) TRY(buf_grow(ctx, s, b, std::max<size_t>(ps * es, 16), es, 0, 0));
+            b.off = 0;
+            NK(ctx, ncclScatter(b.base, b.base, ps * es, ncclUint8, 0, c, s.stream));
+            ctx->stats.nccl_bytes += ps * es * (r == 0 ? D : 1);
+            b.count = want_count(v, SKEL_BLOCK, r);
+            break;
+        }
+        case SKEL_XCHG_BROADCAST: {
+            TRY(buf_grow(ctx, s, b, full_bytes(v), es, r == 0 ? n * es : 0, 0));
+            NK(ctx, ncclBroadcast(b.base, b.base, n * es, ncclUint8, 0, c, s.stream));
+            ctx->stats.nccl_bytes += n * es;
+            b.off = 0;
+            b.count = n;
+            break;
+        }
+        case SKEL_XCHG_GATHER: {
+            if (r == 0) TRY(buf_grow(ctx, s, b, full_bytes(v), es, b.count * es, 0));
+            NK(ctx, ncclGather(b.ptr(es), b.base, ps * es, ncclUint8, 0, c, s.stream));
+            ctx->stats.nccl_bytes += ps * es;
+            b.count = r == 0 ? n : 0;
+            b.off = 0;
+            break;
+        }
+        case SKEL_XCHG_ALLGATHER: {
+            TRY(buf_grow(ctx, s, b, full_bytes(v), es, b.count * es, part_lo(v, r) == std::min(n, r * ps) ? r * ps : 0));
+            NK(ctx, ncclAllGather(b.base + r * ps * es, b.base, ps * es, ncclUint8, c, s.stream));
+            ctx->stats.nccl_bytes += ps * es * D;
+            b.off = 0;
+            b.count = n;
+            break;
+        }
+        case SKEL_XCHG_LOCAL_SLICE: {
+            b.off = part_lo(v, r);
+            b.count = want_count(v, SKEL_BLOCK, r);
+            break;
+        }
+        case SKEL_XCHG_REDUCE_SCATTER: {
+            NK(ctx, ncclReduceScatter(b.base, b.base + r * ps * es, ps, nccl_type(v->dt), nccl_op(combine), c,
+                                      s.stream));
+            ctx->stats.nccl_bytes += ps * es * D;
+            b.off = r * ps;
+            b.count = want_count(v, SKEL_BLOCK, r);
+            break;
+        }
+        case SKEL_XCHG_KEEP_ROOT: {
+            if (r != 0) b.count = 0;
+            break;
+        }
+        case SKEL_XCHG_REDUCE: {
+            NK(ctx, ncclReduce(b.base, b.base, n, nccl_type(v->dt), nccl_op(combine), 0, c, s.stream));
+            ctx->stats.nccl_bytes += n * es;
+            b.count = r == 0 ? n : 0;
+            break;
+        }
+        case SKEL_XCHG_ALLREDUCE: {
+            NK(ctx, ncclAllReduce(b.base, b.base, n, nccl_type(v->dt), nccl_op(combine), c, s.stream));
+            ctx->stats.nccl_bytes += n * es;
+            break;
+        }
+        default: break;
+    }
+    return SKEL_OK;
+}
+
+int set_distribution(skel_vec_s *v, skel_dist dist, skel_combine combine) {
+    skel_ctx_s *ctx = v->ctx;
+    const int x = plan_exchange(v->dist, dist, combine);
+    if (x < 0) return fail(ctx, SKEL_ERR_STATE, "a combine merges per-device copies: the vector must be SKEL_COPY");
+    if (combine != SKEL_COMBINE_NONE && v->dt == SKEL_DT_OPAQUE)
+        return fail(ctx, SKEL_ERR_TYPE, "combine needs a numeric dtype (skel_vector_set_dtype)");
+    if (!v->dev_valid && combine == SKEL_COMBINE_NONE) {  // host-only data: relayout is free (lazy)
+        v->dist = dist;
+        return SKEL_OK;
+    }
+    TRY(ensure_device(v));
+    if (x == SKEL_XCHG_NONE) {
+        v->dist = dist;
+        return SKEL_OK;
+    }
+    const bool diverged = v->diverged;
+    if (ctx->D == 1) {
+        // one device: every distribution is the same storage
+        Buf &b = v->bufs[0];
+        b.off = 0;
+        b.count = v->n;
+    } else if (ctx->rank_mode) {
+        TRY(xchg_rank(v, x, combine));
+    } else {
+        TRY(xchg_local(v, x, combine));
+    }
+    v->dist = dist;
+    v->dev_valid = true;
+    if (combine != SKEL_COMBINE_NONE || diverged) v->host_valid = false;
+    v->diverged = false;
+    return SKEL_OK;
+}
+
+// ---- Arguments (§III-C) ------------------------------------------------------
+int check_args(skel_ctx_s *ctx, const Module *m, const skel_arg *args, int nargs) {
+    const int want = (int)m->sig[6];
+    if (nargs != want)
+        return fail(ctx, SKEL_ERR_TYPE, "user function takes " + std::to_string(want) + " extra argument(s), " +
+                                            std::to_string(nargs) + " given");
+    for (int i = 0; i < nargs; ++i) {
+        const uint64_t size = m->sig[16 + 4 * i], isptr = m->sig[18 + 4 * i];
+        if (args[i].kind == SKEL_ARG_VECTOR) {
+            if (!isptr) return fail(ctx, SKEL_ERR_TYPE, "argument " + std::to_string(i) + ": vector for a by-value parameter");
+            if (!args[i].vec || args[i].vec->ctx != ctx) return fail(ctx, SKEL_ERR_ARG, "argument " + std::to_string(i) + ": bad vector");
+        } else if (args[i].kind == SKEL_ARG_SCALAR) {
+            if (args[i].size != size || !args[i].data)
+                return fail(ctx, SKEL_ERR_TYPE, "argument " + std::to_string(i) + ": " + std::to_string(args[i].size) +
+                                                    " bytes given, parameter has " + std::to_string(size));
+        } else {
+            return fail(ctx, SKEL_ERR_ARG, "argument " + std::to_string(i) + ": bad kind");
+        }
+    }
+    for (int i = 0; i < nargs; ++i)
+        if (args[i].kind == SKEL_ARG_VECTOR) TRY(ensure_device(args[i].vec));
+    return SKEL_OK;
+}
+void pack_args(const Module *m, const skel_arg *args, int nargs, size_t li, std::vector<unsigned char> &buf) {
+    buf.assign(m->sig[7], 0);
+    for (int i = 0; i < nargs; ++i) {
+        const uint64_t off = m->sig[19 + 4 * i];
+        if (args[i].kind == SKEL_ARG_VECTOR) {
+            skel_vec_s *av = args[i].vec;
+            void *p = av->bufs[li].ptr(av->es);
+            memcpy(&buf[off], &p, sizeof p);
+        } else {
+            memcpy(&buf[off], args[i].data, args[i].size);
+        }
+    }
+}
+
+int prepare_output(skel_vec_s *out, size_t n, skel_dist dist, bool same_as_input) {
+    if (!same_as_input) {
+        if (out->n != n) {  // resize: the output gets the input's length
+            out->n = n;
+            if (out->host) {
+                cudaFreeHost(out->host);
+                out->host = nullptr;
+            }
+        }
+        out->dist = dist;
+        TRY(place(out, dist));
+    }
+    out->dev_valid = true;
+    out->host_valid = false;
+    out->diverged = false;
+    return SKEL_OK;
+}
+
+int ew_grid(const Slot &s, size_t chunks, int block) {
+    size_t g = (chunks + block - 1) / block;
+    const size_t cap = (size_t)s.sms * (2048 / block) * 2;
+    g = std::min(g, cap);
+    return (int)std::max<size_t>(g, 1);
+}
+
+int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_s *b, skel_vec_s *out,
+           const skel_arg *args, int nargs) {
+    Module *m = nullptr;
+    TRY(get_module(ctx, kind, src, &m));
+    const uint64_t rsz = m->sig[3];
+    if (m->sig[4] != a->es)
+        return fail(ctx, SKEL_ERR_TYPE, "element size " + std::to_string(a->es) + " != sizeof(parameter 0) = " +
+                                            std::to_string(m->sig[4]));
+    if (b && m->sig[5] != b->es)
+        return fail(ctx, SKEL_ERR_TYPE, "element size of the second vector != sizeof(parameter 1)");
+    if (rsz == 0 && kind == Kind::Zip) return fail(ctx, SKEL_ERR_TYPE, "zip needs a non-void function");
+    if (rsz != 0 && !out) return fail(ctx, SKEL_ERR_ARG, "non-void function needs an output vector");
+    if (rsz != 0 && out->es != rsz)
+        return fail(ctx, SKEL_ERR_TYPE, "output element size " + std::to_string(out->es) + " != sizeof(result) = " +
+                                            std::to_string(rsz));
+    TRY(check_args(ctx, m, args, nargs));
+    TRY(ensure_device(a));
+    if (b) {
+        if (b->dist != a->dist) TRY(set_distribution(b, a->dist, SKEL_COMBINE_NONE));
+        TRY(ensure_device(b));
+    }
+    if (rsz != 0) TRY(prepare_output(out, a->n, a->dist, out == a || out == b));
+    const int block = (int)m->sig[9];
+    const uint64_t E = m->sig[8];
+    std::vector<unsigned char> abuf;
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        uint64_t cnt = a->bufs[li].count;
+        if (!cnt) continue;
+        const void *pa = a->bufs[li].ptr(a->es);
+        const void *pb = b ? b->bufs[li].ptr(b->es) : nullptr;
+        void *po = (rsz != 0) ? out->bufs[li].ptr(out->es) : nullptr;
+        int vec_ok = al16(pa) && (!pb || al16(pb)) && (!po || al16(po));
+        pack_args(m, args, nargs, li, abuf);
+        const size_t chunks = vec_ok ? std::max<uint64_t>(cnt / E, 1) : cnt;
+        const int grid = ew_grid(s, chunks, block);
+        void *params[] = {&pa, &pb, &po, &cnt, &vec_ok, abuf.data()};
+        DevGuard g(s.dev);
+        CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+        ctx->stats.kernel_launches++;
+    }
+    if (rsz != 0) {
+        out->dev_valid = true;
+        out->host_valid = false;
+    }
+    return SKEL_OK;
+}
+
+// ---- Reduce / Scan -------------------------------------------------------------
+using PFN_encode = CUresult (*)(CUtensorMap *, CUtensorMapDataType, cuuint32_t, void *, const cuuint64_t *,
+                                const cuuint64_t *, const cuuint32_t *, const cuuint32_t *, CUtensorMapInterleave,
+                                CUtensorMapSwizzle, CUtensorMapL2promotion, CUtensorMapFloatOOBfill);
+PFN_encode get_encode() {
+    static PFN_encode fn = nullptr;
+    static std::once_flag once;
+    std::call_once(once, [] {
+        void *p = nullptr;
+        cudaDriverEntryPointQueryResult q;
+        if (cudaGetDriverEntryPointByVersion("cuTensorMapEncodeTiled", &p, 12000, cudaEnableDefault, &q) ==
+                cudaSuccess &&
+            q == cudaDriverEntryPointSuccess)
+            fn = reinterpret_cast<PFN_encode>(p);
+    });
+    return fn;
+}
+
+// 2-D view [rows][128 B] of a tile-aligned prefix, 128B swizzle, 256-row boxes
+bool make_tmap(CUtensorMap *map, const void *ptr, uint64_t rows) {
+    memset(map, 0, sizeof *map);
+    PFN_encode enc = get_encode();
+    if (!enc || rows == 0 || !al16(ptr) || rows > 0x7fffffffull) return false;
+    cuuint64_t dims[2] = {32, rows};
+    cuuint64_t strides[1] = {128};
+    cuuint32_t box[2] = {32, 256};
+    cuuint32_t estr[2] = {1, 1};
+    CUresult r = enc(map, CU_TENSOR_MAP_DATA_TYPE_UINT32, 2, const_cast<void *>(ptr), dims, strides, box, estr,
+                     CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_128B, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                     CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    return r == CUDA_SUCCESS;
+}
+
+struct RedLayout {  // per-slot workspace carve-up (bytes)
+    size_t slot;    // sizeof(slot<T>), padded to 16
+    size_t o_res, o_seed, o_gather, o_fold, o_part, o_pvalid, o_aggv, o_incv, total;
+};
+RedLayout red_layout(const Module *m, int D, size_t G, size_t ntiles) {
+    RedLayout L{};
+    L.slot = align_up(m->sig[4], 16);
+    size_t o = 0;
+    L.o_res = o;
+    o += L.slot;
+    L.o_seed = o;
+    o += L.slot;
+    L.o_fold = o;
+    o += L.slot;
+    o = align_up(o, 256);
+    L.o_gather = o;
+    o = align_up(o + (size_t)D * L.slot, 256);
+    L.o_part = o;
+    o = align_up(o + G * L.slot, 256);
+    L.o_pvalid = o;
+    o = align_up(o + G * 4, 256);
+    L.o_aggv = o;
+    o = align_up(o + (m->sig[13] ? 0 : ntiles * L.slot), 256);
+    L.o_incv = o;
+    o = align_up(o + (m->sig[13] ? 0 : ntiles * L.slot), 256);
+    L.total = o;
+    return L;
+}
+int ensure_ws(skel_ctx_s *ctx, Slot &s, size_t bytes) {
+    if (s.ws_cap >= bytes) return SKEL_OK;
+    TRY(dev_free(ctx, s, s.ws));
+    s.ws = nullptr;
+    s.ws_cap = 0;
+    const size_t b = std::max<size_t>(bytes, 1 << 20);
+    TRY(dev_alloc(ctx, s, b, &s.ws));
+    s.ws_cap = b;
+    return SKEL_OK;
+}
+int ensure_status(skel_ctx_s *ctx, Slot &s, size_t ntiles, bool packed) {
+    DevGuard g(s.dev);
+    if (packed && s.st64_cap < ntiles) {
+        TRY(dev_free(ctx, s, reinterpret_cast<char *>(s.st64)));
+        char *p = nullptr;
+        TRY(dev_alloc(ctx, s, ntiles * 8, &p));
+        CK(ctx, cudaMemsetAsync(p, 0, ntiles * 8, s.stream));
+        s.st64 = reinterpret_cast<unsigned long long *>(p);
+        s.st64_cap = ntiles;
+    }
+    if (!packed && s.fl32_cap < ntiles) {
+        TRY(dev_free(ctx, s, reinterpret_cast<char *>(s.fl32)));
+        char *p = nullptr;
+        TRY(dev_alloc(ctx, s, ntiles * 4, &p));
+        CK(ctx, cudaMemsetAsync(p, 0, ntiles * 4, s.stream));
+        s.fl32 = reinterpret_cast<unsigned *>(p);
+        s.fl32_cap = ntiles;
+    }
+    return SKEL_OK;
+}
+int set_smem_attr(skel_ctx_s *ctx, Module *m, const Slot &s) {
+    if (m->attr_set_on.count(s.dev)) return SKEL_OK;
+    DevGuard g(s.dev);
+    const int dsm = (int)m->sig[11];
+    if (dsm > 0) {
+        CK(ctx, cudaFuncSetAttribute((const void *)m->k_main, cudaFuncAttributeMaxDynamicSharedMemorySize, dsm));
+        CK(ctx, cudaFuncSetAttribute((const void *)m->k_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, dsm));
+    }
+    m->attr_set_on.insert(s.dev);
+    return SKEL_OK;
+}
+
+// local reduce of the slot's data into ws[o_res]
+int launch_reduce(skel_ctx_s *ctx, Module *m, Slot &s, const void *in, uint64_t cnt, const RedLayout &L,
+                  std::vector<unsigned char> &abuf) {
+    const uint64_t TILE = m->sig[10];
+    const uint64_t nft = cnt / TILE;
+    const size_t G = (size_t)std::max<uint64_t>(1, std::min<uint64_t>((uint64_t)s.sms, nft));
+    CUtensorMap tin;
+    int use_tma = m->sig[5] && make_tmap(&tin, in, nft * m->sig[9]);
+    char *ws = s.ws;
+    void *partials = ws + L.o_part, *pvalid = ws + L.o_pvalid, *result = ws + L.o_res;
+    unsigned *counter = s.counters + 2;
+    void *params[] = {&tin, &in, &cnt, &use_tma, &partials, &pvalid, &counter, &result, abuf.data()};
+    DevGuard g(s.dev);
+    CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3((unsigned)G), dim3((unsigned)m->sig[9]), params,
+                             use_tma ? m->sig[11] : 0, s.stream));
+    ctx->stats.kernel_launches++;
+    return SKEL_OK;
+}
+
+size_t red_grid(const Module *m, const Slot &s, uint64_t cnt) {
+    return (size_t)std::max<uint64_t>(1, std::min<uint64_t>((uint64_t)s.sms, cnt / m->sig[10]));
+}
+
+// Reduce of `in` leaving the result in every local slot's ws[o_fold]
+// (cross-device: gather of the D partials + ordered fold)
+int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args, int nargs,
+                std::vector<RedLayout> &Ls) {
+    const int D = ctx->D;
+    const bool cross = D > 1 && in->dist == SKEL_BLOCK;
+    std::vector<unsigned char> abuf;
+    Ls.resize(ctx->slots.size());
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        const uint64_t cnt = in->bufs[li].count;
+        Ls[li] = red_layout(m, D, red_grid(m, s, cnt), 0);
+        TRY(ensure_ws(ctx, s, Ls[li].total));
+        TRY(set_smem_attr(ctx, m, s));
+        pack_args(m, args, nargs, li, abuf);
+        if (cnt) TRY(launch_reduce(ctx, m, s, in->bufs[li].ptr(in->es), cnt, Ls[li], abuf));
+    }
+    const size_t es = m->sig[4];
+    const size_t ps = part_size(in->n, D);
+    const int K = cross ? (int)((in->n + ps - 1) / ps) : 1;  // devices holding data
+    if (cross && !ctx->rank_mode) {
+        TRY(join(ctx));
+        std::vector<const void *> src(K);
+        for (int j = 0; j < K; ++j) src[j] = ctx->slots[j].ws + Ls[j].o_res;
+        for (size_t li = 0; li < ctx->slots.size(); ++li) {
+            Slot &s = ctx->slots[li];
+            DevGuard g(s.dev);
+            CK(ctx, launch_gather(s.ws + Ls[li].o_gather, src.data(), K, Ls[li].slot, s.stream));
+            ctx->stats.kernel_launches++;
+        }
+        TRY(join(ctx));
+    } else if (cross) {
+        Slot &s = ctx->slots[0];
+        DevGuard g(s.dev);
+        NK(ctx, ncclAllGather(s.ws + Ls[0].o_res, s.ws + Ls[0].o_gather, Ls[0].slot, ncclUint8, ctx->comm, s.stream));
+        ctx->stats.nccl_bytes += Ls[0].slot * D;
+    }
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        const RedLayout &L = Ls[li];
+        DevGuard g(s.dev);
+        if (cross) {
+            pack_args(m, args, nargs, li, abuf);
+            const void *vals = s.ws + L.o_gather;
+            void *outp = s.ws + L.o_fold;
+            int k = K;
+            void *params[] = {&vals, &k, &outp, abuf.data()};
+            CK(ctx, cudaLaunchKernel((const void *)m->k_fold, dim3(1), dim3(32), params, 0, s.stream));
+            ctx->stats.kernel_launches++;
+        } else if (in->bufs[li].count) {
+            CK(ctx, cudaMemcpyAsync(s.ws + L.o_fold, s.ws + L.o_res, es, cudaMemcpyDeviceToDevice, s.stream));
+        }
+    }
+    return SKEL_OK;
+}
+
+// make every local device's ws[o_fold] hold the Reduce result
+int finish_scalar(skel_ctx_s *ctx, skel_vec_s *in, const std::vector<RedLayout> &Ls) {
+    const bool cross = ctx->D > 1 && in->dist == SKEL_BLOCK;
+    if (cross || ctx->D == 1 || in->dist == SKEL_COPY) return SKEL_OK;
+    // SINGLE on several devices: only logical device 0 computed
+    if (ctx->rank_mode) {
+        Slot &s = ctx->slots[0];
+        DevGuard g(s.dev);
+        char *p = s.ws + Ls[0].o_fold;
+        NK(ctx, ncclBroadcast(p, p, in->es, ncclUint8, 0, ctx->comm, s.stream));
+        ctx->stats.nccl_bytes += in->es;
+        return SKEL_OK;
+    }
+    TRY(join(ctx));
+    for (size_t li = 1; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        DevGuard g(s.dev);
+        CK(ctx, cudaMemcpyAsync(s.ws + Ls[li].o_fold, ctx->slots[0].ws + Ls[0].o_fold, in->es, cudaMemcpyDefault,
+                                s.stream));
+    }
+    return join(ctx);
+}
+
+int check_red(skel_ctx_s *ctx, Module *m, skel_vec_s *in) {
+    if (m->sig[3] != in->es)
+        return fail(ctx, SKEL_ERR_TYPE, "element size " + std::to_string(in->es) + " != sizeof(T) = " +
+                                            std::to_string(m->sig[3]));
+    return SKEL_OK;
+}
+
+}  // namespace
+
+// =============================================================================
+// C-ABI
+// =============================================================================
+extern "C" {
+
+const char *skel_status_string(int st) {
+    switch (st) {
+        case SKEL_OK: return "SKEL_OK";
+        case SKEL_ERR_ARG: return "SKEL_ERR_ARG";
+        case SKEL_ERR_SIZE: return "SKEL_ERR_SIZE";
+        case SKEL_ERR_TYPE: return "SKEL_ERR_TYPE";
+        case SKEL_ERR_COMPILE: return "SKEL_ERR_COMPILE";
+        case SKEL_ERR_CUDA: return "SKEL_ERR_CUDA";
+        case SKEL_ERR_NCCL: return "SKEL_ERR_NCCL";
+        case SKEL_ERR_OOM: return "SKEL_ERR_OOM";
+        case SKEL_ERR_STATE: return "SKEL_ERR_STATE";
+        default: return "SKEL_ERR_UNKNOWN";
+    }
+}
+
+const char *skel_last_error(skel_ctx_t ctx) { return ctx ? ctx->last_error.c_str() : g_last_error.c_str(); }
+
+static int init_slot(skel_ctx_s *ctx, int d, int dev) {
+    Slot s;
+    s.d = d;
+    s.dev = dev;
+    DevGuard g(dev);
+    CK(ctx, cudaDeviceGetAttribute(&s.sms, cudaDevAttrMultiProcessorCount, dev));
+    CK(ctx, cudaStreamCreateWithFlags(&s.stream, cudaStreamNonBlocking));
+    CK(ctx, cudaEventCreateWithFlags(&s.ev, cudaEventDisableTiming));
+    void *p = nullptr;
+    CK(ctx, cudaMalloc(&p, 256));
+    CK(ctx, cudaMemset(p, 0, 256));
+    s.counters = static_cast<unsigned *>(p);
+    ctx->slots.push_back(s);
+    return SKEL_OK;
+}
+
+static void ctx_defaults(skel_ctx_s *ctx) {
+    const char *f = getenv("SKEL_FMAD");
+    ctx->fmad = f && atoi(f) != 0;
+    const char *b = getenv("SKEL_BLOCK_SIZE");
+    if (b) ctx->block_size = atoi(b);
+}
+
+int skel_init(int num_devices, skel_ctx_t *out) {
+    if (!out) return fail(nullptr, SKEL_ERR_ARG, "out is NULL");
+    int ngpu = 0;
+    cudaError_t e = cudaGetDeviceCount(&ngpu);
+    if (e != cudaSuccess || ngpu == 0) {
+        cudaGetLastError();
+        return fail(nullptr, SKEL_ERR_CUDA,
+                    std::string("no CUDA device: ") + (e != cudaSuccess ? cudaGetErrorString(e) : "0 devices"));
+    }
+    const int D = num_devices < 0 ? ngpu : num_devices;
+    if (D < 1 || D > 64) return fail(nullptr, SKEL_ERR_ARG, "num_devices must be -1 or 1..64");
+    auto *ctx = new skel_ctx_s();
+    ctx_defaults(ctx);
+    ctx->D = D;
+    for (int d = 0; d < D; ++d) {
+        int st = init_slot(ctx, d, d % ngpu);
+        if (st != SKEL_OK) {
+            g_last_error = ctx->last_error;
+            delete ctx;
+            return st;
+        }
+    }
+    // peer access between distinct physical devices (NVLink / NVSwitch)
+    for (auto &a : ctx->slots)
+        for (auto &b : ctx->slots)
+            if (a.dev != b.dev) {
+                int can = 0;
+                cudaDeviceCanAccessPeer(&can, a.dev, b.dev);
+                if (can) {
+                    DevGuard g(a.dev);
+                    if (cudaDeviceEnablePeerAccess(b.dev, 0) != cudaSuccess) cudaGetLastError();
+                }
+            }
+    *out = ctx;
+    return SKEL_OK;
+}
+
+int skel_get_unique_id(void *id) {
+    if (!id) return fail(nullptr, SKEL_ERR_ARG, "id is NULL");
+    ncclUniqueId u;
+    ncclResult_t r = ncclGetUniqueId(&u);
+    if (r != ncclSuccess) return fail(nullptr, SKEL_ERR_NCCL, ncclGetErrorString(r));
+    static_assert(sizeof(u) == 128, "ncclUniqueId is 128 bytes");
+    memcpy(id, &u, sizeof u);
+    return SKEL_OK;
+}
+
+int skel_init_rank(int rank, int world, int cuda_device, const void *id, skel_ctx_t *out) {
+    if (!out || world < 1 || rank < 0 || rank >= world) return fail(nullptr, SKEL_ERR_ARG, "bad rank/world");
+    if (world > 1 && !id) return fail(nullptr, SKEL_ERR_ARG, "nccl id required for world > 1");
+    int ngpu = 0;
+    cudaError_t e = cudaGetDeviceCount(&ngpu);
+    if (e != cudaSuccess || ngpu == 0 || cuda_device < 0 || cuda_device >= ngpu) {
+        cudaGetLastError();
+        return fail(nullptr, SKEL_ERR_CUDA, "no such CUDA device");
+    }
+    auto *ctx = new skel_ctx_s();
+    ctx_defaults(ctx);
+    ctx->D = world;
+    ctx->rank_mode = true;
+    ctx->rank = rank;
+    int st = init_slot(ctx, rank, cuda_device);
+    if (st == SKEL_OK && world > 1) {
+        ncclUniqueId u;
+        memcpy(&u, id, sizeof u);
+        DevGuard g(cuda_device);
+        ncclResult_t r = ncclCommInitRank(&ctx->comm, world, u, rank);
+        if (r != ncclSuccess) st = fail(ctx, SKEL_ERR_NCCL, std::string("ncclCommInitRank: ") + ncclGetErrorString(r));
+    }
+    if (st != SKEL_OK) {
+        g_last_error = ctx->last_error;
+        delete ctx;
+        return st;
+    }
+    *out = ctx;
+    return SKEL_OK;
+}
+
+int skel_vector_destroy(skel_vec_t v);
+
+int skel_finalize(skel_ctx_t ctx) {
+    if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
+    sync_all(ctx);
+    std::vector<skel_vec_s *> vs(ctx->vecs.begin(), ctx->vecs.end());
+    for (auto *v : vs) skel_vector_destroy(v);
+    for (auto &kv : ctx->modules)
+        if (kv.second->lib) cudaLibraryUnload(kv.second->lib);
+    if (ctx->comm) ncclCommDestroy(ctx->comm);
+    for (auto &s : ctx->slots) {
+        DevGuard g(s.dev);
+        cudaFree(s.ws);
+        cudaFree(s.scratch);
+        cudaFree(s.counters);
+        cudaFree(s.st64);
+        cudaFree(s.fl32);
+        cudaEventDestroy(s.ev);
+        cudaStreamDestroy(s.stream);
+    }
+    delete ctx;
+    return SKEL_OK;
+}
+
+int skel_num_devices(skel_ctx_t ctx, int *D, int *L) {
+    if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
+    if (D) *D = ctx->D;
+    if (L) *L = (int)ctx->slots.size();
+    return SKEL_OK;
+}
+
+int skel_get_stream(skel_ctx_t ctx, int li, void **stream) {
+    if (!ctx || !stream || li < 0 || li >= (int)ctx->slots.size()) return fail(ctx, SKEL_ERR_ARG, "bad local index");
+    *stream = ctx->slots[li].stream;
+    return SKEL_OK;
+}
+
+int skel_set_block_size(skel_ctx_t ctx, int threads) {
+    if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
+    if (threads != 0 && (threads < 32 || threads > 1024 || threads % 32))
+        return fail(ctx, SKEL_ERR_ARG, "block size must be 0 or a multiple of 32 in [32, 1024]");
+    ctx->block_size = threads;
+    return SKEL_OK;
+}
+
+int skel_set_cache_dir(skel_ctx_t ctx, const char *dir) {
+    if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
+    if (!dir) {
+        ctx->cache_dir.clear();
+        ctx->disk_cache = true;
+    } else if (!*dir) {
+        ctx->disk_cache = false;
+    } else {
+        ctx->cache_dir = dir;
+        ctx->disk_cache = true;
+    }
+    return SKEL_OK;
+}
+
+int skel_clear_kernel_cache(skel_ctx_t ctx) {
+    if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
+    TRY(sync_all(ctx));
+    for (auto &kv : ctx->modules)
+        if (kv.second->lib) cudaLibraryUnload(kv.second->lib);
+    ctx->modules.clear();
+    return SKEL_OK;
+}
+
+int skel_sync(skel_ctx_t ctx) {
+    if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
+    return sync_all(ctx);
+}
+
+int skel_get_stats(skel_ctx_t ctx, skel_stats *out) {
+    if (!ctx || !out) return fail(ctx, SKEL_ERR_ARG, "NULL argument");
+    *out = ctx->stats;
+    return SKEL_OK;
+}
+
+int skel_reset_stats(skel_ctx_t ctx) {
+    if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
+    ctx->stats = skel_stats{};
+    return SKEL_OK;
+}
+
+// ---- vectors -------------------------------------------------------------------
+int skel_vector_create(skel_ctx_t ctx, size_t n, size_t es, skel_vec_t *out) {
+    if (!ctx || !out || es == 0) return fail(ctx, SKEL_ERR_ARG, "bad vector arguments");
+    auto *v = new skel_vec_s();
+    v->ctx = ctx;
+    v->n = n;
+    v->es = es;
+    v->dist = ctx->D == 1 ? SKEL_SINGLE : SKEL_BLOCK;
+    v->bufs.resize(ctx->slots.size());
+    int st = place(v, v->dist);
+    for (size_t li = 0; st == SKEL_OK && li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        Buf &b = v->bufs[li];
+        DevGuard g(s.dev);
+        if (b.cap) {
+            cudaError_t e = cudaMemsetAsync(b.base, 0, b.cap, s.stream);
+            if (e != cudaSuccess) st = fail(ctx, SKEL_ERR_CUDA, cudaGetErrorString(e));
+        }
+    }
+    if (st != SKEL_OK) {
+        for (size_t li = 0; li < v->bufs.size(); ++li) dev_free(ctx, ctx->slots[li], v->bufs[li].base);
+        delete v;
+        return st;
+    }
+    v->dev_valid = true;
+    v->host_valid = false;
+    ctx->vecs.insert(v);
+    *out = v;
+    return SKEL_OK;
+}
+
+int skel_vector_destroy(skel_vec_t v) {
+    if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
+    skel_ctx_s *ctx = v->ctx;
+    for (size_t li = 0; li < v->bufs.size(); ++li) dev_free(ctx, ctx->slots[li], v->bufs[li].base);
+    if (v->host) cudaFreeHost(v->host);
+    ctx->vecs.erase(v);
+    delete v;
+    return SKEL_OK;
+}
+
+int skel_vector_set_dtype(skel_vec_t v, skel_dtype dt) {
+    if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
+    static const size_t sz[] = {0, 4, 8, 4, 4, 8, 8};
+    if ((int)dt < 0 || (int)dt > 6) return fail(v->ctx, SKEL_ERR_ARG, "bad dtype");
+    if (dt != SKEL_DT_OPAQUE && sz[dt] != v->es) return fail(v->ctx, SKEL_ERR_TYPE, "dtype size != elem_size");
+    v->dt = dt;
+    return SKEL_OK;
+}
+
+int skel_vector_size(skel_vec_t v, size_t *n, size_t *es) {
+    if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
+    if (n) *n = v->n;
+    if (es) *es = v->es;
+    return SKEL_OK;
+}
+
+int skel_vector_upload(skel_vec_t v, const void *src, size_t n) {
+    if (!v || (!src && n)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad upload arguments");
+    if (n != v->n) return fail(v->ctx, SKEL_ERR_SIZE, "upload length != vector length");
+    TRY(host_mirror(v));
+    // the host mirror may still be the source of an in-flight H2D copy
+    TRY(sync_all(v->ctx));
+    if (n) memcpy(v->host, src, n * v->es);
+    v->host_valid = true;
+    v->dev_valid = false;  // H2D deferred until a skeleton needs the data
+    v->diverged = false;
+    return SKEL_OK;
+}
+
+int skel_vector_download(skel_vec_t v, void *dst, size_t n) {
+    if (!v || (!dst && n)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad download arguments");
+    if (n != v->n) return fail(v->ctx, SKEL_ERR_SIZE, "download length != vector length");
+    TRY(ensure_host(v));
+    if (n) memcpy(dst, v->host, n * v->es);
+    return SKEL_OK;
+}
+
+int skel_vector_host_ptr(skel_vec_t v, void **host) {
+    if (!v || !host) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad arguments");
+    TRY(ensure_host(v));
+    *host = v->host;
+    return SKEL_OK;
+}
+
+int skel_vector_mark_host_modified(skel_vec_t v) {
+    if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
+    if (!v->host) return fail(v->ctx, SKEL_ERR_STATE, "vector has no host mirror (call skel_vector_host_ptr)");
+    v->host_valid = true;
+    v->dev_valid = false;
+    v->diverged = false;
+    return SKEL_OK;
+}
+
+int skel_vector_fill(skel_vec_t v, const void *value) {
+    if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
+    return skel_vector_fill_dist(v, v->dist, value);
+}
+
+int skel_vector_fill_dist(skel_vec_t v, skel_dist dist, const void *value) {
+    if (!v || !value || (int)dist < 0 || (int)dist > 2)
+        return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad fill arguments");
+    skel_ctx_s *ctx = v->ctx;
+    v->dist = dist;  // old contents are discarded: no exchange needed
+    if (v->es > 64) return fail(ctx, SKEL_ERR_TYPE, "fill supports elements up to 64 bytes");
+    TRY(place(v, v->dist));
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        Buf &b = v->bufs[li];
+        if (!b.count) continue;
+        DevGuard g(s.dev);
+        CK(ctx, launch_fill(b.ptr(v->es), b.count, value, v->es, s.stream));
+        ctx->stats.kernel_launches++;
+    }
+    v->dev_valid = true;
+    v->host_valid = false;
+    v->diverged = false;
+    return SKEL_OK;
+}
+
+int skel_vector_set_distribution(skel_vec_t v, skel_dist dist, skel_combine combine) {
+    if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
+    if ((int)dist < 0 || (int)dist > 2 || (int)combine < 0 || (int)combine > 4)
+        return fail(v->ctx, SKEL_ERR_ARG, "bad distribution or combine");
+    return set_distribution(v, dist, combine);
+}
+
+int skel_vector_get_distribution(skel_vec_t v, skel_dist *dist) {
+    if (!v || !dist) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad arguments");
+    *dist = v->dist;
+    return SKEL_OK;
+}
+
+int skel_vector_mark_device_modified(skel_vec_t v) {
+    if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
+    TRY(ensure_device(v));
+    v->host_valid = false;
+    if (v->dist == SKEL_COPY && v->ctx->D > 1) v->diverged = true;
+    return SKEL_OK;
+}
+
+int skel_vector_part(skel_vec_t v, int d, size_t *lo, size_t *hi) {
+    if (!v || !lo || !hi || d < 0 || d >= v->ctx->D) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad arguments");
+    if (v->dist == SKEL_BLOCK) {
+        part_range(v->n, v->ctx->D, d, lo, hi);
+    } else if (v->dist == SKEL_COPY || d == 0) {
+        *lo = 0;
+        *hi = v->n;
+    } else {
+        *lo = *hi = 0;
+    }
+    return SKEL_OK;
+}
+
+int skel_vector_device_ptr(skel_vec_t v, int li, void **ptr, size_t *count) {
+    if (!v || li < 0 || li >= (int)v->bufs.size()) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad arguments");
+    TRY(ensure_device(v));
+    if (ptr) *ptr = v->bufs[li].ptr(v->es);
+    if (count) *count = v->bufs[li].count;
+    return SKEL_OK;
+}
+
+// ---- skeletons -------------------------------------------------------------------
+int skel_map(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, const skel_arg *args, int nargs) {
+    if (!ctx || !src || !in || in->ctx != ctx || (out && out->ctx != ctx) || (nargs && !args) || nargs < 0)
+        return fail(ctx, SKEL_ERR_ARG, "bad map arguments");
+    return run_ew(ctx, Kind::Map, src, in, nullptr, out, args, nargs);
+}
+
+int skel_zip(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_vec_t out, const skel_arg *args,
+             int nargs) {
+    if (!ctx || !src || !a || !b || !out || a->ctx != ctx || b->ctx != ctx || out->ctx != ctx || (nargs && !args) ||
+        nargs < 0)
+        return fail(ctx, SKEL_ERR_ARG, "bad zip arguments");
+    if (a->n != b->n) return fail(ctx, SKEL_ERR_SIZE, "zip: vectors of unequal length (P:L268-269)");
+    return run_ew(ctx, Kind::Zip, src, a, b, out, args, nargs);
+}
+
+int skel_reduce_to(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t result, const skel_arg *args,
+                   int nargs) {
+    if (!ctx || !src || !in || !result || in->ctx != ctx || result->ctx != ctx || (nargs && !args) || nargs < 0)
+        return fail(ctx, SKEL_ERR_ARG, "bad reduce arguments");
+    if (in->n == 0) return fail(ctx, SKEL_ERR_SIZE, "reduce of an empty vector (eq. 3 has no identity)");
+    Module *m = nullptr;
+    TRY(get_module(ctx, Kind::Red, src, &m));
+    TRY(check_red(ctx, m, in));
+    if (result->es != in->es) return fail(ctx, SKEL_ERR_TYPE, "result element size != input element size");
+    TRY(check_args(ctx, m, args, nargs));
+    TRY(ensure_device(in));
+    std::vector<RedLayout> Ls;
+    TRY(reduce_core(ctx, m, in, args, nargs, Ls));
+    TRY(finish_scalar(ctx, in, Ls));
+    // the result is a 1-element vector with a copy on every local device
+    if (result->n != 1) {
+        result->n = 1;
+        if (result->host) {
+            cudaFreeHost(result->host);
+            result->host = nullptr;
+        }
+    }
+    result->dist = SKEL_COPY;
+    TRY(place(result, SKEL_COPY));
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        DevGuard g(s.dev);
+        CK(ctx, cudaMemcpyAsync(result->bufs[li].ptr(result->es), s.ws + Ls[li].o_fold, in->es,
+                                cudaMemcpyDeviceToDevice, s.stream));
+    }
+    result->dev_valid = true;
+    result->host_valid = false;
+    result->diverged = false;
+    return SKEL_OK;
+}
+
+int skel_reduce(skel_ctx_t ctx, const char *src, skel_vec_t in, void *result_host, const skel_arg *args, int nargs) {
+    if (!ctx || !src || !in || !result_host || in->ctx != ctx || (nargs && !args) || nargs < 0)
+        return fail(ctx, SKEL_ERR_ARG, "bad reduce arguments");
+    if (in->n == 0) return fail(ctx, SKEL_ERR_SIZE, "reduce of an empty vector (eq. 3 has no identity)");
+    Module *m = nullptr;
+    TRY(get_module(ctx, Kind::Red, src, &m));
+    TRY(check_red(ctx, m, in));
+    TRY(check_args(ctx, m, args, nargs));
+    TRY(ensure_device(in));
+    std::vector<RedLayout> Ls;
+    TRY(reduce_core(ctx, m, in, args, nargs, Ls));
+    TRY(finish_scalar(ctx, in, Ls));
+    // Scalar::getValue
+    Slot &s = ctx->slots[0];
+    DevGuard g(s.dev);
+    CK(ctx, cudaMemcpyAsync(result_host, s.ws + Ls[0].o_fold, in->es, cudaMemcpyDeviceToHost, s.stream));
+    ctx->stats.d2h_bytes += in->es;
+    ctx->stats.d2h_copies++;
+    return sync_all(ctx);
+}
+
+int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, const void *identity,
+              const skel_arg *args, int nargs) {
+    if (!ctx || !src || !in || !out || !identity || in->ctx != ctx || out->ctx != ctx || (nargs && !args) ||
+        nargs < 0)
+        return fail(ctx, SKEL_ERR_ARG, "bad scan arguments");
+    Module *m = nullptr;
+    TRY(get_module(ctx, Kind::Red, src, &m));
+    TRY(check_red(ctx, m, in));
+    if (out->es != in->es) return fail(ctx, SKEL_ERR_TYPE, "output element size != input element size");
+    TRY(check_args(ctx, m, args, nargs));
+    TRY(ensure_device(in));
+    TRY(prepare_output(out, in->n, in->dist, out == in));
+    if (in->n == 0) return SKEL_OK;
+    const int D = ctx->D;
+    const bool cross = D > 1 && in->dist == SKEL_BLOCK;
+    std::vector<RedLayout> Ls(ctx->slots.size());
+    std::vector<unsigned char> abuf;
+    // seeds: device k starts from agg_0 (+) ... (+) agg_{k-1} (one exchange of
+    // D partial results)
+    const uint64_t TILE = m->sig[10];
+    const bool packed = m->sig[13] != 0;
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        const uint64_t cnt = in->bufs[li].count;
+        Ls[li] = red_layout(m, D, red_grid(m, s, cnt), (cnt + TILE - 1) / TILE);
+        TRY(ensure_ws(ctx, s, Ls[li].total));
+    }
+    if (cross) {
+        std::vector<RedLayout> Lr;
+        TRY(reduce_core(ctx, m, in, args, nargs, Lr));
+    }
+    if (++ctx->scan_epoch >= (1u << 30) - 1) {
+        ctx->scan_epoch = 1;
+        for (auto &s : ctx->slots) {
+            DevGuard g(s.dev);
+            if (s.st64) CK(ctx, cudaMemsetAsync(s.st64, 0, s.st64_cap * 8, s.stream));
+            if (s.fl32) CK(ctx, cudaMemsetAsync(s.fl32, 0, s.fl32_cap * 4, s.stream));
+        }
+    }
+    unsigned epoch = ctx->scan_epoch;
+    std::vector<unsigned char> idbuf(align_up(m->sig[4], 16), 0);
+    memcpy(idbuf.data(), identity, in->es);
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        uint64_t cnt = in->bufs[li].count;
+        if (!cnt) continue;
+        const uint64_t ntiles = (cnt + TILE - 1) / TILE;
+        const size_t G = (size_t)std::max<uint64_t>(1, std::min<uint64_t>((uint64_t)s.sms, ntiles));
+        const RedLayout &L = Ls[li];
+        TRY(ensure_status(ctx, s, ntiles, packed));
+        TRY(set_smem_attr(ctx, m, s));
+        pack_args(m, args, nargs, li, abuf);
+        DevGuard g(s.dev);
+        const void *seed = nullptr;
+        if (cross) {
+            const void *aggs = s.ws + L.o_gather;
+            int k = s.d;
+            void *seedp = s.ws + L.o_seed;
+            void *params[] = {&aggs, &k, idbuf.data(), &seedp, abuf.data()};
+            CK(ctx, cudaLaunchKernel((const void *)m->k_seed, dim3(1), dim3(32), params, 0, s.stream));
+            ctx->stats.kernel_launches++;
+            seed = seedp;
+        }
+        const void *pin = in->bufs[li].ptr(in->es);
+        void *pout = out->bufs[li].ptr(out->es);
+        CUtensorMap tin, tout;
+        const uint64_t rows = (cnt / TILE) * m->sig[9];
+        int use_tma = m->sig[5] && make_tmap(&tin, pin, rows) && make_tmap(&tout, pout, rows);
+        void *status = s.st64, *flags = s.fl32, *aggv = s.ws + L.o_aggv, *incv = s.ws + L.o_incv;
+        unsigned *counters = s.counters;
+        void *total = nullptr;
+        void *params[] = {&tin, &tout, &pin, &pout, &cnt, &use_tma, idbuf.data(), &seed, &status, &flags,
+                          &aggv, &incv, &counters, &epoch, &total, abuf.data()};
+        CK(ctx, cudaLaunchKernel((const void *)m->k_scan, dim3((unsigned)G), dim3((unsigned)m->sig[9]), params,
+                                 use_tma ? m->sig[11] : 0, s.stream));
+        ctx->stats.kernel_launches++;
+    }
+    out->dev_valid = true;
+    out->host_valid = false;
+    return SKEL_OK;
+}
+
+int skel_prepare(skel_ctx_t ctx, const char *kind, const char *src) {
+    if (!ctx || !kind || !src) return fail(ctx, SKEL_ERR_ARG, "bad arguments");
+    Kind k;
+    if (!strcmp(kind, "map")) k = Kind::Map;
+    else if (!strcmp(kind, "zip")) k = Kind::Zip;
+    else if (!strcmp(kind, "reduce") || !strcmp(kind, "scan")) k = Kind::Red;
+    else return fail(ctx, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan");
+    Module *m = nullptr;
+    return get_module(ctx, k, src, &m);
+}
+
+// ---- pure host logic -------------------------------------------------------------
+int skel_entry_name(const char *src, char *name, size_t cap) {
+    if (!src || !name || cap == 0) return fail(nullptr, SKEL_ERR_ARG, "bad arguments");
+    std::string err;
+    std::string e = entry_name(src, &err);
+    if (e.empty()) return fail(nullptr, SKEL_ERR_COMPILE, err);
+    if (e.size() + 1 > cap) return fail(nullptr, SKEL_ERR_SIZE, "name buffer too small");
+    memcpy(name, e.c_str(), e.size() + 1);
+    return SKEL_OK;
+}
+
+int skel_compile_check(const char *kind, const char *src, int fmad, char *log, size_t cap, size_t *cubin_bytes) {
+    if (!kind || !src) return fail(nullptr, SKEL_ERR_ARG, "bad arguments");
+    Kind k;
+    if (!strcmp(kind, "map")) k = Kind::Map;
+    else if (!strcmp(kind, "zip")) k = Kind::Zip;
+    else if (!strcmp(kind, "reduce") || !strcmp(kind, "scan")) k = Kind::Red;
+    else return fail(nullptr, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan");
+    std::string l;
+    std::vector<char> cubin;
+    const int st = compile_only(k, src, 256, fmad != 0, &l, &cubin);
+    if (log && cap) {
+        const size_t m = std::min(cap - 1, l.size());
+        memcpy(log, l.data(), m);
+        log[m] = 0;
+    }
+    if (cubin_bytes) *cubin_bytes = cubin.size();
+    if (st != SKEL_OK) g_last_error = l;
+    const char *dump = getenv("SKEL_DUMP_CUBIN");  // inspection: cuobjdump -sass / -res-usage
+    if (st == SKEL_OK && dump && *dump) {
+        FILE *f = fopen(dump, "wb");
+        if (f) {
+            fwrite(cubin.data(), 1, cubin.size(), f);
+            fclose(f);
+        }
+    }
+    return st;
+}
+
+int skel_plan_part(size_t n, int D, int k, size_t *lo, size_t *hi) {
+    if (D < 1 || k < 0 || k >= D || !lo || !hi) return fail(nullptr, SKEL_ERR_ARG, "bad arguments");
+    part_range(n, D, k, lo, hi);
+    return SKEL_OK;
+}
+
+int skel_plan_exchange(skel_dist from, skel_dist to, skel_combine combine, int *xchg) {
+    if (!xchg || (int)from < 0 || (int)from > 2 || (int)to < 0 || (int)to > 2 || (int)combine < 0 || (int)combine > 4)
+        return fail(nullptr, SKEL_ERR_ARG, "bad arguments");
+    const int x = plan_exchange(from, to, combine);
+    if (x < 0) return fail(nullptr, SKEL_ERR_STATE, "combine requires a copy-distributed source");
+    *xchg = x;
+    return SKEL_OK;
+}
+
+}  // extern "C"

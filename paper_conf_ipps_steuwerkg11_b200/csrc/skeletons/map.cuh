@@ -1,0 +1,208 @@
+// map.cuh -- Map (eq. (1)) and Zip (eq. (2))
+// skeleton kernel, instantiated by NVRTC for the user function SKEL_FN.
+//
+//   SKEL_NIN == 1:  out[i] = SKEL_FN(a[i], args...)        (void: side effects only)
+//   SKEL_NIN == 2:  out[i] = SKEL_FN(a[i], b[i], args...)
+//
+// B200 mapping (kernel K1): the vector is walked in "chunks" of
+// E consecutive elements, E chosen so one chunk of every operand is one
+// naturally aligned load/store of <= 16 bytes (LDG.E.128 / STG.E.128 for
+// 4-byte elements).  Each thread keeps SKEL_UNROLL chunks in flight
+// (grid-stride loop; the grid is sized by the host to a multiple of the SM
+// count).  Streaming cache hints (.nc / L1::no_allocate loads, .cs stores)
+// keep single-use data from displacing the L2 lines that user functions
+// gather through vector arguments.  Elements whose size is not a power of
+// two, and unaligned views, take the scalar path.
+
+#ifndef SKEL_NIN
+#define SKEL_NIN 1
+#endif
+#ifndef SKEL_BLOCK
+#define SKEL_BLOCK 256
+#endif
+#ifndef SKEL_UNROLL
+#define SKEL_UNROLL 4
+#endif
+
+using skel_F = decltype(&SKEL_FN);
+using skel_FT = skel::fn<skel_F>;
+static_assert(skel_FT::arity >= SKEL_NIN, "user function has too few parameters for this skeleton");
+using skel_A = typename skel_FT::template param<0>;
+#if SKEL_NIN == 2
+using skel_B = typename skel_FT::template param<1>;
+#else
+using skel_B = skel_A;
+#endif
+using skel_R = typename skel_FT::ret;
+constexpr bool skel_void = skel::is_void<skel_R>::value;
+struct skel_none { unsigned char b; };
+template <bool V, class R> struct skel_out_t { using type = skel::decay_t<R>; };
+template <class R> struct skel_out_t<true, R> { using type = skel_none; };
+using skel_O = typename skel_out_t<skel_void, skel_R>::type;
+
+using skel_Args = typename skel::drop<SKEL_NIN, typename skel_FT::params>::type;
+using skel_Lay = skel::args_layout<skel_Args>;
+constexpr skel_u64 SKEL_ARGBYTES = skel::cmax<skel_u64>(16, skel::align_up(skel_Lay::bytes, 16));
+using skel_Buf = skel::argbuf<SKEL_ARGBYTES>;
+using skel_Seq = typename skel::make_iseq<skel_Lay::n>::type;
+
+// ---- chunking ------------------------------------------------------------
+constexpr skel_u64 skel_szA = sizeof(skel_A);
+constexpr skel_u64 skel_szB = (SKEL_NIN == 2) ? sizeof(skel_B) : 1;
+constexpr skel_u64 skel_szO = skel_void ? 1 : sizeof(skel_O);
+constexpr skel_u64 skel_maxsz = skel::cmax(skel_szA, skel::cmax(skel_szB, skel_szO));
+constexpr bool skel_vec_ok = skel::pow2(skel_szA) && skel::pow2(skel_szB) && skel::pow2(skel_szO) && skel_maxsz <= 16;
+#ifndef SKEL_ITEMS
+constexpr int SKEL_E = skel_vec_ok ? (int)(16 / skel_maxsz) : 1;
+#else
+constexpr int SKEL_E = skel_vec_ok ? (SKEL_ITEMS < (int)(16 / skel_maxsz) ? SKEL_ITEMS : (int)(16 / skel_maxsz)) : 1;
+#endif
+
+// ---- signature table, read back by the host once per loaded module ------
+// [0] layout version  [1] NIN  [2] arity  [3] sizeof ret (0 = void)
+// [4] sizeof a  [5] sizeof b  [6] #extra args  [7] arg buffer bytes
+// [8] E (elements per chunk)  [9] block  [10..15] reserved
+// [16 + 4i ..] extra arg i: size, align, is_pointer, offset
+struct skel_sig_t { skel_u64 v[16 + 4 * 32]; };
+constexpr skel_sig_t skel_make_sig() {
+    skel_sig_t s{};
+    s.v[0] = 1;
+    s.v[1] = SKEL_NIN;
+    s.v[2] = skel_FT::arity;
+    s.v[3] = skel_void ? 0 : sizeof(skel_O);
+    s.v[4] = sizeof(skel_A);
+    s.v[5] = (SKEL_NIN == 2) ? sizeof(skel_B) : 0;
+    s.v[6] = skel_Lay::n;
+    s.v[7] = SKEL_ARGBYTES;
+    s.v[8] = SKEL_E;
+    s.v[9] = SKEL_BLOCK;
+    for (int i = 0; i < skel_Lay::n && i < 32; ++i) {
+        s.v[16 + 4 * i] = skel_Lay::size(i);
+        s.v[17 + 4 * i] = skel_Lay::align(i);
+        s.v[18 + 4 * i] = skel_Lay::isptr(i);
+        s.v[19 + 4 * i] = skel_Lay::off(i);
+    }
+    return s;
+}
+extern "C" __device__ skel_sig_t skel_sig = skel_make_sig();
+
+// ---- streaming loads / stores of one chunk ---------------------------------
+template <int N> __device__ __forceinline__ skel::chunk<N> skel_ld(const void *p) {
+    skel::chunk<N> c;
+    if constexpr (N == 16) {
+        asm volatile("ld.global.nc.L1::no_allocate.v4.u32 {%0,%1,%2,%3}, [%4];"
+                     : "=r"(c.v.x), "=r"(c.v.y), "=r"(c.v.z), "=r"(c.v.w)
+                     : "l"(p));
+    } else if constexpr (N == 8) {
+        asm volatile("ld.global.nc.L1::no_allocate.v2.u32 {%0,%1}, [%2];" : "=r"(c.v.x), "=r"(c.v.y) : "l"(p));
+    } else if constexpr (N == 4) {
+        asm volatile("ld.global.nc.L1::no_allocate.u32 %0, [%1];" : "=r"(c.v) : "l"(p));
+    } else {
+        c = *reinterpret_cast<const skel::chunk<N> *>(p);
+    }
+    return c;
+}
+template <int N> __device__ __forceinline__ void skel_st(void *p, const skel::chunk<N> &c) {
+    if constexpr (N == 16) {
+        asm volatile("st.global.cs.v4.u32 [%0], {%1,%2,%3,%4};" ::"l"(p), "r"(c.v.x), "r"(c.v.y), "r"(c.v.z),
+                     "r"(c.v.w)
+                     : "memory");
+    } else if constexpr (N == 8) {
+        asm volatile("st.global.cs.v2.u32 [%0], {%1,%2};" ::"l"(p), "r"(c.v.x), "r"(c.v.y) : "memory");
+    } else if constexpr (N == 4) {
+        asm volatile("st.global.cs.u32 [%0], %1;" ::"l"(p), "r"(c.v) : "memory");
+    } else {
+        *reinterpret_cast<skel::chunk<N> *>(p) = c;
+    }
+}
+
+template <class Tup>
+__device__ __forceinline__ void skel_apply_chunk(const skel_A *xa, const skel_B *xb, skel_O *yo, Tup &t) {
+#pragma unroll
+    for (int e = 0; e < SKEL_E; ++e) {
+        if constexpr (skel_void) {
+#if SKEL_NIN == 2
+            skel::caller<skel_Seq>::call(&SKEL_FN, t, xa[e], xb[e]);
+#else
+            skel::caller<skel_Seq>::call(&SKEL_FN, t, xa[e]);
+#endif
+        } else {
+#if SKEL_NIN == 2
+            yo[e] = skel::caller<skel_Seq>::call(&SKEL_FN, t, xa[e], xb[e]);
+#else
+            yo[e] = skel::caller<skel_Seq>::call(&SKEL_FN, t, xa[e]);
+#endif
+        }
+    }
+}
+
+constexpr int skel_CA = (int)(SKEL_E * skel_szA);
+constexpr int skel_CB = (int)(SKEL_E * skel_szB);
+constexpr int skel_CO = (int)(SKEL_E * skel_szO);
+
+// one chunk: unpack E elements, apply the user function, pack and store
+template <class Tup>
+__device__ __forceinline__ void skel_chunk_op(const skel::chunk<skel_CA> &ca, const skel::chunk<skel_CB> &cb, char *po,
+                                              Tup &t) {
+    auto xa = skel::bit_cast<skel::arr<skel_A, SKEL_E>>(ca);
+    skel::arr<skel_B, SKEL_E> xb;
+    if constexpr (SKEL_NIN == 2) xb = skel::bit_cast<skel::arr<skel_B, SKEL_E>>(cb);
+    skel::arr<skel_O, SKEL_E> yo;
+    skel_apply_chunk(xa.v, xb.v, yo.v, t);
+    if constexpr (!skel_void) skel_st<skel_CO>(po, skel::bit_cast<skel::chunk<skel_CO>>(yo));
+}
+template <class Tup>
+__device__ __forceinline__ void skel_one(const skel_A *a, const skel_B *b, skel_O *out, skel_u64 i, Tup &t) {
+    if constexpr (skel_void) {
+#if SKEL_NIN == 2
+        skel::caller<skel_Seq>::call(&SKEL_FN, t, a[i], b[i]);
+#else
+        skel::caller<skel_Seq>::call(&SKEL_FN, t, a[i]);
+#endif
+    } else {
+#if SKEL_NIN == 2
+        out[i] = skel::caller<skel_Seq>::call(&SKEL_FN, t, a[i], b[i]);
+#else
+        out[i] = skel::caller<skel_Seq>::call(&SKEL_FN, t, a[i]);
+#endif
+    }
+}
+
+extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
+    skel_ew_kernel(const skel_A *__restrict__ a, const skel_B *__restrict__ b, skel_O *__restrict__ out, skel_u64 n,
+                   int vec_ok, const skel_Buf args) {
+    auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
+    const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;
+
+    skel_u64 done = 0;  // elements covered by the chunked path
+    if (SKEL_E > 1 && vec_ok) {
+        const skel_u64 nch = n / SKEL_E;
+        done = nch * SKEL_E;
+        const char *pa = reinterpret_cast<const char *>(a);
+        const char *pb = reinterpret_cast<const char *>(b);
+        char *po = reinterpret_cast<char *>(out);
+        skel_u64 c = tid;
+        for (; c + (SKEL_UNROLL - 1) * stride < nch; c += SKEL_UNROLL * stride) {
+            skel::chunk<skel_CA> ca[SKEL_UNROLL];
+            skel::chunk<skel_CB> cb[SKEL_UNROLL];
+#pragma unroll
+            for (int u = 0; u < SKEL_UNROLL; ++u) {
+                ca[u] = skel_ld<skel_CA>(pa + (c + u * stride) * skel_CA);
+                if constexpr (SKEL_NIN == 2) cb[u] = skel_ld<skel_CB>(pb + (c + u * stride) * skel_CB);
+            }
+#pragma unroll
+            for (int u = 0; u < SKEL_UNROLL; ++u) {
+                skel_chunk_op(ca[u], cb[u], po + (c + u * stride) * skel_CO, t);
+            }
+        }
+        for (; c < nch; c += stride) {
+            skel::chunk<skel_CA> ca = skel_ld<skel_CA>(pa + c * skel_CA);
+            skel::chunk<skel_CB> cb;
+            if constexpr (SKEL_NIN == 2) cb = skel_ld<skel_CB>(pb + c * skel_CB);
+            skel_chunk_op(ca, cb, po + c * skel_CO, t);
+        }
+    }
+    // scalar path: the tail, or everything for non-vectorisable element types
+    for (skel_u64 i = done + tid; i < n; i += stride) skel_one(a, b, out, i, t);
+}

@@ -1,0 +1,112 @@
+"""CPU-side checks of the C-ABI boundary (no GPU needed): the library loads,
+exports every entry point include/skel.h declares, NVRTC injection compiles
+(or rejects) user functions for sm_100a, and the pure planner logic matches
+the oracle's distribution model.  No compute call runs here."""
+import re
+from pathlib import Path
+
+import numpy as np
+import pytest
+
+from oracle import distribution as odist
+from paper_conf_ipps_steuwerkg11_b200 import skel
+from paper_conf_ipps_steuwerkg11_b200.workloads import (LMOSEM_ERROR, LMOSEM_UPDATE, MANDELBROT, SAXPY_F32,
+                                                         SUM_F32)
+
+ROOT = Path(__file__).resolve().parents[1]
+
+
+def declared_symbols():
+    text = (ROOT / "include" / "skel.h").read_text()
+    return sorted(set(re.findall(r"^\s*(?:int|const char \*)\s*(skel_\w+)\s*\(", text, re.M)))
+
+
+def test_library_exports_every_declared_symbol():
+    lib = skel.lib()
+    names = declared_symbols()
+    assert len(names) >= 35
+    missing = [n for n in names if not hasattr(lib, n)]
+    assert not missing, missing
+
+
+def test_status_strings():
+    assert skel.lib().skel_status_string(4) == b"SKEL_ERR_COMPILE"
+
+
+@pytest.mark.parametrize("kind,src", [("map", MANDELBROT), ("map", LMOSEM_ERROR), ("zip", LMOSEM_UPDATE),
+                                      ("zip", SAXPY_F32), ("reduce", SUM_F32), ("scan", SUM_F32)])
+def test_nvrtc_injection_compiles_for_sm100a(kind, src):
+    st, log, nbytes = skel.compile_check(kind, src)
+    assert st == 0, log
+    assert nbytes > 1000
+
+
+def test_listing2_as_printed_is_rejected():
+    st, log, _ = skel.compile_check("map", "float f(float input, float number) { return input * number }")
+    assert st == 4 and 'expected a ";"' in log
+
+
+def test_reduce_operator_shape_is_checked():
+    st, log, _ = skel.compile_check("reduce", "float f(float x){ return x; }")
+    assert st == 4
+
+
+def test_entry_name_is_last_top_level_function():
+    src = """
+    // float decoy(float x) { return x; }
+    #define TWICE(x) ((x) * 2)
+    struct S { int a; int get() const { return a; } };
+    static float helper(float v) { if (v > 0) { return v; } return -v; }
+    /* float nope(float q) { } */
+    float entry(float x, const char* s = "f(x) {") { return helper(x); }
+    """
+    assert skel.entry_name(src) == "entry"
+    assert skel.entry_name(LMOSEM_ERROR) == "lmosem_error"
+    assert skel.entry_name(MANDELBROT) == "mandelbrot"
+
+
+@pytest.mark.parametrize("n", [0, 1, 7, 64, 6_300_000, 2**30 + 5])
+@pytest.mark.parametrize("D", [1, 2, 3, 4, 8])
+def test_plan_part_matches_oracle(n, D):
+    for k in range(D):
+        assert skel.plan_part(n, D, k) == odist.part_range(n, D, k)
+
+
+def test_plan_exchange_table():
+    S, B, C = skel.SINGLE, skel.BLOCK, skel.COPY
+    A = skel.COMBINE_ADD
+    assert skel.plan_exchange(S, B) == "scatter"
+    assert skel.plan_exchange(S, C) == "broadcast"
+    assert skel.plan_exchange(B, S) == "gather"
+    assert skel.plan_exchange(B, C) == "allgather"
+    assert skel.plan_exchange(C, B) == "local_slice"
+    assert skel.plan_exchange(C, B, A) == "reduce_scatter"
+    assert skel.plan_exchange(C, S) == "keep_root"
+    assert skel.plan_exchange(C, S, A) == "reduce"
+    assert skel.plan_exchange(C, C, A) == "allreduce"
+    for d in (S, B, C):
+        assert skel.plan_exchange(d, d) == "none"
+    with pytest.raises(skel.SkelError):
+        skel.plan_exchange(B, B, A)
+
+
+def test_no_cpu_fallback_without_gpu():
+    import torch
+    if torch.cuda.is_available():
+        pytest.skip("a GPU is present")
+    with pytest.raises(skel.SkelError) as e:
+        skel.Context(1)
+    assert e.value.name == "SKEL_ERR_CUDA"
+
+
+def test_oracle_and_product_share_no_code():
+    """The product package never imports the oracle (and vice versa)."""
+    pkg = ROOT / "paper_conf_ipps_steuwerkg11_b200"
+    for p in list(pkg.rglob("*.py")) + list(pkg.rglob("*.cpp")) + list(pkg.rglob("*.cu*")) + list(pkg.rglob("*.h")):
+        text = p.read_text()
+        assert not re.search(r"^\s*(from|import)\s+oracle", text, re.M), p
+        assert "oracle_core" not in text and "skel_oracle" not in text, p
+    osrc = [p for p in (ROOT / "oracle").iterdir() if p.suffix in (".py", ".c", ".hpp")]
+    for p in osrc:
+        assert not re.search(r"^\s*(from|import)\s+paper_conf_ipps_steuwerkg11_b200", p.read_text(), re.M), p
+        assert "skel.h" not in p.read_text() and "libskel" not in p.read_text(), p
