@@ -1,0 +1,438 @@
+#!/usr/bin/env python3
+"""Benchmark of the SkelCL hot path on B200 (BASELINE.json configs).
+
+Headline (BASELINE.json configs[1]): one *step* = Map(x*2+1) + Zip(saxpy) +
+Reduce(+) + Scan(+) over float32 vectors of 2^30 elements per GPU (4 GiB each,
+far larger than the 126 MB L2, so no flush is needed), through libskel's
+C-ABI.  value = aggregate algorithmic GB/s of the step over all GPUs
+(32 bytes/element: Map 8, Zip 12, Reduce 4, Scan 8).  Side measurements in
+the same run: per-skeleton GB/s and %HBM, Mandelbrot 4096x3072 (configs[2],
+Mpix/s) and one LM OSEM subset of 10^6 events (configs[3]/[4], seconds).
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl skel|reference]
+    torchrun --nproc-per-node N bench.py --gpus N ...   (one process per GPU)
+
+`--impl reference` times the CPU oracle (the task's reference arm) on host
+cores for the same metric on a bounded sample.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+BYTES_PER_ELEM = {"map": 8, "zip": 12, "reduce": 4, "scan": 8}
+STEP_BYTES = sum(BYTES_PER_ELEM.values())
+METRIC = "skeleton step GB/s (Map+Zip+Reduce+Scan, float32, 2^30 elements per GPU)"
+SEED = 20110516
+
+
+def bench_config(nloc: int, world: int) -> dict:
+    """The workload description shared by the GPU arm and the reference arm."""
+    return {"workload": "configs[1]: Reduce(+)/Zip(saxpy)/Scan(+) (+ Map x*2+1) sweep point "
+                        "n=2^30 float32 per GPU, one step = all four skeletons",
+            "elements_per_gpu": nloc, "elements_total": nloc * world,
+            "distribution": "single" if world == 1 else "block",
+            "l2": "inputs (4 GiB per vector) far exceed the 126 MB L2; no flush needed"}
+
+
+def env_world():
+    return int(os.environ.get("WORLD_SIZE", "1")), int(os.environ.get("RANK", "0")), \
+        int(os.environ.get("LOCAL_RANK", "0"))
+
+
+def measured_peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    try:
+        with open(p) as fh:
+            d = json.load(fh)
+        return float(d["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs)"
+    except Exception:
+        return 6650.0, "fallback (B200_PROFILING.md: 6.65 TB/s)"
+
+
+def traffic_table():
+    p = os.path.join(ROOT, "profiles", "traffic.json")
+    try:
+        with open(p) as fh:
+            return json.load(fh)
+    except Exception:
+        return {}
+
+
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons sampled during the timed region."""
+
+    FIELDS = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,"
+              "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+              "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, gpu: int):
+        self.gpu = gpu
+        self.proc = None
+        self.lines = []
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(["nvidia-smi", "-i", str(self.gpu), f"--query-gpu={self.FIELDS}",
+                                          "--format=csv,noheader,nounits", "-lms", "100"],
+                                         stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+        except Exception:
+            self.proc = None
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.lines.append(line.strip())
+
+    def stop(self):
+        if not self.proc:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        time.sleep(0.25)
+        self.proc.terminate()
+        try:
+            self.proc.wait(timeout=5)
+        except Exception:
+            self.proc.kill()
+        sm, smax, reasons = [], None, set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for ln in self.lines:
+            f = [x.strip() for x in ln.split(",")]
+            if len(f) < 9:
+                continue
+            try:
+                sm.append(float(f[1]))
+                smax = float(f[2])
+            except ValueError:
+                continue
+            for nm, val in zip(names, f[5:9]):
+                if val.lower().startswith("active"):
+                    reasons.add(nm)
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": smax,
+                "reasons": sorted(reasons), "samples": len(sm)}
+
+
+# ---------------------------------------------------------------------------
+# CPU oracle timing (cpu_baseline and the --impl reference arm)
+# ---------------------------------------------------------------------------
+def oracle_step(x, y):
+    import oracle
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MAP_F32, SAXPY_F32
+    oracle.skel_map(MAP_F32, x, np.float32)
+    oracle.skel_zip(SAXPY_F32, x, y, np.float32, args=[np.float32(2.5)])
+    oracle.sum_f32_exact(x)
+    oracle.exscan_f32_exact(x)
+
+
+def cpu_baseline(total_log2=30, chunk_log2=26):
+    """The oracle as it stands (single-threaded C), timed on this host on a
+    bounded sample: 2^total elements processed in chunks of 2^chunk."""
+    import skel_inputs as si
+    chunks = 1 << (total_log2 - chunk_log2)
+    n = 1 << chunk_log2
+    oracle_step(si.uniform_f32(1024, 1), si.uniform_f32(1024, 2))  # compile the user functions
+    t = 0.0
+    for c in range(chunks):
+        x, y = si.uniform_f32(n, SEED + 2 * c), si.uniform_f32(n, SEED + 2 * c + 1)
+        t0 = time.perf_counter()
+        oracle_step(x, y)
+        t += time.perf_counter() - t0
+    elems = chunks * n
+    return {"value": STEP_BYTES * elems / t / 1e9, "unit": "GB/s", "cores": 1, "kind": "oracle",
+            "sample": f"Map+Zip+Reduce+Scan oracle over 2^{total_log2} float32 elements "
+                      f"({chunks} chunks of 2^{chunk_log2}), {t:.1f} s single-threaded",
+            "host_cpus": os.cpu_count()}
+
+
+def run_reference(args):
+    world, rank, _ = env_world()
+    if rank != 0:
+        return
+    import skel_inputs as si
+    n = 1 << 24
+    x, y = si.uniform_f32(n, SEED), si.uniform_f32(n, SEED + 1)
+    for _ in range(args.warmup):
+        oracle_step(x, y)
+    t0 = time.perf_counter()
+    for _ in range(args.steps):
+        oracle_step(x, y)
+    dt = (time.perf_counter() - t0) / args.steps
+    value = STEP_BYTES * n / dt / 1e9
+    line = {"impl": "reference", "metric": METRIC, "value": value, "unit": "GB/s", "n_gpus": args.gpus,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": dt * 1e3, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "f32", "data": "synthetic",
+            "config": bench_config(1 << args.log2n, args.gpus),
+            "cpu_baseline": {"value": value, "unit": "GB/s", "cores": 1, "kind": "oracle",
+                             "sample": f"bounded: each step runs the oracle on 2^24 of the 2^30 float32 elements "
+                                       f"({args.steps} steps, single-threaded C); value scaled per byte"},
+            "e2e": {"value": value, "unit": "GB/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+# ---------------------------------------------------------------------------
+# GPU arm
+# ---------------------------------------------------------------------------
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--warmup", type=int, default=5)
+    ap.add_argument("--impl", default="skel", choices=["skel", "reference"])
+    ap.add_argument("--log2n", type=int, default=30, help="elements per GPU (log2)")
+    ap.add_argument("--e2e-steps", type=int, default=3)
+    ap.add_argument("--no-extras", action="store_true", help="skip Mandelbrot / LM OSEM side measurements")
+    ap.add_argument("--no-cpu", action="store_true", help="skip the cpu_baseline oracle timing")
+    args = ap.parse_args()
+    args.warmup = max(args.warmup, 3)
+
+    if args.impl == "reference":
+        run_reference(args)
+        return
+
+    import torch
+    import torch.distributed as dist
+
+    from paper_conf_ipps_steuwerkg11_b200 import skel
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MAP_F32, SAXPY_F32, SUM_F32
+
+    world, rank, local = env_world()
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        obj = [skel.unique_id() if rank == 0 else None]
+        dist.broadcast_object_list(obj, src=0)
+        ctx = skel.Context(rank=rank, world=world, device=local, nccl_id=obj[0])
+    else:
+        ctx = skel.Context(1)
+
+    def barrier():
+        if world > 1:
+            dist.barrier()
+
+    def max_over_ranks(v: float) -> float:
+        if world == 1:
+            return v
+        t = torch.tensor([v], device="cuda", dtype=torch.float64)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        return float(t.item())
+
+    stream = torch.cuda.ExternalStream(ctx.stream(0), device=torch.device("cuda", local))
+    nloc = 1 << args.log2n
+    N = nloc * world
+    import skel_inputs as si
+
+    # ---- inputs: this rank's block of x, y (uniform [0,1), PCG64), uploaded once
+    x = ctx.vector(n=N, dtype=np.float32)
+    y = ctx.vector(n=N, dtype=np.float32)
+    lo = rank * nloc
+    if world > 1:
+        x.set_distribution(skel.BLOCK)
+        y.set_distribution(skel.BLOCK)
+    x.upload_part(lo, si.uniform_f32(nloc, SEED + 2 * rank))
+    y.upload_part(lo, si.uniform_f32(nloc, SEED + 2 * rank + 1))
+    m = ctx.vector(n=N, dtype=np.float32)
+    z = ctx.vector(n=N, dtype=np.float32)
+    s = ctx.vector(n=N, dtype=np.float32)
+    r = ctx.vector(n=1, dtype=np.float32)
+    a = np.float32(2.5)
+    for kind, src in (("map", MAP_F32), ("zip", SAXPY_F32), ("reduce", SUM_F32)):
+        ctx.prepare(kind, src)
+
+    def step(ev=None):
+        if ev is not None:
+            ev[0].record(stream)
+        ctx.map(MAP_F32, x, m)
+        if ev is not None:
+            ev[1].record(stream)
+        ctx.zip(SAXPY_F32, x, y, z, args=[a])
+        if ev is not None:
+            ev[2].record(stream)
+        ctx.reduce_to(SUM_F32, x, r)
+        if ev is not None:
+            ev[3].record(stream)
+        ctx.scan(SUM_F32, x, s, np.float32(0))
+        if ev is not None:
+            ev[4].record(stream)
+
+    for _ in range(args.warmup):
+        step()
+    ctx.sync()
+
+    evs = [[torch.cuda.Event(enable_timing=True) for _ in range(5)] for _ in range(args.steps)]
+    t_start, t_stop = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    sampler = ClockSampler(local)
+    launches0 = ctx.stats()["kernel_launches"]
+    xfer0 = ctx.stats()
+    barrier()
+    torch.cuda.synchronize()
+    sampler.start()
+    time.sleep(0.3)
+    t_start.record(stream)
+    for k in range(args.steps):
+        step(evs[k])
+    t_stop.record(stream)
+    ctx.sync()
+    torch.cuda.synchronize()
+    barrier()
+    clocks = sampler.stop()
+    st1 = ctx.stats()
+    launches = st1["kernel_launches"] - launches0
+    assert st1["h2d_bytes"] == xfer0["h2d_bytes"], "inputs were not resident in the timed region"
+    ms_total = max_over_ranks(t_start.elapsed_time(t_stop))
+    ms_step = ms_total / args.steps
+    per = {}
+    for i, name in enumerate(("map", "zip", "reduce", "scan")):
+        ts = [evs[k][i].elapsed_time(evs[k][i + 1]) for k in range(args.steps)]
+        avg = max_over_ranks(sum(ts) / len(ts))
+        per[name] = {"ms": avg, "GBps": BYTES_PER_ELEM[name] * nloc / (avg * 1e-3) / 1e9}
+    value = STEP_BYTES * N / (ms_step * 1e-3) / 1e9
+    peak, peak_src = measured_peaks()
+    for name in per:
+        per[name]["frac_of_hbm"] = per[name]["GBps"] / peak
+    dom = max(per, key=lambda k: per[k]["ms"])
+    traffic = traffic_table().get(dom)
+    roofline = {"bound": "hbm", "kernel": dom, "achieved": per[dom]["GBps"], "peak": peak, "unit": "GB/s",
+                "frac": per[dom]["GBps"] / peak, "peak_source": peak_src,
+                "algorithmic_bytes_per_launch": BYTES_PER_ELEM[dom] * nloc,
+                "traffic": traffic, "traffic_source": "profiles/traffic.json (ncu --set full)" if traffic else None}
+
+    # ---- end to end through the C-ABI: pinned host inputs -> result scalar
+    e2e = None
+    if args.e2e_steps > 0:
+        ctx.sync()
+        barrier()
+        st0 = ctx.stats()
+        torch.cuda.synchronize()
+        t0 = time.perf_counter()
+        for _ in range(args.e2e_steps):
+            x.mark_host_modified()
+            y.mark_host_modified()
+            ctx.map(MAP_F32, x, m)
+            ctx.zip(SAXPY_F32, x, y, z, args=[a])
+            ctx.scan(SUM_F32, x, s, np.float32(0))
+            ctx.reduce(SUM_F32, x)  # blocking: the step's result on the host
+        ctx.sync()
+        dt = max_over_ranks(time.perf_counter() - t0) / args.e2e_steps
+        st1 = ctx.stats()
+        e2e = {"value": STEP_BYTES * N / dt / 1e9, "unit": "GB/s", "ms_per_step": dt * 1e3,
+               "h2d_bytes_per_step": (st1["h2d_bytes"] - st0["h2d_bytes"]) // args.e2e_steps,
+               "d2h_bytes_per_step": (st1["d2h_bytes"] - st0["d2h_bytes"]) // args.e2e_steps,
+               "path": "skel_vector_mark_host_modified on pinned host mirrors, then map/zip/scan/reduce "
+                       "(lazy H2D inside) and skel_reduce's blocking D2H of the scalar"}
+
+    # free the big vectors before the side measurements
+    for v in (x, y, m, z, s):
+        v.destroy()
+
+    extras = {}
+    if not args.no_extras:
+        extras["mandelbrot"] = bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, args)
+        extras["lmosem"] = bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args)
+
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu:
+        cpu = cpu_baseline()
+
+    if rank == 0:
+        line = {"metric": METRIC, "value": value, "unit": "GB/s", "n_gpus": world, "steps": args.steps,
+                "warmup": args.warmup, "ms_per_step": ms_step, "higher_is_better": True, "scaling": "weak",
+                "vs_baseline": None, "dtype": "f32", "data": "synthetic (PCG64 uniform [0,1) float32)",
+                "config": bench_config(nloc, world),
+                "per_skeleton": per, "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e,
+                "gpu_launches": launches, "clocks": clocks, **extras}
+        print(json.dumps(line), flush=True)
+    ctx.close()
+    if world > 1:
+        dist.destroy_process_group()
+
+
+def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
+    """configs[2]: 4096x3072, cap 256, rows block-distributed over the GPUs."""
+    import torch
+    import skel_inputs as si
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT
+    W, H, cap = 4096, 3072, 256
+    pos = si.mandelbrot_positions(W, H)
+    vin = ctx.vector(n=pos.size, dtype=pos.dtype)
+    if world > 1:
+        vin.set_distribution(skel.BLOCK)
+    lo, hi = vin.part(rank) if world > 1 else (0, pos.size)
+    vin.upload_part(lo, pos[lo:hi])
+    out = ctx.vector(n=pos.size, dtype=np.int32)
+    capv = np.int32(cap)
+    ctx.map(MANDELBROT, vin, out, args=[capv])
+    ctx.sync()
+    for _ in range(3):
+        ctx.map(MANDELBROT, vin, out, args=[capv])
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    reps = max(args.steps, 10)
+    barrier()
+    torch.cuda.synchronize()
+    e0.record(stream)
+    for _ in range(reps):
+        ctx.map(MANDELBROT, vin, out, args=[capv])
+    e1.record(stream)
+    ctx.sync()
+    ms = max_over_ranks(e0.elapsed_time(e1) / reps)
+    res = {"config": "configs[2]: 4096x3072, cap 256, block rows", "ms": ms,
+           "Mpix_per_s": W * H / (ms * 1e-3) / 1e6}
+    if rank == 0:
+        counts = out.download()
+        iters = int(counts.astype(np.int64).sum())
+        res["sum_iter"] = iters
+        res["Giter_per_s"] = iters / (ms * 1e-3) / 1e9
+        # FP32 pipe roofline: 8 FP32 ops per iteration as written (3 FMUL, 4 FADD/FSUB, 1 scale)
+        # vs 148 SM x 128 lanes x 1.965 GHz = 37.2 T FP32 instr/s
+        peak_ops = 148 * 128 * 1.965e9
+        res["fp32_frac"] = 8 * iters / (ms * 1e-3) / peak_ops
+    vin.destroy()
+    out.destroy()
+    return res
+
+
+def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
+    """configs[3]/[4]: one subset of 10^6 events into 150x150x280, events block-distributed."""
+    import torch
+    import skel_inputs as si
+    from paper_conf_ipps_steuwerkg11_b200.lmosem import LMOSEM
+    nev = 1_000_000
+    ev = si.lmosem_events(nev, subset=0)
+    rec = LMOSEM(ctx)
+    rec.prepare()
+    evv = ctx.vector(n=nev, dtype=ev.dtype)
+    if world > 1:
+        evv.set_distribution(skel.BLOCK)
+    lo, hi = evv.part(rank) if world > 1 else (0, nev)
+    evv.upload_part(lo, ev[lo:hi])
+    for _ in range(2):
+        rec.subset(evv)
+    ctx.sync()
+    reps = 5
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    barrier()
+    torch.cuda.synchronize()
+    e0.record(stream)
+    for _ in range(reps):
+        rec.subset(evv)
+    e1.record(stream)
+    ctx.sync()
+    ms = max_over_ranks(e0.elapsed_time(e1) / reps)
+    evv.destroy()
+    return {"config": "configs[3]/[4]: one subset, 10^6 events, 150x150x280, events block over GPUs",
+            "subset_s": ms * 1e-3, "events_per_s": nev / (ms * 1e-3),
+            "note": "includes f all-gather, c zero-fill, Siddon Map, c reduce-scatter and update Zip"}
+
+
+if __name__ == "__main__":
+    main()

@@ -154,6 +154,11 @@ int skel_vector_destroy(skel_vec_t v);
 int skel_vector_set_dtype(skel_vec_t v, skel_dtype dt);
 int skel_vector_size(skel_vec_t v, size_t *n, size_t *elem_size);
 int skel_vector_upload(skel_vec_t v, const void *src, size_t n);
+/* upload_part: host data for elements [lo, lo+count) only.  In one-process-
+ * per-GPU mode, uploading exactly this process's block part keeps a host
+ * mirror of that part only (no full-size host copy per process); otherwise
+ * the range is written into the full host copy. */
+int skel_vector_upload_part(skel_vec_t v, size_t lo, const void *src, size_t count);
 int skel_vector_download(skel_vec_t v, void *dst, size_t n);
 int skel_vector_host_ptr(skel_vec_t v, void **host);
 int skel_vector_mark_host_modified(skel_vec_t v);

@@ -104,6 +104,8 @@ struct skel_vec_s {
     skel_dist dist = SKEL_SINGLE;
     skel_dtype dt = SKEL_DT_OPAQUE;
     char *host = nullptr;   // pinned mirror (lazily allocated)
+    size_t host_lo = 0;     // mirror covers elements [host_lo, host_lo + host_n)
+    size_t host_n = 0;      // == n except for a rank-local part mirror (upload_part)
     bool host_valid = false;
     bool dev_valid = true;  // created zero-filled on the devices
     bool diverged = false;  // copy distribution after mark_device_modified

@@ -178,8 +178,16 @@ int join(skel_ctx_s *ctx) {
     return SKEL_OK;
 }
 
+bool partial_mirror(const skel_vec_s *v) { return v->host && v->host_n != v->n; }
+
 int host_mirror(skel_vec_s *v) {
-    if (v->host) return SKEL_OK;
+    if (v->host && !partial_mirror(v)) return SKEL_OK;
+    if (v->host) {  // a rank-local part mirror is replaced by a full one
+        cudaFreeHost(v->host);
+        v->host = nullptr;
+    }
+    v->host_lo = 0;
+    v->host_n = v->n;
     void *p = nullptr;
     cudaError_t e = cudaHostAlloc(&p, std::max<size_t>(v->n * v->es, 16), cudaHostAllocPortable);
     if (e != cudaSuccess) {
@@ -201,9 +209,11 @@ int ensure_device(skel_vec_s *v) {
         Buf &b = v->bufs[li];
         if (!b.count) continue;
         const size_t lo = (v->dist == SKEL_BLOCK) ? part_lo(v, s.d) : 0;
+        if (lo < v->host_lo || lo + b.count > v->host_lo + v->host_n)
+            return fail(ctx, SKEL_ERR_STATE, "host data of this part were not uploaded (upload_part covers another range)");
         DevGuard g(s.dev);
-        CK(ctx, cudaMemcpyAsync(b.ptr(v->es), v->host + lo * v->es, b.count * v->es, cudaMemcpyHostToDevice,
-                                s.stream));
+        CK(ctx, cudaMemcpyAsync(b.ptr(v->es), v->host + (lo - v->host_lo) * v->es, b.count * v->es,
+                                cudaMemcpyHostToDevice, s.stream));
         ctx->stats.h2d_bytes += b.count * v->es;
         ctx->stats.h2d_copies++;
     }
@@ -237,7 +247,11 @@ int scratch(skel_ctx_s *ctx, Slot &s, size_t bytes) {
 
 // lazy D2H into the host mirror
 int ensure_host(skel_vec_s *v) {
-    if (v->host_valid) return SKEL_OK;
+    if (v->host_valid && !partial_mirror(v)) return SKEL_OK;
+    if (partial_mirror(v)) {
+        TRY(ensure_device(v));
+        v->host_valid = false;
+    }
     skel_ctx_s *ctx = v->ctx;
     TRY(host_mirror(v));
     const size_t es = v->es;
@@ -529,7 +543,7 @@ int set_distribution(skel_vec_s *v, skel_dist dist, skel_combine combine) {
     if (x < 0) return fail(ctx, SKEL_ERR_STATE, "a combine merges per-device copies: the vector must be SKEL_COPY");
     if (combine != SKEL_COMBINE_NONE && v->dt == SKEL_DT_OPAQUE)
         return fail(ctx, SKEL_ERR_TYPE, "combine needs a numeric dtype (skel_vector_set_dtype)");
-    if (!v->dev_valid && combine == SKEL_COMBINE_NONE) {  // host-only data: relayout is free (lazy)
+    if (!v->dev_valid && combine == SKEL_COMBINE_NONE && !partial_mirror(v)) {  // host-only data: free relayout
         v->dist = dist;
         return SKEL_OK;
     }
@@ -819,15 +833,15 @@ int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args
         for (size_t li = 0; li < ctx->slots.size(); ++li) {
             Slot &s = ctx->slots[li];
             DevGuard g(s.dev);
-            CK(ctx, launch_gather(s.ws + Ls[li].o_gather, src.data(), K, Ls[li].slot, s.stream));
+            CK(ctx, launch_gather(s.ws + Ls[li].o_gather, src.data(), K, es, s.stream));  // packed slot<T>[K]
             ctx->stats.kernel_launches++;
         }
         TRY(join(ctx));
     } else if (cross) {
         Slot &s = ctx->slots[0];
         DevGuard g(s.dev);
-        NK(ctx, ncclAllGather(s.ws + Ls[0].o_res, s.ws + Ls[0].o_gather, Ls[0].slot, ncclUint8, ctx->comm, s.stream));
-        ctx->stats.nccl_bytes += Ls[0].slot * D;
+        NK(ctx, ncclAllGather(s.ws + Ls[0].o_res, s.ws + Ls[0].o_gather, es, ncclUint8, ctx->comm, s.stream));
+        ctx->stats.nccl_bytes += es * D;
     }
     for (size_t li = 0; li < ctx->slots.size(); ++li) {
         Slot &s = ctx->slots[li];
@@ -1148,7 +1162,7 @@ int skel_vector_size(skel_vec_t v, size_t *n, size_t *es) {
 int skel_vector_upload(skel_vec_t v, const void *src, size_t n) {
     if (!v || (!src && n)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad upload arguments");
     if (n != v->n) return fail(v->ctx, SKEL_ERR_SIZE, "upload length != vector length");
-    TRY(host_mirror(v));
+    TRY(host_mirror(v));  // (replaces a rank-local part mirror)
     // the host mirror may still be the source of an in-flight H2D copy
     TRY(sync_all(v->ctx));
     if (n) memcpy(v->host, src, n * v->es);
@@ -1158,9 +1172,51 @@ int skel_vector_upload(skel_vec_t v, const void *src, size_t n) {
     return SKEL_OK;
 }
 
+int skel_vector_upload_part(skel_vec_t v, size_t lo, const void *src, size_t count) {
+    if (!v || (!src && count)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad upload_part arguments");
+    skel_ctx_s *ctx = v->ctx;
+    if (lo > v->n || count > v->n - lo) return fail(ctx, SKEL_ERR_SIZE, "range outside the vector");
+    size_t plo = 0, phi = 0;
+    if (ctx->rank_mode && v->dist == SKEL_BLOCK) part_range(v->n, ctx->D, ctx->rank, &plo, &phi);
+    TRY(sync_all(ctx));  // the mirror may still feed an in-flight H2D
+    if (ctx->rank_mode && ctx->D > 1 && v->dist == SKEL_BLOCK && lo == plo && count == phi - plo &&
+        !(v->host && !partial_mirror(v) && v->host_valid)) {
+        // this process's part only: a rank-local mirror (no full-size host copy)
+        if (!partial_mirror(v) || v->host_lo != plo) {
+            if (v->host) cudaFreeHost(v->host);
+            v->host = nullptr;
+            void *p = nullptr;
+            cudaError_t e = cudaHostAlloc(&p, std::max<size_t>(count * v->es, 16), cudaHostAllocPortable);
+            if (e != cudaSuccess) {
+                cudaGetLastError();
+                return fail(ctx, SKEL_ERR_OOM, std::string("cudaHostAlloc: ") + cudaGetErrorString(e));
+            }
+            v->host = static_cast<char *>(p);
+            v->host_lo = plo;
+            v->host_n = count;
+        }
+        if (count) memcpy(v->host, src, count * v->es);
+    } else {
+        if (lo == 0 && count == v->n) TRY(host_mirror(v));
+        else if (!v->host_valid) TRY(ensure_host(v));  // the rest of the host copy must be current
+        if (count) memcpy(v->host + lo * v->es, src, count * v->es);
+    }
+    v->host_valid = true;
+    v->dev_valid = false;
+    v->diverged = false;
+    return SKEL_OK;
+}
+
 int skel_vector_download(skel_vec_t v, void *dst, size_t n) {
     if (!v || (!dst && n)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad download arguments");
     if (n != v->n) return fail(v->ctx, SKEL_ERR_SIZE, "download length != vector length");
+    if (partial_mirror(v)) {
+        // rank-local host data: assemble the whole vector on the devices, then read it
+        TRY(ensure_device(v));
+        v->host_valid = false;
+        cudaFreeHost(v->host);
+        v->host = nullptr;
+    }
     TRY(ensure_host(v));
     if (n) memcpy(dst, v->host, n * v->es);
     return SKEL_OK;

@@ -204,24 +204,31 @@ __device__ __forceinline__ void issue_tile(unsigned char *dst, const skel_tmap *
     tma_load_rows(dst + TILE_BYTES / 2, map, row + RB / 2, bar);
 }
 // thread `r` reads its 128-byte row of a 128B-swizzled stage into x[K]
-__device__ __forceinline__ void read_row(const unsigned char *stage, int r, skel_T *x) {
-    const unsigned char *row = stage + (size_t)r * 128;
+// (templates so that element sizes without a TMA path never instantiate them)
+template <bool OK = TMA_OK> __device__ __forceinline__ void read_row(const unsigned char *stage, int r, skel_T *x) {
+    if constexpr (OK) {
+        constexpr int PER = (int)(16 / sizeof(skel_T));
+        const unsigned char *row = stage + (size_t)r * 128;
 #pragma unroll
-    for (int j = 0; j < 8; ++j) {
-        const uint4 q = *reinterpret_cast<const uint4 *>(row + ((j ^ (r & 7)) << 4));
-        const auto e = skel::bit_cast<skel::arr<skel_T, 16 / sizeof(skel_T)>>(q);
+        for (int j = 0; j < 8; ++j) {
+            const uint4 q = *reinterpret_cast<const uint4 *>(row + ((j ^ (r & 7)) << 4));
+            const auto e = skel::bit_cast<skel::arr<skel_T, PER>>(q);
 #pragma unroll
-        for (int k = 0; k < (int)(16 / sizeof(skel_T)); ++k) x[j * (16 / sizeof(skel_T)) + k] = e.v[k];
+            for (int k = 0; k < PER; ++k) x[j * PER + k] = e.v[k];
+        }
     }
 }
-__device__ __forceinline__ void write_row(unsigned char *stage, int r, const skel_T *x) {
-    unsigned char *row = stage + (size_t)r * 128;
+template <bool OK = TMA_OK> __device__ __forceinline__ void write_row(unsigned char *stage, int r, const skel_T *x) {
+    if constexpr (OK) {
+        constexpr int PER = (int)(16 / sizeof(skel_T));
+        unsigned char *row = stage + (size_t)r * 128;
 #pragma unroll
-    for (int j = 0; j < 8; ++j) {
-        skel::arr<skel_T, 16 / sizeof(skel_T)> e;
+        for (int j = 0; j < 8; ++j) {
+            skel::arr<skel_T, PER> e;
 #pragma unroll
-        for (int k = 0; k < (int)(16 / sizeof(skel_T)); ++k) e.v[k] = x[j * (16 / sizeof(skel_T)) + k];
-        *reinterpret_cast<uint4 *>(row + ((j ^ (r & 7)) << 4)) = skel::bit_cast<uint4>(e);
+            for (int k = 0; k < PER; ++k) e.v[k] = x[j * PER + k];
+            *reinterpret_cast<uint4 *>(row + ((j ^ (r & 7)) << 4)) = skel::bit_cast<uint4>(e);
+        }
     }
 }
 __device__ __forceinline__ unsigned char *aligned_stages(unsigned char *p) {

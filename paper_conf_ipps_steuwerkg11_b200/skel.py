@@ -77,7 +77,7 @@ def lib() -> ctypes.CDLL:
             "skel_reset_stats": [P],
             "skel_vector_create": [P, S, S, PP], "skel_vector_destroy": [P], "skel_vector_set_dtype": [P, I],
             "skel_vector_size": [P, ctypes.POINTER(S), ctypes.POINTER(S)], "skel_vector_upload": [P, P, S],
-            "skel_vector_download": [P, P, S], "skel_vector_host_ptr": [P, PP],
+            "skel_vector_download": [P, P, S], "skel_vector_upload_part": [P, S, P, S], "skel_vector_host_ptr": [P, PP],
             "skel_vector_mark_host_modified": [P], "skel_vector_fill": [P, P], "skel_vector_fill_dist": [P, I, P],
             "skel_vector_set_distribution": [P, I, I], "skel_vector_get_distribution": [P, ctypes.POINTER(I)],
             "skel_vector_mark_device_modified": [P],
@@ -240,7 +240,7 @@ class Context:
     def map(self, src: str, vin: "Vector", vout: "Vector | None" = None, args=()):
         """eq. (1): vout[i] = f(vin[i], args...); vout=None for a void (side-effect) Map."""
         a, keep = self._args(args)
-        _check(lib().skel_map(self._h, src.encode(), vin._h, vout._h if vout else None, a, len(args)), self._h)
+        _check(lib().skel_map(self._h, src.encode(), vin._h, vout._h if vout is not None else None, a, len(args)), self._h)
         return vout
 
     def zip(self, src: str, va: "Vector", vb: "Vector", vout: "Vector", args=()):
@@ -303,6 +303,12 @@ class Vector:
     def upload(self, arr):
         a = np.ascontiguousarray(arr, dtype=self.dtype).reshape(-1)
         _check(lib().skel_vector_upload(self._h, a.ctypes.data, a.size), self.ctx._h)
+        return self
+
+    def upload_part(self, lo: int, arr):
+        """Host data for elements [lo, lo + len(arr)) (rank-local mirror in rank mode)."""
+        a = np.ascontiguousarray(arr, dtype=self.dtype).reshape(-1)
+        _check(lib().skel_vector_upload_part(self._h, lo, a.ctypes.data, a.size), self.ctx._h)
         return self
 
     def download(self) -> np.ndarray:

@@ -1,0 +1,194 @@
+"""Distributions and multi-device skeletons (§III-D, Listing 4) on D
+logical devices.  With one physical GPU the logical devices are "virtual"
+(skel_init(D) maps them all onto GPU 0; exchanges use the library's own
+copy/combine kernels).  Every result is checked against the oracle's pure
+distribution model and skeleton definitions; integer results must be
+bit-identical to D = 1."""
+import itertools
+
+import numpy as np
+import pytest
+
+import oracle
+import skel_inputs as si
+from oracle import distribution as odist
+from paper_conf_ipps_steuwerkg11_b200 import skel
+from paper_conf_ipps_steuwerkg11_b200.workloads import MAP_I32, SAXPY_F32, SUM_F32, SUM_I32
+
+pytestmark = pytest.mark.gpu
+
+DISTS = [skel.SINGLE, skel.BLOCK, skel.COPY]
+NAMES = {skel.SINGLE: odist.SINGLE, skel.BLOCK: odist.BLOCK, skel.COPY: odist.COPY}
+IDENT_I32 = "int ident(int x){ return x; }"
+
+
+def on_devices(ctx, x, dist):
+    """A vector whose data live on the devices under `dist` (not just the host)."""
+    v = ctx.vector(x)
+    v.set_distribution(dist)  # lazy: host-only data
+    w = ctx.vector(n=x.size, dtype=x.dtype)
+    ctx.map(IDENT_I32, v, w)  # w: device-valid, distributed like v
+    assert w.distribution == dist
+    return w
+
+
+@pytest.mark.parametrize("D", [2, 3, 4, 8])
+@pytest.mark.parametrize("n", [1, 5, 37, 4099, 100_003])
+def test_every_transition_preserves_the_vector(D, n):
+    x = si.uniform_i32(n, n)
+    with skel.Context(D) as ctx:
+        for a, b in itertools.product(DISTS, DISTS):
+            w = on_devices(ctx, x, a)
+            w.set_distribution(b)
+            assert w.distribution == b
+            assert np.array_equal(w.download(), x), (a, b)
+            # parts follow the planner
+            for d in range(D):
+                lo, hi = w.part(d)
+                if b == skel.BLOCK:
+                    assert (lo, hi) == odist.part_range(n, D, d)
+
+
+@pytest.mark.parametrize("D", [2, 4, 8])
+def test_copy_to_block_add_of_equal_copies(D):
+    x = np.arange(10_001, dtype=np.float32)
+    with skel.Context(D) as ctx:
+        v = ctx.vector(x)
+        v.set_distribution(skel.COPY)
+        w = ctx.vector(n=x.size, dtype=np.float32)
+        ctx.map("float id(float x){ return x; }", v, w)
+        w.set_distribution(skel.BLOCK, skel.COMBINE_ADD)
+        model = odist.redistribute(odist.distribute(x, odist.COPY, D), odist.COPY, odist.BLOCK, "add")
+        assert np.array_equal(w.download(), np.concatenate(model))
+
+
+@pytest.mark.parametrize("D", [2, 3, 4, 8])
+@pytest.mark.parametrize("dst", [skel.BLOCK, skel.SINGLE, skel.COPY])
+def test_combine_of_diverged_copies(D, dst):
+    """Each device writes its own block's indices into its own copy (side-effect
+    Map); the combine then merges the D different copies."""
+    n = 50_001
+    base = np.arange(n, dtype=np.int32) % 1000
+    mark = "void mark(int i, int* c){ c[i] += 1 + i % 7; }"
+    with skel.Context(D) as ctx:
+        c = ctx.vector(base)
+        c.set_distribution(skel.COPY)
+        idx = ctx.vector(np.arange(n, dtype=np.int32))
+        idx.set_distribution(skel.BLOCK)
+        ctx.map(mark, idx, None, args=[c])
+        c.mark_device_modified()
+        c.set_distribution(dst, skel.COMBINE_ADD)
+        copies = []
+        for d in range(D):
+            cd = base.copy()
+            lo, hi = odist.part_range(n, D, d)
+            cd[lo:hi] += 1 + np.arange(lo, hi) % 7
+            copies.append(cd)
+        model = odist.redistribute(copies, odist.COPY, NAMES[dst], "add")
+        assert np.array_equal(c.download(), odist.gather(model, NAMES[dst]))
+
+
+@pytest.mark.parametrize("D", [2, 3, 4, 8])
+def test_copy_to_block_without_combine_keeps_local_slices(D):
+    n = 999
+    mark = "void mark(int i, int* c){ c[i] = 5; }"
+    with skel.Context(D) as ctx:
+        c = ctx.vector(np.zeros(n, np.int32))
+        c.set_distribution(skel.COPY)
+        idx = ctx.vector(np.arange(n, dtype=np.int32))
+        idx.set_distribution(skel.BLOCK)
+        ctx.map(mark, idx, None, args=[c])
+        c.mark_device_modified()
+        c.set_distribution(skel.BLOCK)
+        # each device wrote exactly its own slice, so the local slices are all 5
+        assert (c.download() == 5).all()
+
+
+@pytest.mark.parametrize("D", [2, 3, 4, 8])
+@pytest.mark.parametrize("n", [1, 3, 16385, 1_000_003])
+def test_cross_device_reduce_and_scan_int_bit_identical(D, n):
+    x = si.uniform_int01(n, n + D)
+    want_r = int(oracle.skel_reduce(SUM_I32, x))
+    want_s = oracle.skel_scan(SUM_I32, x, 0)
+    with skel.Context(D) as ctx:
+        v = ctx.vector(x)
+        v.set_distribution(skel.BLOCK)
+        assert int(ctx.reduce(SUM_I32, v)) == want_r
+        out = ctx.vector(n=n, dtype=np.int32)
+        ctx.scan(SUM_I32, v, out, np.int32(0))
+        assert out.distribution == skel.BLOCK
+        assert np.array_equal(out.download(), want_s)
+
+
+@pytest.mark.parametrize("D", [2, 4, 8])
+def test_cross_device_noncommutative_order(D):
+    src = """
+    struct M2 { unsigned a, b, c, d; };
+    M2 matmul(M2 x, M2 y) {
+      M2 r;
+      r.a = x.a*y.a + x.b*y.c;  r.b = x.a*y.b + x.b*y.d;
+      r.c = x.c*y.a + x.d*y.c;  r.d = x.c*y.b + x.d*y.d;
+      return r;
+    }"""
+    M2 = np.dtype([("a", np.uint32), ("b", np.uint32), ("c", np.uint32), ("d", np.uint32)])
+    n = 123_457
+    g = np.random.default_rng(D)
+    m = np.zeros(n, M2)
+    for k in "abcd":
+        m[k] = g.integers(0, 1 << 32, n, dtype=np.uint64).astype(np.uint32)
+    ident = np.zeros(1, M2)
+    ident["a"], ident["d"] = 1, 1
+    with skel.Context(D) as ctx:
+        v = ctx.vector(m)
+        v.set_distribution(skel.BLOCK)
+        assert ctx.reduce(src, v).tobytes() == oracle.skel_reduce(src, m).tobytes()
+        out = ctx.vector(n=n, dtype=M2)
+        ctx.scan(src, v, out, ident[0])
+        assert out.download().tobytes() == oracle.skel_scan(src, m, ident[0]).tobytes()
+
+
+@pytest.mark.parametrize("D", [2, 4])
+def test_cross_device_float_reduce_scan_within_tolerance(D):
+    n = (1 << 20) + 77
+    x = si.uniform_f32(n, 9)
+    with skel.Context(D) as ctx:
+        v = ctx.vector(x)
+        v.set_distribution(skel.BLOCK)
+        r = float(ctx.reduce(SUM_F32, v))
+        assert abs(r - oracle.sum_f32_exact(x)) <= 1e-5 * oracle.abssum_f32(x)
+        out = ctx.vector(n=n, dtype=np.float32)
+        ctx.scan(SUM_F32, v, out, np.float32(0))
+        want, ab = oracle.exscan_f32_exact(x)
+        assert np.all(np.abs(out.download().astype(np.float64) - want) <= 1e-5 * ab)
+
+
+@pytest.mark.parametrize("D", [2, 3, 8])
+def test_zip_brings_b_to_a_distribution(D):
+    n = 77_777
+    x, y = si.uniform_f32(n, 1), si.uniform_f32(n, 2)
+    with skel.Context(D) as ctx:
+        a = ctx.vector(x)
+        a.set_distribution(skel.BLOCK)
+        b = ctx.vector(y)
+        b.set_distribution(skel.COPY)
+        out = ctx.vector(n=n, dtype=np.float32)
+        ctx.zip(SAXPY_F32, a, b, out, args=[np.float32(2.5)])
+        assert b.distribution == skel.BLOCK and out.distribution == skel.BLOCK
+        assert np.array_equal(out.download(), oracle.skel_zip(SAXPY_F32, x, y, np.float32,
+                                                              args=[np.float32(2.5)]))
+
+
+@pytest.mark.parametrize("dist", DISTS)
+def test_map_under_each_distribution(dist):
+    x = si.uniform_i32(30_001, 5)
+    with skel.Context(4) as ctx:
+        v = ctx.vector(x)
+        v.set_distribution(dist)
+        out = ctx.vector(n=x.size, dtype=np.int32)
+        ctx.map(MAP_I32, v, out)
+        assert out.distribution == dist
+        assert np.array_equal(out.download(), oracle.skel_map(MAP_I32, x, np.int32))
+        # copies are computed redundantly: every device holds the full result
+        if dist == skel.COPY:
+            for li in range(4):
+                assert out.device_ptr(li)[1] == x.size

@@ -1,0 +1,56 @@
+"""GPU parity of the Mandelbrot Map (§IV-A, eq. (5)): bit-exact
+iteration counts against the oracle and the golden whole-image pins, on one
+device and block-distributed over virtual devices (rows split)."""
+import json
+import os
+import zlib
+
+import numpy as np
+import pytest
+
+import oracle
+import skel_inputs as si
+from paper_conf_ipps_steuwerkg11_b200 import skel
+from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT
+
+pytestmark = pytest.mark.gpu
+
+
+def run(ctx, pos, cap, dist=None):
+    vin = ctx.vector(pos)
+    if dist is not None:
+        vin.set_distribution(dist)
+    out = ctx.vector(n=pos.size, dtype=np.int32)
+    ctx.map(MANDELBROT, vin, out, args=[np.int32(cap)])
+    return out.download()
+
+
+def test_closed_form_points():
+    cs = [1 + 0j, 2 + 0j, -1.5 + 1.5j, 0j, -1 + 0j, -2 + 0j, 1j, 0.25 + 0j, 3 + 0j]
+    want = [3, 2, 1, 256, 256, 256, 256, 256, 1]
+    pos = np.zeros(len(cs), si.POS_DTYPE)
+    pos["re"] = [c.real for c in cs]
+    pos["im"] = [c.imag for c in cs]
+    with skel.Context(1) as ctx:
+        assert run(ctx, pos, 256).tolist() == want
+
+
+@pytest.mark.parametrize("w,h,cap", [(1024, 768, 256), (4096, 3072, 256), (1024, 768, 4096)])
+def test_whole_image_bit_exact(golden_dir, w, h, cap):
+    pos = si.mandelbrot_positions(w, h)
+    with skel.Context(1) as ctx:
+        got = run(ctx, pos, cap)
+    with open(os.path.join(golden_dir, "mandelbrot.json")) as fh:
+        case = [c for c in json.load(fh)["cases"] if (c["width"], c["height"], c["cap"]) == (w, h, cap)][0]
+    assert zlib.crc32(got.tobytes()) == int(case["crc32"], 16)
+    assert int(got.astype(np.int64).sum()) == case["sum_iter"]
+    if w * h <= 1 << 20:
+        assert np.array_equal(got, oracle.mandelbrot(pos, cap))
+
+
+@pytest.mark.parametrize("D", [2, 3, 4, 8])
+def test_block_rows_on_virtual_devices(D):
+    pos = si.mandelbrot_positions(1024, 768)
+    with skel.Context(D) as ctx:
+        got = run(ctx, pos, 256, skel.BLOCK)
+    assert np.array_equal(got, oracle.mandelbrot(pos, 256))
