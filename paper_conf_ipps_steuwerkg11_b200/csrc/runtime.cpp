@@ -699,13 +699,13 @@ PFN_encode get_encode() {
 }
 
 // 2-D view [rows][128 B] of a tile-aligned prefix, 128B swizzle, 256-row boxes
-bool make_tmap(CUtensorMap *map, const void *ptr, uint64_t rows) {
+bool make_tmap(CUtensorMap *map, const void *ptr, uint64_t rows, uint32_t box_rows = 256) {
     memset(map, 0, sizeof *map);
     PFN_encode enc = get_encode();
     if (!enc || rows == 0 || !al16(ptr) || rows > 0x7fffffffull) return false;
     cuuint64_t dims[2] = {32, rows};
     cuuint64_t strides[1] = {128};
-    cuuint32_t box[2] = {32, 256};
+    cuuint32_t box[2] = {32, box_rows};
     cuuint32_t estr[2] = {1, 1};
     CUresult r = enc(map, CU_TENSOR_MAP_DATA_TYPE_UINT32, 2, const_cast<void *>(ptr), dims, strides, box, estr,
                      CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_128B, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
@@ -777,7 +777,10 @@ int set_smem_attr(skel_ctx_s *ctx, Module *m, const Slot &s) {
     const int dsm = (int)m->sig[11];
     if (dsm > 0) {
         CK(ctx, cudaFuncSetAttribute((const void *)m->k_main, cudaFuncAttributeMaxDynamicSharedMemorySize, dsm));
-        CK(ctx, cudaFuncSetAttribute((const void *)m->k_scan, cudaFuncAttributeMaxDynamicSharedMemorySize, dsm));
+    }
+    if (m->sig[12] > 0) {
+        CK(ctx, cudaFuncSetAttribute((const void *)m->k_scan, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                     (int)m->sig[12]));
     }
     m->attr_set_on.insert(s.dev);
     return SKEL_OK;
@@ -1398,7 +1401,8 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
     std::vector<unsigned char> abuf;
     // seeds: device k starts from agg_0 (+) ... (+) agg_{k-1} (one exchange of
     // D partial results)
-    const uint64_t TILE = m->sig[10];
+    const uint64_t TILE = m->sig[15];  // scan tile (elements)
+    const uint32_t box_rows = (uint32_t)(TILE / m->sig[8] / 2);
     const bool packed = m->sig[13] != 0;
     for (size_t li = 0; li < ctx->slots.size(); ++li) {
         Slot &s = ctx->slots[li];
@@ -1445,15 +1449,15 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         const void *pin = in->bufs[li].ptr(in->es);
         void *pout = out->bufs[li].ptr(out->es);
         CUtensorMap tin, tout;
-        const uint64_t rows = (cnt / TILE) * m->sig[9];
-        int use_tma = m->sig[5] && make_tmap(&tin, pin, rows) && make_tmap(&tout, pout, rows);
+        const uint64_t rows = (cnt / TILE) * 2 * box_rows;
+        int use_tma = m->sig[5] && make_tmap(&tin, pin, rows, box_rows) && make_tmap(&tout, pout, rows, box_rows);
         void *status = s.st64, *flags = s.fl32, *aggv = s.ws + L.o_aggv, *incv = s.ws + L.o_incv;
         unsigned *counters = s.counters;
         void *total = nullptr;
         void *params[] = {&tin, &tout, &pin, &pout, &cnt, &use_tma, idbuf.data(), &seed, &status, &flags,
                           &aggv, &incv, &counters, &epoch, &total, abuf.data()};
-        CK(ctx, cudaLaunchKernel((const void *)m->k_scan, dim3((unsigned)G), dim3((unsigned)m->sig[9]), params,
-                                 use_tma ? m->sig[11] : 0, s.stream));
+        CK(ctx, cudaLaunchKernel((const void *)m->k_scan, dim3((unsigned)G), dim3((unsigned)m->sig[14]), params,
+                                 use_tma ? m->sig[12] : 0, s.stream));
         ctx->stats.kernel_launches++;
     }
     out->dev_valid = true;

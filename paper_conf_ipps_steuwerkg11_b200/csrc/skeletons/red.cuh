@@ -53,6 +53,19 @@ constexpr skel_u64 TILE = (skel_u64)RB * K;
 constexpr unsigned TILE_BYTES = (unsigned)(TILE * sizeof(skel_T));
 constexpr int STAGES = SKEL_STAGES;
 constexpr unsigned DSMEM = TMA_OK ? STAGES * TILE_BYTES + 1024 : 0;
+// Scan: SRB consumer rows per tile, SSTAGES smem stages
+#ifndef SKEL_SCAN_RB
+#define SKEL_SCAN_RB 384
+#endif
+#ifndef SKEL_SCAN_STAGES
+#define SKEL_SCAN_STAGES 4
+#endif
+constexpr int SRB = SKEL_SCAN_RB;
+constexpr int SNW = SRB / 32;
+constexpr int SSTAGES = SKEL_SCAN_STAGES;
+constexpr skel_u64 STILE = (skel_u64)SRB * K;
+constexpr unsigned STILE_BYTES = (unsigned)(STILE * sizeof(skel_T));
+constexpr unsigned SDSMEM = TMA_OK ? SSTAGES * STILE_BYTES + 1024 : 0;
 constexpr bool PACKED = sizeof(skel_S) == 4;  // status = value:32 | epoch:30 | state:2
 
 struct skel_sig_t { skel_u64 v[16 + 4 * 32]; };
@@ -70,8 +83,10 @@ constexpr skel_sig_t skel_make_sig() {
     s.v[9] = RB;
     s.v[10] = TILE;
     s.v[11] = DSMEM;
-    s.v[12] = STAGES;
+    s.v[12] = SDSMEM;
     s.v[13] = PACKED;
+    s.v[14] = SRB + 64;  // scan kernel block size (consumers + producer + look-back warps)
+    s.v[15] = STILE;
     for (int i = 0; i < skel_Lay::n && i < 32; ++i) {
         s.v[16 + 4 * i] = skel_Lay::size(i);
         s.v[17 + 4 * i] = skel_Lay::align(i);
@@ -197,11 +212,13 @@ __device__ __forceinline__ void tma_prefetch_desc(const skel_tmap *map) {
     asm volatile("prefetch.tensormap [%0];" ::"l"(map) : "memory");
 }
 // issue the two 256-row boxes of tile `tile` into stage buffer `dst`
+template <int ROWS = RB>
 __device__ __forceinline__ void issue_tile(unsigned char *dst, const skel_tmap *map, skel_u64 tile, skel_u64 *bar) {
-    skel::mbar_expect_tx(bar, TILE_BYTES);
-    const int row = (int)(tile * RB);
+    constexpr unsigned BYTES = (unsigned)ROWS * 128u;
+    skel::mbar_expect_tx(bar, BYTES);
+    const int row = (int)(tile * ROWS);
     tma_load_rows(dst, map, row, bar);
-    tma_load_rows(dst + TILE_BYTES / 2, map, row + RB / 2, bar);
+    tma_load_rows(dst + BYTES / 2, map, row + ROWS / 2, bar);
 }
 // thread `r` reads its 128-byte row of a 128B-swizzled stage into x[K]
 // (templates so that element sizes without a TMA path never instantiate them)
@@ -369,8 +386,62 @@ extern "C" __global__ void skel_seed_kernel(const skel_S *aggs, int k, const ske
 }
 
 // ============================================================================
-// Scan (single pass, decoupled look-back)
+// Scan (single pass, decoupled look-back, warp-specialised)
+//
+// CTA = RB consumer threads (one 128-byte row of the tile each) + 1 producer
+// warp + 1 look-back warp, one CTA per SM, STAGES smem stages.
+//   producer : takes tile tickets (atomic counter), TMA-loads tiles into free
+//              stages, and TMA-stores finished stages back to global memory;
+//   look-back: as soon as a tile's ticket is known, folds the predecessors'
+//              published aggregates / inclusive prefixes (a 256-tile window
+//              per round trip), then publishes the tile's inclusive prefix;
+//   consumers: in-thread scan of their row, block scan (named barrier 1),
+//              publish the tile aggregate, apply the prefix, write the
+//              outputs back into the stage.
+// Per-stage mbarriers: full (data + ticket), ticket (ticket only), agg
+// (tile aggregate ready), prefix (exclusive prefix ready), written
+// (outputs in smem, RB arrivals).  Parity of use u of a stage is u & 1.
 // ============================================================================
+constexpr int SCAN_THREADS = SRB + 64;
+constexpr int LB_PER_LANE = 8;  // look-back window = 32 * 8 tiles per round trip
+
+__device__ __forceinline__ void cons_sync() { asm volatile("bar.sync 1, %0;" ::"n"(SRB) : "memory"); }
+__device__ __forceinline__ void mbar_arrive(skel_u64 *bar) {
+    asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(skel::smem_addr(bar)) : "memory");
+}
+
+// block exclusive scan among the RB consumer threads (named barrier 1)
+template <class Tup> __device__ __forceinline__ VT cons_exscan(VT x, VT *wsc, VT *total, Tup &t) {
+    const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+    VT inc = x;
+#pragma unroll
+    for (int d = 1; d < 32; d <<= 1) {
+        VT o = vt_shfl_up(inc, d);
+        if (lane >= d) inc = comb(o, inc, t);
+    }
+    VT ex = vt_shfl_up(inc, 1);
+    if (lane == 0) ex.ok = false;
+    if (lane == 31) wsc[w] = inc;
+    cons_sync();
+    if (w == 0) {
+        VT y;
+        y.ok = false;
+        if (lane < SNW) y = wsc[lane];
+        VT yi = y;
+#pragma unroll
+        for (int d = 1; d < 32; d <<= 1) {
+            VT o = vt_shfl_up(yi, d);
+            if (lane >= d) yi = comb(o, yi, t);
+        }
+        VT ye = vt_shfl_up(yi, 1);
+        if (lane == 0) ye.ok = false;
+        if (lane < SNW) wsc[lane] = ye;
+        if (lane == SNW - 1) *total = yi;
+    }
+    cons_sync();
+    return comb(wsc[w], ex, t);
+}
+
 __device__ __forceinline__ void publish(skel_u64 *status, unsigned *flags, skel_S *aggv, skel_S *incv, skel_u64 tile,
                                         unsigned epoch, unsigned state, const skel_T &v) {
     if constexpr (PACKED) {
@@ -383,177 +454,308 @@ __device__ __forceinline__ void publish(skel_u64 *status, unsigned *flags, skel_
         skel::st_release(&flags[tile], (epoch << 2) | state);
     }
 }
-// returns state (0 = not ready, 1 = aggregate, 2 = inclusive prefix)
-__device__ __forceinline__ unsigned peek(const skel_u64 *status, const unsigned *flags, const skel_S *aggv,
-                                         const skel_S *incv, skel_u64 tile, unsigned epoch, skel_T &v) {
+// relaxed read of a tile's status: 0 = not ready, 1 = aggregate, 2 = inclusive
+// prefix.  Packed statuses carry their value in the same 64-bit word; for the
+// others the value is read after an acquire fence (see read_values).
+__device__ __forceinline__ unsigned peek_state(const skel_u64 *status, const unsigned *flags, skel_u64 tile,
+                                               unsigned epoch, skel_T &v) {
     if constexpr (PACKED) {
         skel_u64 word;
-        asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(word) : "l"(status + tile) : "memory");
+        asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(word) : "l"(status + tile) : "memory");
         const unsigned lo = (unsigned)word;
         if ((lo >> 2) != epoch) return 0;
-        const unsigned bits = (unsigned)(word >> 32);
-        v = skel::bit_cast<skel_S>(bits).v;
+        v = skel::bit_cast<skel_S>((unsigned)(word >> 32)).v;
         return lo & 3u;
     } else {
-        const unsigned f = skel::ld_acquire(&flags[tile]);
+        const unsigned f = skel::ld_relaxed_u32(&flags[tile]);
         if ((f >> 2) != epoch) return 0;
-        const unsigned st = f & 3u;
-        if (st == 1) v = skel::ld_value(&aggv[tile]).v;
-        if (st == 2) v = skel::ld_value(&incv[tile]).v;
-        return st;
+        return f & 3u;
     }
 }
 
-extern "C" __global__ void __launch_bounds__(RB, 1)
+extern "C" __global__ void __launch_bounds__(SCAN_THREADS, 1)
     skel_scan_kernel(const __grid_constant__ skel_tmap tin, const __grid_constant__ skel_tmap tout,
                      const skel_T *in, skel_T *out, skel_u64 n, int use_tma, const skel_S identity, const skel_S *seed,
                      skel_u64 *status, unsigned *flags, skel_S *aggv, skel_S *incv, unsigned *counters,
                      unsigned epoch, skel_S *total, const skel_Buf args) {
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
-    __shared__ skel_u64 bars[STAGES];
-    __shared__ skel_u64 tq[STAGES];
-    __shared__ VT wsc[NW];
-    __shared__ VT s_total;
-    __shared__ VT s_prefix;
+    __shared__ skel_u64 full_bar[SSTAGES], tick_bar[SSTAGES], agg_bar[SSTAGES], pre_bar[SSTAGES], wr_bar[SSTAGES];
+    __shared__ skel_u64 tq[SSTAGES];
+    __shared__ VT s_agg[SSTAGES], s_pre[SSTAGES];
+    __shared__ VT wsc[SNW];
+    __shared__ VT s_tot;
     const int t = threadIdx.x, lane = t & 31, w = t >> 5;
-    const skel_u64 ntiles = (n + TILE - 1) / TILE;
+    const skel_u64 ntiles = (n + STILE - 1) / STILE;
     const bool tma = TMA_OK && use_tma;
     unsigned char *stages = aligned_stages(skel_dsmem);
-    unsigned phase = 0;  // per-stage parity bits of TMA-loaded stages
 
     if (t == 0) {
-        if (tma) {
-            for (int s = 0; s < STAGES; ++s) skel::mbar_init(&bars[s], 1);
-            skel::fence_mbar_init();
-            tma_prefetch_desc(&tin);
-            tma_prefetch_desc(&tout);
+        for (int s = 0; s < SSTAGES; ++s) {
+            skel::mbar_init(&full_bar[s], 1);
+            skel::mbar_init(&tick_bar[s], 1);
+            skel::mbar_init(&agg_bar[s], 1);
+            skel::mbar_init(&pre_bar[s], 1);
+            skel::mbar_init(&wr_bar[s], SRB);
         }
-        for (int s = 0; s < STAGES; ++s) {
-            const skel_u64 tk = atomicAdd(&counters[0], 1u);
-            tq[s] = tk;
-            if (tma && (tk + 1) * TILE <= n) issue_tile(stages + s * TILE_BYTES, &tin, tk, &bars[s]);
-        }
+        skel::fence_mbar_init();
     }
     __syncthreads();
 
-    for (skel_u64 i = 0;; ++i) {
-        const int s = (int)(i % STAGES);
-        const skel_u64 tk = tq[s];
-        if (tk >= ntiles) break;
-        const skel_u64 base = tk * TILE;
-        const bool full = base + TILE <= n;
-        const bool staged = tma && full;
-        // refill the stage of the previous tile once its TMA store has read smem
-        if (t == 0 && i > 0) {
-            const int sp = (int)((i - 1) % STAGES);
-            skel::bulk_wait_read0();
-            const skel_u64 nk = atomicAdd(&counters[0], 1u);
-            tq[sp] = nk;
-            if (tma && (nk + 1) * TILE <= n) issue_tile(stages + sp * TILE_BYTES, &tin, nk, &bars[sp]);
-        }
-        // ---- this thread's contiguous items: registers (staged tile) or a
-        //      direct first pass over global memory (ragged / non-TMA tile)
-        skel_T x[K];
-        VT mine;
-        mine.ok = false;
-        skel_u64 first = 0, kt = 0;
-        if (staged) {
-            skel::mbar_wait(&bars[s], (phase >> s) & 1u);
-            phase ^= 1u << s;
-            read_row(stages + s * TILE_BYTES, t, x);
-#pragma unroll
-            for (int k = 1; k < K; ++k) x[k] = opf(x[k - 1], x[k], tup);  // in-thread inclusive scan
-            mine.v = x[K - 1];
-            mine.ok = true;
-        } else {
-            const skel_u64 cnt = full ? TILE : n - base;
-            const skel_u64 per = full ? (skel_u64)K : (cnt + RB - 1) / RB;
-            first = base + (skel_u64)t * per;
-            const skel_u64 end = base + cnt;
-            kt = first >= end ? 0 : ((end - first) < per ? (end - first) : per);
-            for (skel_u64 k = 0; k < kt; ++k) {
-                VT e;
-                e.v = in[first + k];
-                e.ok = true;
-                mine = comb(mine, e, tup);
+    if (w == SNW) {
+        // ------------------------------------------------------------ producer
+        if (lane == 0) {
+            if (tma) {
+                tma_prefetch_desc(&tin);
+                tma_prefetch_desc(&tout);
             }
+            bool done = false;
+            skel_u64 last_i = 0;
+            for (skel_u64 i = 0;; ++i) {
+                const int s = (int)(i % SSTAGES);
+                bool stored = false;
+                if (i >= SSTAGES) {  // retire the tile that used this stage
+                    const skel_u64 old = tq[s];
+                    if (old < ntiles) {
+                        skel::mbar_wait(&wr_bar[s], (unsigned)(((i / SSTAGES) - 1) & 1));
+                        if (tma && (old + 1) * STILE <= n) {
+                            const int row = (int)(old * SRB);
+                            tma_store_rows(&tout, row, stages + s * STILE_BYTES);
+                            tma_store_rows(&tout, row + SRB / 2, stages + s * STILE_BYTES + STILE_BYTES / 2);
+                            skel::bulk_commit();
+                            stored = true;
+                        }
+                    }
+                }
+                // take the ticket only when the stage is about to be refilled (a held
+                // ticket delays every later tile's look-back); its latency overlaps
+                // the TMA store's read of the stage
+                skel_u64 tk = 0;
+                if (!done) tk = atomicAdd(&counters[0], 1u);
+                if (stored) skel::bulk_wait_read0();
+                if (done) {
+                    if (i >= last_i + SSTAGES) break;
+                    tq[s] = ntiles;
+                    continue;
+                }
+                tq[s] = tk;
+                mbar_arrive(&tick_bar[s]);
+                if (tk >= ntiles) {
+                    done = true;
+                    last_i = i;
+                    mbar_arrive(&full_bar[s]);
+                } else if (tma && (tk + 1) * STILE <= n) {
+                    issue_tile<SRB>(stages + s * STILE_BYTES, &tin, tk, &full_bar[s]);
+                } else {
+                    mbar_arrive(&full_bar[s]);
+                }
+            }
+            skel::bulk_wait0();
         }
-        VT excl = block_exscan(mine, wsc, &s_total, tup);
-        // ---- tile prefix: seed for tile 0, decoupled look-back otherwise (warp 0)
-        if (w == 0) {
-            const VT tot = s_total;
+    } else if (w == SNW + 1) {
+        // ------------------------------------------------------------ look-back
+        for (skel_u64 i = 0;; ++i) {
+            const int s = (int)(i % SSTAGES);
+            const unsigned ph = (unsigned)((i / SSTAGES) & 1);
+            skel::mbar_wait(&tick_bar[s], ph);
+            const skel_u64 tk = tq[s];
+            if (tk >= ntiles) break;
             VT prefix;
             if (tk == 0) {
                 prefix.v = seed ? seed->v : identity.v;
                 prefix.ok = true;
             } else {
-                if (lane == 0) publish(status, flags, aggv, incv, tk, epoch, 1u, tot.v);
                 VT acc;
                 acc.ok = false;
                 long long j0 = (long long)tk - 1;
                 for (;;) {
-                    const long long j = j0 - lane;
-                    unsigned st = 0;
-                    skel_T v;
-                    if (j >= 0) {
-                        do {
-                            st = peek(status, flags, aggv, incv, (skel_u64)j, epoch, v);
-                        } while (st == 0);
-                    }
-                    const unsigned pm = __ballot_sync(0xffffffffu, st == 2);
-                    const int last = pm ? __ffs(pm) - 1 : 31;
-                    // fold lanes last..0 (older tiles on the left)
-                    VT wv;
-                    wv.v = v;
-                    wv.ok = (j >= 0) && lane <= last;
+                    // lane covers tiles j0 - lane*8 - q, q = 0..7 (q = 0 nearest)
+                    unsigned st[LB_PER_LANE];
+                    skel_T v[LB_PER_LANE];
 #pragma unroll
-                    for (int d = 1; d < 32; d <<= 1) {
-                        VT o = vt_shfl_down(wv, d);
-                        if ((lane & (2 * d - 1)) == 0) wv = comb(o, wv, tup);
+                    for (int q = 0; q < LB_PER_LANE; ++q) {
+                        const long long j = j0 - (long long)lane * LB_PER_LANE - q;
+                        st[q] = j >= 0 ? peek_state(status, flags, (skel_u64)j, epoch, v[q]) : 3u;
                     }
-                    wv = vt_shfl_idx(wv, 0);
-                    acc = comb(wv, acc, tup);
+                    for (;;) {  // re-poll the ones not ready yet
+                        bool all = true;
+#pragma unroll
+                        for (int q = 0; q < LB_PER_LANE; ++q) {
+                            if (st[q] == 0) {
+                                const long long j = j0 - (long long)lane * LB_PER_LANE - q;
+                                st[q] = peek_state(status, flags, (skel_u64)j, epoch, v[q]);
+                                all = all && st[q] != 0;
+                            }
+                        }
+                        if (all) break;
+                    }
+                    if constexpr (!PACKED) {
+                        __threadfence();  // acquire: values were published before their flags
+#pragma unroll
+                        for (int q = 0; q < LB_PER_LANE; ++q) {
+                            const long long j = j0 - (long long)lane * LB_PER_LANE - q;
+                            if (st[q] == 1) v[q] = skel::ld_value(&aggv[j]).v;
+                            if (st[q] == 2) v[q] = skel::ld_value(&incv[j]).v;
+                        }
+                    }
+                    int qp = LB_PER_LANE;  // nearest inclusive prefix of this lane
+#pragma unroll
+                    for (int q = LB_PER_LANE - 1; q >= 0; --q)
+                        if (st[q] == 2) qp = q;
+                    const unsigned pm = __ballot_sync(0xffffffffu, qp < LB_PER_LANE);
+                    const int lp = pm ? __ffs(pm) - 1 : 32;
+                    VT lf;  // lane fold, older (larger q) on the left
+                    lf.ok = false;
+                    const int qmax = lane < lp ? LB_PER_LANE - 1 : (lane == lp ? qp : -1);
+#pragma unroll
+                    for (int q = LB_PER_LANE - 1; q >= 0; --q) {
+                        if (q <= qmax && st[q] != 3u) {
+                            VT e;
+                            e.v = v[q];
+                            e.ok = true;
+                            lf = comb(lf, e, tup);
+                        }
+                    }
+#pragma unroll
+                    for (int d = 1; d < 32; d <<= 1) {  // window fold, higher lanes (older) left
+                        VT o = vt_shfl_down(lf, d);
+                        if ((lane & (2 * d - 1)) == 0) lf = comb(o, lf, tup);
+                    }
+                    lf = vt_shfl_idx(lf, 0);
+                    acc = comb(lf, acc, tup);
                     if (pm) break;
-                    j0 -= 32;
+                    j0 -= 32 * LB_PER_LANE;
                 }
                 prefix = acc;
             }
-            const VT inc = comb(prefix, tot, tup);
+            skel::mbar_wait(&agg_bar[s], ph);
+            const VT agg = s_agg[s];
+            const VT inc = comb(prefix, agg, tup);
             if (lane == 0) {
                 publish(status, flags, aggv, incv, tk, epoch, 2u, inc.v);
-                s_prefix = prefix;
                 if (tk == ntiles - 1 && total) total->v = inc.v;
+                s_pre[s] = prefix;
+                mbar_arrive(&pre_bar[s]);
             }
+            __syncwarp();
         }
-        __syncthreads();
-        // ---- outputs: o_0 = pre, o_k = pre (+) r_{k-1}
-        const VT pre = comb(s_prefix, excl, tup);
-        if (staged) {
+    } else {
+        // ------------------------------------------------------------ consumers
+        // iteration i: phase A of tile i (local scan, publish its aggregate),
+        // then phase B of tile i-1 (apply its prefix, hand the stage back), so
+        // a tile's aggregate is never held up by the previous tile's look-back.
+        bool pv = false, pstaged = false;  // previous tile pending phase B
+        int ps = 0;
+        unsigned pph = 0;
+        skel_u64 pfirst = 0, pkt = 0;
+        VT pexcl;
+        pexcl.ok = false;
+        for (skel_u64 i = 0;; ++i) {
+            const int s = (int)(i % SSTAGES);
+            const unsigned ph = (unsigned)((i / SSTAGES) & 1);
+            skel::mbar_wait(&full_bar[s], ph);
+            const skel_u64 tk = tq[s];
+            const bool live = tk < ntiles;
+            if (live) {
+                // ---- phase A(i)
+                const skel_u64 base = tk * STILE;
+                const bool full = base + STILE <= n;
+                const bool staged = tma && full;
+                VT mine;
+                mine.ok = false;
+                skel_u64 first = 0, kt = 0;
+                skel_T x[K];
+                if (staged) {
+                    read_row(stages + s * STILE_BYTES, t, x);
 #pragma unroll
-            for (int k = K - 1; k >= 1; --k) x[k] = opf(pre.v, x[k - 1], tup);
-            x[0] = pre.v;
-            write_row(stages + s * TILE_BYTES, t, x);
-            skel::fence_proxy_async();
-            __syncthreads();
-            if (t == 0) {
-                const int row = (int)(tk * RB);
-                tma_store_rows(&tout, row, stages + s * TILE_BYTES);
-                tma_store_rows(&tout, row + RB / 2, stages + s * TILE_BYTES + TILE_BYTES / 2);
-                skel::bulk_commit();
+                    for (int k = 1; k < K; ++k) x[k] = opf(x[k - 1], x[k], tup);
+                    mine.v = x[K - 1];
+                    mine.ok = true;
+                } else {
+                    const skel_u64 cnt = full ? STILE : n - base;
+                    const skel_u64 per = full ? (skel_u64)K : (cnt + SRB - 1) / SRB;
+                    first = base + (skel_u64)t * per;
+                    const skel_u64 end = base + cnt;
+                    kt = first >= end ? 0 : ((end - first) < per ? (end - first) : per);
+                    for (skel_u64 k = 0; k < kt; ++k) {
+                        VT e;
+                        e.v = in[first + k];
+                        e.ok = true;
+                        mine = comb(mine, e, tup);
+                    }
+                }
+                const VT excl = cons_exscan(mine, wsc, &s_tot, tup);
+                if (t == 0) {
+                    const VT tot = s_tot;
+                    if (tk > 0) publish(status, flags, aggv, incv, tk, epoch, 1u, tot.v);
+                    s_agg[s] = tot;
+                    mbar_arrive(&agg_bar[s]);
+                }
+                if (staged) {
+                    // tile-local exclusive results y_k = excl (+) r_{k-1} (y_0 = excl;
+                    // row 0 has no excl: its y_0 slot is unused, y_k = r_{k-1})
+#pragma unroll
+                    for (int k = K - 1; k >= 1; --k) x[k] = excl.ok ? opf(excl.v, x[k - 1], tup) : x[k - 1];
+                    x[0] = excl.v;
+                    write_row(stages + s * STILE_BYTES, t, x);
+                }
+                // ---- phase B(i-1)
+                if (pv) {
+                    skel::mbar_wait(&pre_bar[ps], pph);
+                    const VT prefix = s_pre[ps];
+                    if (pstaged) {
+                        skel_T y[K];
+                        read_row(stages + ps * STILE_BYTES, t, y);
+#pragma unroll
+                        for (int k = 0; k < K; ++k) y[k] = (t == 0 && k == 0) ? prefix.v : opf(prefix.v, y[k], tup);
+                        write_row(stages + ps * STILE_BYTES, t, y);
+                        skel::fence_proxy_async();
+                    } else {
+                        const VT pre = comb(prefix, pexcl, tup);
+                        skel_T run = pre.v;  // second pass (in-place safe: read, then write)
+                        for (skel_u64 k = 0; k < pkt; ++k) {
+                            const skel_T e = in[pfirst + k];
+                            out[pfirst + k] = run;
+                            run = opf(run, e, tup);
+                        }
+                    }
+                    mbar_arrive(&wr_bar[ps]);
+                }
+                pv = true;
+                pstaged = staged;
+                ps = s;
+                pph = ph;
+                pfirst = first;
+                pkt = kt;
+                pexcl = excl;
+            } else {
+                // no more tiles: finish the pending one
+                if (pv) {
+                    skel::mbar_wait(&pre_bar[ps], pph);
+                    const VT prefix = s_pre[ps];
+                    if (pstaged) {
+                        skel_T y[K];
+                        read_row(stages + ps * STILE_BYTES, t, y);
+#pragma unroll
+                        for (int k = 0; k < K; ++k) y[k] = (t == 0 && k == 0) ? prefix.v : opf(prefix.v, y[k], tup);
+                        write_row(stages + ps * STILE_BYTES, t, y);
+                        skel::fence_proxy_async();
+                    } else {
+                        const VT pre = comb(prefix, pexcl, tup);
+                        skel_T run = pre.v;
+                        for (skel_u64 k = 0; k < pkt; ++k) {
+                            const skel_T e = in[pfirst + k];
+                            out[pfirst + k] = run;
+                            run = opf(run, e, tup);
+                        }
+                    }
+                    mbar_arrive(&wr_bar[ps]);
+                }
+                break;
             }
-        } else {
-            // second pass: running prefix from `pre` (in-place safe: read, then write)
-            skel_T run = pre.v;
-            for (skel_u64 k = 0; k < kt; ++k) {
-                const skel_T e = in[first + k];
-                out[first + k] = run;
-                run = opf(run, e, tup);
-            }
-            __syncthreads();
         }
     }
+    __syncthreads();
     if (t == 0) {
-        skel::bulk_wait0();
         __threadfence();
         const unsigned prev = atomicAdd(&counters[1], 1u);
         if (prev == gridDim.x - 1) {
