@@ -1401,13 +1401,18 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
     std::vector<unsigned char> abuf;
     // seeds: device k starts from agg_0 (+) ... (+) agg_{k-1} (one exchange of
     // D partial results)
-    const uint64_t TILE = m->sig[15];  // scan tile (elements)
-    const uint32_t box_rows = (uint32_t)(TILE / m->sig[8] / 2);
+    const uint64_t TILE = m->sig[10];
+    const uint64_t CH = m->sig[15];  // tiles per CTA per slice
     const bool packed = m->sig[13] != 0;
+    // one aggregate status word per (slice, CTA)
+    auto scan_slots = [&](const Slot &s, uint64_t cnt) -> uint64_t {
+        const uint64_t per_slice = (uint64_t)s.sms * CH, nft = cnt / TILE;
+        return std::max<uint64_t>(1, (nft + per_slice - 1) / per_slice) * (uint64_t)s.sms;
+    };
     for (size_t li = 0; li < ctx->slots.size(); ++li) {
         Slot &s = ctx->slots[li];
         const uint64_t cnt = in->bufs[li].count;
-        Ls[li] = red_layout(m, D, red_grid(m, s, cnt), (cnt + TILE - 1) / TILE);
+        Ls[li] = red_layout(m, D, red_grid(m, s, cnt), scan_slots(s, cnt));
         TRY(ensure_ws(ctx, s, Ls[li].total));
     }
     if (cross) {
@@ -1429,10 +1434,9 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         Slot &s = ctx->slots[li];
         uint64_t cnt = in->bufs[li].count;
         if (!cnt) continue;
-        const uint64_t ntiles = (cnt + TILE - 1) / TILE;
-        const size_t G = (size_t)std::max<uint64_t>(1, std::min<uint64_t>((uint64_t)s.sms, ntiles));
+        const size_t G = (size_t)s.sms;  // persistent: one CTA per SM
         const RedLayout &L = Ls[li];
-        TRY(ensure_status(ctx, s, ntiles, packed));
+        TRY(ensure_status(ctx, s, scan_slots(s, cnt), packed));
         TRY(set_smem_attr(ctx, m, s));
         pack_args(m, args, nargs, li, abuf);
         DevGuard g(s.dev);
@@ -1449,8 +1453,8 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         const void *pin = in->bufs[li].ptr(in->es);
         void *pout = out->bufs[li].ptr(out->es);
         CUtensorMap tin, tout;
-        const uint64_t rows = (cnt / TILE) * 2 * box_rows;
-        int use_tma = m->sig[5] && make_tmap(&tin, pin, rows, box_rows) && make_tmap(&tout, pout, rows, box_rows);
+        const uint64_t rows = (cnt / TILE) * m->sig[9];
+        int use_tma = m->sig[5] && make_tmap(&tin, pin, rows) && make_tmap(&tout, pout, rows);
         void *status = s.st64, *flags = s.fl32, *aggv = s.ws + L.o_aggv, *incv = s.ws + L.o_incv;
         unsigned *counters = s.counters;
         void *total = nullptr;

@@ -53,19 +53,11 @@ constexpr skel_u64 TILE = (skel_u64)RB * K;
 constexpr unsigned TILE_BYTES = (unsigned)(TILE * sizeof(skel_T));
 constexpr int STAGES = SKEL_STAGES;
 constexpr unsigned DSMEM = TMA_OK ? STAGES * TILE_BYTES + 1024 : 0;
-// Scan: SRB consumer rows per tile, SSTAGES smem stages
-#ifndef SKEL_SCAN_RB
-#define SKEL_SCAN_RB 384
+// Scan: tiles per CTA per slice (see the Scan section)
+#ifndef SKEL_SCAN_CH
+#define SKEL_SCAN_CH 3
 #endif
-#ifndef SKEL_SCAN_STAGES
-#define SKEL_SCAN_STAGES 4
-#endif
-constexpr int SRB = SKEL_SCAN_RB;
-constexpr int SNW = SRB / 32;
-constexpr int SSTAGES = SKEL_SCAN_STAGES;
-constexpr skel_u64 STILE = (skel_u64)SRB * K;
-constexpr unsigned STILE_BYTES = (unsigned)(STILE * sizeof(skel_T));
-constexpr unsigned SDSMEM = TMA_OK ? SSTAGES * STILE_BYTES + 1024 : 0;
+constexpr int SCAN_CH = SKEL_SCAN_CH;
 constexpr bool PACKED = sizeof(skel_S) == 4;  // status = value:32 | epoch:30 | state:2
 
 struct skel_sig_t { skel_u64 v[16 + 4 * 32]; };
@@ -83,10 +75,10 @@ constexpr skel_sig_t skel_make_sig() {
     s.v[9] = RB;
     s.v[10] = TILE;
     s.v[11] = DSMEM;
-    s.v[12] = SDSMEM;
+    s.v[12] = DSMEM;
     s.v[13] = PACKED;
-    s.v[14] = SRB + 64;  // scan kernel block size (consumers + producer + look-back warps)
-    s.v[15] = STILE;
+    s.v[14] = RB;  // scan kernel block size
+    s.v[15] = SCAN_CH;
     for (int i = 0; i < skel_Lay::n && i < 32; ++i) {
         s.v[16 + 4 * i] = skel_Lay::size(i);
         s.v[17 + 4 * i] = skel_Lay::align(i);
@@ -386,381 +378,323 @@ extern "C" __global__ void skel_seed_kernel(const skel_S *aggs, int k, const ske
 }
 
 // ============================================================================
-// Scan (single pass, decoupled look-back, warp-specialised)
+// Scan: single pass over HBM with an L2-resident second read
 //
-// CTA = RB consumer threads (one 128-byte row of the tile each) + 1 producer
-// warp + 1 look-back warp, one CTA per SM, STAGES smem stages.
-//   producer : takes tile tickets (atomic counter), TMA-loads tiles into free
-//              stages, and TMA-stores finished stages back to global memory;
-//   look-back: as soon as a tile's ticket is known, folds the predecessors'
-//              published aggregates / inclusive prefixes (a 256-tile window
-//              per round trip), then publishes the tile's inclusive prefix;
-//   consumers: in-thread scan of their row, block scan (named barrier 1),
-//              publish the tile aggregate, apply the prefix, write the
-//              outputs back into the stage.
-// Per-stage mbarriers: full (data + ticket), ticket (ticket only), agg
-// (tile aggregate ready), prefix (exclusive prefix ready), written
-// (outputs in smem, RB arrivals).  Parity of use u of a stage is u & 1.
+// A persistent grid of G CTAs (one per SM) walks the vector in *slices* of
+// G x CH tiles; CTA c owns the CH consecutive tiles (s*G + c)*CH ... of slice
+// s.  Per slice and CTA:
+//   P1(s): fold the CTA's tiles in order (TMA loads with an L2 evict_last
+//          policy, so the slice stays in L2) and publish the aggregate A(s,c);
+//   P2(s): prefix(s,c) = carry(s) (+) A(s,0) (+) ... (+) A(s,c-1), with
+//          carry(s) = carry(s-1) (+) A(s-1,0) (+) ... (+) A(s-1,G-1); then
+//          re-read the tiles (L2 hits, evict_first), scan them with a running
+//          prefix and TMA-store the outputs (evict_first).
+// Work order per CTA: P1(0), P1(1), P2(0), P1(2), P2(1), ... so each CTA's
+// wait for its predecessors' aggregates of slice s is covered by its own
+// P1(s+1): no CTA waits on another in the steady state, HBM sees each input
+// byte read once and each output byte written once (8 B/element for float),
+// and every element's prefix chain has one carry link per slice (float
+// rounding stays far below 1e-5 at 2^30 elements).
+// The ragged last tile is scanned by CTA G-1 with direct loads; element sizes
+// without a TMA path use direct loads for every tile.
 // ============================================================================
-constexpr int SCAN_THREADS = SRB + 64;
-constexpr int LB_PER_LANE = 8;  // look-back window = 32 * 8 tiles per round trip
-
-__device__ __forceinline__ void cons_sync() { asm volatile("bar.sync 1, %0;" ::"n"(SRB) : "memory"); }
-__device__ __forceinline__ void mbar_arrive(skel_u64 *bar) {
-    asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(skel::smem_addr(bar)) : "memory");
+__device__ __forceinline__ skel_u64 policy_evict_last() {
+    skel_u64 p;
+    asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
+__device__ __forceinline__ skel_u64 policy_evict_first() {
+    skel_u64 p;
+    asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
+__device__ __forceinline__ void tma_load_rows_hint(void *dst, const skel_tmap *map, int row, skel_u64 *bar,
+                                                   skel_u64 pol) {
+    asm volatile(
+        "cp.async.bulk.tensor.2d.shared::cluster.global.tile.mbarrier::complete_tx::bytes.L2::cache_hint"
+        " [%0], [%1, {%2, %3}], [%4], %5;" ::"r"(skel::smem_addr(dst)),
+        "l"(map), "r"(0), "r"(row), "r"(skel::smem_addr(bar)), "l"(pol)
+        : "memory");
+}
+__device__ __forceinline__ void tma_store_rows_hint(const skel_tmap *map, int row, const void *src, skel_u64 pol) {
+    asm volatile("cp.async.bulk.tensor.2d.global.shared::cta.tile.bulk_group.L2::cache_hint [%0, {%1, %2}], [%3], %4;" ::"l"(
+                     map),
+                 "r"(0), "r"(row), "r"(skel::smem_addr(src)), "l"(pol)
+                 : "memory");
 }
 
-// block exclusive scan among the RB consumer threads (named barrier 1)
-template <class Tup> __device__ __forceinline__ VT cons_exscan(VT x, VT *wsc, VT *total, Tup &t) {
-    const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-    VT inc = x;
-#pragma unroll
-    for (int d = 1; d < 32; d <<= 1) {
-        VT o = vt_shfl_up(inc, d);
-        if (lane >= d) inc = comb(o, inc, t);
-    }
-    VT ex = vt_shfl_up(inc, 1);
-    if (lane == 0) ex.ok = false;
-    if (lane == 31) wsc[w] = inc;
-    cons_sync();
-    if (w == 0) {
-        VT y;
-        y.ok = false;
-        if (lane < SNW) y = wsc[lane];
-        VT yi = y;
-#pragma unroll
-        for (int d = 1; d < 32; d <<= 1) {
-            VT o = vt_shfl_up(yi, d);
-            if (lane >= d) yi = comb(o, yi, t);
-        }
-        VT ye = vt_shfl_up(yi, 1);
-        if (lane == 0) ye.ok = false;
-        if (lane < SNW) wsc[lane] = ye;
-        if (lane == SNW - 1) *total = yi;
-    }
-    cons_sync();
-    return comb(wsc[w], ex, t);
-}
-
-__device__ __forceinline__ void publish(skel_u64 *status, unsigned *flags, skel_S *aggv, skel_S *incv, skel_u64 tile,
-                                        unsigned epoch, unsigned state, const skel_T &v) {
+// status of A(s,c): state 1 = value, 2 = empty sub-chunk
+__device__ __forceinline__ void publish_agg(skel_u64 *st64, unsigned *fl32, skel_S *vals, skel_u64 idx, unsigned epoch,
+                                            const VT &a) {
+    const unsigned state = a.ok ? 1u : 2u;
     if constexpr (PACKED) {
-        skel_S sv{v};
+        skel_S sv{a.v};
         const unsigned bits = skel::bit_cast<unsigned>(sv);
         const skel_u64 word = ((skel_u64)bits << 32) | (skel_u64)((epoch << 2) | state);
-        asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(status + tile), "l"(word) : "memory");
+        asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(st64 + idx), "l"(word) : "memory");
     } else {
-        skel::st_value(state == 1 ? &aggv[tile] : &incv[tile], skel_S{v});
-        skel::st_release(&flags[tile], (epoch << 2) | state);
+        if (a.ok) skel::st_value(&vals[idx], skel_S{a.v});
+        skel::st_release(&fl32[idx], (epoch << 2) | state);
     }
 }
-// relaxed read of a tile's status: 0 = not ready, 1 = aggregate, 2 = inclusive
-// prefix.  Packed statuses carry their value in the same 64-bit word; for the
-// others the value is read after an acquire fence (see read_values).
-__device__ __forceinline__ unsigned peek_state(const skel_u64 *status, const unsigned *flags, skel_u64 tile,
-                                               unsigned epoch, skel_T &v) {
+// spin until A(idx) is published; returns it
+__device__ __forceinline__ VT wait_agg(const skel_u64 *st64, const unsigned *fl32, const skel_S *vals, skel_u64 idx,
+                                       unsigned epoch) {
+    VT r;
     if constexpr (PACKED) {
         skel_u64 word;
-        asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(word) : "l"(status + tile) : "memory");
-        const unsigned lo = (unsigned)word;
-        if ((lo >> 2) != epoch) return 0;
-        v = skel::bit_cast<skel_S>((unsigned)(word >> 32)).v;
-        return lo & 3u;
+        do {
+            asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(word) : "l"(st64 + idx) : "memory");
+        } while (((unsigned)word >> 2) != epoch);
+        r.ok = ((unsigned)word & 3u) == 1u;
+        r.v = skel::bit_cast<skel_S>((unsigned)(word >> 32)).v;
     } else {
-        const unsigned f = skel::ld_relaxed_u32(&flags[tile]);
-        if ((f >> 2) != epoch) return 0;
-        return f & 3u;
+        unsigned f;
+        do {
+            f = skel::ld_acquire(&fl32[idx]);
+        } while ((f >> 2) != epoch);
+        r.ok = (f & 3u) == 1u;
+        if (r.ok) r.v = skel::ld_value(&vals[idx]).v;
     }
+    return r;
+}
+// ordered fold of A(base .. base+cnt-1) by one warp; result in every lane
+template <class Tup>
+__device__ __forceinline__ VT warp_fold_aggs(const skel_u64 *st64, const unsigned *fl32, const skel_S *vals,
+                                             skel_u64 base, int cnt, unsigned epoch, int lane, Tup &t) {
+    const int per = (cnt + 31) / 32;
+    VT a;
+    a.ok = false;
+    for (int k = 0; k < per; ++k) {
+        const int i = lane * per + k;
+        if (i < cnt) a = comb(a, wait_agg(st64, fl32, vals, base + i, epoch), t);
+    }
+    a = warp_fold(a, lane, t);
+    return vt_shfl_idx(a, 0);
 }
 
-extern "C" __global__ void __launch_bounds__(SCAN_THREADS, 1)
+// work item q of a CTA's sequence: P1(0) x CH, then per slice s: P1(s+1) x CH
+// (if any), P2(s) x CH.  Returns false past the end.
+__device__ __forceinline__ bool scan_item(skel_u64 q, skel_u64 nslices, int &phase, skel_u64 &s, int &j) {
+    const skel_u64 L = SCAN_CH;
+    if (nslices == 0) return false;
+    if (q < L) {
+        phase = 1;
+        s = 0;
+        j = (int)q;
+        return true;
+    }
+    const skel_u64 k = q - L, blk = k / (2 * L), r = k % (2 * L);
+    if (blk >= nslices) return false;
+    if (blk + 1 < nslices) {
+        phase = r < L ? 1 : 2;
+        s = r < L ? blk + 1 : blk;
+        j = (int)(r < L ? r : r - L);
+        return true;
+    }
+    if (r >= L) return false;  // last slice: P2 only
+    phase = 2;
+    s = blk;
+    j = (int)r;
+    return true;
+}
+
+extern "C" __global__ void __launch_bounds__(RB, 1)
     skel_scan_kernel(const __grid_constant__ skel_tmap tin, const __grid_constant__ skel_tmap tout,
                      const skel_T *in, skel_T *out, skel_u64 n, int use_tma, const skel_S identity, const skel_S *seed,
                      skel_u64 *status, unsigned *flags, skel_S *aggv, skel_S *incv, unsigned *counters,
                      unsigned epoch, skel_S *total, const skel_Buf args) {
+    (void)incv;
+    (void)counters;
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
-    __shared__ skel_u64 full_bar[SSTAGES], tick_bar[SSTAGES], agg_bar[SSTAGES], pre_bar[SSTAGES], wr_bar[SSTAGES];
-    __shared__ skel_u64 tq[SSTAGES];
-    __shared__ VT s_agg[SSTAGES], s_pre[SSTAGES];
-    __shared__ VT wsc[SNW];
-    __shared__ VT s_tot;
+    __shared__ skel_u64 bars[STAGES];
+    __shared__ VT wsc[NW];
+    __shared__ VT s_tot, s_run, s_carry;
     const int t = threadIdx.x, lane = t & 31, w = t >> 5;
-    const skel_u64 ntiles = (n + STILE - 1) / STILE;
+    const skel_u64 G = gridDim.x, c = blockIdx.x;
+    const skel_u64 nft = n / TILE;                    // full tiles
+    const skel_u64 per_slice = G * SCAN_CH;
+    const skel_u64 nslices = (nft + per_slice - 1) / per_slice;
     const bool tma = TMA_OK && use_tma;
     unsigned char *stages = aligned_stages(skel_dsmem);
-
-    if (t == 0) {
-        for (int s = 0; s < SSTAGES; ++s) {
-            skel::mbar_init(&full_bar[s], 1);
-            skel::mbar_init(&tick_bar[s], 1);
-            skel::mbar_init(&agg_bar[s], 1);
-            skel::mbar_init(&pre_bar[s], 1);
-            skel::mbar_init(&wr_bar[s], SRB);
-        }
+    auto tile_of = [&](skel_u64 s, int j) -> skel_u64 { return (s * G + c) * SCAN_CH + (skel_u64)j; };
+    // valid tiles of CTA c in slice s: j < jn(s)
+    auto jn = [&](skel_u64 s) -> int {
+        const skel_u64 first = (s * G + c) * SCAN_CH;
+        if (first >= nft) return 0;
+        const skel_u64 left = nft - first;
+        return (int)(left < (skel_u64)SCAN_CH ? left : (skel_u64)SCAN_CH);
+    };
+    skel_u64 pol_keep = 0, pol_drop = 0;
+    if (tma && t == 0) {
+        pol_keep = policy_evict_last();
+        pol_drop = policy_evict_first();
+        for (int st = 0; st < STAGES; ++st) skel::mbar_init(&bars[st], 1);
         skel::fence_mbar_init();
+        tma_prefetch_desc(&tin);
+        tma_prefetch_desc(&tout);
+    }
+    if (t == 0) {
+        VT cz;
+        cz.v = seed ? seed->v : identity.v;
+        cz.ok = true;
+        s_carry = cz;  // carry(0)
     }
     __syncthreads();
 
-    if (w == SNW) {
-        // ------------------------------------------------------------ producer
-        if (lane == 0) {
+    // the producer (thread 0) walks the same item sequence, STAGES valid items ahead
+    skel_u64 pq = 0;  // next sequence position to load
+    auto issue_next = [&](int stage) {
+        int ph, j;
+        skel_u64 s;
+        while (scan_item(pq, nslices, ph, s, j)) {
+            ++pq;
+            if (j < jn(s)) {
+                const int row = (int)(tile_of(s, j) * RB);
+                unsigned char *dst = stages + stage * TILE_BYTES;
+                const skel_u64 pol = ph == 1 ? pol_keep : pol_drop;
+                skel::mbar_expect_tx(&bars[stage], TILE_BYTES);
+                tma_load_rows_hint(dst, &tin, row, &bars[stage], pol);
+                tma_load_rows_hint(dst + TILE_BYTES / 2, &tin, row + RB / 2, &bars[stage], pol);
+                return;
+            }
+        }
+    };
+    if (tma && t == 0)
+        for (int st = 0; st < STAGES; ++st) issue_next(st);
+
+    skel_u64 v = 0;  // valid items consumed
+    VT run1;         // P1 running aggregate (thread 0)
+    run1.ok = false;
+    int ph;
+    skel_u64 s;
+    int j;
+    for (skel_u64 q = 0; scan_item(q, nslices, ph, s, j); ++q) {
+        const int nj = jn(s);
+        if (ph == 2 && j == 0) {
+            // ---- prefix(s, c) = carry(s) (+) A(s,0..c-1); carry(s+1) prepared
+            if (w == 0) {
+                VT carry = s_carry;
+                if (s > 0) {
+                    const VT prev = warp_fold_aggs(status, flags, aggv, (s - 1) * G, (int)G, epoch, lane, tup);
+                    carry = comb(carry, prev, tup);
+                }
+                const VT mine = warp_fold_aggs(status, flags, aggv, s * G, (int)c, epoch, lane, tup);
+                if (lane == 0) {
+                    s_carry = carry;
+                    s_run = comb(carry, mine, tup);
+                }
+            }
+            __syncthreads();
+        }
+        if (j >= nj) {
+            // no tile of this CTA in slice s: publish an empty aggregate once
+            if (ph == 1 && j == 0 && nj == 0 && t == 0) {
+                VT e;
+                e.ok = false;
+                publish_agg(status, flags, aggv, s * G + c, epoch, e);
+            }
+            continue;
+        }
+        const int stage = (int)(v % STAGES);
+        const skel_u64 tile = tile_of(s, j);
+        skel_T x[K];
+        if (tma) {
+            skel::mbar_wait(&bars[stage], (unsigned)((v / STAGES) & 1));
+            read_row(stages + stage * TILE_BYTES, t, x);
+        } else {
+            const skel_T *p = in + tile * TILE + (skel_u64)t * K;
+#pragma unroll
+            for (int k = 0; k < K; ++k) x[k] = p[k];
+        }
+        if (ph == 1) {
+            // ---- P1: ordered fold of the tile
+            VT a;
+            a.v = x[0];
+            a.ok = true;
+#pragma unroll
+            for (int k = 1; k < K; ++k) a.v = opf(a.v, x[k], tup);
+            __syncthreads();  // stage consumed
+            if (tma && t == 0) issue_next(stage);
+            const VT tv = block_fold(a, wsc, tup);
+            if (t == 0) {
+                run1 = comb(run1, tv, tup);
+                if (j == SCAN_CH - 1 || j == nj - 1) {
+                    publish_agg(status, flags, aggv, s * G + c, epoch, run1);
+                    run1.ok = false;
+                }
+            }
+        } else {
+            // ---- P2: scan of the tile with the running prefix
+#pragma unroll
+            for (int k = 1; k < K; ++k) x[k] = opf(x[k - 1], x[k], tup);
+            VT mine;
+            mine.v = x[K - 1];
+            mine.ok = true;
+            const VT excl = block_exscan(mine, wsc, &s_tot, tup);
+            const VT pre = comb(s_run, excl, tup);
+#pragma unroll
+            for (int k = K - 1; k >= 1; --k) x[k] = opf(pre.v, x[k - 1], tup);
+            x[0] = pre.v;
             if (tma) {
-                tma_prefetch_desc(&tin);
-                tma_prefetch_desc(&tout);
-            }
-            bool done = false;
-            skel_u64 last_i = 0;
-            for (skel_u64 i = 0;; ++i) {
-                const int s = (int)(i % SSTAGES);
-                bool stored = false;
-                if (i >= SSTAGES) {  // retire the tile that used this stage
-                    const skel_u64 old = tq[s];
-                    if (old < ntiles) {
-                        skel::mbar_wait(&wr_bar[s], (unsigned)(((i / SSTAGES) - 1) & 1));
-                        if (tma && (old + 1) * STILE <= n) {
-                            const int row = (int)(old * SRB);
-                            tma_store_rows(&tout, row, stages + s * STILE_BYTES);
-                            tma_store_rows(&tout, row + SRB / 2, stages + s * STILE_BYTES + STILE_BYTES / 2);
-                            skel::bulk_commit();
-                            stored = true;
-                        }
-                    }
-                }
-                // take the ticket only when the stage is about to be refilled (a held
-                // ticket delays every later tile's look-back); its latency overlaps
-                // the TMA store's read of the stage
-                skel_u64 tk = 0;
-                if (!done) tk = atomicAdd(&counters[0], 1u);
-                if (stored) skel::bulk_wait_read0();
-                if (done) {
-                    if (i >= last_i + SSTAGES) break;
-                    tq[s] = ntiles;
-                    continue;
-                }
-                tq[s] = tk;
-                mbar_arrive(&tick_bar[s]);
-                if (tk >= ntiles) {
-                    done = true;
-                    last_i = i;
-                    mbar_arrive(&full_bar[s]);
-                } else if (tma && (tk + 1) * STILE <= n) {
-                    issue_tile<SRB>(stages + s * STILE_BYTES, &tin, tk, &full_bar[s]);
-                } else {
-                    mbar_arrive(&full_bar[s]);
-                }
-            }
-            skel::bulk_wait0();
-        }
-    } else if (w == SNW + 1) {
-        // ------------------------------------------------------------ look-back
-        for (skel_u64 i = 0;; ++i) {
-            const int s = (int)(i % SSTAGES);
-            const unsigned ph = (unsigned)((i / SSTAGES) & 1);
-            skel::mbar_wait(&tick_bar[s], ph);
-            const skel_u64 tk = tq[s];
-            if (tk >= ntiles) break;
-            VT prefix;
-            if (tk == 0) {
-                prefix.v = seed ? seed->v : identity.v;
-                prefix.ok = true;
+                write_row(stages + stage * TILE_BYTES, t, x);
+                skel::fence_proxy_async();
             } else {
-                VT acc;
-                acc.ok = false;
-                long long j0 = (long long)tk - 1;
-                for (;;) {
-                    // lane covers tiles j0 - lane*8 - q, q = 0..7 (q = 0 nearest)
-                    unsigned st[LB_PER_LANE];
-                    skel_T v[LB_PER_LANE];
+                skel_T *o = out + tile * TILE + (skel_u64)t * K;
 #pragma unroll
-                    for (int q = 0; q < LB_PER_LANE; ++q) {
-                        const long long j = j0 - (long long)lane * LB_PER_LANE - q;
-                        st[q] = j >= 0 ? peek_state(status, flags, (skel_u64)j, epoch, v[q]) : 3u;
-                    }
-                    for (;;) {  // re-poll the ones not ready yet
-                        bool all = true;
-#pragma unroll
-                        for (int q = 0; q < LB_PER_LANE; ++q) {
-                            if (st[q] == 0) {
-                                const long long j = j0 - (long long)lane * LB_PER_LANE - q;
-                                st[q] = peek_state(status, flags, (skel_u64)j, epoch, v[q]);
-                                all = all && st[q] != 0;
-                            }
-                        }
-                        if (all) break;
-                    }
-                    if constexpr (!PACKED) {
-                        __threadfence();  // acquire: values were published before their flags
-#pragma unroll
-                        for (int q = 0; q < LB_PER_LANE; ++q) {
-                            const long long j = j0 - (long long)lane * LB_PER_LANE - q;
-                            if (st[q] == 1) v[q] = skel::ld_value(&aggv[j]).v;
-                            if (st[q] == 2) v[q] = skel::ld_value(&incv[j]).v;
-                        }
-                    }
-                    int qp = LB_PER_LANE;  // nearest inclusive prefix of this lane
-#pragma unroll
-                    for (int q = LB_PER_LANE - 1; q >= 0; --q)
-                        if (st[q] == 2) qp = q;
-                    const unsigned pm = __ballot_sync(0xffffffffu, qp < LB_PER_LANE);
-                    const int lp = pm ? __ffs(pm) - 1 : 32;
-                    VT lf;  // lane fold, older (larger q) on the left
-                    lf.ok = false;
-                    const int qmax = lane < lp ? LB_PER_LANE - 1 : (lane == lp ? qp : -1);
-#pragma unroll
-                    for (int q = LB_PER_LANE - 1; q >= 0; --q) {
-                        if (q <= qmax && st[q] != 3u) {
-                            VT e;
-                            e.v = v[q];
-                            e.ok = true;
-                            lf = comb(lf, e, tup);
-                        }
-                    }
-#pragma unroll
-                    for (int d = 1; d < 32; d <<= 1) {  // window fold, higher lanes (older) left
-                        VT o = vt_shfl_down(lf, d);
-                        if ((lane & (2 * d - 1)) == 0) lf = comb(o, lf, tup);
-                    }
-                    lf = vt_shfl_idx(lf, 0);
-                    acc = comb(lf, acc, tup);
-                    if (pm) break;
-                    j0 -= 32 * LB_PER_LANE;
-                }
-                prefix = acc;
+                for (int k = 0; k < K; ++k) o[k] = x[k];
             }
-            skel::mbar_wait(&agg_bar[s], ph);
-            const VT agg = s_agg[s];
-            const VT inc = comb(prefix, agg, tup);
-            if (lane == 0) {
-                publish(status, flags, aggv, incv, tk, epoch, 2u, inc.v);
-                if (tk == ntiles - 1 && total) total->v = inc.v;
-                s_pre[s] = prefix;
-                mbar_arrive(&pre_bar[s]);
-            }
-            __syncwarp();
-        }
-    } else {
-        // ------------------------------------------------------------ consumers
-        // iteration i: phase A of tile i (local scan, publish its aggregate),
-        // then phase B of tile i-1 (apply its prefix, hand the stage back), so
-        // a tile's aggregate is never held up by the previous tile's look-back.
-        bool pv = false, pstaged = false;  // previous tile pending phase B
-        int ps = 0;
-        unsigned pph = 0;
-        skel_u64 pfirst = 0, pkt = 0;
-        VT pexcl;
-        pexcl.ok = false;
-        for (skel_u64 i = 0;; ++i) {
-            const int s = (int)(i % SSTAGES);
-            const unsigned ph = (unsigned)((i / SSTAGES) & 1);
-            skel::mbar_wait(&full_bar[s], ph);
-            const skel_u64 tk = tq[s];
-            const bool live = tk < ntiles;
-            if (live) {
-                // ---- phase A(i)
-                const skel_u64 base = tk * STILE;
-                const bool full = base + STILE <= n;
-                const bool staged = tma && full;
-                VT mine;
-                mine.ok = false;
-                skel_u64 first = 0, kt = 0;
-                skel_T x[K];
-                if (staged) {
-                    read_row(stages + s * STILE_BYTES, t, x);
-#pragma unroll
-                    for (int k = 1; k < K; ++k) x[k] = opf(x[k - 1], x[k], tup);
-                    mine.v = x[K - 1];
-                    mine.ok = true;
-                } else {
-                    const skel_u64 cnt = full ? STILE : n - base;
-                    const skel_u64 per = full ? (skel_u64)K : (cnt + SRB - 1) / SRB;
-                    first = base + (skel_u64)t * per;
-                    const skel_u64 end = base + cnt;
-                    kt = first >= end ? 0 : ((end - first) < per ? (end - first) : per);
-                    for (skel_u64 k = 0; k < kt; ++k) {
-                        VT e;
-                        e.v = in[first + k];
-                        e.ok = true;
-                        mine = comb(mine, e, tup);
-                    }
+            __syncthreads();  // outputs staged, s_run / s_tot read by everyone
+            if (t == 0) {
+                s_run = comb(s_run, s_tot, tup);
+                if (tma) {
+                    const int row = (int)(tile * RB);
+                    tma_store_rows_hint(&tout, row, stages + stage * TILE_BYTES, pol_drop);
+                    tma_store_rows_hint(&tout, row + RB / 2, stages + stage * TILE_BYTES + TILE_BYTES / 2, pol_drop);
+                    skel::bulk_commit();
+                    skel::bulk_wait_read0();
+                    issue_next(stage);
                 }
-                const VT excl = cons_exscan(mine, wsc, &s_tot, tup);
-                if (t == 0) {
-                    const VT tot = s_tot;
-                    if (tk > 0) publish(status, flags, aggv, incv, tk, epoch, 1u, tot.v);
-                    s_agg[s] = tot;
-                    mbar_arrive(&agg_bar[s]);
-                }
-                if (staged) {
-                    // tile-local exclusive results y_k = excl (+) r_{k-1} (y_0 = excl;
-                    // row 0 has no excl: its y_0 slot is unused, y_k = r_{k-1})
-#pragma unroll
-                    for (int k = K - 1; k >= 1; --k) x[k] = excl.ok ? opf(excl.v, x[k - 1], tup) : x[k - 1];
-                    x[0] = excl.v;
-                    write_row(stages + s * STILE_BYTES, t, x);
-                }
-                // ---- phase B(i-1)
-                if (pv) {
-                    skel::mbar_wait(&pre_bar[ps], pph);
-                    const VT prefix = s_pre[ps];
-                    if (pstaged) {
-                        skel_T y[K];
-                        read_row(stages + ps * STILE_BYTES, t, y);
-#pragma unroll
-                        for (int k = 0; k < K; ++k) y[k] = (t == 0 && k == 0) ? prefix.v : opf(prefix.v, y[k], tup);
-                        write_row(stages + ps * STILE_BYTES, t, y);
-                        skel::fence_proxy_async();
-                    } else {
-                        const VT pre = comb(prefix, pexcl, tup);
-                        skel_T run = pre.v;  // second pass (in-place safe: read, then write)
-                        for (skel_u64 k = 0; k < pkt; ++k) {
-                            const skel_T e = in[pfirst + k];
-                            out[pfirst + k] = run;
-                            run = opf(run, e, tup);
-                        }
-                    }
-                    mbar_arrive(&wr_bar[ps]);
-                }
-                pv = true;
-                pstaged = staged;
-                ps = s;
-                pph = ph;
-                pfirst = first;
-                pkt = kt;
-                pexcl = excl;
-            } else {
-                // no more tiles: finish the pending one
-                if (pv) {
-                    skel::mbar_wait(&pre_bar[ps], pph);
-                    const VT prefix = s_pre[ps];
-                    if (pstaged) {
-                        skel_T y[K];
-                        read_row(stages + ps * STILE_BYTES, t, y);
-#pragma unroll
-                        for (int k = 0; k < K; ++k) y[k] = (t == 0 && k == 0) ? prefix.v : opf(prefix.v, y[k], tup);
-                        write_row(stages + ps * STILE_BYTES, t, y);
-                        skel::fence_proxy_async();
-                    } else {
-                        const VT pre = comb(prefix, pexcl, tup);
-                        skel_T run = pre.v;
-                        for (skel_u64 k = 0; k < pkt; ++k) {
-                            const skel_T e = in[pfirst + k];
-                            out[pfirst + k] = run;
-                            run = opf(run, e, tup);
-                        }
-                    }
-                    mbar_arrive(&wr_bar[ps]);
-                }
-                break;
             }
         }
+        ++v;
     }
-    __syncthreads();
-    if (t == 0) {
-        __threadfence();
-        const unsigned prev = atomicAdd(&counters[1], 1u);
-        if (prev == gridDim.x - 1) {
-            counters[0] = 0;
-            counters[1] = 0;
+    // ---- ragged last tile and the device total: CTA G-1
+    if (c == G - 1) {
+        if (w == 0) {
+            VT carry = s_carry;
+            if (nslices > 0) {
+                const VT prev = warp_fold_aggs(status, flags, aggv, (nslices - 1) * G, (int)G, epoch, lane, tup);
+                carry = comb(carry, prev, tup);
+            }
+            if (lane == 0) s_run = carry;
         }
+        __syncthreads();
+        const skel_u64 base = nft * TILE;
+        VT mine;
+        mine.ok = false;
+        skel_u64 first = 0, kt = 0;
+        if (base < n) {
+            const skel_u64 cnt = n - base, per = (cnt + RB - 1) / RB;
+            first = base + (skel_u64)t * per;
+            const skel_u64 end = n;
+            kt = first >= end ? 0 : ((end - first) < per ? (end - first) : per);
+            for (skel_u64 k = 0; k < kt; ++k) {
+                VT e;
+                e.v = in[first + k];
+                e.ok = true;
+                mine = comb(mine, e, tup);
+            }
+        }
+        const VT excl = block_exscan(mine, wsc, &s_tot, tup);
+        const VT pre = comb(s_run, excl, tup);
+        skel_T r = pre.v;  // second pass (in-place safe: read, then write)
+        for (skel_u64 k = 0; k < kt; ++k) {
+            const skel_T e = in[first + k];
+            out[first + k] = r;
+            r = opf(r, e, tup);
+        }
+        if (t == 0 && total) total->v = comb(s_run, s_tot, tup).v;
     }
+    if (tma && t == 0) skel::bulk_wait0();
 }
