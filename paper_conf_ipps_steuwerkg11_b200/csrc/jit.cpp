@@ -177,6 +177,12 @@ static int assemble(Kind kind, const std::string &user, int block, bool fmad, st
     if (entry.empty()) return SKEL_ERR_COMPILE;
     *opts = {"--gpu-architecture=sm_100a", "-default-device", "-std=c++17", "-lineinfo",
              fmad ? "--fmad=true" : "--fmad=false"};
+    // tuning experiments: extra -D options for the skeleton templates (part of the cache key)
+    if (const char *extra = getenv("SKEL_NVRTC_DEFINES")) {
+        std::stringstream ss(extra);
+        std::string tok;
+        while (ss >> tok) opts->push_back(tok);
+    }
     std::string defs;
     if (kind == Kind::Map) defs = "#define SKEL_NIN 1\n#define SKEL_BLOCK " + std::to_string(block) + "\n";
     if (kind == Kind::Zip) defs = "#define SKEL_NIN 2\n#define SKEL_BLOCK " + std::to_string(block) + "\n";

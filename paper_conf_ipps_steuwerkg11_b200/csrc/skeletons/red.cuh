@@ -398,14 +398,24 @@ extern "C" __global__ void skel_seed_kernel(const skel_S *aggs, int k, const ske
 // The ragged last tile is scanned by CTA G-1 with direct loads; element sizes
 // without a TMA path use direct loads for every tile.
 // ============================================================================
+#ifndef SKEL_SCAN_KEEP_POLICY
+#define SKEL_SCAN_KEEP_POLICY evict_last
+#endif
+#ifndef SKEL_SCAN_DROP_POLICY
+#define SKEL_SCAN_DROP_POLICY evict_first
+#endif
+#define SKEL_STR2(x) #x
+#define SKEL_STR(x) SKEL_STR2(x)
+// L2 policy of the P1 loads (the slice must survive until P2 re-reads it)
 __device__ __forceinline__ skel_u64 policy_evict_last() {
     skel_u64 p;
-    asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+    asm volatile("createpolicy.fractional.L2::" SKEL_STR(SKEL_SCAN_KEEP_POLICY) ".b64 %0, 1.0;" : "=l"(p));
     return p;
 }
+// L2 policy of the P2 loads and of the output stores (dead after use)
 __device__ __forceinline__ skel_u64 policy_evict_first() {
     skel_u64 p;
-    asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
+    asm volatile("createpolicy.fractional.L2::" SKEL_STR(SKEL_SCAN_DROP_POLICY) ".b64 %0, 1.0;" : "=l"(p));
     return p;
 }
 __device__ __forceinline__ void tma_load_rows_hint(void *dst, const skel_tmap *map, int row, skel_u64 *bar,
@@ -563,7 +573,8 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
     if (tma && t == 0)
         for (int st = 0; st < STAGES; ++st) issue_next(st);
 
-    skel_u64 v = 0;  // valid items consumed
+    int pending = -1;  // thread 0: stage whose TMA store may still be reading it
+    skel_u64 v = 0;    // valid items consumed
     VT run1;         // P1 running aggregate (thread 0)
     run1.ok = false;
     int ph;
@@ -615,7 +626,14 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
 #pragma unroll
             for (int k = 1; k < K; ++k) a.v = opf(a.v, x[k], tup);
             __syncthreads();  // stage consumed
-            if (tma && t == 0) issue_next(stage);
+            if (tma && t == 0) {
+                if (pending >= 0) {  // a stored stage waiting for its refill goes first (sequence order)
+                    skel::bulk_wait_read0();
+                    issue_next(pending);
+                    pending = -1;
+                }
+                issue_next(stage);
+            }
             const VT tv = block_fold(a, wsc, tup);
             if (t == 0) {
                 run1 = comb(run1, tv, tup);
@@ -652,8 +670,13 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
                     tma_store_rows_hint(&tout, row, stages + stage * TILE_BYTES, pol_drop);
                     tma_store_rows_hint(&tout, row + RB / 2, stages + stage * TILE_BYTES + TILE_BYTES / 2, pol_drop);
                     skel::bulk_commit();
-                    skel::bulk_wait_read0();
-                    issue_next(stage);
+                    // refill the stage of the previous store once that store has read it;
+                    // this one's stage is refilled after the next tile (off the critical path)
+                    if (pending >= 0) {
+                        asm volatile("cp.async.bulk.wait_group.read 1;" ::: "memory");
+                        issue_next(pending);
+                    }
+                    pending = stage;
                 }
             }
         }
