@@ -77,7 +77,7 @@ constexpr skel_sig_t skel_make_sig() {
     s.v[11] = DSMEM;
     s.v[12] = DSMEM;
     s.v[13] = PACKED;
-    s.v[14] = RB;  // scan kernel block size
+    s.v[14] = RB + 32;  // scan kernel block size (consumers + TMA producer warp)
     s.v[15] = SCAN_CH;
     for (int i = 0; i < skel_Lay::n && i < 32; ++i) {
         s.v[16 + 4 * i] = skel_Lay::size(i);
@@ -509,7 +509,61 @@ __device__ __forceinline__ bool scan_item(skel_u64 q, skel_u64 nslices, int &pha
     return true;
 }
 
-extern "C" __global__ void __launch_bounds__(RB, 1)
+// consumers = the RB threads of warps 0..NW-1; warp NW is the TMA producer
+constexpr int SCAN_THREADS = RB + 32;
+__device__ __forceinline__ void cons_sync() { asm volatile("bar.sync 1, %0;" ::"n"(RB) : "memory"); }
+__device__ __forceinline__ void mbar_arrive(skel_u64 *bar) {
+    asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(skel::smem_addr(bar)) : "memory");
+}
+// ordered fold over the consumers; result in thread 0
+template <class Tup> __device__ __forceinline__ VT cons_fold(VT x, VT *wpart, Tup &t) {
+    const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+    x = warp_fold(x, lane, t);
+    if (lane == 0) wpart[w] = x;
+    cons_sync();
+    VT r;
+    r.ok = false;
+    if (w == 0) {
+        VT y;
+        y.ok = false;
+        if (lane < NW) y = wpart[lane];
+        r = warp_fold(y, lane, t);
+    }
+    return r;
+}
+// ordered exclusive scan over the consumers; block total to *total
+template <class Tup> __device__ __forceinline__ VT cons_exscan(VT x, VT *wsc, VT *total, Tup &t) {
+    const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+    VT inc = x;
+#pragma unroll
+    for (int d = 1; d < 32; d <<= 1) {
+        VT o = vt_shfl_up(inc, d);
+        if (lane >= d) inc = comb(o, inc, t);
+    }
+    VT ex = vt_shfl_up(inc, 1);
+    if (lane == 0) ex.ok = false;
+    if (lane == 31) wsc[w] = inc;
+    cons_sync();
+    if (w == 0) {
+        VT y;
+        y.ok = false;
+        if (lane < NW) y = wsc[lane];
+        VT yi = y;
+#pragma unroll
+        for (int d = 1; d < 32; d <<= 1) {
+            VT o = vt_shfl_up(yi, d);
+            if (lane >= d) yi = comb(o, yi, t);
+        }
+        VT ye = vt_shfl_up(yi, 1);
+        if (lane == 0) ye.ok = false;
+        if (lane < NW) wsc[lane] = ye;
+        if (lane == NW - 1) *total = yi;
+    }
+    cons_sync();
+    return comb(wsc[w], ex, t);
+}
+
+extern "C" __global__ void __launch_bounds__(SCAN_THREADS, 1)
     skel_scan_kernel(const __grid_constant__ skel_tmap tin, const __grid_constant__ skel_tmap tout,
                      const skel_T *in, skel_T *out, skel_u64 n, int use_tma, const skel_S identity, const skel_S *seed,
                      skel_u64 *status, unsigned *flags, skel_S *aggv, skel_S *incv, unsigned *counters,
@@ -517,102 +571,112 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
     (void)incv;
     (void)counters;
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
-    __shared__ skel_u64 bars[STAGES];
+    __shared__ skel_u64 full_bar[STAGES], done_bar[STAGES];
     __shared__ VT wsc[NW];
-    __shared__ VT s_tot, s_run, s_carry;
+    __shared__ VT s_tot, s_run;
     const int t = threadIdx.x, lane = t & 31, w = t >> 5;
     const skel_u64 G = gridDim.x, c = blockIdx.x;
-    const skel_u64 nft = n / TILE;                    // full tiles
+    const skel_u64 nft = n / TILE;  // full tiles
     const skel_u64 per_slice = G * SCAN_CH;
     const skel_u64 nslices = (nft + per_slice - 1) / per_slice;
     const bool tma = TMA_OK && use_tma;
     unsigned char *stages = aligned_stages(skel_dsmem);
     auto tile_of = [&](skel_u64 s, int j) -> skel_u64 { return (s * G + c) * SCAN_CH + (skel_u64)j; };
-    // valid tiles of CTA c in slice s: j < jn(s)
-    auto jn = [&](skel_u64 s) -> int {
+    auto jn = [&](skel_u64 s) -> int {  // valid tiles of this CTA in slice s
         const skel_u64 first = (s * G + c) * SCAN_CH;
         if (first >= nft) return 0;
         const skel_u64 left = nft - first;
         return (int)(left < (skel_u64)SCAN_CH ? left : (skel_u64)SCAN_CH);
     };
-    skel_u64 pol_keep = 0, pol_drop = 0;
-    if (tma && t == 0) {
-        pol_keep = policy_evict_last();
-        pol_drop = policy_evict_first();
-        for (int st = 0; st < STAGES; ++st) skel::mbar_init(&bars[st], 1);
-        skel::fence_mbar_init();
-        tma_prefetch_desc(&tin);
-        tma_prefetch_desc(&tout);
-    }
     if (t == 0) {
-        VT cz;
-        cz.v = seed ? seed->v : identity.v;
-        cz.ok = true;
-        s_carry = cz;  // carry(0)
+        for (int st = 0; st < STAGES; ++st) {
+            skel::mbar_init(&full_bar[st], 1);
+            skel::mbar_init(&done_bar[st], RB);
+        }
+        skel::fence_mbar_init();
     }
     __syncthreads();
 
-    // the producer (thread 0) walks the same item sequence, STAGES valid items ahead
-    skel_u64 pq = 0;  // next sequence position to load
-    auto issue_next = [&](int stage) {
-        int ph, j;
-        skel_u64 s;
-        while (scan_item(pq, nslices, ph, s, j)) {
-            ++pq;
-            if (j < jn(s)) {
-                const int row = (int)(tile_of(s, j) * RB);
-                unsigned char *dst = stages + stage * TILE_BYTES;
+    if (w == NW) {
+        // ================================================ TMA producer warp
+        if (tma && lane == 0) {
+            const skel_u64 pol_keep = policy_evict_last(), pol_drop = policy_evict_first();
+            tma_prefetch_desc(&tin);
+            tma_prefetch_desc(&tout);
+            skel_u64 ring_tile[STAGES];
+            int ring_ph[STAGES];
+            skel_u64 v = 0;
+            int ph, j;
+            skel_u64 s;
+            auto retire = [&](int st, skel_u64 use) {  // wait until the consumers are done with a stage
+                skel::mbar_wait(&done_bar[st], (unsigned)(use & 1));
+                if (ring_ph[st] == 2) {  // P2: the stage holds outputs
+                    const int row = (int)(ring_tile[st] * RB);
+                    tma_store_rows_hint(&tout, row, stages + st * TILE_BYTES, pol_drop);
+                    tma_store_rows_hint(&tout, row + RB / 2, stages + st * TILE_BYTES + TILE_BYTES / 2, pol_drop);
+                    skel::bulk_commit();
+                    skel::bulk_wait_read0();
+                }
+            };
+            for (skel_u64 q = 0; scan_item(q, nslices, ph, s, j); ++q) {
+                if (j >= jn(s)) continue;
+                const int st = (int)(v % STAGES);
+                if (v >= STAGES) retire(st, v / STAGES - 1);
+                const skel_u64 tile = tile_of(s, j);
+                ring_tile[st] = tile;
+                ring_ph[st] = ph;
+                const int row = (int)(tile * RB);
+                unsigned char *dst = stages + st * TILE_BYTES;
                 const skel_u64 pol = ph == 1 ? pol_keep : pol_drop;
-                skel::mbar_expect_tx(&bars[stage], TILE_BYTES);
-                tma_load_rows_hint(dst, &tin, row, &bars[stage], pol);
-                tma_load_rows_hint(dst + TILE_BYTES / 2, &tin, row + RB / 2, &bars[stage], pol);
-                return;
+                skel::mbar_expect_tx(&full_bar[st], TILE_BYTES);
+                tma_load_rows_hint(dst, &tin, row, &full_bar[st], pol);
+                tma_load_rows_hint(dst + TILE_BYTES / 2, &tin, row + RB / 2, &full_bar[st], pol);
+                ++v;
             }
+            const skel_u64 first = v > STAGES ? v - STAGES : 0;
+            for (skel_u64 u = first; u < v; ++u) retire((int)(u % STAGES), u / STAGES);
+            skel::bulk_wait0();
         }
-    };
-    if (tma && t == 0)
-        for (int st = 0; st < STAGES; ++st) issue_next(st);
+        return;
+    }
 
-    int pending = -1;  // thread 0: stage whose TMA store may still be reading it
-    skel_u64 v = 0;    // valid items consumed
-    VT run1;         // P1 running aggregate (thread 0)
+    // ==================================================== consumer warps
+    skel_u64 v = 0;  // valid items consumed
+    VT run1;         // P1 running aggregate of this CTA's sub-chunk (thread 0)
     run1.ok = false;
-    int ph;
+    VT run;          // P2 running prefix (identical in every consumer thread)
+    run.ok = false;
+    VT carry;        // carry(s) (warp 0)
+    carry.v = seed ? seed->v : identity.v;
+    carry.ok = true;
+    int ph, j;
     skel_u64 s;
-    int j;
     for (skel_u64 q = 0; scan_item(q, nslices, ph, s, j); ++q) {
         const int nj = jn(s);
         if (ph == 2 && j == 0) {
-            // ---- prefix(s, c) = carry(s) (+) A(s,0..c-1); carry(s+1) prepared
+            // prefix(s, c) = carry(s) (+) A(s,0..c-1), carry(s) = carry(s-1) (+) A(s-1, 0..G-1)
             if (w == 0) {
-                VT carry = s_carry;
-                if (s > 0) {
-                    const VT prev = warp_fold_aggs(status, flags, aggv, (s - 1) * G, (int)G, epoch, lane, tup);
-                    carry = comb(carry, prev, tup);
-                }
+                if (s > 0) carry = comb(carry, warp_fold_aggs(status, flags, aggv, (s - 1) * G, (int)G, epoch, lane, tup), tup);
                 const VT mine = warp_fold_aggs(status, flags, aggv, s * G, (int)c, epoch, lane, tup);
-                if (lane == 0) {
-                    s_carry = carry;
-                    s_run = comb(carry, mine, tup);
-                }
+                if (lane == 0) s_run = comb(carry, mine, tup);
             }
-            __syncthreads();
+            cons_sync();
+            run = s_run;
         }
         if (j >= nj) {
-            // no tile of this CTA in slice s: publish an empty aggregate once
-            if (ph == 1 && j == 0 && nj == 0 && t == 0) {
+            if (ph == 1 && j == 0 && nj == 0 && t == 0) {  // empty sub-chunk: publish once
                 VT e;
                 e.ok = false;
                 publish_agg(status, flags, aggv, s * G + c, epoch, e);
             }
             continue;
         }
-        const int stage = (int)(v % STAGES);
+        const int st = (int)(v % STAGES);
         const skel_u64 tile = tile_of(s, j);
         skel_T x[K];
         if (tma) {
-            skel::mbar_wait(&bars[stage], (unsigned)((v / STAGES) & 1));
-            read_row(stages + stage * TILE_BYTES, t, x);
+            skel::mbar_wait(&full_bar[st], (unsigned)((v / STAGES) & 1));
+            read_row(stages + st * TILE_BYTES, t, x);
         } else {
             const skel_T *p = in + tile * TILE + (skel_u64)t * K;
 #pragma unroll
@@ -620,24 +684,16 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
         }
         if (ph == 1) {
             // ---- P1: ordered fold of the tile
+            if (tma) mbar_arrive(&done_bar[st]);  // stage read: free for the producer
             VT a;
             a.v = x[0];
             a.ok = true;
 #pragma unroll
             for (int k = 1; k < K; ++k) a.v = opf(a.v, x[k], tup);
-            __syncthreads();  // stage consumed
-            if (tma && t == 0) {
-                if (pending >= 0) {  // a stored stage waiting for its refill goes first (sequence order)
-                    skel::bulk_wait_read0();
-                    issue_next(pending);
-                    pending = -1;
-                }
-                issue_next(stage);
-            }
-            const VT tv = block_fold(a, wsc, tup);
+            const VT tv = cons_fold(a, wsc, tup);
             if (t == 0) {
                 run1 = comb(run1, tv, tup);
-                if (j == SCAN_CH - 1 || j == nj - 1) {
+                if (j == nj - 1) {
                     publish_agg(status, flags, aggv, s * G + c, epoch, run1);
                     run1.ok = false;
                 }
@@ -649,35 +705,20 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
             VT mine;
             mine.v = x[K - 1];
             mine.ok = true;
-            const VT excl = block_exscan(mine, wsc, &s_tot, tup);
-            const VT pre = comb(s_run, excl, tup);
+            const VT excl = cons_exscan(mine, wsc, &s_tot, tup);
+            const VT pre = comb(run, excl, tup);
+            run = comb(run, s_tot, tup);
 #pragma unroll
             for (int k = K - 1; k >= 1; --k) x[k] = opf(pre.v, x[k - 1], tup);
             x[0] = pre.v;
             if (tma) {
-                write_row(stages + stage * TILE_BYTES, t, x);
+                write_row(stages + st * TILE_BYTES, t, x);
                 skel::fence_proxy_async();
+                mbar_arrive(&done_bar[st]);  // outputs staged: the producer stores them
             } else {
                 skel_T *o = out + tile * TILE + (skel_u64)t * K;
 #pragma unroll
                 for (int k = 0; k < K; ++k) o[k] = x[k];
-            }
-            __syncthreads();  // outputs staged, s_run / s_tot read by everyone
-            if (t == 0) {
-                s_run = comb(s_run, s_tot, tup);
-                if (tma) {
-                    const int row = (int)(tile * RB);
-                    tma_store_rows_hint(&tout, row, stages + stage * TILE_BYTES, pol_drop);
-                    tma_store_rows_hint(&tout, row + RB / 2, stages + stage * TILE_BYTES + TILE_BYTES / 2, pol_drop);
-                    skel::bulk_commit();
-                    // refill the stage of the previous store once that store has read it;
-                    // this one's stage is refilled after the next tile (off the critical path)
-                    if (pending >= 0) {
-                        asm volatile("cp.async.bulk.wait_group.read 1;" ::: "memory");
-                        issue_next(pending);
-                    }
-                    pending = stage;
-                }
             }
         }
         ++v;
@@ -685,14 +726,12 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
     // ---- ragged last tile and the device total: CTA G-1
     if (c == G - 1) {
         if (w == 0) {
-            VT carry = s_carry;
-            if (nslices > 0) {
-                const VT prev = warp_fold_aggs(status, flags, aggv, (nslices - 1) * G, (int)G, epoch, lane, tup);
-                carry = comb(carry, prev, tup);
-            }
+            if (nslices > 0)
+                carry = comb(carry, warp_fold_aggs(status, flags, aggv, (nslices - 1) * G, (int)G, epoch, lane, tup), tup);
             if (lane == 0) s_run = carry;
         }
-        __syncthreads();
+        cons_sync();
+        const VT carry_end = s_run;
         const skel_u64 base = nft * TILE;
         VT mine;
         mine.ok = false;
@@ -700,8 +739,7 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
         if (base < n) {
             const skel_u64 cnt = n - base, per = (cnt + RB - 1) / RB;
             first = base + (skel_u64)t * per;
-            const skel_u64 end = n;
-            kt = first >= end ? 0 : ((end - first) < per ? (end - first) : per);
+            kt = first >= n ? 0 : ((n - first) < per ? (n - first) : per);
             for (skel_u64 k = 0; k < kt; ++k) {
                 VT e;
                 e.v = in[first + k];
@@ -709,15 +747,14 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
                 mine = comb(mine, e, tup);
             }
         }
-        const VT excl = block_exscan(mine, wsc, &s_tot, tup);
-        const VT pre = comb(s_run, excl, tup);
+        const VT excl = cons_exscan(mine, wsc, &s_tot, tup);
+        const VT pre = comb(carry_end, excl, tup);
         skel_T r = pre.v;  // second pass (in-place safe: read, then write)
         for (skel_u64 k = 0; k < kt; ++k) {
             const skel_T e = in[first + k];
             out[first + k] = r;
             r = opf(r, e, tup);
         }
-        if (t == 0 && total) total->v = comb(s_run, s_tot, tup).v;
+        if (t == 0 && total) total->v = comb(carry_end, s_tot, tup).v;
     }
-    if (tma && t == 0) skel::bulk_wait0();
 }
