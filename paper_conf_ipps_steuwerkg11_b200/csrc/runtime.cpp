@@ -1401,13 +1401,25 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
     std::vector<unsigned char> abuf;
     // seeds: device k starts from agg_0 (+) ... (+) agg_{k-1} (one exchange of
     // D partial results)
-    const uint64_t TILE = m->sig[10];
-    const uint64_t CH = m->sig[15];  // tiles per CTA per slice
+    const uint64_t SRB = m->sig[15] & 0xffff;  // rows (consumer threads) per scan tile
+    const uint64_t TILE = SRB * m->sig[8];      // scan tile (elements)
+    const uint64_t CH = m->sig[15] >> 16;       // tiles per CTA per slice
     const bool packed = m->sig[13] != 0;
+    TRY(set_smem_attr(ctx, m, ctx->slots[0]));
+    int occ = 1;  // persistent grid: SMs x resident CTAs per SM
+    {
+        DevGuard g(ctx->slots[0].dev);
+        if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, (const void *)m->k_scan, (int)m->sig[14],
+                                                          (size_t)m->sig[12]) != cudaSuccess || occ < 1) {
+            cudaGetLastError();
+            occ = 1;
+        }
+    }
+    auto scan_grid = [&](const Slot &s) -> uint64_t { return (uint64_t)s.sms * (uint64_t)occ; };
     // one aggregate status word per (slice, CTA)
     auto scan_slots = [&](const Slot &s, uint64_t cnt) -> uint64_t {
-        const uint64_t per_slice = (uint64_t)s.sms * CH, nft = cnt / TILE;
-        return std::max<uint64_t>(1, (nft + per_slice - 1) / per_slice) * (uint64_t)s.sms;
+        const uint64_t per_slice = scan_grid(s) * CH, nft = cnt / TILE;
+        return std::max<uint64_t>(1, (nft + per_slice - 1) / per_slice) * scan_grid(s);
     };
     for (size_t li = 0; li < ctx->slots.size(); ++li) {
         Slot &s = ctx->slots[li];
@@ -1434,7 +1446,7 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         Slot &s = ctx->slots[li];
         uint64_t cnt = in->bufs[li].count;
         if (!cnt) continue;
-        const size_t G = (size_t)s.sms;  // persistent: one CTA per SM
+        const size_t G = (size_t)scan_grid(s);
         const RedLayout &L = Ls[li];
         TRY(ensure_status(ctx, s, scan_slots(s, cnt), packed));
         TRY(set_smem_attr(ctx, m, s));
@@ -1453,8 +1465,9 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         const void *pin = in->bufs[li].ptr(in->es);
         void *pout = out->bufs[li].ptr(out->es);
         CUtensorMap tin, tout;
-        const uint64_t rows = (cnt / TILE) * m->sig[9];
-        int use_tma = m->sig[5] && make_tmap(&tin, pin, rows) && make_tmap(&tout, pout, rows);
+        const uint64_t rows = (cnt / TILE) * SRB;
+        int use_tma = m->sig[5] && make_tmap(&tin, pin, rows, (uint32_t)(SRB / 2)) &&
+                      make_tmap(&tout, pout, rows, (uint32_t)(SRB / 2));
         void *status = s.st64, *flags = s.fl32, *aggv = s.ws + L.o_aggv, *incv = s.ws + L.o_incv;
         unsigned *counters = s.counters;
         void *total = nullptr;

@@ -55,9 +55,21 @@ constexpr int STAGES = SKEL_STAGES;
 constexpr unsigned DSMEM = TMA_OK ? STAGES * TILE_BYTES + 1024 : 0;
 // Scan: tiles per CTA per slice (see the Scan section)
 #ifndef SKEL_SCAN_CH
-#define SKEL_SCAN_CH 3
+#define SKEL_SCAN_CH 2
 #endif
 constexpr int SCAN_CH = SKEL_SCAN_CH;
+#ifndef SKEL_SCAN_RB
+#define SKEL_SCAN_RB 512
+#endif
+#ifndef SKEL_SCAN_STAGES
+#define SKEL_SCAN_STAGES 3
+#endif
+constexpr int SRB = SKEL_SCAN_RB;  // consumer threads = rows per scan tile
+constexpr int SNW = SRB / 32;
+constexpr int SSTAGES = SKEL_SCAN_STAGES;
+constexpr skel_u64 STILE = (skel_u64)SRB * K;
+constexpr unsigned STILE_BYTES = (unsigned)(STILE * sizeof(skel_T));
+constexpr unsigned SDSMEM = TMA_OK ? SSTAGES * STILE_BYTES + 1024 : 0;
 constexpr bool PACKED = sizeof(skel_S) == 4;  // status = value:32 | epoch:30 | state:2
 
 struct skel_sig_t { skel_u64 v[16 + 4 * 32]; };
@@ -75,10 +87,10 @@ constexpr skel_sig_t skel_make_sig() {
     s.v[9] = RB;
     s.v[10] = TILE;
     s.v[11] = DSMEM;
-    s.v[12] = DSMEM;
+    s.v[12] = SDSMEM;
     s.v[13] = PACKED;
-    s.v[14] = RB + 32;  // scan kernel block size (consumers + TMA producer warp)
-    s.v[15] = SCAN_CH;
+    s.v[14] = SRB + 64;  // scan kernel block size (consumers + producer + prefix warps); tile = SRB * K
+    s.v[15] = (skel_u64)SRB | ((skel_u64)SCAN_CH << 16);  // scan rows per tile | tiles per CTA per slice
     for (int i = 0; i < skel_Lay::n && i < 32; ++i) {
         s.v[16 + 4 * i] = skel_Lay::size(i);
         s.v[17 + 4 * i] = skel_Lay::align(i);
@@ -468,50 +480,93 @@ __device__ __forceinline__ VT wait_agg(const skel_u64 *st64, const unsigned *fl3
     }
     return r;
 }
-// ordered fold of A(base .. base+cnt-1) by one warp; result in every lane
+// relaxed probe of A(idx): true once published in this epoch
+__device__ __forceinline__ bool probe_agg(const skel_u64 *st64, const unsigned *fl32, const skel_S *vals, skel_u64 idx,
+                                          unsigned epoch, VT &r) {
+    if constexpr (PACKED) {
+        skel_u64 word;
+        asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(word) : "l"(st64 + idx) : "memory");
+        if (((unsigned)word >> 2) != epoch) return false;
+        r.ok = ((unsigned)word & 3u) == 1u;
+        r.v = skel::bit_cast<skel_S>((unsigned)(word >> 32)).v;
+        return true;
+    } else {
+        const unsigned f = skel::ld_acquire(&fl32[idx]);
+        if ((f >> 2) != epoch) return false;
+        r.ok = (f & 3u) == 1u;
+        if (r.ok) r.v = skel::ld_value(&vals[idx]).v;
+        return true;
+    }
+}
+// ordered fold of A(base .. base+cnt-1) by one warp (cnt <= 32*AGG_PER);
+// every lane issues all of its probes before waiting; result in every lane
+constexpr int AGG_PER = 16;
 template <class Tup>
 __device__ __forceinline__ VT warp_fold_aggs(const skel_u64 *st64, const unsigned *fl32, const skel_S *vals,
                                              skel_u64 base, int cnt, unsigned epoch, int lane, Tup &t) {
     const int per = (cnt + 31) / 32;
+    VT e[AGG_PER];
+    bool got[AGG_PER];
+#pragma unroll
+    for (int k = 0; k < AGG_PER; ++k) got[k] = !(k < per && lane * per + k < cnt);
+    for (unsigned ns = 32;; ns = ns < 1024 ? 2 * ns : ns) {
+        bool all = true;
+#pragma unroll
+        for (int k = 0; k < AGG_PER; ++k) {
+            if (!got[k]) {
+                got[k] = probe_agg(st64, fl32, vals, base + lane * per + k, epoch, e[k]);
+                all = all && got[k];
+            }
+        }
+        if (__all_sync(0xffffffffu, all)) break;
+        __nanosleep(ns);  // back off: many CTAs poll the same status lines
+    }
     VT a;
     a.ok = false;
-    for (int k = 0; k < per; ++k) {
-        const int i = lane * per + k;
-        if (i < cnt) a = comb(a, wait_agg(st64, fl32, vals, base + i, epoch), t);
-    }
+#pragma unroll
+    for (int k = 0; k < AGG_PER; ++k)
+        if (k < per && lane * per + k < cnt) a = comb(a, e[k], t);
     a = warp_fold(a, lane, t);
     return vt_shfl_idx(a, 0);
 }
 
-// work item q of a CTA's sequence: P1(0) x CH, then per slice s: P1(s+1) x CH
-// (if any), P2(s) x CH.  Returns false past the end.
+// work item q of a CTA's sequence: P1 of slices 0..LAG-1, then per slice s:
+// P1(s+LAG) x CH (if that slice exists), P2(s) x CH.  Returns false past the
+// end.  LAG slices of slack absorb the CTAs' speed differences.
+#ifndef SKEL_SCAN_LAG
+#define SKEL_SCAN_LAG 2
+#endif
+constexpr int SCAN_LAG = SKEL_SCAN_LAG;
 __device__ __forceinline__ bool scan_item(skel_u64 q, skel_u64 nslices, int &phase, skel_u64 &s, int &j) {
     const skel_u64 L = SCAN_CH;
-    if (nslices == 0) return false;
-    if (q < L) {
+    const skel_u64 P = nslices < (skel_u64)SCAN_LAG ? nslices : (skel_u64)SCAN_LAG;
+    if (q < P * L) {
         phase = 1;
-        s = 0;
-        j = (int)q;
+        s = q / L;
+        j = (int)(q % L);
         return true;
     }
-    const skel_u64 k = q - L, blk = k / (2 * L), r = k % (2 * L);
-    if (blk >= nslices) return false;
-    if (blk + 1 < nslices) {
+    const skel_u64 k = q - P * L;
+    const skel_u64 F = nslices > (skel_u64)SCAN_LAG ? nslices - SCAN_LAG : 0;
+    if (k < F * 2 * L) {
+        const skel_u64 blk = k / (2 * L), r = k % (2 * L);
         phase = r < L ? 1 : 2;
-        s = r < L ? blk + 1 : blk;
+        s = r < L ? blk + SCAN_LAG : blk;
         j = (int)(r < L ? r : r - L);
         return true;
     }
-    if (r >= L) return false;  // last slice: P2 only
+    const skel_u64 k2 = k - F * 2 * L;
+    s = F + k2 / L;
+    if (s >= nslices) return false;
     phase = 2;
-    s = blk;
-    j = (int)r;
+    j = (int)(k2 % L);
     return true;
 }
 
-// consumers = the RB threads of warps 0..NW-1; warp NW is the TMA producer
-constexpr int SCAN_THREADS = RB + 32;
-__device__ __forceinline__ void cons_sync() { asm volatile("bar.sync 1, %0;" ::"n"(RB) : "memory"); }
+// consumers = the SRB threads of warps 0..SNW-1; warp SNW is the TMA producer,
+// warp SNW+1 computes the slice prefixes ahead of the consumers
+constexpr int SCAN_THREADS = SRB + 64;
+__device__ __forceinline__ void cons_sync() { asm volatile("bar.sync 1, %0;" ::"n"(SRB) : "memory"); }
 __device__ __forceinline__ void mbar_arrive(skel_u64 *bar) {
     asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(skel::smem_addr(bar)) : "memory");
 }
@@ -526,7 +581,7 @@ template <class Tup> __device__ __forceinline__ VT cons_fold(VT x, VT *wpart, Tu
     if (w == 0) {
         VT y;
         y.ok = false;
-        if (lane < NW) y = wpart[lane];
+        if (lane < SNW) y = wpart[lane];
         r = warp_fold(y, lane, t);
     }
     return r;
@@ -547,7 +602,7 @@ template <class Tup> __device__ __forceinline__ VT cons_exscan(VT x, VT *wsc, VT
     if (w == 0) {
         VT y;
         y.ok = false;
-        if (lane < NW) y = wsc[lane];
+        if (lane < SNW) y = wsc[lane];
         VT yi = y;
 #pragma unroll
         for (int d = 1; d < 32; d <<= 1) {
@@ -556,14 +611,17 @@ template <class Tup> __device__ __forceinline__ VT cons_exscan(VT x, VT *wsc, VT
         }
         VT ye = vt_shfl_up(yi, 1);
         if (lane == 0) ye.ok = false;
-        if (lane < NW) wsc[lane] = ye;
-        if (lane == NW - 1) *total = yi;
+        if (lane < SNW) wsc[lane] = ye;
+        if (lane == SNW - 1) *total = yi;
     }
     cons_sync();
     return comb(wsc[w], ex, t);
 }
 
-extern "C" __global__ void __launch_bounds__(SCAN_THREADS, 1)
+#ifndef SKEL_SCAN_MINB
+#define SKEL_SCAN_MINB 1
+#endif
+extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
     skel_scan_kernel(const __grid_constant__ skel_tmap tin, const __grid_constant__ skel_tmap tout,
                      const skel_T *in, skel_T *out, skel_u64 n, int use_tma, const skel_S identity, const skel_S *seed,
                      skel_u64 *status, unsigned *flags, skel_S *aggv, skel_S *incv, unsigned *counters,
@@ -571,12 +629,12 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, 1)
     (void)incv;
     (void)counters;
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
-    __shared__ skel_u64 full_bar[STAGES], done_bar[STAGES];
-    __shared__ VT wsc[NW];
-    __shared__ VT s_tot, s_run;
+    __shared__ skel_u64 full_bar[SSTAGES], done_bar[SSTAGES], pre_full[2], pre_empty[2];
+    __shared__ VT wsc[SNW];
+    __shared__ VT s_tot, s_pre[2];
     const int t = threadIdx.x, lane = t & 31, w = t >> 5;
     const skel_u64 G = gridDim.x, c = blockIdx.x;
-    const skel_u64 nft = n / TILE;  // full tiles
+    const skel_u64 nft = n / STILE;  // full tiles
     const skel_u64 per_slice = G * SCAN_CH;
     const skel_u64 nslices = (nft + per_slice - 1) / per_slice;
     const bool tma = TMA_OK && use_tma;
@@ -589,53 +647,80 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, 1)
         return (int)(left < (skel_u64)SCAN_CH ? left : (skel_u64)SCAN_CH);
     };
     if (t == 0) {
-        for (int st = 0; st < STAGES; ++st) {
+        for (int st = 0; st < SSTAGES; ++st) {
             skel::mbar_init(&full_bar[st], 1);
-            skel::mbar_init(&done_bar[st], RB);
+            skel::mbar_init(&done_bar[st], SRB);
+        }
+        for (int k = 0; k < 2; ++k) {
+            skel::mbar_init(&pre_full[k], 1);
+            skel::mbar_init(&pre_empty[k], SRB);
         }
         skel::fence_mbar_init();
     }
     __syncthreads();
 
-    if (w == NW) {
+    if (w == SNW) {
         // ================================================ TMA producer warp
         if (tma && lane == 0) {
             const skel_u64 pol_keep = policy_evict_last(), pol_drop = policy_evict_first();
             tma_prefetch_desc(&tin);
             tma_prefetch_desc(&tout);
-            skel_u64 ring_tile[STAGES];
-            int ring_ph[STAGES];
+            skel_u64 ring_tile[SSTAGES];
+            int ring_ph[SSTAGES];
             skel_u64 v = 0;
             int ph, j;
             skel_u64 s;
             auto retire = [&](int st, skel_u64 use) {  // wait until the consumers are done with a stage
                 skel::mbar_wait(&done_bar[st], (unsigned)(use & 1));
                 if (ring_ph[st] == 2) {  // P2: the stage holds outputs
-                    const int row = (int)(ring_tile[st] * RB);
-                    tma_store_rows_hint(&tout, row, stages + st * TILE_BYTES, pol_drop);
-                    tma_store_rows_hint(&tout, row + RB / 2, stages + st * TILE_BYTES + TILE_BYTES / 2, pol_drop);
+                    const int row = (int)(ring_tile[st] * SRB);
+                    tma_store_rows_hint(&tout, row, stages + st * STILE_BYTES, pol_drop);
+                    tma_store_rows_hint(&tout, row + SRB / 2, stages + st * STILE_BYTES + STILE_BYTES / 2, pol_drop);
                     skel::bulk_commit();
                     skel::bulk_wait_read0();
                 }
             };
             for (skel_u64 q = 0; scan_item(q, nslices, ph, s, j); ++q) {
                 if (j >= jn(s)) continue;
-                const int st = (int)(v % STAGES);
-                if (v >= STAGES) retire(st, v / STAGES - 1);
+                const int st = (int)(v % SSTAGES);
+                if (v >= SSTAGES) retire(st, v / SSTAGES - 1);
                 const skel_u64 tile = tile_of(s, j);
                 ring_tile[st] = tile;
                 ring_ph[st] = ph;
-                const int row = (int)(tile * RB);
-                unsigned char *dst = stages + st * TILE_BYTES;
+                const int row = (int)(tile * SRB);
+                unsigned char *dst = stages + st * STILE_BYTES;
                 const skel_u64 pol = ph == 1 ? pol_keep : pol_drop;
-                skel::mbar_expect_tx(&full_bar[st], TILE_BYTES);
+                skel::mbar_expect_tx(&full_bar[st], STILE_BYTES);
                 tma_load_rows_hint(dst, &tin, row, &full_bar[st], pol);
-                tma_load_rows_hint(dst + TILE_BYTES / 2, &tin, row + RB / 2, &full_bar[st], pol);
+                tma_load_rows_hint(dst + STILE_BYTES / 2, &tin, row + SRB / 2, &full_bar[st], pol);
                 ++v;
             }
-            const skel_u64 first = v > STAGES ? v - STAGES : 0;
-            for (skel_u64 u = first; u < v; ++u) retire((int)(u % STAGES), u / STAGES);
+            const skel_u64 first = v > SSTAGES ? v - SSTAGES : 0;
+            for (skel_u64 u = first; u < v; ++u) retire((int)(u % SSTAGES), u / SSTAGES);
             skel::bulk_wait0();
+        }
+        return;
+    }
+
+    if (w == SNW + 1) {
+        // ================================================ prefix warp
+        // prefix(s, c) = carry(s) (+) A(s,0..c-1), carry(s) = carry(s-1) (+) A(s-1,0..G-1);
+        // slot s&1 of s_pre; one extra round (s = nslices) gives CTA G-1 the carry of the tail
+        VT carry;
+        carry.v = seed ? seed->v : identity.v;
+        carry.ok = true;
+        const skel_u64 rounds = nslices + (c == G - 1 ? 1 : 0);
+        for (skel_u64 s = 0; s < rounds; ++s) {
+            const int slot = (int)(s & 1);
+            if (s >= 2) skel::mbar_wait(&pre_empty[slot], (unsigned)(((s >> 1) - 1) & 1));
+            if (s > 0) carry = comb(carry, warp_fold_aggs(status, flags, aggv, (s - 1) * G, (int)G, epoch, lane, tup), tup);
+            VT p = carry;
+            if (s < nslices) p = comb(carry, warp_fold_aggs(status, flags, aggv, s * G, (int)c, epoch, lane, tup), tup);
+            if (lane == 0) {
+                s_pre[slot] = p;
+                mbar_arrive(&pre_full[slot]);
+            }
+            __syncwarp();
         }
         return;
     }
@@ -646,22 +731,15 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, 1)
     run1.ok = false;
     VT run;          // P2 running prefix (identical in every consumer thread)
     run.ok = false;
-    VT carry;        // carry(s) (warp 0)
-    carry.v = seed ? seed->v : identity.v;
-    carry.ok = true;
     int ph, j;
     skel_u64 s;
     for (skel_u64 q = 0; scan_item(q, nslices, ph, s, j); ++q) {
         const int nj = jn(s);
-        if (ph == 2 && j == 0) {
-            // prefix(s, c) = carry(s) (+) A(s,0..c-1), carry(s) = carry(s-1) (+) A(s-1, 0..G-1)
-            if (w == 0) {
-                if (s > 0) carry = comb(carry, warp_fold_aggs(status, flags, aggv, (s - 1) * G, (int)G, epoch, lane, tup), tup);
-                const VT mine = warp_fold_aggs(status, flags, aggv, s * G, (int)c, epoch, lane, tup);
-                if (lane == 0) s_run = comb(carry, mine, tup);
-            }
-            cons_sync();
-            run = s_run;
+        if (ph == 2 && j == 0) {  // the slice prefix, computed ahead by the prefix warp
+            const int slot = (int)(s & 1);
+            skel::mbar_wait(&pre_full[slot], (unsigned)((s >> 1) & 1));
+            run = s_pre[slot];
+            mbar_arrive(&pre_empty[slot]);
         }
         if (j >= nj) {
             if (ph == 1 && j == 0 && nj == 0 && t == 0) {  // empty sub-chunk: publish once
@@ -671,14 +749,14 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, 1)
             }
             continue;
         }
-        const int st = (int)(v % STAGES);
+        const int st = (int)(v % SSTAGES);
         const skel_u64 tile = tile_of(s, j);
         skel_T x[K];
         if (tma) {
-            skel::mbar_wait(&full_bar[st], (unsigned)((v / STAGES) & 1));
-            read_row(stages + st * TILE_BYTES, t, x);
+            skel::mbar_wait(&full_bar[st], (unsigned)((v / SSTAGES) & 1));
+            read_row(stages + st * STILE_BYTES, t, x);
         } else {
-            const skel_T *p = in + tile * TILE + (skel_u64)t * K;
+            const skel_T *p = in + tile * STILE + (skel_u64)t * K;
 #pragma unroll
             for (int k = 0; k < K; ++k) x[k] = p[k];
         }
@@ -712,11 +790,11 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, 1)
             for (int k = K - 1; k >= 1; --k) x[k] = opf(pre.v, x[k - 1], tup);
             x[0] = pre.v;
             if (tma) {
-                write_row(stages + st * TILE_BYTES, t, x);
+                write_row(stages + st * STILE_BYTES, t, x);
                 skel::fence_proxy_async();
                 mbar_arrive(&done_bar[st]);  // outputs staged: the producer stores them
             } else {
-                skel_T *o = out + tile * TILE + (skel_u64)t * K;
+                skel_T *o = out + tile * STILE + (skel_u64)t * K;
 #pragma unroll
                 for (int k = 0; k < K; ++k) o[k] = x[k];
             }
@@ -725,19 +803,15 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, 1)
     }
     // ---- ragged last tile and the device total: CTA G-1
     if (c == G - 1) {
-        if (w == 0) {
-            if (nslices > 0)
-                carry = comb(carry, warp_fold_aggs(status, flags, aggv, (nslices - 1) * G, (int)G, epoch, lane, tup), tup);
-            if (lane == 0) s_run = carry;
-        }
-        cons_sync();
-        const VT carry_end = s_run;
-        const skel_u64 base = nft * TILE;
+        const int slot = (int)(nslices & 1);
+        skel::mbar_wait(&pre_full[slot], (unsigned)((nslices >> 1) & 1));
+        const VT carry_end = s_pre[slot];
+        const skel_u64 base = nft * STILE;
         VT mine;
         mine.ok = false;
         skel_u64 first = 0, kt = 0;
         if (base < n) {
-            const skel_u64 cnt = n - base, per = (cnt + RB - 1) / RB;
+            const skel_u64 cnt = n - base, per = (cnt + SRB - 1) / SRB;
             first = base + (skel_u64)t * per;
             kt = first >= n ? 0 : ((n - first) < per ? (n - first) : per);
             for (skel_u64 k = 0; k < kt; ++k) {
