@@ -64,6 +64,7 @@ def core() -> ctypes.CDLL:
         lib.oracle_abssum_f32.argtypes = [P, ctypes.c_size_t]
         lib.oracle_abssum_f32.restype = ctypes.c_double
         lib.oracle_exscan_f32_exact.argtypes = [P, P, P, ctypes.c_size_t]
+        lib.oracle_exscan_f32_sampled.argtypes = [P, ctypes.c_size_t, P, ctypes.c_size_t, P, P]
         _core = lib
     return _core
 
@@ -263,6 +264,16 @@ def exscan_f32_exact(x: np.ndarray):
     if x.size:
         core().oracle_exscan_f32_exact(_ptr(x), _ptr(out), _ptr(ab), x.size)
     return out, ab
+
+
+def exscan_f32_sampled(x: np.ndarray, idx: np.ndarray):
+    """Exact (float64) exclusive prefix sums of x at the sorted positions idx."""
+    x = np.ascontiguousarray(x, dtype=np.float32)
+    idx = np.ascontiguousarray(np.sort(idx), dtype=np.int64)
+    pre = np.empty(idx.size, np.float64)
+    ab = np.empty(idx.size, np.float64)
+    core().oracle_exscan_f32_sampled(_ptr(x), x.size, _ptr(idx), idx.size, _ptr(pre), _ptr(ab))
+    return idx, pre, ab
 
 
 # ---------------------------------------------------------------------------

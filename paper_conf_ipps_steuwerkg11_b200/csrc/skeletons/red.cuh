@@ -534,7 +534,7 @@ __device__ __forceinline__ VT warp_fold_aggs(const skel_u64 *st64, const unsigne
 // P1(s+LAG) x CH (if that slice exists), P2(s) x CH.  Returns false past the
 // end.  LAG slices of slack absorb the CTAs' speed differences.
 #ifndef SKEL_SCAN_LAG
-#define SKEL_SCAN_LAG 2
+#define SKEL_SCAN_LAG 1
 #endif
 constexpr int SCAN_LAG = SKEL_SCAN_LAG;
 __device__ __forceinline__ bool scan_item(skel_u64 q, skel_u64 nslices, int &phase, skel_u64 &s, int &j) {
