@@ -337,6 +337,7 @@ def main():
 
     extras = {}
     if not args.no_extras:
+        extras["sweep"] = bench_sweep(ctx, skel, stream, world, rank, barrier, max_over_ranks, args)
         extras["mandelbrot"] = bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, args)
         extras["lmosem"] = bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args)
 
@@ -355,6 +356,60 @@ def main():
     ctx.close()
     if world > 1:
         dist.destroy_process_group()
+
+
+def bench_sweep(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
+    """configs[1] sweep: GB/s per skeleton, n = 2^20 .. 2^30 per GPU, float32 and int32.
+    Vectors are filled on the device (values do not change the memory traffic).
+    Sizes below 4x L2 are timed with a 512 MB L2 flush between repetitions."""
+    import torch
+    from paper_conf_ipps_steuwerkg11_b200.workloads import (MAP_F32, MAP_I32, SAXPY_F32, SAXPY_I32, SUM_F32,
+                                                             SUM_I32)
+    funcs = {np.float32: (MAP_F32, SAXPY_F32, SUM_F32), np.int32: (MAP_I32, SAXPY_I32, SUM_I32)}
+    peak, _ = measured_peaks()
+    flush = torch.empty(512 << 20, dtype=torch.uint8, device="cuda")
+    out = []
+    for dt, (fm, fz, fs) in funcs.items():
+        for k in range(20, 31, 2):
+            nloc = 1 << k
+            N = nloc * world
+            vs = [ctx.vector(n=N, dtype=dt) for _ in range(4)]
+            x, y, o, r = vs[0], vs[1], vs[2], ctx.vector(n=1, dtype=dt)
+            for v, val in ((x, 1), (y, 2)):
+                if world > 1:
+                    v.fill_dist(skel.BLOCK, dt(val))
+                else:
+                    v.fill(dt(val))
+            a = dt(3)
+            ops = {"map": lambda: ctx.map(fm, x, o), "zip": lambda: ctx.zip(fz, x, y, o, args=[a]),
+                   "reduce": lambda: ctx.reduce_to(fs, x, r), "scan": lambda: ctx.scan(fs, x, o, dt(0))}
+            small = nloc * 4 < 4 * 126e6
+            reps = 10 if k < 30 else 5
+            row = {"dtype": np.dtype(dt).name, "log2n": k, "l2": "flushed" if small else "exceeds L2"}
+            for name, fn in ops.items():
+                for _ in range(2):
+                    fn()
+                ctx.sync()
+                tot = 0.0
+                for _ in range(reps):
+                    if small:
+                        flush.zero_()
+                        torch.cuda.synchronize()
+                    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                    e0.record(stream)
+                    fn()
+                    e1.record(stream)
+                    ctx.sync()
+                    tot += e0.elapsed_time(e1)
+                ms = max_over_ranks(tot / reps)
+                gbs = BYTES_PER_ELEM[name] * N / (ms * 1e-3) / 1e9
+                row[name] = {"ms": round(ms, 5), "GBps": round(gbs, 1), "frac": round(gbs / world / peak, 4)}
+            out.append(row)
+            for v in vs:
+                v.destroy()
+            r.destroy()
+    del flush
+    return out
 
 
 def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):

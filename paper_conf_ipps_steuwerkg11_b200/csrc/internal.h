@@ -10,6 +10,7 @@
 #include <memory>
 #include <set>
 #include <string>
+#include <unordered_map>
 #include <vector>
 
 #include "skel.h"
@@ -94,6 +95,7 @@ struct skel_ctx_s {
     skel_stats stats{};
     std::string last_error;
     std::map<std::string, std::unique_ptr<skelrt::Module>> modules;
+    std::unordered_map<std::string, skelrt::Module *> fast_modules;  // (kind, options, user text) -> module
     std::set<skel_vec_s *> vecs;
     unsigned scan_epoch = 0;
 };

@@ -137,6 +137,8 @@ std::string entry_name(const std::string &src, std::string *err) {
     return last;
 }
 
+int get_module_slow(skel_ctx_s *ctx, Kind kind, const char *src, Module **out);
+
 static const char *kind_name(Kind k) {
     switch (k) {
         case Kind::Map: return "map";
@@ -238,6 +240,30 @@ int compile_only(Kind kind, const char *src, int block, bool fmad, std::string *
 }
 
 int get_module(skel_ctx_s *ctx, Kind kind, const char *src, Module **out) {
+    // fast path: the same user text with the same options was loaded before
+    // (skips assembling and hashing the ~50 KB translation unit on every call)
+    const char *extra = getenv("SKEL_NVRTC_DEFINES");
+    std::string fast;
+    fast.reserve(64 + strlen(src));
+    fast += kind_name(kind);
+    fast += '|';
+    fast += std::to_string(ctx->block_size);
+    fast += ctx->fmad ? "|f1|" : "|f0|";
+    fast += extra ? extra : "";
+    fast += '|';
+    fast += src;
+    auto fit = ctx->fast_modules.find(fast);
+    if (fit != ctx->fast_modules.end()) {
+        ctx->stats.compile_mem_hits++;
+        *out = fit->second;
+        return SKEL_OK;
+    }
+    int st = get_module_slow(ctx, kind, src, out);
+    if (st == SKEL_OK) ctx->fast_modules[fast] = *out;
+    return st;
+}
+
+int get_module_slow(skel_ctx_s *ctx, Kind kind, const char *src, Module **out) {
     std::string err;
     const std::string user(src);
     const int block = ctx->block_size > 0 ? ctx->block_size : 256;

@@ -1085,6 +1085,7 @@ int skel_clear_kernel_cache(skel_ctx_t ctx) {
     for (auto &kv : ctx->modules)
         if (kv.second->lib) cudaLibraryUnload(kv.second->lib);
     ctx->modules.clear();
+    ctx->fast_modules.clear();
     return SKEL_OK;
 }
 
