@@ -1,0 +1,73 @@
+"""The LM OSEM customizing function (workloads/lmosem_error.cu) is plain C++
+apart from atomicAdd/__ldg; compiled for the host with three one-line shims
+it can be checked against the oracle on the CPU (tiny grids with exact
+plane/edge/corner ties, and the paper-sized volume).  This tests the walk's
+logic only; the GPU parity tests run the same text through NVRTC."""
+import ctypes
+import subprocess
+from pathlib import Path
+
+import numpy as np
+import pytest
+
+import oracle
+import skel_inputs as si
+
+ROOT = Path(__file__).resolve().parents[1]
+SHIM = r'''
+#include <cmath>
+#include <algorithm>
+using std::min; using std::max; using std::fmin; using std::fmax;
+static float atomicAdd(float* p, float v) { float o = *p; *p += v; return o; }
+template <class T> static T __ldg(const T* p) { return *p; }
+#include "SRC"
+extern "C" void run(const float* ev, int n, const float* f, float* c, int nx, int ny, int nz) {
+    for (int i = 0; i < n; ++i) {
+        Event e{ev[6*i], ev[6*i+1], ev[6*i+2], ev[6*i+3], ev[6*i+4], ev[6*i+5]};
+        lmosem_error(e, f, c, nx, ny, nz);
+    }
+}
+'''
+
+
+@pytest.fixture(scope="module")
+def walk(tmp_path_factory):
+    d = tmp_path_factory.mktemp("walk")
+    src = d / "shim.cpp"
+    src.write_text(SHIM.replace("SRC", str(ROOT / "paper_conf_ipps_steuwerkg11_b200" / "workloads" / "lmosem_error.cu")))
+    so = d / "walk.so"
+    subprocess.run(["g++", "-O2", "-std=c++17", "-ffp-contract=off", "-shared", "-fPIC", str(src), "-o", str(so)],
+                   check=True)
+    lib = ctypes.CDLL(str(so))
+    P, I = ctypes.c_void_p, ctypes.c_int
+    lib.run.argtypes = [P, I, P, P, I, I, I]
+
+    def run(ev, f, dims):
+        c = np.zeros(int(np.prod(dims)), np.float32)
+        f32 = np.ascontiguousarray(f, np.float32)
+        lib.run(ev.ctypes.data, ev.size, f32.ctypes.data, c.ctypes.data, *dims)
+        return c
+    return run
+
+
+@pytest.mark.parametrize("quarter", [False, True])
+def test_tiny_grid_with_ties(walk, quarter):
+    g = np.random.default_rng(5 + quarter)
+    dims = (4, 3, 5)
+    e = np.zeros(500, si.EVENT_DTYPE)
+    for k in ("x1", "y1", "z1", "x2", "y2", "z2"):
+        e[k] = g.integers(-8, 28, 500) / 4.0 if quarter else g.uniform(-2, 7, 500)
+    f = g.uniform(0.5, 2, int(np.prod(dims))).astype(np.float32)
+    c = walk(e, f, dims)
+    want, _ = oracle.lmosem_error_image(e, f.astype(np.float64), dims)
+    assert np.array_equal(c > 0, want > 0)  # same voxels touched
+    assert np.linalg.norm(c - want) <= 1e-6 * np.linalg.norm(want)
+
+
+def test_paper_volume_no_flips(walk):
+    ev = si.lmosem_events(5000, subset=4)
+    dims = (150, 150, 280)
+    c = walk(ev, np.ones(int(np.prod(dims))), dims)
+    want, _ = oracle.lmosem_error_image(ev, np.ones(int(np.prod(dims))), dims)
+    assert np.array_equal(c > 0, want > 0)
+    assert np.linalg.norm(c - want) <= 1e-6 * np.linalg.norm(want)
