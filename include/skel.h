@@ -204,6 +204,19 @@ int skel_reduce_to(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t re
 int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out,
               const void *identity, const skel_arg *args, int nargs);
 
+/* ---- CUDA graphs ------------------------------------------------------------
+ * capture_begin/end record every skeleton, distribution change and fill issued
+ * in between (on all local devices, NCCL collectives included) into a graph;
+ * graph_launch replays that device work.  Host-side bookkeeping (lazy
+ * transfers, allocations, compilation) happens once, at capture time, so run
+ * the sequence eagerly once before capturing it; calls that would block,
+ * reallocate or compile inside a capture fail with SKEL_ERR_STATE. */
+typedef struct skel_graph_s *skel_graph_t;
+int skel_capture_begin(skel_ctx_t ctx);
+int skel_capture_end(skel_ctx_t ctx, skel_graph_t *out);
+int skel_graph_launch(skel_graph_t graph);
+int skel_graph_destroy(skel_graph_t graph);
+
 /* Compile (or fetch from the caches) the kernels of a skeleton without
  * running them; kind = "map" | "zip" | "reduce" | "scan".  Used to move the
  * one-time NVRTC cost out of timed regions. */

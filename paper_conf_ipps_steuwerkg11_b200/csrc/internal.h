@@ -59,7 +59,7 @@ struct Slot {
     // grow-only workspace for reduce/scan partials, look-back status, seeds
     char *ws = nullptr;
     size_t ws_cap = 0;
-    unsigned *counters = nullptr;  // [0] scan ticket, [1] scan done, [2] reduce done, [3] pad
+    unsigned *counters = nullptr;  // [1] scan done, [2] reduce done, [3] scan epoch (device-resident)
     // look-back status words (only ever hold status words; zeroed at allocation)
     unsigned long long *st64 = nullptr;
     size_t st64_cap = 0;  // entries
@@ -97,7 +97,16 @@ struct skel_ctx_s {
     std::map<std::string, std::unique_ptr<skelrt::Module>> modules;
     std::unordered_map<std::string, skelrt::Module *> fast_modules;  // (kind, options, user text) -> module
     std::set<skel_vec_s *> vecs;
-    unsigned scan_epoch = 0;
+    bool capturing = false;  // between skel_capture_begin and skel_capture_end
+    std::vector<std::pair<skel_vec_s *, uint64_t>> captured;  // vectors written inside the capture
+    uint64_t next_serial = 0;
+};
+
+struct skel_graph_s {
+    skel_ctx_s *ctx = nullptr;
+    cudaGraph_t graph = nullptr;
+    cudaGraphExec_t exec = nullptr;
+    std::vector<std::pair<skel_vec_s *, uint64_t>> written;  // (vector, serial) the graph writes
 };
 
 struct skel_vec_s {
@@ -112,6 +121,7 @@ struct skel_vec_s {
     bool dev_valid = true;  // created zero-filled on the devices
     bool diverged = false;  // copy distribution after mark_device_modified
     std::vector<skelrt::Buf> bufs;  // indexed like ctx->slots
+    uint64_t serial = 0;            // unique per context (graphs refer to vectors by it)
 };
 
 namespace skelrt {

@@ -258,6 +258,10 @@ int get_module(skel_ctx_s *ctx, Kind kind, const char *src, Module **out) {
         *out = fit->second;
         return SKEL_OK;
     }
+    if (ctx->capturing) {
+        ctx->last_error = "user function not compiled yet: call skel_prepare (or run once) before capturing";
+        return SKEL_ERR_STATE;
+    }
     int st = get_module_slow(ctx, kind, src, out);
     if (st == SKEL_OK) ctx->fast_modules[fast] = *out;
     return st;

@@ -102,6 +102,9 @@ int dev_alloc(skel_ctx_s *ctx, Slot &s, size_t bytes, char **out) {
 }
 int dev_free(skel_ctx_s *ctx, Slot &s, char *p) {
     if (!p) return SKEL_OK;
+    if (ctx->capturing)
+        return fail(ctx, SKEL_ERR_STATE, "a buffer would be reallocated inside a capture: run the sequence once "
+                                         "eagerly before capturing it");
     DevGuard g(s.dev);
     CK(ctx, cudaStreamSynchronize(s.stream));
     CK(ctx, cudaFree(p));
@@ -180,6 +183,13 @@ int join(skel_ctx_s *ctx) {
 
 bool partial_mirror(const skel_vec_s *v) { return v->host && v->host_n != v->n; }
 
+// the devices now hold newer data than the host; inside a capture the vector
+// is also remembered, so that replaying the graph invalidates its host copy
+void device_wrote(skel_vec_s *v) {
+    v->host_valid = false;
+    if (v->ctx->capturing) v->ctx->captured.emplace_back(v, v->serial);
+}
+
 int host_mirror(skel_vec_s *v) {
     if (v->host && !partial_mirror(v)) return SKEL_OK;
     if (v->host) {  // a rank-local part mirror is replaced by a full one
@@ -223,6 +233,7 @@ int ensure_device(skel_vec_s *v) {
 }
 
 int sync_all(skel_ctx_s *ctx) {
+    if (ctx->capturing) return fail(ctx, SKEL_ERR_STATE, "blocking call inside a capture (skel_capture_begin)");
     for (auto &s : ctx->slots) {
         DevGuard g(s.dev);
         CK(ctx, cudaStreamSynchronize(s.stream));
@@ -565,7 +576,7 @@ int set_distribution(skel_vec_s *v, skel_dist dist, skel_combine combine) {
     }
     v->dist = dist;
     v->dev_valid = true;
-    if (combine != SKEL_COMBINE_NONE || diverged) v->host_valid = false;
+    if (combine != SKEL_COMBINE_NONE || diverged) device_wrote(v);
     v->diverged = false;
     return SKEL_OK;
 }
@@ -620,7 +631,7 @@ int prepare_output(skel_vec_s *out, size_t n, skel_dist dist, bool same_as_input
         TRY(place(out, dist));
     }
     out->dev_valid = true;
-    out->host_valid = false;
+    device_wrote(out);
     out->diverged = false;
     return SKEL_OK;
 }
@@ -675,7 +686,7 @@ int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_
     }
     if (rsz != 0) {
         out->dev_valid = true;
-        out->host_valid = false;
+        device_wrote(out);
     }
     return SKEL_OK;
 }
@@ -931,6 +942,8 @@ static int init_slot(skel_ctx_s *ctx, int d, int dev) {
     CK(ctx, cudaMalloc(&p, 256));
     CK(ctx, cudaMemset(p, 0, 256));
     s.counters = static_cast<unsigned *>(p);
+    const unsigned first_epoch = 1;  // status words are zeroed: epoch 0 must never be live
+    CK(ctx, cudaMemcpy(s.counters + 3, &first_epoch, sizeof first_epoch, cudaMemcpyHostToDevice));
     ctx->slots.push_back(s);
     return SKEL_OK;
 }
@@ -1111,6 +1124,7 @@ int skel_vector_create(skel_ctx_t ctx, size_t n, size_t es, skel_vec_t *out) {
     if (!ctx || !out || es == 0) return fail(ctx, SKEL_ERR_ARG, "bad vector arguments");
     auto *v = new skel_vec_s();
     v->ctx = ctx;
+    v->serial = ++ctx->next_serial;
     v->n = n;
     v->es = es;
     v->dist = ctx->D == 1 ? SKEL_SINGLE : SKEL_BLOCK;
@@ -1263,7 +1277,7 @@ int skel_vector_fill_dist(skel_vec_t v, skel_dist dist, const void *value) {
         ctx->stats.kernel_launches++;
     }
     v->dev_valid = true;
-    v->host_valid = false;
+    device_wrote(v);
     v->diverged = false;
     return SKEL_OK;
 }
@@ -1284,7 +1298,7 @@ int skel_vector_get_distribution(skel_vec_t v, skel_dist *dist) {
 int skel_vector_mark_device_modified(skel_vec_t v) {
     if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
     TRY(ensure_device(v));
-    v->host_valid = false;
+    device_wrote(v);
     if (v->dist == SKEL_COPY && v->ctx->D > 1) v->diverged = true;
     return SKEL_OK;
 }
@@ -1357,7 +1371,7 @@ int skel_reduce_to(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t re
                                 cudaMemcpyDeviceToDevice, s.stream));
     }
     result->dev_valid = true;
-    result->host_valid = false;
+    device_wrote(result);
     result->diverged = false;
     return SKEL_OK;
 }
@@ -1432,15 +1446,7 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         std::vector<RedLayout> Lr;
         TRY(reduce_core(ctx, m, in, args, nargs, Lr));
     }
-    if (++ctx->scan_epoch >= (1u << 30) - 1) {
-        ctx->scan_epoch = 1;
-        for (auto &s : ctx->slots) {
-            DevGuard g(s.dev);
-            if (s.st64) CK(ctx, cudaMemsetAsync(s.st64, 0, s.st64_cap * 8, s.stream));
-            if (s.fl32) CK(ctx, cudaMemsetAsync(s.fl32, 0, s.fl32_cap * 4, s.stream));
-        }
-    }
-    unsigned epoch = ctx->scan_epoch;
+
     std::vector<unsigned char> idbuf(align_up(m->sig[4], 16), 0);
     memcpy(idbuf.data(), identity, in->es);
     for (size_t li = 0; li < ctx->slots.size(); ++li) {
@@ -1471,15 +1477,16 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
                       make_tmap(&tout, pout, rows, (uint32_t)(SRB / 2));
         void *status = s.st64, *flags = s.fl32, *aggv = s.ws + L.o_aggv, *incv = s.ws + L.o_incv;
         unsigned *counters = s.counters;
+        unsigned *epoch_ptr = s.counters + 3;  // device-resident scan epoch (graph-replay safe)
         void *total = nullptr;
         void *params[] = {&tin, &tout, &pin, &pout, &cnt, &use_tma, idbuf.data(), &seed, &status, &flags,
-                          &aggv, &incv, &counters, &epoch, &total, abuf.data()};
+                          &aggv, &incv, &counters, &epoch_ptr, &total, abuf.data()};
         CK(ctx, cudaLaunchKernel((const void *)m->k_scan, dim3((unsigned)G), dim3((unsigned)m->sig[14]), params,
                                  use_tma ? m->sig[12] : 0, s.stream));
         ctx->stats.kernel_launches++;
     }
     out->dev_valid = true;
-    out->host_valid = false;
+    device_wrote(out);
     return SKEL_OK;
 }
 
@@ -1492,6 +1499,89 @@ int skel_prepare(skel_ctx_t ctx, const char *kind, const char *src) {
     else return fail(ctx, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan");
     Module *m = nullptr;
     return get_module(ctx, k, src, &m);
+}
+
+// ---- CUDA graphs: capture a skeleton sequence once, replay it ------------------------
+int skel_capture_begin(skel_ctx_t ctx) {
+    if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
+    if (ctx->capturing) return fail(ctx, SKEL_ERR_STATE, "already capturing");
+    TRY(sync_all(ctx));
+    Slot &s0 = ctx->slots[0];
+    {
+        DevGuard g(s0.dev);
+        CK(ctx, cudaStreamBeginCapture(s0.stream, cudaStreamCaptureModeRelaxed));
+        CK(ctx, cudaEventRecord(s0.ev, s0.stream));
+    }
+    for (size_t li = 1; li < ctx->slots.size(); ++li) {  // fork: the other streams join the capture
+        DevGuard g(ctx->slots[li].dev);
+        CK(ctx, cudaStreamWaitEvent(ctx->slots[li].stream, s0.ev, 0));
+    }
+    ctx->captured.clear();
+    ctx->capturing = true;
+    return SKEL_OK;
+}
+
+int skel_capture_end(skel_ctx_t ctx, skel_graph_t *out) {
+    if (!ctx || !out) return fail(ctx, SKEL_ERR_ARG, "bad arguments");
+    if (!ctx->capturing) return fail(ctx, SKEL_ERR_STATE, "not capturing");
+    ctx->capturing = false;
+    Slot &s0 = ctx->slots[0];
+    for (size_t li = 1; li < ctx->slots.size(); ++li) {  // join back into the origin stream
+        Slot &s = ctx->slots[li];
+        DevGuard g(s.dev);
+        CK(ctx, cudaEventRecord(s.ev, s.stream));
+        DevGuard g0(s0.dev);
+        CK(ctx, cudaStreamWaitEvent(s0.stream, s.ev, 0));
+    }
+    DevGuard g(s0.dev);
+    auto *gr = new skel_graph_s();
+    gr->ctx = ctx;
+    cudaError_t e = cudaStreamEndCapture(s0.stream, &gr->graph);
+    if (e == cudaSuccess) e = cudaGraphInstantiate(&gr->exec, gr->graph, 0);
+    if (e != cudaSuccess) {
+        if (gr->graph) cudaGraphDestroy(gr->graph);
+        delete gr;
+        return fail(ctx, SKEL_ERR_CUDA, std::string("capture: ") + cudaGetErrorString(e));
+    }
+    gr->written.swap(ctx->captured);
+    *out = gr;
+    return SKEL_OK;
+}
+
+int skel_graph_launch(skel_graph_t g) {
+    if (!g) return fail(nullptr, SKEL_ERR_ARG, "graph is NULL");
+    skel_ctx_s *ctx = g->ctx;
+    Slot &s0 = ctx->slots[0];
+    for (size_t li = 1; li < ctx->slots.size(); ++li) {  // earlier work on the other streams first
+        Slot &s = ctx->slots[li];
+        DevGuard gd(s.dev);
+        CK(ctx, cudaEventRecord(s.ev, s.stream));
+        DevGuard g0(s0.dev);
+        CK(ctx, cudaStreamWaitEvent(s0.stream, s.ev, 0));
+    }
+    {
+        DevGuard gd(s0.dev);
+        CK(ctx, cudaGraphLaunch(g->exec, s0.stream));
+        CK(ctx, cudaEventRecord(s0.ev, s0.stream));
+    }
+    for (size_t li = 1; li < ctx->slots.size(); ++li) {  // later work on the other streams after it
+        DevGuard gd(ctx->slots[li].dev);
+        CK(ctx, cudaStreamWaitEvent(ctx->slots[li].stream, s0.ev, 0));
+    }
+    for (auto &w : g->written)  // the replay rewrote these vectors on the devices
+        if (ctx->vecs.count(w.first) && w.first->serial == w.second) {
+            w.first->host_valid = false;
+            w.first->dev_valid = true;
+        }
+    return SKEL_OK;
+}
+
+int skel_graph_destroy(skel_graph_t g) {
+    if (!g) return fail(nullptr, SKEL_ERR_ARG, "graph is NULL");
+    if (g->exec) cudaGraphExecDestroy(g->exec);
+    if (g->graph) cudaGraphDestroy(g->graph);
+    delete g;
+    return SKEL_OK;
 }
 
 // ---- pure host logic -------------------------------------------------------------

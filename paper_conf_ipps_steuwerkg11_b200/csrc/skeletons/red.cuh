@@ -625,10 +625,13 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
     skel_scan_kernel(const __grid_constant__ skel_tmap tin, const __grid_constant__ skel_tmap tout,
                      const skel_T *in, skel_T *out, skel_u64 n, int use_tma, const skel_S identity, const skel_S *seed,
                      skel_u64 *status, unsigned *flags, skel_S *aggv, skel_S *incv, unsigned *counters,
-                     unsigned epoch, skel_S *total, const skel_Buf args) {
+                     unsigned *epoch_ptr, skel_S *total, const skel_Buf args) {
     (void)incv;
-    (void)counters;
+    // the launch's epoch lives in device memory (graph replays must see a new
+    // one): every CTA reads it before publishing anything; the last CTA to
+    // finish advances it (all CTAs have read it by then)
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    __shared__ unsigned s_epoch;
     __shared__ skel_u64 full_bar[SSTAGES], done_bar[SSTAGES], pre_full[2], pre_empty[2];
     __shared__ VT wsc[SNW];
     __shared__ VT s_tot, s_pre[2];
@@ -656,8 +659,10 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
             skel::mbar_init(&pre_empty[k], SRB);
         }
         skel::fence_mbar_init();
+        s_epoch = *(volatile unsigned *)epoch_ptr;
     }
     __syncthreads();
+    const unsigned epoch = s_epoch;
 
     if (w == SNW) {
         // ================================================ TMA producer warp
@@ -830,5 +835,15 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
             r = opf(r, e, tup);
         }
         if (t == 0 && total) total->v = comb(carry_end, s_tot, tup).v;
+    }
+    cons_sync();
+    if (t == 0) {
+        __threadfence();
+        const unsigned prev = atomicAdd(&counters[1], 1u);
+        if (prev == gridDim.x - 1) {
+            counters[1] = 0;
+            *epoch_ptr = epoch >= (1u << 30) - 1 ? 1u : epoch + 1;
+            __threadfence();
+        }
     }
 }

@@ -90,6 +90,8 @@ def lib() -> ctypes.CDLL:
             "skel_compile_check": [ctypes.c_char_p, ctypes.c_char_p, I, ctypes.c_char_p, S, ctypes.POINTER(S)],
             "skel_plan_part": [S, I, I, ctypes.POINTER(S), ctypes.POINTER(S)],
             "skel_plan_exchange": [I, I, I, ctypes.POINTER(I)],
+            "skel_capture_begin": [P], "skel_capture_end": [P, PP], "skel_graph_launch": [P],
+            "skel_graph_destroy": [P],
         }
         for name, argt in sig.items():
             f = getattr(L, name)
@@ -215,6 +217,28 @@ class Context:
     def prepare(self, kind: str, src: str):
         _check(lib().skel_prepare(self._h, kind.encode(), src.encode()), self._h)
 
+    # -- CUDA graphs
+    def capture_begin(self):
+        _check(lib().skel_capture_begin(self._h), self._h)
+
+    def capture_end(self) -> "Graph":
+        g = ctypes.c_void_p()
+        _check(lib().skel_capture_end(self._h, ctypes.byref(g)), self._h)
+        return Graph(self, g)
+
+    def capture(self, fn) -> "Graph":
+        """Record the device work of fn() into a replayable graph."""
+        self.capture_begin()
+        try:
+            fn()
+        except BaseException:
+            try:
+                self.capture_end().destroy()
+            except SkelError:
+                pass
+            raise
+        return self.capture_end()
+
     # -- vectors
     def vector(self, data=None, *, n: int | None = None, dtype=None) -> "Vector":
         if data is not None:
@@ -267,6 +291,27 @@ class Context:
         idv = np.ascontiguousarray(np.asarray(identity, dtype=vin.dtype).reshape(1))
         _check(lib().skel_scan(self._h, src.encode(), vin._h, vout._h, idv.ctypes.data, a, len(args)), self._h)
         return vout
+
+
+class Graph:
+    """A captured skeleton sequence (CUDA graph) that can be replayed."""
+
+    def __init__(self, ctx: Context, h):
+        self.ctx, self._h = ctx, h
+
+    def launch(self):
+        _check(lib().skel_graph_launch(self._h), self.ctx._h)
+
+    def destroy(self):
+        if self._h and self._h.value:
+            lib().skel_graph_destroy(self._h)
+        self._h = ctypes.c_void_p()
+
+    def __del__(self):
+        try:
+            self.destroy()
+        except Exception:
+            pass
 
 
 class Vector:
