@@ -338,6 +338,8 @@ def main():
     extras = {}
     if not args.no_extras:
         extras["sweep"] = bench_sweep(ctx, skel, stream, world, rank, barrier, max_over_ranks, args)
+        if world == 1:
+            extras["overhead"] = bench_overhead(ctx, skel, stream, args)
         extras["mandelbrot"] = bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, args)
         extras["lmosem"] = bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args)
 
@@ -414,6 +416,76 @@ def bench_sweep(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
             r.destroy()
     del flush
     return out
+
+
+def bench_overhead(ctx, skel, stream, args):
+    """NEXT-3: (a) the skeletons vs the same operations hand-written in CUDA C++
+    (nvcc, float4 loops) and CUB's DeviceScan, on the same device buffers and
+    stream -- the analog of the paper's SkelCL-vs-OpenCL overhead (P:L472-481);
+    (b) NVRTC build time vs loading the cubin from the disk cache."""
+    import ctypes
+    import tempfile
+    import torch
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MAP_F32, SAXPY_F32, SUM_F32
+    hw = ctypes.CDLL(os.path.join(ROOT, "paper_conf_ipps_steuwerkg11_b200", "libhandwritten.so"))
+    P, S = ctypes.c_void_p, ctypes.c_size_t
+    hw.hw_map_f32.argtypes = [P, P, S, P]
+    hw.hw_saxpy_f32.argtypes = [P, P, P, ctypes.c_float, S, P]
+    hw.hw_sum_f32.argtypes = [P, S, P, P]
+    hw.hw_exscan_f32.argtypes = [P, P, S, P]
+    n = 1 << args.log2n
+    x, y, o, r = (ctx.vector(n=n, dtype=np.float32) for _ in range(4))
+    x.fill(np.float32(0.5))
+    y.fill(np.float32(0.25))
+    px, py, po = x.device_ptr()[0], y.device_ptr()[0], o.device_ptr()[0]
+    tmp = torch.empty(1, dtype=torch.float32, device="cuda")
+    sp = ctx.stream(0)
+    a = np.float32(2.5)
+    pairs = {
+        "map": (lambda: ctx.map(MAP_F32, x, o), lambda: hw.hw_map_f32(px, po, n, sp)),
+        "zip": (lambda: ctx.zip(SAXPY_F32, x, y, o, args=[a]), lambda: hw.hw_saxpy_f32(px, py, po, 2.5, n, sp)),
+        "reduce": (lambda: ctx.reduce_to(SUM_F32, x, r), lambda: hw.hw_sum_f32(px, n, tmp.data_ptr(), sp)),
+        "scan": (lambda: ctx.scan(SUM_F32, x, o, np.float32(0)), lambda: hw.hw_exscan_f32(px, po, n, sp)),
+    }
+    res = {}
+    for name, (fs, fh) in pairs.items():
+        times = []
+        for fn in (fs, fh):
+            for _ in range(3):
+                fn()
+            ctx.sync()
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            e0.record(stream)
+            for _ in range(10):
+                fn()
+            e1.record(stream)
+            ctx.sync()
+            times.append(e0.elapsed_time(e1) / 10)
+        res[name] = {"skeleton_ms": round(times[0], 4), "handwritten_ms": round(times[1], 4),
+                     "skeleton_over_handwritten": round(times[0] / times[1], 4)}
+    res["handwritten"] = "nvcc float4 grid-stride kernels (map, saxpy), block-reduce + atomicAdd (sum, any order), " \
+                         "CUB DeviceScan::ExclusiveSum (scan)"
+    for v in (x, y, o, r):
+        v.destroy()
+    # disk cache: build from source vs load (fresh cache directory)
+    srcs = [("map", MAP_F32), ("zip", SAXPY_F32), ("reduce", SUM_F32)]
+    with tempfile.TemporaryDirectory() as d:
+        c1 = skel.Context(1)
+        c1.set_cache_dir(d)
+        for k, src in srcs:
+            c1.prepare(k, src)
+        st1 = c1.stats()
+        c1.close()
+        c2 = skel.Context(1)
+        c2.set_cache_dir(d)
+        for k, src in srcs:
+            c2.prepare(k, src)
+        st2 = c2.stats()
+        c2.close()
+    res["kernel_cache"] = {"nvrtc_build_ms": round(st1["compile_ms"], 1), "disk_load_ms": round(st2["disk_load_ms"], 2),
+                           "load_speedup": round(st1["compile_ms"] / max(st2["disk_load_ms"], 1e-6), 1),
+                           "kernels": [k for k, _ in srcs], "paper": "loading is at least 5x faster (P:L248-250)"}
+    return res
 
 
 def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):

@@ -637,8 +637,12 @@ int prepare_output(skel_vec_s *out, size_t n, skel_dist dist, bool same_as_input
 }
 
 int ew_grid(const Slot &s, size_t chunks, int block) {
+    static const int waves = [] {
+        const char *e = getenv("SKEL_EW_WAVES");  // tuning hook: grid = SMs x (2048/block) x waves
+        return e ? std::max(1, atoi(e)) : 32;
+    }();
     size_t g = (chunks + block - 1) / block;
-    const size_t cap = (size_t)s.sms * (2048 / block) * 2;
+    const size_t cap = (size_t)s.sms * (2048 / block) * waves;
     g = std::min(g, cap);
     return (int)std::max<size_t>(g, 1);
 }

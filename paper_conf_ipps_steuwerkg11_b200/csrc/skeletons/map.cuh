@@ -87,30 +87,36 @@ constexpr skel_sig_t skel_make_sig() {
 extern "C" __device__ skel_sig_t skel_sig = skel_make_sig();
 
 // ---- streaming loads / stores of one chunk ---------------------------------
+#ifndef SKEL_LD_HINT
+#define SKEL_LD_HINT ".nc.L1::no_allocate"
+#endif
 template <int N> __device__ __forceinline__ skel::chunk<N> skel_ld(const void *p) {
     skel::chunk<N> c;
     if constexpr (N == 16) {
-        asm volatile("ld.global.nc.L1::no_allocate.v4.u32 {%0,%1,%2,%3}, [%4];"
+        asm volatile("ld.global" SKEL_LD_HINT ".v4.u32 {%0,%1,%2,%3}, [%4];"
                      : "=r"(c.v.x), "=r"(c.v.y), "=r"(c.v.z), "=r"(c.v.w)
                      : "l"(p));
     } else if constexpr (N == 8) {
-        asm volatile("ld.global.nc.L1::no_allocate.v2.u32 {%0,%1}, [%2];" : "=r"(c.v.x), "=r"(c.v.y) : "l"(p));
+        asm volatile("ld.global" SKEL_LD_HINT ".v2.u32 {%0,%1}, [%2];" : "=r"(c.v.x), "=r"(c.v.y) : "l"(p));
     } else if constexpr (N == 4) {
-        asm volatile("ld.global.nc.L1::no_allocate.u32 %0, [%1];" : "=r"(c.v) : "l"(p));
+        asm volatile("ld.global" SKEL_LD_HINT ".u32 %0, [%1];" : "=r"(c.v) : "l"(p));
     } else {
         c = *reinterpret_cast<const skel::chunk<N> *>(p);
     }
     return c;
 }
+#ifndef SKEL_ST_HINT
+#define SKEL_ST_HINT ".cs"
+#endif
 template <int N> __device__ __forceinline__ void skel_st(void *p, const skel::chunk<N> &c) {
     if constexpr (N == 16) {
-        asm volatile("st.global.cs.v4.u32 [%0], {%1,%2,%3,%4};" ::"l"(p), "r"(c.v.x), "r"(c.v.y), "r"(c.v.z),
-                     "r"(c.v.w)
+        asm volatile("st.global" SKEL_ST_HINT ".v4.u32 [%0], {%1,%2,%3,%4};" ::"l"(p), "r"(c.v.x), "r"(c.v.y),
+                     "r"(c.v.z), "r"(c.v.w)
                      : "memory");
     } else if constexpr (N == 8) {
-        asm volatile("st.global.cs.v2.u32 [%0], {%1,%2};" ::"l"(p), "r"(c.v.x), "r"(c.v.y) : "memory");
+        asm volatile("st.global" SKEL_ST_HINT ".v2.u32 [%0], {%1,%2};" ::"l"(p), "r"(c.v.x), "r"(c.v.y) : "memory");
     } else if constexpr (N == 4) {
-        asm volatile("st.global.cs.u32 [%0], %1;" ::"l"(p), "r"(c.v) : "memory");
+        asm volatile("st.global" SKEL_ST_HINT ".u32 [%0], %1;" ::"l"(p), "r"(c.v) : "memory");
     } else {
         *reinterpret_cast<skel::chunk<N> *>(p) = c;
     }
