@@ -18,7 +18,7 @@ SHIM = r'''
 #include <cmath>
 #include <algorithm>
 using std::min; using std::max; using std::fmin; using std::fmax;
-static float atomicAdd(float* p, float v) { float o = *p; *p += v; return o; }
+#define __forceinline__ inline
 template <class T> static T __ldg(const T* p) { return *p; }
 #include "SRC"
 extern "C" void run(const float* ev, int n, const float* f, float* c, int nx, int ny, int nz) {
