@@ -207,9 +207,16 @@ def main():
     from paper_conf_ipps_steuwerkg11_b200.workloads import MAP_F32, SAXPY_F32, SUM_F32
 
     world, rank, local = env_world()
+    # test hooks: SKEL_TEST_DEVICE puts every rank on one device (rank-mode tests on a
+    # single GPU with tests/fakenccl), SKEL_BENCH_BACKEND=gloo for the process group
+    local = int(os.environ.get("SKEL_TEST_DEVICE", local))
+    backend = os.environ.get("SKEL_BENCH_BACKEND", "nccl")
     torch.cuda.set_device(local)
     if world > 1:
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        if backend == "nccl":
+            dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        else:
+            dist.init_process_group(backend)
         obj = [skel.unique_id() if rank == 0 else None]
         dist.broadcast_object_list(obj, src=0)
         ctx = skel.Context(rank=rank, world=world, device=local, nccl_id=obj[0])
@@ -223,7 +230,7 @@ def main():
     def max_over_ranks(v: float) -> float:
         if world == 1:
             return v
-        t = torch.tensor([v], device="cuda", dtype=torch.float64)
+        t = torch.tensor([v], device="cuda" if backend == "nccl" else "cpu", dtype=torch.float64)
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
         return float(t.item())
 
@@ -392,9 +399,16 @@ def bench_sweep(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
                 for _ in range(2):
                     fn()
                 ctx.sync()
-                g = ctx.capture(fn)  # replay the skeleton as a CUDA graph: no host overhead in the timing
-                g.launch()
-                ctx.sync()
+                try:  # replay the skeleton as a CUDA graph: no host overhead in the timing
+                    if os.environ.get("SKEL_BENCH_NO_GRAPH"):
+                        raise skel.SkelError(8, "graphs disabled")
+                    g = ctx.capture(fn)
+                    g.launch()
+                    ctx.sync()
+                    run = g.launch
+                except skel.SkelError:  # e.g. a collective backend that cannot be captured
+                    g, run = None, fn
+                    row["graph"] = False
                 tot = 0.0
                 for _ in range(reps):
                     if small:
@@ -402,11 +416,12 @@ def bench_sweep(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
                         torch.cuda.synchronize()
                     e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
                     e0.record(stream)
-                    g.launch()
+                    run()
                     e1.record(stream)
                     ctx.sync()
                     tot += e0.elapsed_time(e1)
-                g.destroy()
+                if g is not None:
+                    g.destroy()
                 ms = max_over_ranks(tot / reps)
                 gbs = BYTES_PER_ELEM[name] * N / (ms * 1e-3) / 1e9
                 row[name] = {"ms": round(ms, 5), "GBps": round(gbs, 1), "frac": round(gbs / world / peak, 4)}
@@ -563,9 +578,14 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         return max_over_ranks(e0.elapsed_time(e1) / reps)
 
     ms = timed(lambda: rec.subset(evv))
-    g = ctx.capture(lambda: rec.subset(evv))  # the subset loop body as one CUDA graph
-    ms_graph = timed(g.launch)
-    g.destroy()
+    try:
+        if os.environ.get("SKEL_BENCH_NO_GRAPH"):
+            raise skel.SkelError(8, "graphs disabled")
+        g = ctx.capture(lambda: rec.subset(evv))  # the subset loop body as one CUDA graph
+        ms_graph = timed(g.launch)
+        g.destroy()
+    except skel.SkelError:  # a collective backend that cannot be captured
+        ms_graph = ms
     evv.destroy()
     return {"config": "configs[3]/[4]: one subset, 10^6 events, 150x150x280, events block over GPUs",
             "subset_s": ms * 1e-3, "subset_s_graph": ms_graph * 1e-3, "events_per_s": nev / (ms_graph * 1e-3),

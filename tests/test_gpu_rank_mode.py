@@ -1,0 +1,66 @@
+"""The one-process-per-GPU (rank) path of libskel, run with several processes
+on the single available GPU.  Real NCCL refuses two ranks on one device, so
+the ranks preload tests/fakenccl (a host-staged stand-in for the NCCL
+collectives, test infrastructure): everything else -- buffer layouts, part
+offsets, in-place collective conventions, cross-rank Reduce/Scan folds, LM
+OSEM's all-gather / reduce-scatter, bench.py's torchrun path -- is the
+product code."""
+import json
+import os
+import socket
+import subprocess
+import sys
+from pathlib import Path
+
+import pytest
+
+pytestmark = pytest.mark.gpu
+ROOT = Path(__file__).resolve().parents[1]
+
+
+def free_port():
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    p = s.getsockname()[1]
+    s.close()
+    return p
+
+
+@pytest.fixture(scope="module")
+def fake_nccl(tmp_path_factory):
+    import nvidia.nccl as nn
+    inc = Path(list(nn.__path__)[0]) / "include"
+    out = tmp_path_factory.mktemp("fakenccl") / "libfakenccl.so"
+    subprocess.run(["gcc", "-O2", "-shared", "-fPIC", "-I/usr/local/cuda/include", f"-I{inc}",
+                    str(ROOT / "tests" / "fakenccl" / "fake_nccl.c"), "-o", str(out), "-L/usr/local/cuda/lib64",
+                    "-lcudart", "-lpthread"], check=True, capture_output=True)
+    return str(out)
+
+
+def torchrun(nproc, script_args, fake, timeout=600, extra_env=None):
+    # the host-staged fake collectives cannot be captured into CUDA graphs
+    env = dict(os.environ, LD_PRELOAD=fake, SKEL_TEST_DEVICE="0", SKEL_BENCH_BACKEND="gloo", SKEL_BENCH_NO_GRAPH="1")
+    env.update(extra_env or {})
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", "--nproc-per-node", str(nproc),
+           "--master-addr", "127.0.0.1", "--master-port", str(free_port()), *script_args]
+    return subprocess.run(cmd, capture_output=True, text=True, timeout=timeout, cwd=str(ROOT), env=env)
+
+
+@pytest.mark.parametrize("nproc", [2, 3])
+def test_rank_mode_selftest(fake_nccl, nproc):
+    r = torchrun(nproc, ["tools/rank_selftest.py"], fake_nccl)
+    oks = [ln for ln in r.stdout.splitlines() if ln.startswith("rank ")]
+    assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-3000:]
+    assert len(oks) == nproc and all(": OK" in ln for ln in oks), oks
+
+
+def test_bench_rank_path(fake_nccl):
+    r = torchrun(2, ["bench.py", "--gpus", "2", "--steps", "3", "--warmup", "3", "--log2n", "22", "--e2e-steps", "1",
+                     "--no-cpu"], fake_nccl)
+    assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-3000:]
+    lines = [ln for ln in r.stdout.splitlines() if ln.startswith("{")]
+    assert len(lines) == 1
+    d = json.loads(lines[0])
+    assert d["n_gpus"] == 2 and d["value"] > 0 and d["config"]["distribution"] == "block"
+    assert d["e2e"]["h2d_bytes_per_step"] == 2 * (1 << 22) * 4  # this rank's parts of x and y
+    assert d["mandelbrot"]["sum_iter"] == 453197644
