@@ -197,6 +197,19 @@ int skel_map(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out,
              const skel_arg *args, int nargs);
 int skel_zip(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_vec_t out,
              const skel_arg *args, int nargs);
+/* Fused form of Listing 4's tail:
+ *   b.set_distribution(BLOCK, combine); out = zip(src, a, b); out -> COPY
+ * as ONE kernel per device over peer memory: device k combines the D copies of
+ * b on its part (peer loads), keeps the combined part of b, applies the Zip
+ * function and stores the result into every device's copy of out (peer
+ * stores).  b must be SKEL_COPY with a numeric dtype; a is SKEL_COPY or
+ * SKEL_BLOCK (out may be a when a is SKEL_COPY).  Afterwards b is SKEL_BLOCK
+ * (combined) and out is SKEL_COPY.  One-process-per-GPU contexts reach the
+ * peers' buffers through CUDA IPC (opened once per allocation, collectively)
+ * and order the kernel between two one-word all-reduce barriers.  With D = 1,
+ * more than 16 devices, or inside a capture, the unfused sequence runs. */
+int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_combine combine,
+                     skel_vec_t out, const skel_arg *args, int nargs);
 int skel_reduce(skel_ctx_t ctx, const char *src, skel_vec_t in, void *result_host,
                 const skel_arg *args, int nargs);
 int skel_reduce_to(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t result,

@@ -105,9 +105,17 @@ _SIZES = ('extern "C" void oracle_sizes(size_t* out, int* np) '
           '{{ skel_oracle::sizes_of(&{f}, out, np); }}')
 
 
+def _strip_comments(src: str) -> str:
+    src = re.sub(r"/\*.*?\*/", " ", src, flags=re.S)
+    src = re.sub(r"//[^\n]*", " ", src)
+    src = re.sub(r'"(\\.|[^"\\])*"', '""', src)
+    return re.sub(r"^\s*#[^\n]*", " ", src, flags=re.M)
+
+
 def entry_name(src: str) -> str:
     """The oracle is told nothing but the text: the user function is the last
     top-level function definition in it (the convention stated in DESIGN.md §1)."""
+    src = _strip_comments(src)
     names = re.findall(r"([A-Za-z_]\w*)\s*\([^;{}]*\)\s*\{", src)
     names = [n for n in names if n not in ("if", "for", "while", "switch", "return")]
     if not names:

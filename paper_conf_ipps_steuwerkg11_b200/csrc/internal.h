@@ -38,6 +38,7 @@ struct Module {
     cudaKernel_t k_scan = nullptr;
     cudaKernel_t k_fold = nullptr;
     cudaKernel_t k_seed = nullptr;
+    cudaKernel_t k_zipcomb = nullptr;  // Zip modules: fused combine + zip + broadcast
     uint64_t sig[16 + 4 * 32] = {0};
     std::set<int> attr_set_on;  // devices on which smem attributes were set
 };
@@ -76,6 +77,9 @@ struct Buf {  // one logical device's storage of a vector
     size_t off = 0;    // element offset of the live data inside base
     size_t count = 0;  // live elements
     char *ptr(size_t es) const { return base ? base + off * es : nullptr; }
+    // rank mode: every rank's `base` of this vector, opened through CUDA IPC
+    std::vector<char *> peers;
+    char *peers_of = nullptr;  // the local base the peer table was built for
 };
 
 }  // namespace skelrt

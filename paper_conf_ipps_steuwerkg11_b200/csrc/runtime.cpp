@@ -695,6 +695,52 @@ int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_
     return SKEL_OK;
 }
 
+// ---- fused copy->block combine + Zip + block->copy (NEXT-1) ---------------------
+int ensure_ws(skel_ctx_s *ctx, Slot &s, size_t bytes);
+// rank mode: a stream-ordered barrier over all ranks (a one-word all-reduce)
+int rank_barrier(skel_ctx_s *ctx, Slot &s) {
+    DevGuard g(s.dev);
+    NK(ctx, ncclAllReduce(s.counters + 8, s.counters + 8, 1, ncclInt32, ncclSum, ctx->comm, s.stream));
+    return SKEL_OK;
+}
+
+void close_peers(Buf &b) {
+    for (size_t r = 0; r < b.peers.size(); ++r)
+        if (b.peers[r] && b.peers[r] != b.base) cudaIpcCloseMemHandle(b.peers[r]);
+    b.peers.clear();
+    b.peers_of = nullptr;
+}
+
+// rank mode: open every rank's allocation of this buffer through CUDA IPC
+// (collective: all ranks call it for the same vector)
+int ipc_peers(skel_ctx_s *ctx, Slot &s, Buf &b) {
+    if (b.peers_of == b.base && (int)b.peers.size() == ctx->D) return SKEL_OK;
+    close_peers(b);
+    DevGuard g(s.dev);
+    TRY(sync_all(ctx));
+    cudaIpcMemHandle_t mine;
+    CK(ctx, cudaIpcGetMemHandle(&mine, b.base));
+    const size_t hb = sizeof(cudaIpcMemHandle_t);
+    TRY(ensure_ws(ctx, s, std::max<size_t>(s.ws_cap, hb * (ctx->D + 1))));
+    CK(ctx, cudaMemcpy(s.ws, &mine, hb, cudaMemcpyHostToDevice));
+    NK(ctx, ncclAllGather(s.ws, s.ws + hb, hb, ncclUint8, ctx->comm, s.stream));
+    std::vector<cudaIpcMemHandle_t> all(ctx->D);
+    CK(ctx, cudaMemcpyAsync(all.data(), s.ws + hb, hb * ctx->D, cudaMemcpyDeviceToHost, s.stream));
+    CK(ctx, cudaStreamSynchronize(s.stream));
+    b.peers.assign(ctx->D, nullptr);
+    for (int r = 0; r < ctx->D; ++r) {
+        if (r == ctx->rank) {
+            b.peers[r] = b.base;
+            continue;
+        }
+        void *p = nullptr;
+        CK(ctx, cudaIpcOpenMemHandle(&p, all[r], cudaIpcMemLazyEnablePeerAccess));
+        b.peers[r] = static_cast<char *>(p);
+    }
+    b.peers_of = b.base;
+    return SKEL_OK;
+}
+
 // ---- Reduce / Scan -------------------------------------------------------------
 using PFN_encode = CUresult (*)(CUtensorMap *, CUtensorMapDataType, cuuint32_t, void *, const cuuint64_t *,
                                 const cuuint64_t *, const cuuint32_t *, const cuuint32_t *, CUtensorMapInterleave,
@@ -1158,6 +1204,7 @@ int skel_vector_create(skel_ctx_t ctx, size_t n, size_t es, skel_vec_t *out) {
 int skel_vector_destroy(skel_vec_t v) {
     if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
     skel_ctx_s *ctx = v->ctx;
+    for (auto &b : v->bufs) close_peers(b);
     for (size_t li = 0; li < v->bufs.size(); ++li) dev_free(ctx, ctx->slots[li], v->bufs[li].base);
     if (v->host) cudaFreeHost(v->host);
     ctx->vecs.erase(v);
@@ -1342,6 +1389,118 @@ int skel_zip(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_v
         return fail(ctx, SKEL_ERR_ARG, "bad zip arguments");
     if (a->n != b->n) return fail(ctx, SKEL_ERR_SIZE, "zip: vectors of unequal length (P:L268-269)");
     return run_ew(ctx, Kind::Zip, src, a, b, out, args, nargs);
+}
+
+int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_combine combine,
+                     skel_vec_t out, const skel_arg *args, int nargs) {
+    if (!ctx || !src || !a || !b || !out || a->ctx != ctx || b->ctx != ctx || out->ctx != ctx || (nargs && !args) ||
+        nargs < 0 || (int)combine < 1 || (int)combine > 4 || out == b)
+        return fail(ctx, SKEL_ERR_ARG, "bad zip_combine arguments");
+    if (a->n != b->n) return fail(ctx, SKEL_ERR_SIZE, "zip: vectors of unequal length (P:L268-269)");
+    if (b->dt == SKEL_DT_OPAQUE) return fail(ctx, SKEL_ERR_TYPE, "combine needs a numeric dtype (skel_vector_set_dtype)");
+    if (b->dist != SKEL_COPY && ctx->D > 1)
+        return fail(ctx, SKEL_ERR_STATE, "a combine merges per-device copies: b must be SKEL_COPY");
+    const int D = ctx->D;
+    const bool fused = D > 1 && D <= 16 && (a->dist == SKEL_COPY || a->dist == SKEL_BLOCK) &&
+                       (out != a || a->dist == SKEL_COPY) && !ctx->capturing;
+    if (!fused) {  // the same result as the unfused sequence
+        if (D > 1) TRY(set_distribution(b, SKEL_BLOCK, combine));
+        if (a->dist != b->dist) TRY(set_distribution(a, b->dist, SKEL_COMBINE_NONE));
+        TRY(run_ew(ctx, Kind::Zip, src, a, b, out, args, nargs));
+        return D > 1 ? set_distribution(out, SKEL_COPY, SKEL_COMBINE_NONE) : SKEL_OK;
+    }
+    Module *m = nullptr;
+    TRY(get_module(ctx, Kind::Zip, src, &m));
+    if (m->sig[4] != a->es || m->sig[5] != b->es)
+        return fail(ctx, SKEL_ERR_TYPE, "element sizes do not match the zip function's parameters");
+    if (m->sig[3] == 0 || m->sig[3] != out->es)
+        return fail(ctx, SKEL_ERR_TYPE, "output element size != sizeof(result)");
+    TRY(check_args(ctx, m, args, nargs));
+    TRY(ensure_device(a));
+    TRY(ensure_device(b));
+    const size_t n = a->n, esa = a->es, esb = b->es, eso = out->es;
+    if (out != a) {
+        if (out->n != n) {
+            out->n = n;
+            if (out->host) {
+                cudaFreeHost(out->host);
+                out->host = nullptr;
+            }
+        }
+        out->dist = SKEL_COPY;
+        TRY(place(out, SKEL_COPY));
+    }
+    const int block = (int)m->sig[9];
+    const uint64_t E = m->sig[8];
+    std::vector<unsigned char> abuf;
+    struct Ptrs {
+        void *p[16];
+    };
+    auto launch = [&](Slot &s, size_t li, const Ptrs &bs, void *bown, const Ptrs &os, const void *pa,
+                      uint64_t cnt) -> int {
+        int vec_ok = al16(pa) && al16(bown);
+        for (int j = 0; j < D; ++j) vec_ok = vec_ok && al16(bs.p[j]) && al16(os.p[j]);
+        pack_args(m, args, nargs, li, abuf);
+        const size_t chunks = vec_ok ? std::max<uint64_t>(cnt / E, 1) : cnt;
+        const int grid = ew_grid(s, chunks, block);
+        int nsrc = D, ndst = D, op = (int)combine;
+        void *params[] = {&pa, (void *)&bs, &nsrc, &bown, (void *)&os, &ndst, &cnt, &op, &vec_ok, abuf.data()};
+        DevGuard g(s.dev);
+        CK(ctx, cudaLaunchKernel((const void *)m->k_zipcomb, dim3(grid), dim3(block), params, 0, s.stream));
+        ctx->stats.kernel_launches++;
+        ctx->stats.d2d_bytes += (uint64_t)(D - 1) * cnt * (esb + eso);
+        return SKEL_OK;
+    };
+    if (!ctx->rank_mode) {
+        TRY(join(ctx));
+        for (size_t li = 0; li < ctx->slots.size(); ++li) {
+            Slot &s = ctx->slots[li];
+            const int k = s.d;
+            const size_t lo = part_lo(a, k), cnt = want_count(a, SKEL_BLOCK, k);
+            if (!cnt) continue;
+            Ptrs bs{}, os{};
+            for (int j = 0; j < D; ++j) {
+                bs.p[j] = b->bufs[j].base + lo * esb;
+                os.p[j] = out->bufs[j].base + lo * eso;
+            }
+            const void *pa = a->dist == SKEL_COPY ? a->bufs[li].base + lo * esa : a->bufs[li].ptr(esa);
+            TRY(launch(s, li, bs, b->bufs[li].base + lo * esb, os, pa, cnt));
+        }
+        TRY(join(ctx));
+    } else {
+        Slot &s = ctx->slots[0];
+        const int k = ctx->rank;
+        TRY(ipc_peers(ctx, s, b->bufs[0]));
+        TRY(ipc_peers(ctx, s, out->bufs[0]));
+        TRY(rank_barrier(ctx, s));  // every rank's copy of b is complete
+        const size_t lo = part_lo(a, k), cnt = want_count(a, SKEL_BLOCK, k);
+        if (cnt) {
+            Ptrs bs{}, os{};
+            for (int j = 0; j < D; ++j) {
+                bs.p[j] = b->bufs[0].peers[j] + lo * esb;
+                os.p[j] = out->bufs[0].peers[j] + lo * eso;
+            }
+            const void *pa = a->dist == SKEL_COPY ? a->bufs[0].base + lo * esa : a->bufs[0].ptr(esa);
+            TRY(launch(s, 0, bs, b->bufs[0].base + lo * esb, os, pa, cnt));
+        }
+        TRY(rank_barrier(ctx, s));  // every rank's part of out has landed everywhere
+    }
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        const int k = ctx->slots[li].d;
+        b->bufs[li].off = part_lo(b, k);
+        b->bufs[li].count = want_count(b, SKEL_BLOCK, k);
+        out->bufs[li].off = 0;
+        out->bufs[li].count = n;
+    }
+    b->dist = SKEL_BLOCK;
+    b->dev_valid = true;
+    b->diverged = false;
+    device_wrote(b);
+    out->dist = SKEL_COPY;
+    out->dev_valid = true;
+    out->diverged = false;
+    device_wrote(out);
+    return SKEL_OK;
 }
 
 int skel_reduce_to(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t result, const skel_arg *args,

@@ -212,3 +212,74 @@ extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
     // scalar path: the tail, or everything for non-vectorisable element types
     for (skel_u64 i = done + tid; i < n; i += stride) skel_one(a, b, out, i, t);
 }
+
+#if SKEL_NIN == 2
+// ---------------------------------------------------------------------------
+// Fused copy->block combine + Zip + block->copy (Listing 4
+// P:L542-548 as one kernel).  Device k owns part [lo, hi): for each element it
+// combines the D copies of b (peer loads over NVLink when the copies live on
+// other GPUs), keeps the combined value in its own part of b, applies the Zip
+// function to a and the combined b, and stores the result into the part of
+// every device's copy of out (peer stores).  Replaces reduce-scatter + Zip +
+// all-gather: each byte crosses the interconnect once and no intermediate
+// round trip through HBM is needed.
+// ---------------------------------------------------------------------------
+#define SKEL_MAXDEV 16
+struct skel_ptrs { void *p[SKEL_MAXDEV]; };
+
+template <class T> __device__ __forceinline__ T skel_comb_op(T x, T y, int op) {
+    if constexpr (skel::is_arith<T>::value) {
+        if (op == 1) return x + y;
+        if (op == 2) return y < x ? y : x;
+        if (op == 3) return x < y ? y : x;
+        return x * y;
+    } else {
+        return x;  // never launched: the host requires a numeric dtype for a combine
+    }
+}
+
+template <class Tup>
+__device__ __forceinline__ void skel_zipcomb_elem(const skel_A &xa, const skel_ptrs &bs, int nsrc, skel_B *bown,
+                                                  const skel_ptrs &os, int ndst, skel_u64 i, int op, Tup &t) {
+    skel_B acc = static_cast<const skel_B *>(bs.p[0])[i];
+    for (int d = 1; d < nsrc; ++d) acc = skel_comb_op(acc, static_cast<const skel_B *>(bs.p[d])[i], op);
+    bown[i] = acc;
+    if constexpr (!skel_void) {
+        const skel_O r = skel::caller<skel_Seq>::call(&SKEL_FN, t, xa, acc);
+        for (int d = 0; d < ndst; ++d) static_cast<skel_O *>(os.p[d])[i] = r;
+    }
+}
+
+extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
+    skel_zipcomb_kernel(const skel_A *__restrict__ a, const skel_ptrs bsrc, int nsrc, skel_B *bown,
+                        const skel_ptrs odst, int ndst, skel_u64 n, int op, int vec_ok, const skel_Buf args) {
+    auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
+    const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;
+    skel_u64 done = 0;
+    if constexpr (SKEL_E > 1 && !skel_void) {
+        if (vec_ok) {
+            const skel_u64 nch = n / SKEL_E;
+            done = nch * SKEL_E;
+            for (skel_u64 c = tid; c < nch; c += stride) {
+                const auto xa = skel::bit_cast<skel::arr<skel_A, SKEL_E>>(
+                    skel_ld<skel_CA>(reinterpret_cast<const char *>(a) + c * skel_CA));
+                auto acc = skel::bit_cast<skel::arr<skel_B, SKEL_E>>(
+                    *reinterpret_cast<const skel::chunk<skel_CB> *>(static_cast<const char *>(bsrc.p[0]) + c * skel_CB));
+                for (int d = 1; d < nsrc; ++d) {
+                    const auto y = skel::bit_cast<skel::arr<skel_B, SKEL_E>>(
+                        *reinterpret_cast<const skel::chunk<skel_CB> *>(static_cast<const char *>(bsrc.p[d]) + c * skel_CB));
+#pragma unroll
+                    for (int e = 0; e < SKEL_E; ++e) acc.v[e] = skel_comb_op(acc.v[e], y.v[e], op);
+                }
+                skel_st<skel_CB>(reinterpret_cast<char *>(bown) + c * skel_CB, skel::bit_cast<skel::chunk<skel_CB>>(acc));
+                skel::arr<skel_O, SKEL_E> yo;
+                skel_apply_chunk(xa.v, acc.v, yo.v, t);
+                const auto co = skel::bit_cast<skel::chunk<skel_CO>>(yo);
+                for (int d = 0; d < ndst; ++d) skel_st<skel_CO>(static_cast<char *>(odst.p[d]) + c * skel_CO, co);
+            }
+        }
+    }
+    for (skel_u64 i = done + tid; i < n; i += stride) skel_zipcomb_elem(a[i], bsrc, nsrc, bown, odst, ndst, i, op, t);
+}
+#endif

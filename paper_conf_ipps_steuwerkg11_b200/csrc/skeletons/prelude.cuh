@@ -33,6 +33,15 @@ template <class T> struct is_ptr { static constexpr bool value = false; };
 template <class T> struct is_ptr<T *> { static constexpr bool value = true; };
 template <class T> struct is_void { static constexpr bool value = false; };
 template <> struct is_void<void> { static constexpr bool value = true; };
+template <class T> struct is_arith { static constexpr bool value = false; };
+template <> struct is_arith<float> { static constexpr bool value = true; };
+template <> struct is_arith<double> { static constexpr bool value = true; };
+template <> struct is_arith<int> { static constexpr bool value = true; };
+template <> struct is_arith<unsigned> { static constexpr bool value = true; };
+template <> struct is_arith<long long> { static constexpr bool value = true; };
+template <> struct is_arith<unsigned long long> { static constexpr bool value = true; };
+template <> struct is_arith<long> { static constexpr bool value = true; };
+template <> struct is_arith<unsigned long> { static constexpr bool value = true; };
 template <class A, class B> struct same { static constexpr bool value = false; };
 template <class A> struct same<A, A> { static constexpr bool value = true; };
 

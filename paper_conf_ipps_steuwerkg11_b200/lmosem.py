@@ -37,13 +37,17 @@ class LMOSEM:
         v.set_distribution(skel.BLOCK)
         return v
 
-    def subset(self, events: skel.Vector):
-        """One iteration of Listing 4's loop body."""
+    def subset(self, events: skel.Vector, fused: bool = False):
+        """One iteration of Listing 4's loop body.  fused=True runs the tail
+        (combine c, update f, redistribute f) as one peer-memory kernel."""
         ctx, f, c = self.ctx, self.f, self.c
-        f.set_distribution(skel.COPY)                     # block -> copy: all-gather
+        f.set_distribution(skel.COPY)                     # block -> copy: all-gather (no-op after a fused tail)
         c.fill_dist(skel.COPY, np.float32(0))             # fresh zero copy on every device
         ctx.map(LMOSEM_ERROR, events, None, args=[f, c, *self.dims_args])
         c.mark_device_modified()                          # dataOnDevicesModified()
+        if fused:
+            ctx.zip_combine(LMOSEM_UPDATE, f, c, skel.COMBINE_ADD, f)
+            return
         f.set_distribution(skel.BLOCK)                    # copy -> block: local slice
         c.set_distribution(skel.BLOCK, skel.COMBINE_ADD)  # copy -> block + add: reduce-scatter
         ctx.zip(LMOSEM_UPDATE, f, c, f)                   # f[j] *= c[j] where c[j] > 0

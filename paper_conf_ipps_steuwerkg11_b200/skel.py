@@ -84,7 +84,8 @@ def lib() -> ctypes.CDLL:
             "skel_vector_part": [P, I, ctypes.POINTER(S), ctypes.POINTER(S)],
             "skel_vector_device_ptr": [P, I, PP, ctypes.POINTER(S)],
             "skel_map": [P, ctypes.c_char_p, P, P, P, I], "skel_zip": [P, ctypes.c_char_p, P, P, P, P, I],
-            "skel_reduce": [P, ctypes.c_char_p, P, P, P, I], "skel_reduce_to": [P, ctypes.c_char_p, P, P, P, I],
+            "skel_reduce": [P, ctypes.c_char_p, P, P, P, I],
+            "skel_zip_combine": [P, ctypes.c_char_p, P, P, I, P, P, I], "skel_reduce_to": [P, ctypes.c_char_p, P, P, P, I],
             "skel_scan": [P, ctypes.c_char_p, P, P, P, P, I], "skel_prepare": [P, ctypes.c_char_p, ctypes.c_char_p],
             "skel_entry_name": [ctypes.c_char_p, ctypes.c_char_p, S],
             "skel_compile_check": [ctypes.c_char_p, ctypes.c_char_p, I, ctypes.c_char_p, S, ctypes.POINTER(S)],
@@ -271,6 +272,12 @@ class Context:
         """eq. (2): vout[i] = f(va[i], vb[i], args...)."""
         a, keep = self._args(args)
         _check(lib().skel_zip(self._h, src.encode(), va._h, vb._h, vout._h, a, len(args)), self._h)
+        return vout
+
+    def zip_combine(self, src: str, va: "Vector", vb: "Vector", combine: int, vout: "Vector", args=()):
+        """vb.set_distribution(BLOCK, combine); vout = zip(va, vb); vout -> COPY, fused (NEXT-1)."""
+        a, keep = self._args(args)
+        _check(lib().skel_zip_combine(self._h, src.encode(), va._h, vb._h, combine, vout._h, a, len(args)), self._h)
         return vout
 
     def reduce(self, src: str, vin: "Vector", args=()):

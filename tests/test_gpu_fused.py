@@ -1,0 +1,92 @@
+"""skel_zip_combine: Listing 4's tail (copy->block+combine, update Zip,
+block->copy) fused into one peer-memory kernel per device (NEXT-1).  It must
+give bit-for-bit what the unfused sequence gives (same summation order)."""
+import numpy as np
+import pytest
+
+import oracle
+import skel_inputs as si
+from paper_conf_ipps_steuwerkg11_b200 import skel
+from paper_conf_ipps_steuwerkg11_b200.lmosem import LMOSEM
+from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_UPDATE
+
+pytestmark = pytest.mark.gpu
+MARK = "void mark(int i, float* c, float s){ c[i] += s * (float)(1 + i % 5); }"
+
+
+def diverged_copies(ctx, n, seed):
+    """A copy-distributed float vector whose D copies differ (side-effect Map)."""
+    base = si.uniform_f32(n, seed)
+    c = ctx.vector(base)
+    c.set_distribution(skel.COPY)
+    idx = ctx.vector(np.arange(n, dtype=np.int32))
+    idx.set_distribution(skel.BLOCK)
+    ctx.map(MARK, idx, None, args=[c, np.float32(0.25)])
+    c.mark_device_modified()
+    return c
+
+
+@pytest.mark.parametrize("D", [2, 3, 4, 8])
+@pytest.mark.parametrize("inplace", [True, False])
+def test_fused_equals_unfused(D, inplace):
+    n = 123_457
+    f0 = si.uniform_f32(n, 3)
+    res = []
+    for fused in (True, False):
+        with skel.Context(D) as ctx:
+            f = ctx.vector(f0)
+            f.set_distribution(skel.COPY)
+            c = diverged_copies(ctx, n, 9)
+            out = f if inplace else ctx.vector(n=n, dtype=np.float32)
+            if fused:
+                ctx.zip_combine(LMOSEM_UPDATE, f, c, skel.COMBINE_ADD, out)
+            else:
+                c.set_distribution(skel.BLOCK, skel.COMBINE_ADD)
+                f.set_distribution(skel.BLOCK)
+                ctx.zip(LMOSEM_UPDATE, f, c, out)
+                out.set_distribution(skel.COPY)
+            assert out.distribution == skel.COPY and c.distribution == skel.BLOCK
+            res.append((out.download(), c.download()))
+            # every device holds the full result
+            for li in range(D):
+                assert out.device_ptr(li)[1] == n
+    assert np.array_equal(res[0][0], res[1][0]) and np.array_equal(res[0][1], res[1][1])
+    # and against the definition: c = sum of the copies, out = update(f, c)
+    copies = [si.uniform_f32(n, 9) for _ in range(D)]
+    for d in range(D):
+        lo, hi = (d * -(-n // D), min(n, (d + 1) * -(-n // D)))
+        copies[d][lo:hi] += np.float32(0.25) * (1 + np.arange(lo, hi) % 5).astype(np.float32)
+    csum = copies[0].copy()
+    for d in range(1, D):
+        csum = (csum + copies[d]).astype(np.float32)
+    assert np.array_equal(res[0][1], csum)
+    assert np.array_equal(res[0][0], oracle.skel_zip(LMOSEM_UPDATE, f0, csum, np.float32))
+
+
+def test_fused_min_max_int():
+    n = 10_001
+    src = "int keep(int a, int b){ return a > b ? a : b; }"
+    with skel.Context(4) as ctx:
+        a = ctx.vector(np.arange(n, dtype=np.int32))
+        a.set_distribution(skel.BLOCK)
+        c = ctx.vector(np.zeros(n, np.int32))
+        c.set_distribution(skel.COPY)
+        idx = ctx.vector(np.arange(n, dtype=np.int32))
+        idx.set_distribution(skel.BLOCK)
+        ctx.map("void m(int i, int* c){ c[i] = 3 * i; }", idx, None, args=[c])
+        c.mark_device_modified()
+        out = ctx.vector(n=n, dtype=np.int32)
+        ctx.zip_combine(src, a, c, skel.COMBINE_MAX, out)
+        assert np.array_equal(out.download(), 3 * np.arange(n, dtype=np.int32))
+
+
+@pytest.mark.parametrize("D", [2, 4])
+def test_lmosem_fused_subsets_match_oracle(D):
+    subsets = [si.lmosem_events(10_000, subset=l) for l in range(2)]
+    with skel.Context(D) as ctx:
+        rec = LMOSEM(ctx)
+        for ev in subsets:
+            rec.subset(rec.events(ev), fused=True)
+        img = rec.image()
+    want = oracle.lmosem_reconstruct(subsets)
+    assert np.linalg.norm(img - want) <= 1e-4 * np.linalg.norm(want)

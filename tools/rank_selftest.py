@@ -76,7 +76,7 @@ for dst in (skel.BLOCK, skel.SINGLE, skel.COPY):
             print(f"rank {rank}: combine->{dst} rep {rep}: {bad.size} bad, first {bad[:5]}, got {got[bad[:5]]}, "
                   f"want {want[bad[:5]]}, parts {[c.part(d) for d in range(world)]}", flush=True)
         check(f"combine->{dst}", ok)
-# LM OSEM one subset
+# LM OSEM one subset, then two more with the fused peer-memory tail (CUDA IPC)
 ev = si.lmosem_events(20_000, subset=1)
 rec = LMOSEM(ctx)
 rec.subset(rec.events(ev))
@@ -84,6 +84,13 @@ img = rec.image()
 want, _, _ = oracle.lmosem_subset(ev, np.ones(150 * 150 * 280))
 rel = float(np.linalg.norm(img - want) / np.linalg.norm(want))
 check("lmosem", rel <= 1e-4)
+subsets = [si.lmosem_events(8_000, subset=l) for l in range(2)]
+rec2 = LMOSEM(ctx)
+for sub in subsets:
+    rec2.subset(rec2.events(sub), fused=True)
+want2 = oracle.lmosem_reconstruct(subsets)
+rel2 = float(np.linalg.norm(rec2.image() - want2) / np.linalg.norm(want2))
+check("lmosem_fused", rel2 <= 1e-4)
 print(f"rank {rank}/{world} device {dev}: {'OK' if not fails else 'FAIL ' + ','.join(fails)} (lmosem relL2 {rel:.2e})",
       flush=True)
 ctx.close()
