@@ -578,6 +578,9 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         return max_over_ranks(e0.elapsed_time(e1) / reps)
 
     ms = timed(lambda: rec.subset(evv))
+    for _ in range(2):
+        rec.subset(evv, fused=True)
+    ms_fused = timed(lambda: rec.subset(evv, fused=True))
     try:
         if os.environ.get("SKEL_BENCH_NO_GRAPH"):
             raise skel.SkelError(8, "graphs disabled")
@@ -588,9 +591,11 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         ms_graph = ms
     evv.destroy()
     return {"config": "configs[3]/[4]: one subset, 10^6 events, 150x150x280, events block over GPUs",
-            "subset_s": ms * 1e-3, "subset_s_graph": ms_graph * 1e-3, "events_per_s": nev / (ms_graph * 1e-3),
+            "subset_s": ms * 1e-3, "subset_s_graph": ms_graph * 1e-3, "subset_s_fused": ms_fused * 1e-3,
+            "events_per_s": nev / (min(ms_graph, ms_fused) * 1e-3),
             "note": "includes f all-gather, c zero-fill, Siddon Map, c reduce-scatter and update Zip; "
-                    "subset_s = eager calls, subset_s_graph = the same subset replayed as a CUDA graph"}
+                    "subset_s = eager calls, subset_s_graph = the same subset replayed as a CUDA graph, "
+                    "subset_s_fused = the tail as one peer-memory kernel (skel_zip_combine, NEXT-1)"}
 
 
 if __name__ == "__main__":

@@ -722,7 +722,8 @@ int ipc_peers(skel_ctx_s *ctx, Slot &s, Buf &b) {
     CK(ctx, cudaIpcGetMemHandle(&mine, b.base));
     const size_t hb = sizeof(cudaIpcMemHandle_t);
     TRY(ensure_ws(ctx, s, std::max<size_t>(s.ws_cap, hb * (ctx->D + 1))));
-    CK(ctx, cudaMemcpy(s.ws, &mine, hb, cudaMemcpyHostToDevice));
+    // stream-ordered: the all-gather below runs on s.stream
+    CK(ctx, cudaMemcpyAsync(s.ws, &mine, hb, cudaMemcpyHostToDevice, s.stream));
     NK(ctx, ncclAllGather(s.ws, s.ws + hb, hb, ncclUint8, ctx->comm, s.stream));
     std::vector<cudaIpcMemHandle_t> all(ctx->D);
     CK(ctx, cudaMemcpyAsync(all.data(), s.ws + hb, hb * ctx->D, cudaMemcpyDeviceToHost, s.stream));
@@ -990,10 +991,11 @@ static int init_slot(skel_ctx_s *ctx, int d, int dev) {
     CK(ctx, cudaEventCreateWithFlags(&s.ev, cudaEventDisableTiming));
     void *p = nullptr;
     CK(ctx, cudaMalloc(&p, 256));
-    CK(ctx, cudaMemset(p, 0, 256));
+    CK(ctx, cudaMemsetAsync(p, 0, 256, s.stream));  // ordered with the epoch write below
     s.counters = static_cast<unsigned *>(p);
     const unsigned first_epoch = 1;  // status words are zeroed: epoch 0 must never be live
-    CK(ctx, cudaMemcpy(s.counters + 3, &first_epoch, sizeof first_epoch, cudaMemcpyHostToDevice));
+    CK(ctx, cudaMemcpyAsync(s.counters + 3, &first_epoch, sizeof first_epoch, cudaMemcpyHostToDevice, s.stream));
+    CK(ctx, cudaStreamSynchronize(s.stream));
     ctx->slots.push_back(s);
     return SKEL_OK;
 }
