@@ -586,8 +586,12 @@ template <class Tup> __device__ __forceinline__ VT cons_fold(VT x, VT *wpart, Tu
     }
     return r;
 }
-// ordered exclusive scan over the consumers; block total to *total
-template <class Tup> __device__ __forceinline__ VT cons_exscan(VT x, VT *wsc, VT *total, Tup &t) {
+// ordered exclusive scan over the consumers with ONE barrier: warp totals go
+// to wbuf, then every warp scans the SNW totals itself (redundantly) to get
+// its warp prefix and the block total.  Callers alternate two wbuf buffers
+// between consecutive tiles, so a buffer is rewritten only after a barrier
+// that every reader of its previous contents has passed.
+template <class Tup> __device__ __forceinline__ VT cons_exscan1(VT x, VT *wbuf, VT &total, Tup &t) {
     const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
     VT inc = x;
 #pragma unroll
@@ -597,25 +601,20 @@ template <class Tup> __device__ __forceinline__ VT cons_exscan(VT x, VT *wsc, VT
     }
     VT ex = vt_shfl_up(inc, 1);
     if (lane == 0) ex.ok = false;
-    if (lane == 31) wsc[w] = inc;
+    if (lane == 31) wbuf[w] = inc;
     cons_sync();
-    if (w == 0) {
-        VT y;
-        y.ok = false;
-        if (lane < SNW) y = wsc[lane];
-        VT yi = y;
+    VT yi;
+    yi.ok = false;
+    if (lane < SNW) yi = wbuf[lane];
 #pragma unroll
-        for (int d = 1; d < 32; d <<= 1) {
-            VT o = vt_shfl_up(yi, d);
-            if (lane >= d) yi = comb(o, yi, t);
-        }
-        VT ye = vt_shfl_up(yi, 1);
-        if (lane == 0) ye.ok = false;
-        if (lane < SNW) wsc[lane] = ye;
-        if (lane == SNW - 1) *total = yi;
+    for (int d = 1; d < SNW; d <<= 1) {
+        VT o = vt_shfl_up(yi, d);
+        if (lane >= d) yi = comb(o, yi, t);
     }
-    cons_sync();
-    return comb(wsc[w], ex, t);
+    VT wpre = vt_shfl_idx(yi, w > 0 ? w - 1 : 0);
+    if (w == 0) wpre.ok = false;
+    total = vt_shfl_idx(yi, SNW - 1);
+    return comb(wpre, ex, t);
 }
 
 #ifndef SKEL_SCAN_MINB
@@ -633,7 +632,7 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     __shared__ unsigned s_epoch;
     __shared__ skel_u64 full_bar[SSTAGES], done_bar[SSTAGES], pre_full[2], pre_empty[2];
-    __shared__ VT wsc[SNW];
+    __shared__ VT wsc[2][SNW];  // warp partials, alternated between consecutive tiles
     __shared__ VT s_tot, s_pre[2];
     const int t = threadIdx.x, lane = t & 31, w = t >> 5;
     const skel_u64 G = gridDim.x, c = blockIdx.x;
@@ -773,7 +772,7 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
             a.ok = true;
 #pragma unroll
             for (int k = 1; k < K; ++k) a.v = opf(a.v, x[k], tup);
-            const VT tv = cons_fold(a, wsc, tup);
+            const VT tv = cons_fold(a, wsc[v & 1], tup);
             if (t == 0) {
                 run1 = comb(run1, tv, tup);
                 if (j == nj - 1) {
@@ -788,9 +787,10 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
             VT mine;
             mine.v = x[K - 1];
             mine.ok = true;
-            const VT excl = cons_exscan(mine, wsc, &s_tot, tup);
+            VT tot;
+            const VT excl = cons_exscan1(mine, wsc[v & 1], tot, tup);
             const VT pre = comb(run, excl, tup);
-            run = comb(run, s_tot, tup);
+            run = comb(run, tot, tup);
 #pragma unroll
             for (int k = K - 1; k >= 1; --k) x[k] = opf(pre.v, x[k - 1], tup);
             x[0] = pre.v;
@@ -826,7 +826,9 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
                 mine = comb(mine, e, tup);
             }
         }
-        const VT excl = cons_exscan(mine, wsc, &s_tot, tup);
+        cons_sync();  // the last tile's readers of wsc are done
+        VT tot;
+        const VT excl = cons_exscan1(mine, wsc[0], tot, tup);
         const VT pre = comb(carry_end, excl, tup);
         skel_T r = pre.v;  // second pass (in-place safe: read, then write)
         for (skel_u64 k = 0; k < kt; ++k) {
@@ -834,7 +836,7 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
             out[first + k] = r;
             r = opf(r, e, tup);
         }
-        if (t == 0 && total) total->v = comb(carry_end, s_tot, tup).v;
+        if (t == 0 && total) total->v = comb(carry_end, tot, tup).v;
     }
     cons_sync();
     if (t == 0) {
