@@ -194,7 +194,9 @@ static int assemble(Kind kind, const std::string &user, int block, bool fmad, st
     *text += kPreludeSrc;
     *text += "\n#line 1 \"user_function\"\n";
     *text += user;
-    *text += "\n#line 1 \"skel_skeleton.cuh\"\n#define SKEL_FN " + entry + "\n" + defs;
+    // "::entry": the user's function is a top-level one, so a template local of
+    // the same name (e.g. a parameter `op`) cannot shadow it
+    *text += "\n#line 1 \"skel_skeleton.cuh\"\n#define SKEL_FN ::" + entry + "\n" + defs;
     *text += (kind == Kind::Red) ? kRedSrc : kMapSrc;
     return SKEL_OK;
 }

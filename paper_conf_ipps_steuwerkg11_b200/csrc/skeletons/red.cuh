@@ -228,7 +228,7 @@ __device__ __forceinline__ void issue_tile(unsigned char *dst, const skel_tmap *
 // (templates so that element sizes without a TMA path never instantiate them)
 template <bool OK = TMA_OK> __device__ __forceinline__ void read_row(const unsigned char *stage, int r, skel_T *x) {
     if constexpr (OK) {
-        constexpr int PER = (int)(16 / sizeof(skel_T));
+        constexpr int PER = OK ? (int)(16 / sizeof(skel_T)) : 1;  // dependent: no arr<T,0> when !OK
         const unsigned char *row = stage + (size_t)r * 128;
 #pragma unroll
         for (int j = 0; j < 8; ++j) {
@@ -241,7 +241,7 @@ template <bool OK = TMA_OK> __device__ __forceinline__ void read_row(const unsig
 }
 template <bool OK = TMA_OK> __device__ __forceinline__ void write_row(unsigned char *stage, int r, const skel_T *x) {
     if constexpr (OK) {
-        constexpr int PER = (int)(16 / sizeof(skel_T));
+        constexpr int PER = OK ? (int)(16 / sizeof(skel_T)) : 1;  // dependent: no arr<T,0> when !OK
         unsigned char *row = stage + (size_t)r * 128;
 #pragma unroll
         for (int j = 0; j < 8; ++j) {

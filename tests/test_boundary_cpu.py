@@ -110,3 +110,21 @@ def test_oracle_and_product_share_no_code():
     for p in osrc:
         assert not re.search(r"^\s*(from|import)\s+paper_conf_ipps_steuwerkg11_b200", p.read_text(), re.M), p
         assert "skel.h" not in p.read_text() and "libskel" not in p.read_text(), p
+
+
+@pytest.mark.parametrize("kind,nbytes", [(k, b) for k in ("map", "zip") for b in (1, 2, 3, 6, 12, 20, 24, 48, 64, 256)]
+                         + [("reduce", b) for b in (1, 2, 3, 6, 8, 12, 16, 20, 24, 32)])
+def test_every_element_size_instantiates(kind, nbytes):
+    """The reduce/scan templates (one module) pick a TMA path for 4/8/16-byte
+    elements and a direct path for every other size; each must instantiate
+    (no zero-length arrays, no instantiation of the unused path).  The entry is
+    named `op` on purpose: the templates have a parameter of that name, which
+    must not shadow the user's function."""
+    n = nbytes
+    src = (f"struct E {{ unsigned char b[{n}]; }};\n"
+           f"E op(E x, E y) {{ E r = x; r.b[0] += y.b[0]; r.b[{n - 1}] ^= y.b[{n - 1}]; return r; }}\n")
+    if kind == "map":
+        src = src.replace("E op(E x, E y)", "E op(E x)").replace("y.b", "x.b")
+    st, log, nb = skel.compile_check(kind, src)
+    assert st == 0, log
+    assert nb > 1000

@@ -192,3 +192,49 @@ def test_map_under_each_distribution(dist):
         if dist == skel.COPY:
             for li in range(4):
                 assert out.device_ptr(li)[1] == x.size
+
+
+@pytest.mark.parametrize("D", [3, 5, 7])
+@pytest.mark.parametrize("n", [1001, 70_003])
+def test_skeletons_on_unaligned_block_views(D, n):
+    """copy -> block keeps each device's part inside its full buffer at offset
+    k*ceil(n/D) (no data movement); for these (n, D) the parts start at
+    addresses that are not 16-byte aligned, which must route every skeleton to
+    its unaligned path."""
+    xi = si.uniform_int01(n, 1)
+    xf = si.uniform_f32(n, 2)
+    with skel.Context(D) as ctx:
+        vi = ctx.vector(xi)
+        vi.set_distribution(skel.COPY)
+        wi = ctx.vector(n=n, dtype=np.int32)
+        ctx.map(IDENT_I32, vi, wi)  # device-valid copies
+        wi.set_distribution(skel.BLOCK)  # local slices, aliased
+        assert int(ctx.reduce(SUM_I32, wi)) == int(xi.sum())
+        out = ctx.vector(n=n, dtype=np.int32)
+        ctx.scan(SUM_I32, wi, out, np.int32(0))
+        assert np.array_equal(out.download(), oracle.skel_scan(SUM_I32, xi, 0))
+        m = ctx.vector(n=n, dtype=np.int32)
+        ctx.map(MAP_I32, wi, m)
+        assert np.array_equal(m.download(), oracle.skel_map(MAP_I32, xi, np.int32))
+        vf = ctx.vector(xf)
+        vf.set_distribution(skel.COPY)
+        wf = ctx.vector(n=n, dtype=np.float32)
+        ctx.map("float id(float x){ return x; }", vf, wf)
+        wf.set_distribution(skel.BLOCK)
+        z = ctx.vector(n=n, dtype=np.float32)
+        ctx.zip(SAXPY_F32, wf, wf, z, args=[np.float32(2.5)])
+        assert np.array_equal(z.download(), oracle.skel_zip(SAXPY_F32, xf, xf, np.float32, args=[np.float32(2.5)]))
+
+
+def test_more_devices_than_elements():
+    x = np.arange(3, dtype=np.int32)
+    with skel.Context(8) as ctx:
+        v = ctx.vector(x)
+        v.set_distribution(skel.BLOCK)
+        assert int(ctx.reduce(SUM_I32, v)) == 3
+        out = ctx.vector(n=3, dtype=np.int32)
+        ctx.scan(SUM_I32, v, out, np.int32(0))
+        assert out.download().tolist() == [0, 0, 1]
+        v.set_distribution(skel.COPY)
+        v.set_distribution(skel.SINGLE)
+        assert v.download().tolist() == [0, 1, 2]

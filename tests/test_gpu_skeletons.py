@@ -327,3 +327,41 @@ def test_scan_last_plus_x_equals_reduce(ctx):
     vx = ctx.vector(x)
     ctx.scan(src, vx, out, np.uint32(0))
     assert np.uint32(out.download()[-1] + x[-1]) == ctx.reduce(src, vx)
+
+
+BIG = """
+struct Big { double a[3]; unsigned n; unsigned p; };   /* 32-byte element, direct path */
+/* .a: exact float64 sums; (.n, .p): base-3 Horner digits mod 2^32 -- associative, not commutative */
+Big bsum(Big x, Big y) { Big r; for (int i = 0; i < 3; ++i) r.a[i] = x.a[i] + y.a[i]; r.n = x.n * y.p + y.n; r.p = x.p * y.p; return r; }
+"""
+BIG_DT = np.dtype([("a", np.float64, (3,)), ("n", np.uint32), ("p", np.uint32)])
+
+
+@pytest.mark.parametrize("n", [1, 100, 5000, 200_003])
+def test_32byte_elements_reduce_scan(ctx, n):
+    g = np.random.default_rng(n)
+    x = np.zeros(n, BIG_DT)
+    x["a"] = g.integers(0, 1000, (n, 3)).astype(np.float64)  # exact in float64: any order
+    x["n"] = g.integers(0, 3, n).astype(np.uint32)
+    x["p"] = 3
+    r = ctx.reduce(BIG, ctx.vector(x))
+    want = oracle.skel_reduce(BIG, x)
+    assert r.tobytes() == want.tobytes()  # .n is order-sensitive, .a exact
+    ident = np.zeros(1, BIG_DT)
+    ident["p"] = 1
+    out = ctx.vector(n=n, dtype=BIG_DT)
+    ctx.scan(BIG, ctx.vector(x), out, ident[0])
+    assert out.download().tobytes() == oracle.skel_scan(BIG, x, ident[0]).tobytes()
+
+
+@pytest.mark.parametrize("n", [3, 16385, 1_000_001])
+def test_double_reduce_scan(ctx, n):
+    src = "double add(double a, double b){ return a + b; }"
+    x = si.uniform_f32(n, 4).astype(np.float64)
+    r = float(ctx.reduce(src, ctx.vector(x)))
+    assert abs(r - float(np.sum(x))) <= 1e-12 * float(np.sum(np.abs(x)))
+    out = ctx.vector(n=n, dtype=np.float64)
+    ctx.scan(src, ctx.vector(x), out, np.float64(0))
+    want = oracle.skel_scan(src, x, 0.0)  # left-to-right float64 prefix
+    got = out.download()
+    assert np.all(np.abs(got - want) <= 1e-12 * np.concatenate([[0], np.cumsum(np.abs(x))[:-1]]) + 1e-300)
