@@ -1583,7 +1583,8 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
     // D partial results)
     const uint64_t SRB = m->sig[15] & 0xffff;  // rows (consumer threads) per scan tile
     const uint64_t TILE = SRB * m->sig[8];      // scan tile (elements)
-    const uint64_t CH = m->sig[15] >> 16;       // tiles per CTA per slice
+    const uint64_t CH = (m->sig[15] >> 16) & 0xffff;                     // tiles per CTA per slice
+    const uint64_t REPL = std::max<uint64_t>(1, (m->sig[15] >> 32) & 0xff);  // copies of each status word
     const bool packed = m->sig[13] != 0;
     TRY(set_smem_attr(ctx, m, ctx->slots[0]));
     int occ = 1;  // persistent grid: SMs x resident CTAs per SM
@@ -1620,7 +1621,7 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         if (!cnt) continue;
         const size_t G = (size_t)scan_grid(s);
         const RedLayout &L = Ls[li];
-        TRY(ensure_status(ctx, s, scan_slots(s, cnt), packed));
+        TRY(ensure_status(ctx, s, REPL * (scan_slots(s, cnt) + 64), packed));
         TRY(set_smem_attr(ctx, m, s));
         pack_args(m, args, nargs, li, abuf);
         DevGuard g(s.dev);

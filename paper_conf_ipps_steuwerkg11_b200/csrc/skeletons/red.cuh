@@ -55,9 +55,13 @@ constexpr int STAGES = SKEL_STAGES;
 constexpr unsigned DSMEM = TMA_OK ? STAGES * TILE_BYTES + 1024 : 0;
 // Scan: tiles per CTA per slice (see the Scan section)
 #ifndef SKEL_SCAN_CH
-#define SKEL_SCAN_CH 2
+#define SKEL_SCAN_CH 1
 #endif
 constexpr int SCAN_CH = SKEL_SCAN_CH;
+#ifndef SKEL_SCAN_PW
+#define SKEL_SCAN_PW 1
+#endif
+constexpr int PW = SKEL_SCAN_PW;  // Scan window warps (slices folded concurrently)
 #ifndef SKEL_SCAN_RB
 #define SKEL_SCAN_RB 512
 #endif
@@ -71,6 +75,12 @@ constexpr skel_u64 STILE = (skel_u64)SRB * K;
 constexpr unsigned STILE_BYTES = (unsigned)(STILE * sizeof(skel_T));
 constexpr unsigned SDSMEM = TMA_OK ? SSTAGES * STILE_BYTES + 1024 : 0;
 constexpr bool PACKED = sizeof(skel_S) == 4;  // status = value:32 | epoch:30 | state:2
+#ifndef SKEL_SCAN_REPL
+#define SKEL_SCAN_REPL 8
+#endif
+// copies of every packed status word: CTA c polls copy c % REPL, so the few L2
+// lines a slice's status occupies are not hammered by all G CTAs at once
+constexpr int REPL = PACKED ? SKEL_SCAN_REPL : 1;
 
 struct skel_sig_t { skel_u64 v[16 + 4 * 32]; };
 constexpr skel_sig_t skel_make_sig() {
@@ -89,8 +99,8 @@ constexpr skel_sig_t skel_make_sig() {
     s.v[11] = DSMEM;
     s.v[12] = SDSMEM;
     s.v[13] = PACKED;
-    s.v[14] = SRB + 64;  // scan kernel block size (consumers + producer + prefix warps); tile = SRB * K
-    s.v[15] = (skel_u64)SRB | ((skel_u64)SCAN_CH << 16);  // scan rows per tile | tiles per CTA per slice
+    s.v[14] = SRB + 64 + 32 * PW;  // scan block size (consumers, producer, store and window warps); tile = SRB * K
+    s.v[15] = (skel_u64)SRB | ((skel_u64)SCAN_CH << 16) | ((skel_u64)REPL << 32);  // scan rows/tile | tiles/CTA/slice | status copies
     for (int i = 0; i < skel_Lay::n && i < 32; ++i) {
         s.v[16 + 4 * i] = skel_Lay::size(i);
         s.v[17 + 4 * i] = skel_Lay::align(i);
@@ -453,7 +463,11 @@ __device__ __forceinline__ void publish_agg(skel_u64 *st64, unsigned *fl32, skel
         skel_S sv{a.v};
         const unsigned bits = skel::bit_cast<unsigned>(sv);
         const skel_u64 word = ((skel_u64)bits << 32) | (skel_u64)((epoch << 2) | state);
-        asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(st64 + idx), "l"(word) : "memory");
+        // value, epoch and state travel in ONE 64-bit word, so nothing else has
+        // to be ordered before it: a relaxed store suffices (a release would
+        // cost a GPU-scope fence -- microseconds under streaming load -- on the
+        // consumers' critical path)
+        asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(st64 + idx), "l"(word) : "memory");
     } else {
         if (a.ok) skel::st_value(&vals[idx], skel_S{a.v});
         skel::st_release(&fl32[idx], (epoch << 2) | state);
@@ -498,9 +512,20 @@ __device__ __forceinline__ bool probe_agg(const skel_u64 *st64, const unsigned *
         return true;
     }
 }
+constexpr int AGG_PER = 16;  // status words one prefix-warp lane polls at most
+#ifndef SKEL_SCAN_NPRE
+#define SKEL_SCAN_NPRE 4
+#endif
+constexpr int NPRE = SKEL_SCAN_NPRE;  // slice windows buffered for the consumers
+#ifndef SKEL_SCAN_BACKOFF_MIN
+#define SKEL_SCAN_BACKOFF_MIN 32
+#endif
+#ifndef SKEL_SCAN_BACKOFF_MAX
+#define SKEL_SCAN_BACKOFF_MAX 1024
+#endif
+
 // ordered fold of A(base .. base+cnt-1) by one warp (cnt <= 32*AGG_PER);
 // every lane issues all of its probes before waiting; result in every lane
-constexpr int AGG_PER = 16;
 template <class Tup>
 __device__ __forceinline__ VT warp_fold_aggs(const skel_u64 *st64, const unsigned *fl32, const skel_S *vals,
                                              skel_u64 base, int cnt, unsigned epoch, int lane, Tup &t) {
@@ -509,7 +534,7 @@ __device__ __forceinline__ VT warp_fold_aggs(const skel_u64 *st64, const unsigne
     bool got[AGG_PER];
 #pragma unroll
     for (int k = 0; k < AGG_PER; ++k) got[k] = !(k < per && lane * per + k < cnt);
-    for (unsigned ns = 32;; ns = ns < 1024 ? 2 * ns : ns) {
+    for (unsigned ns = SKEL_SCAN_BACKOFF_MIN;; ns = ns < SKEL_SCAN_BACKOFF_MAX ? 2 * ns : ns) {
         bool all = true;
 #pragma unroll
         for (int k = 0; k < AGG_PER; ++k) {
@@ -530,11 +555,12 @@ __device__ __forceinline__ VT warp_fold_aggs(const skel_u64 *st64, const unsigne
     return vt_shfl_idx(a, 0);
 }
 
+
 // work item q of a CTA's sequence: P1 of slices 0..LAG-1, then per slice s:
 // P1(s+LAG) x CH (if that slice exists), P2(s) x CH.  Returns false past the
 // end.  LAG slices of slack absorb the CTAs' speed differences.
 #ifndef SKEL_SCAN_LAG
-#define SKEL_SCAN_LAG 1
+#define SKEL_SCAN_LAG 2
 #endif
 constexpr int SCAN_LAG = SKEL_SCAN_LAG;
 __device__ __forceinline__ bool scan_item(skel_u64 q, skel_u64 nslices, int &phase, skel_u64 &s, int &j) {
@@ -563,9 +589,24 @@ __device__ __forceinline__ bool scan_item(skel_u64 q, skel_u64 nslices, int &pha
     return true;
 }
 
+#ifdef SKEL_SCAN_TRACE
+// lab instrumentation (tools/scan_lab.cu): globaltimer stamps per (slice, CTA)
+//   0 = P1 aggregate published, 1 = prefix ready, 2 = P2 start, 3 = P2 done,
+//   4 = prefix warp starts the slice
+__device__ skel_u64 skel_scan_trace[6 * 148 * 1024];
+__device__ __forceinline__ void scan_stamp(int ev, skel_u64 s, skel_u64 c) {
+    skel_u64 t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    if (s < 1024 && c < 148) skel_scan_trace[(ev * 1024 + s) * 148 + c] = t;
+}
+#define SKEL_STAMP(ev, s, c) scan_stamp(ev, s, c)
+#else
+#define SKEL_STAMP(ev, s, c)
+#endif
 // consumers = the SRB threads of warps 0..SNW-1; warp SNW is the TMA producer,
-// warp SNW+1 computes the slice prefixes ahead of the consumers
-constexpr int SCAN_THREADS = SRB + 64;
+// warp SNW+1 issues the TMA stores of scanned tiles and hands their stages back,
+// warps SNW+2 .. SNW+1+PW fold the slice windows ahead of the consumers
+constexpr int SCAN_THREADS = SRB + 64 + 32 * PW;
 __device__ __forceinline__ void cons_sync() { asm volatile("bar.sync 1, %0;" ::"n"(SRB) : "memory"); }
 __device__ __forceinline__ void mbar_arrive(skel_u64 *bar) {
     asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(skel::smem_addr(bar)) : "memory");
@@ -631,14 +672,17 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
     // finish advances it (all CTAs have read it by then)
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     __shared__ unsigned s_epoch;
-    __shared__ skel_u64 full_bar[SSTAGES], done_bar[SSTAGES], pre_full[2], pre_empty[2];
+    // full: TMA load landed; empty: stage free (P1: consumers done reading,
+    // P2: the store of its outputs has read it); outs: P2 outputs staged
+    __shared__ skel_u64 full_bar[SSTAGES], empty_bar[SSTAGES], outs_bar[SSTAGES], pre_full[NPRE], pre_empty[NPRE];
     __shared__ VT wsc[2][SNW];  // warp partials, alternated between consecutive tiles
-    __shared__ VT s_tot, s_pre[2];
+    __shared__ VT s_pre[NPRE];
     const int t = threadIdx.x, lane = t & 31, w = t >> 5;
     const skel_u64 G = gridDim.x, c = blockIdx.x;
     const skel_u64 nft = n / STILE;  // full tiles
     const skel_u64 per_slice = G * SCAN_CH;
     const skel_u64 nslices = (nft + per_slice - 1) / per_slice;
+    const skel_u64 rstride = (nslices * G + 63) / 64 * 64;  // status words per copy
     const bool tma = TMA_OK && use_tma;
     unsigned char *stages = aligned_stages(skel_dsmem);
     auto tile_of = [&](skel_u64 s, int j) -> skel_u64 { return (s * G + c) * SCAN_CH + (skel_u64)j; };
@@ -651,9 +695,10 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
     if (t == 0) {
         for (int st = 0; st < SSTAGES; ++st) {
             skel::mbar_init(&full_bar[st], 1);
-            skel::mbar_init(&done_bar[st], SRB);
+            skel::mbar_init(&empty_bar[st], 1);
+            skel::mbar_init(&outs_bar[st], SRB);
         }
-        for (int k = 0; k < 2; ++k) {
+        for (int k = 0; k < NPRE; ++k) {
             skel::mbar_init(&pre_full[k], 1);
             skel::mbar_init(&pre_empty[k], SRB);
         }
@@ -668,30 +713,14 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
         if (tma && lane == 0) {
             const skel_u64 pol_keep = policy_evict_last(), pol_drop = policy_evict_first();
             tma_prefetch_desc(&tin);
-            tma_prefetch_desc(&tout);
-            skel_u64 ring_tile[SSTAGES];
-            int ring_ph[SSTAGES];
             skel_u64 v = 0;
             int ph, j;
             skel_u64 s;
-            auto retire = [&](int st, skel_u64 use) {  // wait until the consumers are done with a stage
-                skel::mbar_wait(&done_bar[st], (unsigned)(use & 1));
-                if (ring_ph[st] == 2) {  // P2: the stage holds outputs
-                    const int row = (int)(ring_tile[st] * SRB);
-                    tma_store_rows_hint(&tout, row, stages + st * STILE_BYTES, pol_drop);
-                    tma_store_rows_hint(&tout, row + SRB / 2, stages + st * STILE_BYTES + STILE_BYTES / 2, pol_drop);
-                    skel::bulk_commit();
-                    skel::bulk_wait_read0();
-                }
-            };
             for (skel_u64 q = 0; scan_item(q, nslices, ph, s, j); ++q) {
                 if (j >= jn(s)) continue;
                 const int st = (int)(v % SSTAGES);
-                if (v >= SSTAGES) retire(st, v / SSTAGES - 1);
-                const skel_u64 tile = tile_of(s, j);
-                ring_tile[st] = tile;
-                ring_ph[st] = ph;
-                const int row = (int)(tile * SRB);
+                if (v >= SSTAGES) skel::mbar_wait(&empty_bar[st], (unsigned)((v / SSTAGES - 1) & 1));
+                const int row = (int)(tile_of(s, j) * SRB);
                 unsigned char *dst = stages + st * STILE_BYTES;
                 const skel_u64 pol = ph == 1 ? pol_keep : pol_drop;
                 skel::mbar_expect_tx(&full_bar[st], STILE_BYTES);
@@ -699,29 +728,64 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
                 tma_load_rows_hint(dst + STILE_BYTES / 2, &tin, row + SRB / 2, &full_bar[st], pol);
                 ++v;
             }
-            const skel_u64 first = v > SSTAGES ? v - SSTAGES : 0;
-            for (skel_u64 u = first; u < v; ++u) retire((int)(u % SSTAGES), u / SSTAGES);
-            skel::bulk_wait0();
         }
         return;
     }
 
     if (w == SNW + 1) {
-        // ================================================ prefix warp
-        // prefix(s, c) = carry(s) (+) A(s,0..c-1), carry(s) = carry(s-1) (+) A(s-1,0..G-1);
-        // slot s&1 of s_pre; one extra round (s = nslices) gives CTA G-1 the carry of the tail
-        VT carry;
-        carry.v = seed ? seed->v : identity.v;
-        carry.ok = true;
-        const skel_u64 rounds = nslices + (c == G - 1 ? 1 : 0);
-        for (skel_u64 s = 0; s < rounds; ++s) {
-            const int slot = (int)(s & 1);
-            if (s >= 2) skel::mbar_wait(&pre_empty[slot], (unsigned)(((s >> 1) - 1) & 1));
-            if (s > 0) carry = comb(carry, warp_fold_aggs(status, flags, aggv, (s - 1) * G, (int)G, epoch, lane, tup), tup);
-            VT p = carry;
-            if (s < nslices) p = comb(carry, warp_fold_aggs(status, flags, aggv, s * G, (int)c, epoch, lane, tup), tup);
+        // ================================================ TMA store warp
+        // stores each scanned tile as soon as its outputs are staged; the
+        // stage goes back to the producer once the store has read it
+        if (tma && lane == 0) {
+            const skel_u64 pol_drop = policy_evict_first();
+            tma_prefetch_desc(&tout);
+            skel_u64 v = 0;
+            unsigned par = 0;  // phase parity of outs_bar[st], one bit per stage
+            int ph, j;
+            skel_u64 s;
+            for (skel_u64 q = 0; scan_item(q, nslices, ph, s, j); ++q) {
+                if (j >= jn(s)) continue;
+                const int st = (int)(v % SSTAGES);
+                ++v;
+                if (ph != 2) continue;
+                skel::mbar_wait(&outs_bar[st], (par >> st) & 1u);
+                par ^= 1u << st;
+                const int row = (int)(tile_of(s, j) * SRB);
+                unsigned char *src = stages + st * STILE_BYTES;
+                tma_store_rows_hint(&tout, row, src, pol_drop);
+                tma_store_rows_hint(&tout, row + SRB / 2, src + STILE_BYTES / 2, pol_drop);
+                skel::bulk_commit();
+                skel::bulk_wait_read0();
+                mbar_arrive(&empty_bar[st]);
+            }
+            skel::bulk_wait0();
+        }
+        return;
+    }
+
+    if (w >= SNW + 2) {
+        // ================================================ window warps
+        // The consumers carry the running prefix from slice to slice: after P2(s-1)
+        // their prefix is p(s-1) (+) A(s-1,c), so
+        //   p(s) = that (+) A(s-1,c+1..G-1) (+) A(s,0..c-1)  =: that (+) W(s),
+        // a window of G-1 consecutive aggregates (W(0) = A(0,0..c-1)).  Windows of
+        // different slices are independent, so PW warps fold them concurrently
+        // (warp k takes s = k, k+PW, ...): an L2 poll takes microseconds while the
+        // SM streams, and one warp folding one window per round trip would pace
+        // the whole grid.  Results go to a ring of NPRE slots the consumers drain.
+        const int k = w - (SNW + 2);
+        for (skel_u64 s = (skel_u64)k; s < nslices; s += PW) {
+            const int slot = (int)(s % NPRE);
+            if (s >= (skel_u64)NPRE) skel::mbar_wait(&pre_empty[slot], (unsigned)((s / NPRE - 1) & 1));
+            if (lane == 0) SKEL_STAMP(4, s, c);
+            const skel_u64 base = s == 0 ? 0 : (s - 1) * G + c + 1;
+            const int cnt = s == 0 ? (int)c : (int)G - 1;
+            VT win;
+            win.ok = false;
+            if (cnt > 0) win = warp_fold_aggs(status + (c % REPL) * rstride, flags, aggv, base, cnt, epoch, lane, tup);
             if (lane == 0) {
-                s_pre[slot] = p;
+                SKEL_STAMP(1, s, c);
+                s_pre[slot] = win;
                 mbar_arrive(&pre_full[slot]);
             }
             __syncwarp();
@@ -734,22 +798,24 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
     VT run1;         // P1 running aggregate of this CTA's sub-chunk (thread 0)
     run1.ok = false;
     VT run;          // P2 running prefix (identical in every consumer thread)
-    run.ok = false;
+    run.v = seed ? seed->v : identity.v;
+    run.ok = true;
     int ph, j;
     skel_u64 s;
     for (skel_u64 q = 0; scan_item(q, nslices, ph, s, j); ++q) {
         const int nj = jn(s);
-        if (ph == 2 && j == 0) {  // the slice prefix, computed ahead by the prefix warp
-            const int slot = (int)(s & 1);
-            skel::mbar_wait(&pre_full[slot], (unsigned)((s >> 1) & 1));
-            run = s_pre[slot];
+        if (ph == 2 && j == 0) {  // p(s) = p(s-1) (+) own A(s-1,c) (+) W(s), W folded ahead
+            const int slot = (int)(s % NPRE);
+            skel::mbar_wait(&pre_full[slot], (unsigned)((s / NPRE) & 1));
+            run = comb(run, s_pre[slot], tup);
             mbar_arrive(&pre_empty[slot]);
+            if (t == 0) SKEL_STAMP(2, s, c);
         }
         if (j >= nj) {
             if (ph == 1 && j == 0 && nj == 0 && t == 0) {  // empty sub-chunk: publish once
                 VT e;
                 e.ok = false;
-                publish_agg(status, flags, aggv, s * G + c, epoch, e);
+                for (int r = 0; r < REPL; ++r) publish_agg(status + r * rstride, flags, aggv, s * G + c, epoch, e);
             }
             continue;
         }
@@ -766,17 +832,19 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
         }
         if (ph == 1) {
             // ---- P1: ordered fold of the tile
-            if (tma) mbar_arrive(&done_bar[st]);  // stage read: free for the producer
             VT a;
             a.v = x[0];
             a.ok = true;
 #pragma unroll
             for (int k = 1; k < K; ++k) a.v = opf(a.v, x[k], tup);
-            const VT tv = cons_fold(a, wsc[v & 1], tup);
+            const VT tv = cons_fold(a, wsc[v & 1], tup);  // its barrier: every row is read
             if (t == 0) {
+                if (tma) mbar_arrive(&empty_bar[st]);  // stage free for the producer
                 run1 = comb(run1, tv, tup);
                 if (j == nj - 1) {
-                    publish_agg(status, flags, aggv, s * G + c, epoch, run1);
+                    SKEL_STAMP(0, s, c);
+                    for (int r = 0; r < REPL; ++r)
+                        publish_agg(status + r * rstride, flags, aggv, s * G + c, epoch, run1);
                     run1.ok = false;
                 }
             }
@@ -797,7 +865,8 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
             if (tma) {
                 write_row(stages + st * STILE_BYTES, t, x);
                 skel::fence_proxy_async();
-                mbar_arrive(&done_bar[st]);  // outputs staged: the producer stores them
+                mbar_arrive(&outs_bar[st]);  // outputs staged: the store warp writes them
+                if (t == 0 && j == nj - 1) SKEL_STAMP(3, s, c);
             } else {
                 skel_T *o = out + tile * STILE + (skel_u64)t * K;
 #pragma unroll
@@ -808,9 +877,7 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
     }
     // ---- ragged last tile and the device total: CTA G-1
     if (c == G - 1) {
-        const int slot = (int)(nslices & 1);
-        skel::mbar_wait(&pre_full[slot], (unsigned)((nslices >> 1) & 1));
-        const VT carry_end = s_pre[slot];
+        const VT carry_end = run;  // p(nslices): CTA G-1 has no later aggregates in its window
         const skel_u64 base = nft * STILE;
         VT mine;
         mine.ok = false;
