@@ -589,13 +589,76 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         g.destroy()
     except skel.SkelError:  # a collective backend that cannot be captured
         ms_graph = ms
+    roof = lmosem_roofline(ctx, skel, rec, evv, timed, world)
     evv.destroy()
     return {"config": "configs[3]/[4]: one subset, 10^6 events, 150x150x280, events block over GPUs",
             "subset_s": ms * 1e-3, "subset_s_graph": ms_graph * 1e-3, "subset_s_fused": ms_fused * 1e-3,
+            "roofline": roof,
             "events_per_s": nev / (min(ms_graph, ms_fused) * 1e-3),
             "note": "includes f all-gather, c zero-fill, Siddon Map, c reduce-scatter and update Zip; "
                     "subset_s = eager calls, subset_s_graph = the same subset replayed as a CUDA graph, "
                     "subset_s_fused = the tail as one peer-memory kernel (skel_zip_combine, NEXT-1)"}
+
+
+def lmosem_roofline(ctx, skel, rec, evv, timed, nd):
+    """Roofline of the error-image Map.  Every voxel visit of a
+    path is one scattered 4-byte request in each walk (a gather of f forward,
+    a red.add into c backward) and the lanes of a warp are on different rays,
+    so the Map is bound by how fast the SMs' L1TEX units can issue scattered
+    requests to L2.  The peaks are measured in the same run by two probe
+    Maps (workloads/probe_*.cu) issuing random scattered gathers / reductions
+    into an image-sized buffer; the Map's ideal time is V/peak_gather +
+    V/peak_red for V voxel visits, counted by a Map over the same events."""
+    from paper_conf_ipps_steuwerkg11_b200.workloads import (LMOSEM_ERROR, LMOSEM_VISITS, PROBE_GATHER,
+                                                            PROBE_K, PROBE_SCATTER_RED, SUM_I32)
+    dims = rec.dims_args
+    nvis = ctx.vector(n=evv.n, dtype=np.int32)
+    if evv.distribution == skel.BLOCK:
+        nvis.set_distribution(skel.BLOCK)
+    ctx.map(LMOSEM_VISITS, evv, nvis, args=dims)
+    visits = int(ctx.reduce(SUM_I32, nvis))  # all ranks' events
+    nvis.destroy()
+    f, c = rec.f, rec.c
+    f.set_distribution(skel.COPY)
+    c.fill_dist(skel.COPY, np.float32(0))
+    ctx.map(LMOSEM_ERROR, evv, None, args=[f, c, *dims])
+    ms_map = timed(lambda: ctx.map(LMOSEM_ERROR, evv, None, args=[f, c, *dims]))
+    c.mark_device_modified()
+    # probes: 2^20 elements x PROBE_K scattered requests each (per GPU), into (a) an
+    # image-sized 25 MB buffer (random lines: L2 hit/miss and far-partition traffic
+    # included) and (b) a small buffer (64 KB gathers: L1-resident; 1 MB reductions:
+    # L2-resident), which isolates the SM's rate of issuing scattered requests
+    npr = 1 << 20
+    idx = ctx.vector(np.arange(npr, dtype=np.uint32))
+    img = ctx.vector(n=rec.nvox, dtype=np.float32)  # whole buffers on every GPU (copy)
+    img.fill_dist(skel.COPY, np.float32(1))
+    acc = ctx.vector(n=rec.nvox, dtype=np.float32)
+    acc.fill_dist(skel.COPY, np.float32(0))
+    gout = ctx.vector(n=npr, dtype=np.float32)
+    probes = {}
+    for tag, ng, nr in (("image", rec.nvox, rec.nvox), ("resident", 1 << 14, 1 << 18)):
+        ng, nr = np.uint32(ng), np.uint32(nr)
+        for _ in range(2):
+            ctx.map(PROBE_GATHER, idx, gout, args=[img, ng])
+            ctx.map(PROBE_SCATTER_RED, idx, None, args=[acc, nr])
+        ms_g = timed(lambda: ctx.map(PROBE_GATHER, idx, gout, args=[img, ng]))
+        ms_r = timed(lambda: ctx.map(PROBE_SCATTER_RED, idx, None, args=[acc, nr]))
+        probes[tag] = (npr * PROBE_K / (ms_g * 1e-3) / 1e9, npr * PROBE_K / (ms_r * 1e-3) / 1e9)
+    for v in (idx, img, acc, gout):
+        v.destroy()
+    peak_g = max(p[0] for p in probes.values())  # G requests/s per GPU
+    peak_r = max(p[1] for p in probes.values())
+    ideal_ms = (visits / nd) / (peak_g * 1e9) * 1e3 + (visits / nd) / (peak_r * 1e9) * 1e3
+    achieved = 2 * visits / nd / (ms_map * 1e-3) / 1e9
+    peak = 2 / (1 / peak_g + 1 / peak_r)
+    return {"kernel": "LM OSEM error-image Map (skel_ew_kernel + lmosem_error)", "bound": "l1tex",
+            "achieved": achieved, "peak": peak, "unit": "G scattered requests/s per GPU",
+            "frac": ideal_ms / ms_map, "map_ms": ms_map, "visits_per_subset": visits,
+            "peak_gather": peak_g, "peak_red": peak_r,
+            "probes_Greq_per_s": {k: {"gather": v[0], "red": v[1]} for k, v in probes.items()},
+            "peak_source": "measured in this run: probe Maps workloads/probe_gather.cu, probe_scatter.cu "
+                           "(random 4-byte gathers / red.add.f32, 32 lanes on 32 lines; best of a 25 MB "
+                           "image-sized buffer and an L1/L2-resident one)"}
 
 
 if __name__ == "__main__":

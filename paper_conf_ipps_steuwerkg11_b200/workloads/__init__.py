@@ -14,6 +14,29 @@ def source(name: str) -> str:
 MANDELBROT = source("mandelbrot")
 LMOSEM_ERROR = source("lmosem_error")
 LMOSEM_UPDATE = source("lmosem_update")
+# voxel visits of one event's path (measurement only: the LM OSEM roofline
+# counts one scattered request per visit in each of the two walks)
+LMOSEM_VISITS = LMOSEM_ERROR + """
+int lmosem_visits(Event e, int nx, int ny, int nz) {
+    Walk w;
+    if (!walk_init(e, nx, ny, nz, w)) return 0;
+    double an0 = w.an[0], an1 = w.an[1], an2 = w.an[2], ac = w.amin;
+    const double aend = w.amax - 1.0e-12;
+    int n = 0;
+    for (int it = 0; it < w.n_steps && ac < aend; ++it) {
+        const double a1 = dmin(dmin(dmin(an0, an1), an2), w.amax);
+        an0 = an0 == a1 ? an0 + w.da[0] : an0;
+        an1 = an1 == a1 ? an1 + w.da[1] : an1;
+        an2 = an2 == a1 ? an2 + w.da[2] : an2;
+        ac = a1;
+        ++n;
+    }
+    return n;
+}
+"""
+PROBE_SCATTER_RED = source("probe_scatter")
+PROBE_GATHER = source("probe_gather")
+PROBE_K = 64
 
 # Listing 1 (P:L198-201), verbatim
 SUM_F32 = "float sum (float x,float y){return x+y;}"

@@ -1,5 +1,5 @@
 """The LM OSEM customizing function (workloads/lmosem_error.cu) is plain C++
-apart from atomicAdd/__ldg; compiled for the host with three one-line shims
+apart from atomicAdd/__ldg/float4; compiled for the host with a few one-line shims
 it can be checked against the oracle on the CPU (tiny grids with exact
 plane/edge/corner ties, and the paper-sized volume).  This tests the walk's
 logic only; the GPU parity tests run the same text through NVRTC."""
@@ -20,6 +20,8 @@ SHIM = r'''
 using std::min; using std::max; using std::fmin; using std::fmax;
 #define __forceinline__ inline
 template <class T> static T __ldg(const T* p) { return *p; }
+struct float4 { float x, y, z, w; };
+static inline float4 make_float4(float a, float b, float c, float d) { return float4{a, b, c, d}; }
 #include "SRC"
 extern "C" void run(const float* ev, int n, const float* f, float* c, int nx, int ny, int nz) {
     for (int i = 0; i < n; ++i) {
