@@ -41,6 +41,15 @@ struct Module {
     cudaKernel_t k_zipcomb = nullptr;  // Zip modules: fused combine + zip + broadcast
     uint64_t sig[16 + 4 * 32] = {0};
     std::set<int> attr_set_on;  // devices on which smem attributes were set
+    // element-wise grid policy per size class (log2 of the chunk count), chosen
+    // by measurement: 0 = UNROLL chunks in flight per thread (bandwidth-bound
+    // user functions), 1 = one chunk per thread (compute-bound, divergent ones)
+    struct EwTune {
+        int trial = 0;   // launches timed so far (policies alternate 0,1,0,1)
+        int best = -1;   // decided policy, -1 while measuring
+        cudaEvent_t ev[8] = {};
+    };
+    std::map<int, EwTune> ew_tune;
 };
 
 // signature accessors (layout documented in map.cuh / red.cuh)

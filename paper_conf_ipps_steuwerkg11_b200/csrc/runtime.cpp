@@ -636,12 +636,27 @@ int prepare_output(skel_vec_s *out, size_t n, skel_dist dist, bool same_as_input
     return SKEL_OK;
 }
 
-int ew_grid(const Slot &s, size_t chunks, int block) {
+// grid of the element-wise kernels: one chunk per thread, or -- when the kernel
+// keeps `per_thread` chunks in flight per thread (vectorised path) -- just
+// enough threads to give each of them that many, but never less than one full
+// resident wave while there is work for it; capped at `waves` resident waves
+// (a grid-stride loop covers the rest)
+int ew_grid(const Slot &s, size_t chunks, int block, int per_thread = 1) {
     static const int waves = [] {
         const char *e = getenv("SKEL_EW_WAVES");  // tuning hook: grid = SMs x (2048/block) x waves
         return e ? std::max(1, atoi(e)) : 32;
     }();
+    static const int pt_env = [] {
+        const char *e = getenv("SKEL_EW_PER_THREAD");  // tuning hook: chunks per thread for the sizing
+        return e ? atoi(e) : 0;
+    }();
+    if (pt_env > 0 && per_thread > 1) per_thread = std::min(per_thread, pt_env);
     size_t g = (chunks + block - 1) / block;
+    if (per_thread > 1) {
+        const size_t resident = (size_t)s.sms * (2048 / block);
+        const size_t gu = (chunks + (size_t)block * per_thread - 1) / ((size_t)block * per_thread);
+        g = std::max(gu, std::min(g, resident));
+    }
     const size_t cap = (size_t)s.sms * (2048 / block) * waves;
     g = std::min(g, cap);
     return (int)std::max<size_t>(g, 1);
@@ -682,10 +697,40 @@ int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_
         int vec_ok = al16(pa) && (!pb || al16(pb)) && (!po || al16(po));
         pack_args(m, args, nargs, li, abuf);
         const size_t chunks = vec_ok ? std::max<uint64_t>(cnt / E, 1) : cnt;
-        const int grid = ew_grid(s, chunks, block);
-        void *params[] = {&pa, &pb, &po, &cnt, &vec_ok, abuf.data()};
+        const int unroll = std::max<int>(1, (int)m->sig[10]);
         DevGuard g(s.dev);
+        // grid policy (Module::EwTune): the first launches of a size class time
+        // both policies alternately on the first device; later ones use the faster
+        Module::EwTune *tu = nullptr;
+        int policy = 0, tslot = -1;
+        if (vec_ok && E > 1 && unroll > 1) {
+            tu = &m->ew_tune[64 - __builtin_clzll((unsigned long long)chunks)];
+            cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
+            cudaStreamIsCapturing(s.stream, &cs);
+            if (tu->best < 0 && li == 0 && cs == cudaStreamCaptureStatusNone) {
+                if (tu->trial == 4) {  // all four samples recorded: decide (one wait, once per class)
+                    CK(ctx, cudaEventSynchronize(tu->ev[7]));
+                    float t[4] = {0, 0, 0, 0};
+                    for (int k = 0; k < 4; ++k) CK(ctx, cudaEventElapsedTime(&t[k], tu->ev[2 * k], tu->ev[2 * k + 1]));
+                    tu->best = std::min(t[1], t[3]) < 0.97f * std::min(t[0], t[2]) ? 1 : 0;
+                    for (cudaEvent_t &e : tu->ev) {
+                        cudaEventDestroy(e);
+                        e = nullptr;
+                    }
+                } else {
+                    tslot = tu->trial++;
+                    policy = tslot & 1;
+                    for (int k = 0; k < 2; ++k)
+                        if (!tu->ev[2 * tslot + k]) CK(ctx, cudaEventCreate(&tu->ev[2 * tslot + k]));
+                }
+            }
+            if (tu->best >= 0) policy = tu->best;
+        }
+        const int grid = ew_grid(s, chunks, block, policy == 0 && vec_ok && E > 1 ? unroll : 1);
+        void *params[] = {&pa, &pb, &po, &cnt, &vec_ok, abuf.data()};
+        if (tslot >= 0) CK(ctx, cudaEventRecord(tu->ev[2 * tslot], s.stream));
         CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+        if (tslot >= 0) CK(ctx, cudaEventRecord(tu->ev[2 * tslot + 1], s.stream));
         ctx->stats.kernel_launches++;
     }
     if (rsz != 0) {
@@ -848,16 +893,16 @@ int set_smem_attr(skel_ctx_s *ctx, Module *m, const Slot &s) {
     return SKEL_OK;
 }
 
-// local reduce of the slot's data into ws[o_res]
+// local reduce of the slot's data into dst
 int launch_reduce(skel_ctx_s *ctx, Module *m, Slot &s, const void *in, uint64_t cnt, const RedLayout &L,
-                  std::vector<unsigned char> &abuf) {
+                  std::vector<unsigned char> &abuf, void *dst) {
     const uint64_t TILE = m->sig[10];
     const uint64_t nft = cnt / TILE;
     const size_t G = (size_t)std::max<uint64_t>(1, std::min<uint64_t>((uint64_t)s.sms, nft));
     CUtensorMap tin;
     int use_tma = m->sig[5] && make_tmap(&tin, in, nft * m->sig[9]);
     char *ws = s.ws;
-    void *partials = ws + L.o_part, *pvalid = ws + L.o_pvalid, *result = ws + L.o_res;
+    void *partials = ws + L.o_part, *pvalid = ws + L.o_pvalid, *result = dst;
     unsigned *counter = s.counters + 2;
     void *params[] = {&tin, &in, &cnt, &use_tma, &partials, &pvalid, &counter, &result, abuf.data()};
     DevGuard g(s.dev);
@@ -872,9 +917,10 @@ size_t red_grid(const Module *m, const Slot &s, uint64_t cnt) {
 }
 
 // Reduce of `in` leaving the result in every local slot's ws[o_fold]
-// (cross-device: gather of the D partials + ordered fold)
+// (cross-device: gather of the D partials + ordered fold), or --
+// one local device and `direct` given -- written by the kernel straight to `direct`
 int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args, int nargs,
-                std::vector<RedLayout> &Ls) {
+                std::vector<RedLayout> &Ls, void *direct = nullptr) {
     const int D = ctx->D;
     const bool cross = D > 1 && in->dist == SKEL_BLOCK;
     std::vector<unsigned char> abuf;
@@ -886,7 +932,8 @@ int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args
         TRY(ensure_ws(ctx, s, Ls[li].total));
         TRY(set_smem_attr(ctx, m, s));
         pack_args(m, args, nargs, li, abuf);
-        if (cnt) TRY(launch_reduce(ctx, m, s, in->bufs[li].ptr(in->es), cnt, Ls[li], abuf));
+        char *dst = cross ? s.ws + Ls[li].o_res : (direct && D == 1 ? static_cast<char *>(direct) : s.ws + Ls[li].o_fold);
+        if (cnt) TRY(launch_reduce(ctx, m, s, in->bufs[li].ptr(in->es), cnt, Ls[li], abuf, dst));
     }
     const size_t es = m->sig[4];
     const size_t ps = part_size(in->n, D);
@@ -920,8 +967,6 @@ int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args
             void *params[] = {&vals, &k, &outp, abuf.data()};
             CK(ctx, cudaLaunchKernel((const void *)m->k_fold, dim3(1), dim3(32), params, 0, s.stream));
             ctx->stats.kernel_launches++;
-        } else if (in->bufs[li].count) {
-            CK(ctx, cudaMemcpyAsync(s.ws + L.o_fold, s.ws + L.o_res, es, cudaMemcpyDeviceToDevice, s.stream));
         }
     }
     return SKEL_OK;
@@ -1092,8 +1137,12 @@ int skel_finalize(skel_ctx_t ctx) {
     sync_all(ctx);
     std::vector<skel_vec_s *> vs(ctx->vecs.begin(), ctx->vecs.end());
     for (auto *v : vs) skel_vector_destroy(v);
-    for (auto &kv : ctx->modules)
+    for (auto &kv : ctx->modules) {
         if (kv.second->lib) cudaLibraryUnload(kv.second->lib);
+        for (auto &t : kv.second->ew_tune)
+            for (cudaEvent_t e : t.second.ev)
+                if (e) cudaEventDestroy(e);
+    }
     if (ctx->comm) ncclCommDestroy(ctx->comm);
     for (auto &s : ctx->slots) {
         DevGuard g(s.dev);
@@ -1147,8 +1196,12 @@ int skel_set_cache_dir(skel_ctx_t ctx, const char *dir) {
 int skel_clear_kernel_cache(skel_ctx_t ctx) {
     if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
     TRY(sync_all(ctx));
-    for (auto &kv : ctx->modules)
+    for (auto &kv : ctx->modules) {
         if (kv.second->lib) cudaLibraryUnload(kv.second->lib);
+        for (auto &t : kv.second->ew_tune)
+            for (cudaEvent_t e : t.second.ev)
+                if (e) cudaEventDestroy(e);
+    }
     ctx->modules.clear();
     ctx->fast_modules.clear();
     return SKEL_OK;
@@ -1516,9 +1569,6 @@ int skel_reduce_to(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t re
     if (result->es != in->es) return fail(ctx, SKEL_ERR_TYPE, "result element size != input element size");
     TRY(check_args(ctx, m, args, nargs));
     TRY(ensure_device(in));
-    std::vector<RedLayout> Ls;
-    TRY(reduce_core(ctx, m, in, args, nargs, Ls));
-    TRY(finish_scalar(ctx, in, Ls));
     // the result is a 1-element vector with a copy on every local device
     if (result->n != 1) {
         result->n = 1;
@@ -1529,11 +1579,19 @@ int skel_reduce_to(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t re
     }
     result->dist = SKEL_COPY;
     TRY(place(result, SKEL_COPY));
-    for (size_t li = 0; li < ctx->slots.size(); ++li) {
-        Slot &s = ctx->slots[li];
-        DevGuard g(s.dev);
-        CK(ctx, cudaMemcpyAsync(result->bufs[li].ptr(result->es), s.ws + Ls[li].o_fold, in->es,
-                                cudaMemcpyDeviceToDevice, s.stream));
+    std::vector<RedLayout> Ls;
+    if (ctx->D == 1) {
+        // one device: the Reduce kernel writes the result element itself
+        TRY(reduce_core(ctx, m, in, args, nargs, Ls, result->bufs[0].ptr(result->es)));
+    } else {
+        TRY(reduce_core(ctx, m, in, args, nargs, Ls));
+        TRY(finish_scalar(ctx, in, Ls));
+        for (size_t li = 0; li < ctx->slots.size(); ++li) {
+            Slot &s = ctx->slots[li];
+            DevGuard g(s.dev);
+            CK(ctx, cudaMemcpyAsync(result->bufs[li].ptr(result->es), s.ws + Ls[li].o_fold, in->es,
+                                    cudaMemcpyDeviceToDevice, s.stream));
+        }
     }
     result->dev_valid = true;
     device_wrote(result);

@@ -61,7 +61,7 @@ constexpr int SKEL_E = skel_vec_ok ? (SKEL_ITEMS < (int)(16 / skel_maxsz) ? SKEL
 // ---- signature table, read back by the host once per loaded module ------
 // [0] layout version  [1] NIN  [2] arity  [3] sizeof ret (0 = void)
 // [4] sizeof a  [5] sizeof b  [6] #extra args  [7] arg buffer bytes
-// [8] E (elements per chunk)  [9] block  [10..15] reserved
+// [8] E (elements per chunk)  [9] block  [10] chunks in flight per thread  [11..15] reserved
 // [16 + 4i ..] extra arg i: size, align, is_pointer, offset
 struct skel_sig_t { skel_u64 v[16 + 4 * 32]; };
 constexpr skel_sig_t skel_make_sig() {
@@ -76,6 +76,7 @@ constexpr skel_sig_t skel_make_sig() {
     s.v[7] = SKEL_ARGBYTES;
     s.v[8] = SKEL_E;
     s.v[9] = SKEL_BLOCK;
+    s.v[10] = SKEL_UNROLL;
     for (int i = 0; i < skel_Lay::n && i < 32; ++i) {
         s.v[16 + 4 * i] = skel_Lay::size(i);
         s.v[17 + 4 * i] = skel_Lay::align(i);
