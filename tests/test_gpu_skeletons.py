@@ -365,3 +365,24 @@ def test_double_reduce_scan(ctx, n):
     want = oracle.skel_scan(src, x, 0.0)  # left-to-right float64 prefix
     got = out.download()
     assert np.all(np.abs(got - want) <= 1e-12 * np.concatenate([[0], np.cumsum(np.abs(x))[:-1]]) + 1e-300)
+
+
+@pytest.mark.parametrize("n", [(1 << 22) + 5, 1 << 24])
+def test_map_zip_grid_policy_trials_bit_identical(n):
+    """The element-wise grid policy is chosen per module and size class by timing
+    both candidates on the first launches (K1/K2): every launch --
+    trials of either policy and the decided one -- must give the same bits."""
+    with skel.Context(1) as c:
+        x, y = si.uniform_f32(n, 11), si.uniform_f32(n, 12)
+        vx, vy = c.vector(x), c.vector(y)
+        want_m = oracle.skel_map(MAP_F32, x, np.float32)
+        want_z = oracle.skel_zip(SAXPY_F32, x, y, np.float32, args=[np.float32(2.5)])
+        for _ in range(7):
+            vm = c.vector(n=n, dtype=np.float32)
+            vz = c.vector(n=n, dtype=np.float32)
+            c.map(MAP_F32, vx, vm)
+            c.zip(SAXPY_F32, vx, vy, vz, args=[np.float32(2.5)])
+            assert np.array_equal(vm.download(), want_m)
+            assert np.array_equal(vz.download(), want_z)
+            vm.destroy()
+            vz.destroy()
