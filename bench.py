@@ -617,18 +617,22 @@ def lmosem_roofline(ctx, skel, rec, evv, timed, nd):
     path is one scattered 4-byte request in each walk (a gather of f forward,
     a red.add into c backward) and the lanes of a warp are on different rays,
     so the Map is bound by how fast the SMs' L1TEX units can issue scattered
-    requests to L2.  The peaks are measured in the same run by two probe
-    Maps (workloads/probe_*.cu) issuing random scattered gathers / reductions
-    into an image-sized buffer; the Map's ideal time is V/peak_gather +
-    V/peak_red for V voxel visits, counted by a Map over the same events."""
-    from paper_conf_ipps_steuwerkg11_b200.workloads import (LMOSEM_ERROR, LMOSEM_VISITS, PROBE_GATHER,
-                                                            PROBE_K, PROBE_SCATTER_RED, SUM_I32)
+    requests to L2.  The peaks are measured in the same run by probe Maps
+    (workloads/probe_*.cu) issuing random scattered gathers / scalar and
+    vector reductions; the Map's ideal time is V/peak_gather + R/peak_red_v4
+    for V voxel visits and R vector reductions (4-float groups entered),
+    both counted by Maps over the same events."""
+    from paper_conf_ipps_steuwerkg11_b200.workloads import (LMOSEM_ERROR, LMOSEM_GROUPS, LMOSEM_VISITS,
+                                                            PROBE_GATHER, PROBE_K, PROBE_SCATTER_RED,
+                                                            PROBE_SCATTER_RED4, SUM_I32)
     dims = rec.dims_args
     nvis = ctx.vector(n=evv.n, dtype=np.int32)
     if evv.distribution == skel.BLOCK:
         nvis.set_distribution(skel.BLOCK)
     ctx.map(LMOSEM_VISITS, evv, nvis, args=dims)
     visits = int(ctx.reduce(SUM_I32, nvis))  # all ranks' events
+    ctx.map(LMOSEM_GROUPS, evv, nvis, args=dims)
+    groups = int(ctx.reduce(SUM_I32, nvis))  # vector reductions of the back projection
     nvis.destroy()
     f, c = rec.f, rec.c
     f.set_distribution(skel.COPY)
@@ -653,24 +657,31 @@ def lmosem_roofline(ctx, skel, rec, evv, timed, nd):
         for _ in range(2):
             ctx.map(PROBE_GATHER, idx, gout, args=[img, ng])
             ctx.map(PROBE_SCATTER_RED, idx, None, args=[acc, nr])
+            ctx.map(PROBE_SCATTER_RED4, idx, None, args=[acc, nr])
         ms_g = timed(lambda: ctx.map(PROBE_GATHER, idx, gout, args=[img, ng]))
         ms_r = timed(lambda: ctx.map(PROBE_SCATTER_RED, idx, None, args=[acc, nr]))
-        probes[tag] = (npr * PROBE_K / (ms_g * 1e-3) / 1e9, npr * PROBE_K / (ms_r * 1e-3) / 1e9)
+        ms_r4 = timed(lambda: ctx.map(PROBE_SCATTER_RED4, idx, None, args=[acc, nr]))
+        probes[tag] = tuple(npr * PROBE_K / (t * 1e-3) / 1e9 for t in (ms_g, ms_r, ms_r4))
     for v in (idx, img, acc, gout):
         v.destroy()
     peak_g = max(p[0] for p in probes.values())  # G requests/s per GPU
     peak_r = max(p[1] for p in probes.values())
-    ideal_ms = (visits / nd) / (peak_g * 1e9) * 1e3 + (visits / nd) / (peak_r * 1e9) * 1e3
-    achieved = 2 * visits / nd / (ms_map * 1e-3) / 1e9
-    peak = 2 / (1 / peak_g + 1 / peak_r)
+    peak_r4 = max(p[2] for p in probes.values())
+    # requests of the Map: one gather per visit (forward), one vector reduction per
+    # 4-float group entered (back projection); ideal = each at its measured peak
+    reqs = (visits + groups) / nd
+    ideal_ms = (visits / nd) / (peak_g * 1e9) * 1e3 + (groups / nd) / (peak_r4 * 1e9) * 1e3
+    achieved = reqs / (ms_map * 1e-3) / 1e9
+    peak = reqs / (ideal_ms * 1e-3) / 1e9
     return {"kernel": "LM OSEM error-image Map (skel_ew_kernel + lmosem_error)", "bound": "l1tex",
             "achieved": achieved, "peak": peak, "unit": "G scattered requests/s per GPU",
-            "frac": ideal_ms / ms_map, "map_ms": ms_map, "visits_per_subset": visits,
-            "peak_gather": peak_g, "peak_red": peak_r,
-            "probes_Greq_per_s": {k: {"gather": v[0], "red": v[1]} for k, v in probes.items()},
-            "peak_source": "measured in this run: probe Maps workloads/probe_gather.cu, probe_scatter.cu "
-                           "(random 4-byte gathers / red.add.f32, 32 lanes on 32 lines; best of a 25 MB "
-                           "image-sized buffer and an L1/L2-resident one)"}
+            "frac": ideal_ms / ms_map, "map_ms": ms_map, "ideal_ms": ideal_ms, "visits_per_subset": visits,
+            "vector_reductions_per_subset": groups, "peak_gather": peak_g, "peak_red_v4": peak_r4,
+            "peak_red": peak_r,
+            "probes_Greq_per_s": {k: {"gather": v[0], "red": v[1], "red_v4": v[2]} for k, v in probes.items()},
+            "peak_source": "measured in this run: probe Maps workloads/probe_gather.cu, probe_scatter.cu, "
+                           "probe_scatter4.cu (random 4-byte gathers / red.add.f32 / red.add.v4.f32, 32 lanes on "
+                           "32 lines; best of a 25 MB image-sized buffer and an L1/L2-resident one)"}
 
 
 if __name__ == "__main__":
