@@ -168,6 +168,20 @@ int skel_vector_fill(skel_vec_t v, const void *value);
  * LM OSEM, reading R10(i)). */
 int skel_vector_fill_dist(skel_vec_t v, skel_dist dist, const void *value);
 int skel_vector_set_distribution(skel_vec_t v, skel_dist dist, skel_combine combine);
+/* set_distribution_fn: leave SKEL_COPY with a
+ * USER-DEFINED element-wise combine instead of the built-in ones.  combine_src
+ * is source text of an associative function  T f(T x, T y)  (the last
+ * top-level function, as for the skeletons; sizeof(T) = the element size, no
+ * further parameters).  The D copies are folded in device order,
+ *   result[i] = f(...f(f(copy_0[i], copy_1[i]), copy_2[i])..., copy_{D-1}[i]),
+ * so f need not be commutative (P:L283-288 asks only associativity of a
+ * customizing operator).  dist = BLOCK: device k folds part k of every copy
+ * (peer reads; one process per GPU: part k of every rank is gathered on rank
+ * k over NCCL first); SINGLE: device 0 folds the whole copies; COPY: BLOCK then
+ * all-gather.  Works on any element type (no dtype needed).
+ * Errors: SKEL_ERR_STATE if the vector is not SKEL_COPY; SKEL_ERR_TYPE if f
+ * is not T f(T, T) for this element size; SKEL_ERR_COMPILE with the NVRTC log. */
+int skel_vector_set_distribution_fn(skel_vec_t v, skel_dist dist, const char *combine_src);
 int skel_vector_get_distribution(skel_vec_t v, skel_dist *dist);
 int skel_vector_mark_device_modified(skel_vec_t v);
 /* Range [lo, hi) of the vector held by logical device d under the current

@@ -57,17 +57,21 @@ def redistribute(parts: list, src: str, dst: str, combine: str | None = None) ->
     """Change the distribution of a vector held as `parts` from src to dst.
 
     combine = "add" merges the D copies element-wise (Listing 4)
-    and is only meaningful from `copy`.
+    and is only meaningful from `copy`; a callable f(acc, x) is a user-defined
+    element-wise combine, folded over the copies in device order.
     """
     D = len(parts)
-    if combine not in (None, "add"):
+    if combine is not None and combine != "add" and not callable(combine):
         raise ValueError(combine)
-    if combine == "add" and src != COPY:
+    if combine is not None and src != COPY:
         raise ValueError("a combine merges per-device copies: source must be copy")
-    if src == COPY and combine == "add":
+    if src == COPY and combine is not None:
+        # element-wise, folded over the copies in device order (a callable is a
+        # user combine f(acc, x) applied to whole arrays, NEXT-2)
+        f = (lambda a, b: a + b) if combine == "add" else combine
         total = parts[0].copy()
         for d in range(1, D):
-            total = total + parts[d]
+            total = f(total, parts[d])
         return distribute(total, dst, D)
     if src == COPY and dst == BLOCK:
         # each device keeps its own slice of its own copy (no data exchange)

@@ -581,6 +581,130 @@ int set_distribution(skel_vec_s *v, skel_dist dist, skel_combine combine) {
     return SKEL_OK;
 }
 
+// ---- user-defined combine ---------------------------------
+// The paper's combine is "element-wise add"; here any associative
+// user function T f(T, T) given as source text (an NVRTC-built Zip module) merges
+// the copies element-wise, folded in device order 0..D-1 (non-commutative f ok).
+
+int ew_grid(const Slot &s, size_t chunks, int block, int per_thread = 1);
+int ensure_ws(skel_ctx_s *ctx, Slot &s, size_t bytes);
+
+// one Zip launch out[i] = f(a[i], b[i]) on raw device pointers (out may alias a or b)
+int zip_raw(skel_ctx_s *ctx, Module *m, Slot &s, const void *pa, const void *pb, void *po, uint64_t cnt) {
+    if (!cnt) return SKEL_OK;
+    std::vector<unsigned char> abuf(std::max<uint64_t>(m->sig[7], 16), 0);
+    const int block = (int)m->sig[9];
+    const uint64_t E = m->sig[8];
+    int vec_ok = al16(pa) && al16(pb) && al16(po);
+    const size_t chunks = vec_ok ? std::max<uint64_t>(cnt / E, 1) : cnt;
+    const int grid = ew_grid(s, chunks, block, vec_ok && E > 1 ? std::max<int>(1, (int)m->sig[10]) : 1);
+    void *params[] = {&pa, &pb, &po, &cnt, &vec_ok, abuf.data()};
+    DevGuard g(s.dev);
+    CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+    ctx->stats.kernel_launches++;
+    return SKEL_OK;
+}
+
+// dst = f(...f(f(src[0], src[1]), src[2])..., src[D-1]) over cnt elements on slot s
+int fold_raw(skel_ctx_s *ctx, Module *m, Slot &s, const std::vector<const char *> &src, char *dst, uint64_t cnt) {
+    TRY(zip_raw(ctx, m, s, src[0], src[1], dst, cnt));
+    for (size_t j = 2; j < src.size(); ++j) TRY(zip_raw(ctx, m, s, dst, src[j], dst, cnt));
+    return SKEL_OK;
+}
+
+int set_distribution_fn(skel_vec_s *v, skel_dist dist, const char *src) {
+    skel_ctx_s *ctx = v->ctx;
+    if (v->dist != SKEL_COPY) return fail(ctx, SKEL_ERR_STATE, "a combine merges per-device copies: the vector must be SKEL_COPY");
+    Module *m = nullptr;
+    TRY(get_module(ctx, Kind::Zip, src, &m));
+    if (m->sig[6] != 0) return fail(ctx, SKEL_ERR_TYPE, "a combine function takes exactly two parameters");
+    if (m->sig[3] != v->es || m->sig[4] != v->es || m->sig[5] != v->es)
+        return fail(ctx, SKEL_ERR_TYPE, "combine function must have the form T f(T, T) with sizeof(T) = element size");
+    TRY(ensure_device(v));
+    const int D = ctx->D;
+    const size_t es = v->es, n = v->n;
+    if (D == 1) {  // one copy: nothing to merge
+        Buf &b = v->bufs[0];
+        b.off = 0;
+        b.count = n;
+    } else if (!ctx->rank_mode) {
+        auto &S = ctx->slots;
+        auto &B = v->bufs;
+        TRY(join(ctx));
+        if (dist == SKEL_SINGLE) {
+            std::vector<const char *> srcs(D);
+            for (int j = 0; j < D; ++j) srcs[j] = B[j].base;
+            TRY(fold_raw(ctx, m, S[0], srcs, B[0].base, n));
+            ctx->stats.d2d_bytes += (D - 1) * n * es;
+            TRY(join(ctx));
+            for (int d = 1; d < D; ++d) B[d].count = 0;
+            B[0].off = 0;
+            B[0].count = n;
+        } else {
+            // device d merges part d of every copy into part d of its own copy; for
+            // d >= 2 its own copy is a later operand of the fold, so the fold runs in
+            // the slot's workspace and is copied over afterwards
+            for (int d = 0; d < D; ++d) {
+                const size_t lo = part_lo(v, d), cnt = want_count(v, SKEL_BLOCK, d);
+                if (!cnt) continue;
+                std::vector<const char *> srcs(D);
+                for (int j = 0; j < D; ++j) srcs[j] = B[j].base + lo * es;
+                char *own = B[d].base + lo * es;
+                if (d < 2) {
+                    TRY(fold_raw(ctx, m, S[d], srcs, own, cnt));
+                } else {
+                    TRY(ensure_ws(ctx, S[d], cnt * es + 256));
+                    TRY(fold_raw(ctx, m, S[d], srcs, S[d].ws, cnt));
+                    DevGuard g(S[d].dev);
+                    CK(ctx, cudaMemcpyAsync(own, S[d].ws, cnt * es, cudaMemcpyDeviceToDevice, S[d].stream));
+                }
+                ctx->stats.d2d_bytes += (D - 1) * cnt * es;
+            }
+            TRY(join(ctx));
+            for (int d = 0; d < D; ++d) {
+                B[d].off = part_lo(v, d);
+                B[d].count = want_count(v, SKEL_BLOCK, d);
+            }
+            if (dist == SKEL_COPY) TRY(xchg_local(v, SKEL_XCHG_ALLGATHER, SKEL_COMBINE_NONE));
+        }
+    } else {
+        // one process per GPU: every rank's part r of its copy is gathered on rank r
+        // (D gathers, one per root), then folded there in rank order
+        Slot &s = ctx->slots[0];
+        Buf &b = v->bufs[0];
+        const int r = ctx->rank;
+        const size_t ps = part_size(n, D);
+        const size_t piece = dist == SKEL_SINGLE ? n : ps;
+        TRY(ensure_ws(ctx, s, (size_t)D * piece * es + 256));
+        char *stage = s.ws;
+        DevGuard g(s.dev);
+        if (dist == SKEL_SINGLE) {
+            NK(ctx, ncclGather(b.base, stage, n * es, ncclUint8, 0, ctx->comm, s.stream));
+            ctx->stats.nccl_bytes += n * es;
+        } else {
+            for (int j = 0; j < D; ++j) {
+                NK(ctx, ncclGather(b.base + (size_t)j * ps * es, stage, ps * es, ncclUint8, j, ctx->comm, s.stream));
+                ctx->stats.nccl_bytes += ps * es;
+            }
+        }
+        const size_t lo = dist == SKEL_SINGLE ? 0 : part_lo(v, r);
+        const size_t cnt = dist == SKEL_SINGLE ? (r == 0 ? n : 0) : want_count(v, SKEL_BLOCK, r);
+        if (cnt) {
+            std::vector<const char *> srcs(D);
+            for (int j = 0; j < D; ++j) srcs[j] = stage + (size_t)j * piece * es;
+            TRY(fold_raw(ctx, m, s, srcs, b.base + lo * es, cnt));
+        }
+        b.off = lo;
+        b.count = cnt;
+        if (dist == SKEL_COPY) TRY(xchg_rank(v, SKEL_XCHG_ALLGATHER, SKEL_COMBINE_NONE));
+    }
+    v->dist = dist;
+    v->dev_valid = true;
+    device_wrote(v);
+    v->diverged = false;
+    return SKEL_OK;
+}
+
 // ---- Arguments (§III-C) ------------------------------------------------------
 int check_args(skel_ctx_s *ctx, const Module *m, const skel_arg *args, int nargs) {
     const int want = (int)m->sig[6];
@@ -641,7 +765,7 @@ int prepare_output(skel_vec_s *out, size_t n, skel_dist dist, bool same_as_input
 // enough threads to give each of them that many, but never less than one full
 // resident wave while there is work for it; capped at `waves` resident waves
 // (a grid-stride loop covers the rest)
-int ew_grid(const Slot &s, size_t chunks, int block, int per_thread = 1) {
+int ew_grid(const Slot &s, size_t chunks, int block, int per_thread) {
     static const int waves = [] {
         const char *e = getenv("SKEL_EW_WAVES");  // tuning hook: grid = SMs x (2048/block) x waves
         return e ? std::max(1, atoi(e)) : 32;
@@ -1393,6 +1517,12 @@ int skel_vector_set_distribution(skel_vec_t v, skel_dist dist, skel_combine comb
     if ((int)dist < 0 || (int)dist > 2 || (int)combine < 0 || (int)combine > 4)
         return fail(v->ctx, SKEL_ERR_ARG, "bad distribution or combine");
     return set_distribution(v, dist, combine);
+}
+
+int skel_vector_set_distribution_fn(skel_vec_t v, skel_dist dist, const char *combine_src) {
+    if (!v || !combine_src) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad arguments");
+    if ((int)dist < 0 || (int)dist > 2) return fail(v->ctx, SKEL_ERR_ARG, "bad distribution");
+    return set_distribution_fn(v, dist, combine_src);
 }
 
 int skel_vector_get_distribution(skel_vec_t v, skel_dist *dist) {

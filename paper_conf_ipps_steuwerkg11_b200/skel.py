@@ -80,6 +80,7 @@ def lib() -> ctypes.CDLL:
             "skel_vector_download": [P, P, S], "skel_vector_upload_part": [P, S, P, S], "skel_vector_host_ptr": [P, PP],
             "skel_vector_mark_host_modified": [P], "skel_vector_fill": [P, P], "skel_vector_fill_dist": [P, I, P],
             "skel_vector_set_distribution": [P, I, I], "skel_vector_get_distribution": [P, ctypes.POINTER(I)],
+            "skel_vector_set_distribution_fn": [P, I, ctypes.c_char_p],
             "skel_vector_mark_device_modified": [P],
             "skel_vector_part": [P, I, ctypes.POINTER(S), ctypes.POINTER(S)],
             "skel_vector_device_ptr": [P, I, PP, ctypes.POINTER(S)],
@@ -390,8 +391,13 @@ class Vector:
         _check(lib().skel_vector_fill_dist(self._h, dist, b.ctypes.data), self.ctx._h)
         return self
 
-    def set_distribution(self, dist: int, combine: int = COMBINE_NONE):
-        _check(lib().skel_vector_set_distribution(self._h, dist, combine), self.ctx._h)
+    def set_distribution(self, dist: int, combine: "int | str" = COMBINE_NONE):
+        """combine: a built-in skel_combine, or source text of a user function
+        T f(T, T) (skel_vector_set_distribution_fn, NEXT-2)."""
+        if isinstance(combine, str):
+            _check(lib().skel_vector_set_distribution_fn(self._h, dist, combine.encode()), self.ctx._h)
+        else:
+            _check(lib().skel_vector_set_distribution(self._h, dist, combine), self.ctx._h)
         return self
 
     @property

@@ -238,3 +238,97 @@ def test_more_devices_than_elements():
         v.set_distribution(skel.COPY)
         v.set_distribution(skel.SINGLE)
         assert v.download().tolist() == [0, 1, 2]
+
+
+# NEXT-2: user-defined combine functions (skel_vector_set_distribution_fn)
+MAX_I32 = "int mx(int a, int b){ return a > b ? a : b; }"
+AFF2_SRC = """
+struct A2 { unsigned a, b; };
+A2 comp2(A2 f, A2 g) { A2 r; r.a = f.a * g.a; r.b = f.b * g.a + g.b; return r; }
+"""
+A2 = np.dtype([("a", np.uint32), ("b", np.uint32)])
+
+
+def diverged_copies_i32(ctx, base, D):
+    """copy d = base with part d overwritten by a side-effect Map (device d's events)"""
+    n = base.size
+    c = ctx.vector(base)
+    c.set_distribution(skel.COPY)
+    idx = ctx.vector(np.arange(n, dtype=np.int32))
+    idx.set_distribution(skel.BLOCK)
+    ctx.map("void mark(int i, int* c){ c[i] = (i * 7919) % 1000 - 500; }", idx, None, args=[c])
+    c.mark_device_modified()
+    copies = []
+    for d in range(D):
+        cd = base.copy()
+        lo, hi = odist.part_range(n, D, d)
+        cd[lo:hi] = (np.arange(lo, hi) * 7919) % 1000 - 500
+        copies.append(cd)
+    return c, copies
+
+
+@pytest.mark.parametrize("D", [2, 3, 4])
+@pytest.mark.parametrize("dst", [skel.BLOCK, skel.SINGLE, skel.COPY])
+def test_user_combine_max_of_diverged_copies(D, dst):
+    n = 30_011
+    base = (np.arange(n, dtype=np.int32) % 613) - 300
+    with skel.Context(D) as ctx:
+        c, copies = diverged_copies_i32(ctx, base, D)
+        c.set_distribution(dst, MAX_I32)
+        assert c.distribution == dst
+        f = lambda a, b: oracle.skel_zip(MAX_I32, a, b, np.int32)
+        model = odist.redistribute(copies, odist.COPY, NAMES[dst], f)
+        assert np.array_equal(c.download(), odist.gather(model, NAMES[dst]))
+
+
+@pytest.mark.parametrize("D", [2, 3, 4])
+@pytest.mark.parametrize("dst", [skel.BLOCK, skel.SINGLE])
+def test_user_combine_noncommutative_struct_in_device_order(D, dst):
+    """8-byte affine maps composed across the copies: only the device order
+    0..D-1 gives the oracle's result (the function is not commutative)."""
+    n = 4099
+    g = np.random.default_rng(7)
+    base = np.zeros(n, A2)
+    base["a"] = g.integers(1, 1 << 16, n)
+    base["b"] = g.integers(0, 1 << 16, n)
+    mk = """
+struct A2 { unsigned a, b; };
+void mk(int i, A2* c){ c[i].a = 2u * (unsigned)i + 3u; c[i].b = (unsigned)i * 40503u; }
+"""
+    with skel.Context(D) as ctx:
+        c = ctx.vector(base)
+        c.set_distribution(skel.COPY)
+        idx = ctx.vector(np.arange(n, dtype=np.int32))
+        idx.set_distribution(skel.BLOCK)
+        ctx.map(mk, idx, None, args=[c])
+        c.mark_device_modified()
+        copies = []
+        for d in range(D):
+            cd = base.copy()
+            lo, hi = odist.part_range(n, D, d)
+            i = np.arange(lo, hi, dtype=np.uint64)
+            cd["a"][lo:hi] = (2 * i + 3).astype(np.uint32)
+            cd["b"][lo:hi] = ((i * 40503) % (1 << 32)).astype(np.uint32)
+            copies.append(cd)
+        c.set_distribution(dst, AFF2_SRC)
+        f = lambda a, b: oracle.skel_zip(AFF2_SRC, a, b, A2)
+        want = odist.gather(odist.redistribute(copies, odist.COPY, NAMES[dst], f), NAMES[dst])
+        assert c.download().tobytes() == want.tobytes()
+        rev = odist.gather(odist.redistribute(copies[::-1], odist.COPY, NAMES[dst], f), NAMES[dst])
+        assert want.tobytes() != rev.tobytes()  # the order matters for this data
+
+
+def test_user_combine_errors():
+    with skel.Context(2) as ctx:
+        v = ctx.vector(np.arange(10, dtype=np.int32))
+        v.set_distribution(skel.BLOCK)
+        with pytest.raises(skel.SkelError) as e:
+            v.set_distribution(skel.BLOCK, MAX_I32)  # not copy-distributed
+        assert e.value.status == 8  # SKEL_ERR_STATE
+        v.set_distribution(skel.COPY)
+        with pytest.raises(skel.SkelError) as e:
+            v.set_distribution(skel.BLOCK, "double f(double a, double b){ return a + b; }")
+        assert e.value.status == 3  # SKEL_ERR_TYPE
+        with pytest.raises(skel.SkelError) as e:
+            v.set_distribution(skel.BLOCK, "int f(int a, int b, int k){ return a + b + k; }")
+        assert e.value.status == 3  # SKEL_ERR_TYPE

@@ -52,3 +52,34 @@ def test_copy_to_block_without_combine_is_local_slice():
 def test_combine_requires_copy_source():
     with pytest.raises(ValueError):
         dist.redistribute(dist.distribute(np.ones(4), dist.BLOCK, 2), dist.BLOCK, dist.COPY, "add")
+
+
+@pytest.mark.parametrize("D", [2, 3, 5])
+def test_user_combine_folds_in_device_order(D):
+    """NEXT-2 user combine: element-wise fold over the copies in device order.
+    Pinned by 2x2 integer matrix products (associative, not commutative):
+    folding copy d = [[1, d+1], [0, 1]] gives [[1, D(D+1)/2], [0, 1]], and
+    reversing the order of non-commuting factors changes the result."""
+    n = 4
+    copies = []
+    for d in range(D):
+        m = np.zeros((n, 2, 2), dtype=np.int64)
+        m[:, 0, 0] = m[:, 1, 1] = 1
+        m[:, 0, 1] = d + 1
+        copies.append(m)
+    matmul = lambda a, b: np.einsum("nij,njk->nik", a, b)
+    out = dist.gather(dist.redistribute(copies, dist.COPY, dist.BLOCK, matmul), dist.BLOCK)
+    assert (out[:, 0, 1] == D * (D + 1) // 2).all() and (out[:, 0, 0] == 1).all() and (out[:, 1, 0] == 0).all()
+    # a non-commuting case: upper- then lower-triangular differs from the reverse
+    u = np.array([[[1, 1], [0, 1]]] * n)
+    low = np.array([[[1, 0], [1, 1]]] * n)
+    fwd = dist.gather(dist.redistribute([u, low], dist.COPY, dist.SINGLE, matmul), dist.SINGLE)
+    rev = dist.gather(dist.redistribute([low, u], dist.COPY, dist.SINGLE, matmul), dist.SINGLE)
+    assert fwd[0].tolist() == [[2, 1], [1, 1]] and rev[0].tolist() == [[1, 1], [1, 2]]
+
+
+def test_user_add_equals_builtin_add():
+    parts = [np.arange(10, dtype=np.int32) * (d + 1) for d in range(3)]
+    a = dist.redistribute(parts, dist.COPY, dist.COPY, "add")
+    b = dist.redistribute(parts, dist.COPY, dist.COPY, lambda x, y: x + y)
+    assert all(np.array_equal(p, q) for p, q in zip(a, b))

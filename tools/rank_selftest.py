@@ -76,6 +76,22 @@ for dst in (skel.BLOCK, skel.SINGLE, skel.COPY):
             print(f"rank {rank}: combine->{dst} rep {rep}: {bad.size} bad, first {bad[:5]}, got {got[bad[:5]]}, "
                   f"want {want[bad[:5]]}, parts {[c.part(d) for d in range(world)]}", flush=True)
         check(f"combine->{dst}", ok)
+# NEXT-2: user-defined combine (gathered on each part's rank, folded in rank order)
+MX = "int mx(int a, int b){ return a > b ? a : b; }"
+for dst in (skel.BLOCK, skel.SINGLE, skel.COPY):
+    base = ((np.arange(n) % 613) - 300).astype(np.int32)
+    c = ctx.vector(base)
+    c.set_distribution(skel.COPY)
+    idx = ctx.vector(np.arange(n, dtype=np.int32))
+    idx.set_distribution(skel.BLOCK)
+    ctx.map("void mark(int i, int* c){ c[i] = (i * 7919) % 1000 - 500; }", idx, None, args=[c])
+    c.mark_device_modified()
+    c.set_distribution(dst, MX)
+    want = base.copy()
+    for d in range(world):
+        lo, hi = odist.part_range(n, world, d)
+        want[lo:hi] = np.maximum(base[lo:hi], ((np.arange(lo, hi) * 7919) % 1000 - 500).astype(np.int32))
+    check(f"user combine->{dst}", np.array_equal(c.download(), want))
 # LM OSEM one subset, then two more with the fused peer-memory tail (CUDA IPC)
 ev = si.lmosem_events(20_000, subset=1)
 rec = LMOSEM(ctx)
