@@ -545,6 +545,23 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
     ms = max_over_ranks(e0.elapsed_time(e1) / reps)
     res = {"config": "configs[2]: 4096x3072, cap 256, block rows", "ms": ms,
            "Mpix_per_s": W * H / (ms * 1e-3) / 1e6}
+    # NEXT-4: the same image from an index Map (c computed in-kernel, no position vector)
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_INDEX
+    oi = ctx.vector(n=pos.size, dtype=np.int32)
+    if world > 1:
+        oi.set_distribution(skel.BLOCK)
+    iargs = [np.int32(W), np.int32(H), capv]
+    for _ in range(3):
+        ctx.map_index(MANDELBROT_INDEX, W * H, oi, args=iargs)
+    barrier()
+    torch.cuda.synchronize()
+    e0.record(stream)
+    for _ in range(reps):
+        ctx.map_index(MANDELBROT_INDEX, W * H, oi, args=iargs)
+    e1.record(stream)
+    ctx.sync()
+    res["index_map_ms"] = max_over_ranks(e0.elapsed_time(e1) / reps)
+    oi.destroy()
     counts = out.download()  # collective in rank mode: every rank takes part
     if rank == 0:
         iters = int(counts.astype(np.int64).sum())

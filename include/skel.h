@@ -209,6 +209,14 @@ int skel_vector_device_ptr(skel_vec_t v, int local_index, void **ptr, size_t *co
  * arguments and the function's parameters -> SKEL_ERR_TYPE. */
 int skel_map(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out,
              const skel_arg *args, int nargs);
+/* map_index: Map over the index range [0, n) without an
+ * input vector: out[i] = f(i, args...), f given as source text whose first
+ * parameter is an integer index (4- or 8-byte; a 4-byte index needs
+ * n <= 2^31 - 1, else SKEL_ERR_SIZE).  i is the GLOBAL index: under a block
+ * distribution of out, device k evaluates its part's indices.  out takes length
+ * n and keeps its distribution; out = NULL for a void f (side effects only),
+ * which runs over a block partition of [0, n).  Errors as skel_map. */
+int skel_map_index(skel_ctx_t ctx, const char *src, size_t n, skel_vec_t out, const skel_arg *args, int nargs);
 int skel_zip(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_vec_t out,
              const skel_arg *args, int nargs);
 /* Fused form of Listing 4's tail:

@@ -143,6 +143,7 @@ static const char *kind_name(Kind k) {
     switch (k) {
         case Kind::Map: return "map";
         case Kind::Zip: return "zip";
+        case Kind::Idx: return "idx";
         default: return "red";
     }
 }
@@ -188,6 +189,7 @@ static int assemble(Kind kind, const std::string &user, int block, bool fmad, st
     std::string defs;
     if (kind == Kind::Map) defs = "#define SKEL_NIN 1\n#define SKEL_BLOCK " + std::to_string(block) + "\n";
     if (kind == Kind::Zip) defs = "#define SKEL_NIN 2\n#define SKEL_BLOCK " + std::to_string(block) + "\n";
+    if (kind == Kind::Idx) defs = "#define SKEL_NIN 0\n#define SKEL_BLOCK " + std::to_string(block) + "\n";
     text->clear();
     text->reserve(user.size() + 65536);
     *text += "#line 1 \"skel_prelude.cuh\"\n";

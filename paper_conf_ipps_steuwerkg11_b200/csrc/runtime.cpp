@@ -1567,6 +1567,61 @@ int skel_map(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, con
     return run_ew(ctx, Kind::Map, src, in, nullptr, out, args, nargs);
 }
 
+// index Map: out[i] = f(i, args...) for i in [0, n) without an
+// input vector; each device computes the indices of its part of out (block: its
+// part, copy: all, single: device 0); a void f runs over a block partition of [0, n)
+int skel_map_index(skel_ctx_t ctx, const char *src, size_t n, skel_vec_t out, const skel_arg *args, int nargs) {
+    if (!ctx || !src || (out && out->ctx != ctx) || (nargs && !args) || nargs < 0)
+        return fail(ctx, SKEL_ERR_ARG, "bad map_index arguments");
+    Module *m = nullptr;
+    TRY(get_module(ctx, Kind::Idx, src, &m));
+    const uint64_t rsz = m->sig[3];
+    if (rsz != 0 && !out) return fail(ctx, SKEL_ERR_ARG, "non-void function needs an output vector");
+    if (rsz != 0 && out->es != rsz)
+        return fail(ctx, SKEL_ERR_TYPE, "output element size " + std::to_string(out->es) + " != sizeof(result) = " +
+                                            std::to_string(rsz));
+    if (m->sig[4] < 8 && n > 0x7fffffffull)
+        return fail(ctx, SKEL_ERR_SIZE, "index range exceeds a 4-byte index parameter");
+    TRY(check_args(ctx, m, args, nargs));
+    skel_dist dist = ctx->D == 1 ? SKEL_SINGLE : SKEL_BLOCK;
+    if (rsz != 0) {
+        dist = out->dist;
+        TRY(prepare_output(out, n, dist, false));
+    }
+    const int block = (int)m->sig[9];
+    const uint64_t E = m->sig[8];
+    std::vector<unsigned char> abuf;
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        uint64_t cnt, base;
+        void *po = nullptr;
+        if (rsz != 0) {
+            cnt = out->bufs[li].count;
+            base = dist == SKEL_BLOCK ? part_lo(out, s.d) : 0;
+            po = out->bufs[li].ptr(out->es);
+        } else {
+            size_t lo, hi;
+            part_range(n, ctx->D, s.d, &lo, &hi);
+            cnt = hi - lo;
+            base = lo;
+        }
+        if (!cnt) continue;
+        int vec_ok = !po || al16(po);
+        pack_args(m, args, nargs, li, abuf);
+        const size_t chunks = vec_ok && rsz != 0 ? std::max<uint64_t>(cnt / E, 1) : cnt;
+        const int grid = ew_grid(s, chunks, block, 1);
+        void *params[] = {&po, &cnt, &base, &vec_ok, abuf.data()};
+        DevGuard g(s.dev);
+        CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+        ctx->stats.kernel_launches++;
+    }
+    if (rsz != 0) {
+        out->dev_valid = true;
+        device_wrote(out);
+    }
+    return SKEL_OK;
+}
+
 int skel_zip(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_vec_t out, const skel_arg *args,
              int nargs) {
     if (!ctx || !src || !a || !b || !out || a->ctx != ctx || b->ctx != ctx || out->ctx != ctx || (nargs && !args) ||
@@ -1850,7 +1905,8 @@ int skel_prepare(skel_ctx_t ctx, const char *kind, const char *src) {
     if (!strcmp(kind, "map")) k = Kind::Map;
     else if (!strcmp(kind, "zip")) k = Kind::Zip;
     else if (!strcmp(kind, "reduce") || !strcmp(kind, "scan")) k = Kind::Red;
-    else return fail(ctx, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan");
+    else if (!strcmp(kind, "index")) k = Kind::Idx;
+    else return fail(ctx, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan|index");
     Module *m = nullptr;
     return get_module(ctx, k, src, &m);
 }
@@ -1955,7 +2011,8 @@ int skel_compile_check(const char *kind, const char *src, int fmad, char *log, s
     if (!strcmp(kind, "map")) k = Kind::Map;
     else if (!strcmp(kind, "zip")) k = Kind::Zip;
     else if (!strcmp(kind, "reduce") || !strcmp(kind, "scan")) k = Kind::Red;
-    else return fail(nullptr, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan");
+    else if (!strcmp(kind, "index")) k = Kind::Idx;
+    else return fail(nullptr, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan|index");
     std::string l;
     std::vector<char> cubin;
     const int st = compile_only(k, src, 256, fmad != 0, &l, &cubin);

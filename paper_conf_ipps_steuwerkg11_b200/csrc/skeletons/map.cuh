@@ -3,6 +3,8 @@
 //
 //   SKEL_NIN == 1:  out[i] = SKEL_FN(a[i], args...)        (void: side effects only)
 //   SKEL_NIN == 2:  out[i] = SKEL_FN(a[i], b[i], args...)
+//   SKEL_NIN == 0:  out[i] = SKEL_FN(i, args...)           (index Map over [0, n), NEXT-4;
+//                   i is the GLOBAL index, the part's offset is passed in)
 //
 // B200 mapping (kernel K1): the vector is walked in "chunks" of
 // E consecutive elements, E chosen so one chunk of every operand is one
@@ -26,7 +28,8 @@
 
 using skel_F = decltype(&SKEL_FN);
 using skel_FT = skel::fn<skel_F>;
-static_assert(skel_FT::arity >= SKEL_NIN, "user function has too few parameters for this skeleton");
+constexpr int SKEL_NPOS = SKEL_NIN == 0 ? 1 : SKEL_NIN;  // positional (element / index) parameters
+static_assert(skel_FT::arity >= SKEL_NPOS, "user function has too few parameters for this skeleton");
 using skel_A = typename skel_FT::template param<0>;
 #if SKEL_NIN == 2
 using skel_B = typename skel_FT::template param<1>;
@@ -40,14 +43,14 @@ template <bool V, class R> struct skel_out_t { using type = skel::decay_t<R>; };
 template <class R> struct skel_out_t<true, R> { using type = skel_none; };
 using skel_O = typename skel_out_t<skel_void, skel_R>::type;
 
-using skel_Args = typename skel::drop<SKEL_NIN, typename skel_FT::params>::type;
+using skel_Args = typename skel::drop<SKEL_NPOS, typename skel_FT::params>::type;
 using skel_Lay = skel::args_layout<skel_Args>;
 constexpr skel_u64 SKEL_ARGBYTES = skel::cmax<skel_u64>(16, skel::align_up(skel_Lay::bytes, 16));
 using skel_Buf = skel::argbuf<SKEL_ARGBYTES>;
 using skel_Seq = typename skel::make_iseq<skel_Lay::n>::type;
 
 // ---- chunking ------------------------------------------------------------
-constexpr skel_u64 skel_szA = sizeof(skel_A);
+constexpr skel_u64 skel_szA = SKEL_NIN == 0 ? 1 : sizeof(skel_A);  // the index is not loaded
 constexpr skel_u64 skel_szB = (SKEL_NIN == 2) ? sizeof(skel_B) : 1;
 constexpr skel_u64 skel_szO = skel_void ? 1 : sizeof(skel_O);
 constexpr skel_u64 skel_maxsz = skel::cmax(skel_szA, skel::cmax(skel_szB, skel_szO));
@@ -175,6 +178,46 @@ __device__ __forceinline__ void skel_one(const skel_A *a, const skel_B *b, skel_
     }
 }
 
+#if SKEL_NIN == 0
+static_assert(skel::is_arith<skel::decay_t<skel_A>>::value, "an index Map's first parameter must be an integer index");
+// index Map: element c*E + e of this part is index base + c*E + e; outputs are
+// staged per chunk and stored with one 128-bit store, like Map.  (The bodies are
+// templates on "void result" so that the discarded branch is never checked.)
+template <bool V = skel_void, class Tup>
+__device__ __forceinline__ skel_u64 skel_idx_chunks(skel_O *out, skel_u64 n, skel_u64 base, skel_u64 tid,
+                                                    skel_u64 stride, Tup &t) {
+    using I = skel::decay_t<skel_A>;
+    if constexpr (SKEL_E > 1 && !V) {
+        const skel_u64 nch = n / SKEL_E;
+        for (skel_u64 c = tid; c < nch; c += stride) {
+            skel::arr<skel_O, SKEL_E> yo;
+#pragma unroll
+            for (int e = 0; e < SKEL_E; ++e) yo.v[e] = skel::caller<skel_Seq>::call(&SKEL_FN, t, (I)(base + c * SKEL_E + e));
+            skel_st<skel_CO>(reinterpret_cast<char *>(out) + c * skel_CO, skel::bit_cast<skel::chunk<skel_CO>>(yo));
+        }
+        return nch * SKEL_E;
+    } else {
+        return 0;
+    }
+}
+template <bool V = skel_void, class Tup>
+__device__ __forceinline__ void skel_idx_one(skel_O *out, skel_u64 i, skel_u64 base, Tup &t) {
+    using I = skel::decay_t<skel_A>;
+    if constexpr (V) {
+        skel::caller<skel_Seq>::call(&SKEL_FN, t, (I)(base + i));
+    } else {
+        out[i] = skel::caller<skel_Seq>::call(&SKEL_FN, t, (I)(base + i));
+    }
+}
+extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
+    skel_ew_kernel(skel_O *__restrict__ out, skel_u64 n, skel_u64 base, int vec_ok, const skel_Buf args) {
+    auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
+    const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;
+    const skel_u64 done = vec_ok ? skel_idx_chunks(out, n, base, tid, stride, t) : 0;
+    for (skel_u64 i = done + tid; i < n; i += stride) skel_idx_one(out, i, base, t);
+}
+#else
 extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
     skel_ew_kernel(const skel_A *__restrict__ a, const skel_B *__restrict__ b, skel_O *__restrict__ out, skel_u64 n,
                    int vec_ok, const skel_Buf args) {
@@ -213,6 +256,7 @@ extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
     // scalar path: the tail, or everything for non-vectorisable element types
     for (skel_u64 i = done + tid; i < n; i += stride) skel_one(a, b, out, i, t);
 }
+#endif  // SKEL_NIN == 0
 
 #if SKEL_NIN == 2
 // ---------------------------------------------------------------------------

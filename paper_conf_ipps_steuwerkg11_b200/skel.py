@@ -85,6 +85,7 @@ def lib() -> ctypes.CDLL:
             "skel_vector_part": [P, I, ctypes.POINTER(S), ctypes.POINTER(S)],
             "skel_vector_device_ptr": [P, I, PP, ctypes.POINTER(S)],
             "skel_map": [P, ctypes.c_char_p, P, P, P, I], "skel_zip": [P, ctypes.c_char_p, P, P, P, P, I],
+            "skel_map_index": [P, ctypes.c_char_p, S, P, P, I],
             "skel_reduce": [P, ctypes.c_char_p, P, P, P, I],
             "skel_zip_combine": [P, ctypes.c_char_p, P, P, I, P, P, I], "skel_reduce_to": [P, ctypes.c_char_p, P, P, P, I],
             "skel_scan": [P, ctypes.c_char_p, P, P, P, P, I], "skel_prepare": [P, ctypes.c_char_p, ctypes.c_char_p],
@@ -267,6 +268,13 @@ class Context:
         """eq. (1): vout[i] = f(vin[i], args...); vout=None for a void (side-effect) Map."""
         a, keep = self._args(args)
         _check(lib().skel_map(self._h, src.encode(), vin._h, vout._h if vout is not None else None, a, len(args)), self._h)
+        return vout
+
+    def map_index(self, src: str, n: int, vout: "Vector | None" = None, args=()):
+        """NEXT-4: out[i] = f(i, args...) for i in [0, n), no input vector."""
+        a, keep = self._args(args)
+        _check(lib().skel_map_index(self._h, src.encode(), n, vout._h if vout is not None else None, a, len(args)),
+               self._h)
         return vout
 
     def zip(self, src: str, va: "Vector", vb: "Vector", vout: "Vector", args=()):

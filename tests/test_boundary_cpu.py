@@ -10,7 +10,7 @@ import pytest
 
 from oracle import distribution as odist
 from paper_conf_ipps_steuwerkg11_b200 import skel
-from paper_conf_ipps_steuwerkg11_b200.workloads import (LMOSEM_ERROR, LMOSEM_UPDATE, MANDELBROT, SAXPY_F32,
+from paper_conf_ipps_steuwerkg11_b200.workloads import (LMOSEM_ERROR, LMOSEM_UPDATE, MANDELBROT, MANDELBROT_INDEX, SAXPY_F32,
                                                          SUM_F32)
 
 ROOT = Path(__file__).resolve().parents[1]
@@ -34,7 +34,8 @@ def test_status_strings():
 
 
 @pytest.mark.parametrize("kind,src", [("map", MANDELBROT), ("map", LMOSEM_ERROR), ("zip", LMOSEM_UPDATE),
-                                      ("zip", SAXPY_F32), ("reduce", SUM_F32), ("scan", SUM_F32)])
+                                      ("zip", SAXPY_F32), ("reduce", SUM_F32), ("scan", SUM_F32),
+                                      ("index", MANDELBROT_INDEX)])
 def test_nvrtc_injection_compiles_for_sm100a(kind, src):
     st, log, nbytes = skel.compile_check(kind, src)
     assert st == 0, log

@@ -54,3 +54,19 @@ def test_block_rows_on_virtual_devices(D):
     with skel.Context(D) as ctx:
         got = run(ctx, pos, 256, skel.BLOCK)
     assert np.array_equal(got, oracle.mandelbrot(pos, 256))
+
+
+@pytest.mark.parametrize("w,h,cap,D", [(1024, 768, 256, 1), (4096, 3072, 256, 1), (1024, 768, 256, 3)])
+def test_index_map_variant_matches_the_golden_image(golden_dir, w, h, cap, D):
+    """NEXT-4: the same image from an index Map (c computed in the kernel from
+    the pixel index, no position vector) -- bit-identical to the golden pins."""
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_INDEX
+    with skel.Context(D) as ctx:
+        out = ctx.vector(n=w * h, dtype=np.int32)
+        if D > 1:
+            out.set_distribution(skel.BLOCK)
+        ctx.map_index(MANDELBROT_INDEX, w * h, out, args=[np.int32(w), np.int32(h), np.int32(cap)])
+        got = out.download()
+    with open(os.path.join(golden_dir, "mandelbrot.json")) as fh:
+        case = [c for c in json.load(fh)["cases"] if (c["width"], c["height"], c["cap"]) == (w, h, cap)][0]
+    assert zlib.crc32(got.tobytes()) == int(case["crc32"], 16)

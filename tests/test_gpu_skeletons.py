@@ -386,3 +386,31 @@ def test_map_zip_grid_policy_trials_bit_identical(n):
             assert np.array_equal(vz.download(), want_z)
             vm.destroy()
             vz.destroy()
+
+
+IDX_I64 = "long long poly(long long i, long long k){ return i * i - k * i + 7; }"
+
+
+@pytest.mark.parametrize("D,dist", [(1, None), (2, skel.BLOCK), (3, skel.BLOCK), (3, skel.COPY), (2, skel.SINGLE)])
+@pytest.mark.parametrize("n", [1, 5, 4097, (1 << 20) + 3])
+def test_index_map_is_map_over_the_index_vector(D, dist, n):
+    """NEXT-4: map_index(f, n) equals Map(f) over [0, 1, ..., n-1] (eq. (1)), with
+    global indices under a block distribution of the output."""
+    want = oracle.skel_map(IDX_I64, np.arange(n, dtype=np.int64), np.int64, args=[np.int64(5)])
+    with skel.Context(D) as c:
+        out = c.vector(n=n, dtype=np.int64)
+        if dist is not None:
+            out.set_distribution(dist)
+        c.map_index(IDX_I64, n, out, args=[np.int64(5)])
+        assert np.array_equal(out.download(), want)
+
+
+def test_void_index_map_side_effects():
+    n = 10_007
+    with skel.Context(2) as c:
+        acc = c.vector(np.zeros(n, np.int32))
+        acc.set_distribution(skel.COPY)
+        c.map_index("void touch(int i, int* a){ a[i] += i % 5 + 1; }", n, None, args=[acc])
+        acc.mark_device_modified()
+        acc.set_distribution(skel.BLOCK, skel.COMBINE_ADD)
+        assert np.array_equal(acc.download(), (np.arange(n) % 5 + 1).astype(np.int32))
