@@ -78,3 +78,18 @@ int hw_exscan_f32(const float *x, float *y, size_t n, void *stream) {
     return (int)cudaGetLastError();
 }
 }
+
+// CUB's two-kernel DeviceReduce::Sum (small-size comparison, tools/small_n_probe.py)
+extern "C" int hw_cubsum_f32(const float *x, size_t n, float *out, void *stream) {
+    static void *tmp = nullptr;
+    static size_t tmp_bytes = 0;
+    size_t need = 0;
+    cub::DeviceReduce::Sum(nullptr, need, x, out, (int64_t)n, (cudaStream_t)stream);
+    if (need > tmp_bytes) {
+        if (tmp) cudaFree(tmp);
+        cudaMalloc(&tmp, need);
+        tmp_bytes = need;
+    }
+    cub::DeviceReduce::Sum(tmp, tmp_bytes, x, out, (int64_t)n, (cudaStream_t)stream);
+    return (int)cudaGetLastError();
+}

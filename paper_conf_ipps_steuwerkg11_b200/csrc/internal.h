@@ -50,6 +50,7 @@ struct Module {
         cudaEvent_t ev[8] = {};
     };
     std::map<int, EwTune> ew_tune;
+    int red_occ = 0;  // resident Reduce CTAs per SM (0 = not yet queried)
 };
 
 // signature accessors (layout documented in map.cuh / red.cuh)

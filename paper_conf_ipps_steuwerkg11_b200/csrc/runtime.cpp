@@ -1017,27 +1017,67 @@ int set_smem_attr(skel_ctx_s *ctx, Module *m, const Slot &s) {
     return SKEL_OK;
 }
 
+// resident Reduce CTAs per SM (the grid is SMs x this, capped by the tile count)
+int red_occupancy(Module *m, const Slot &s) {
+    if (m->red_occ > 0) return m->red_occ;
+    int occ = 1;
+    DevGuard g(s.dev);
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, (const void *)m->k_main, (int)m->sig[9],
+                                                      (size_t)m->sig[11]) != cudaSuccess || occ < 1) {
+        cudaGetLastError();
+        occ = 1;
+    }
+    if (const char *e = getenv("SKEL_RED_OCC")) occ = std::max(1, std::min(occ, atoi(e)));  // tuning hook
+    m->red_occ = occ;
+    return occ;
+}
+
+// Reduce grid.  Up to ~55 tiles per SM: one CTA per resident slot, static
+// contiguous tile ranges.  Larger vectors: oversubscribe (2/4/8 CTAs per slot,
+// still contiguous ranges) so the hardware scheduler hands the last ranges to
+// whichever SMs finish first -- measured at 2^28/2^29/2^30 floats: 168->161,
+// 326->310, 629->605 us; below that the pipeline fill of each extra CTA costs
+// more than the balance gains (tools/red_variants.sh).
+size_t red_grid(Module *m, const Slot &s, uint64_t cnt) {
+    static const int os_env = [] {  // tuning hook SKEL_RED_OVERSUB (CTAs per resident slot)
+        const char *e = getenv("SKEL_RED_OVERSUB");
+        return e ? std::max(1, atoi(e)) : 0;
+    }();
+    const uint64_t slots = (uint64_t)s.sms * (uint64_t)red_occupancy(m, s);
+    const uint64_t nft = cnt / m->sig[10];
+    uint64_t os = os_env;
+    if (!os) os = std::min<uint64_t>(8, std::max<uint64_t>(1, nft / (slots * 55)));
+    if (os > 2 && os < 8) os = os < 6 ? 4 : 8;  // powers of two (measured points)
+    return (size_t)std::max<uint64_t>(1, std::min<uint64_t>(slots * os, nft));
+}
+
+// partial results the Reduce kernel publishes: one per CTA, or one per tile
+// (+ the ragged tail) in the interleaved tile order (sig[15] bit 48)
+size_t red_parts(Module *m, const Slot &s, uint64_t cnt) {
+    const size_t G = red_grid(m, s, cnt);
+    if (!((m->sig[15] >> 48) & 1)) return G;
+    return std::max<size_t>(G, (size_t)(cnt / m->sig[10]) + 1);
+}
+
 // local reduce of the slot's data into dst
 int launch_reduce(skel_ctx_s *ctx, Module *m, Slot &s, const void *in, uint64_t cnt, const RedLayout &L,
                   std::vector<unsigned char> &abuf, void *dst) {
-    const uint64_t TILE = m->sig[10];
+    const uint64_t TILE = m->sig[10], RB = m->sig[9];
     const uint64_t nft = cnt / TILE;
-    const size_t G = (size_t)std::max<uint64_t>(1, std::min<uint64_t>((uint64_t)s.sms, nft));
+    const size_t G = red_grid(m, s, cnt);
     CUtensorMap tin;
-    int use_tma = m->sig[5] && make_tmap(&tin, in, nft * m->sig[9]);
+    memset(&tin, 0, sizeof tin);
+    const bool direct = (m->sig[15] >> 49) & 1;  // direct 128-bit loads: `use_tma` = 16-byte aligned
+    int use_tma = m->sig[5] && (direct ? al16(in) : make_tmap(&tin, in, nft * RB, (uint32_t)(RB / 2)));
     char *ws = s.ws;
     void *partials = ws + L.o_part, *pvalid = ws + L.o_pvalid, *result = dst;
     unsigned *counter = s.counters + 2;
     void *params[] = {&tin, &in, &cnt, &use_tma, &partials, &pvalid, &counter, &result, abuf.data()};
     DevGuard g(s.dev);
-    CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3((unsigned)G), dim3((unsigned)m->sig[9]), params,
+    CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3((unsigned)G), dim3((unsigned)RB), params,
                              use_tma ? m->sig[11] : 0, s.stream));
     ctx->stats.kernel_launches++;
     return SKEL_OK;
-}
-
-size_t red_grid(const Module *m, const Slot &s, uint64_t cnt) {
-    return (size_t)std::max<uint64_t>(1, std::min<uint64_t>((uint64_t)s.sms, cnt / m->sig[10]));
 }
 
 // Reduce of `in` leaving the result in every local slot's ws[o_fold]
@@ -1052,9 +1092,9 @@ int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args
     for (size_t li = 0; li < ctx->slots.size(); ++li) {
         Slot &s = ctx->slots[li];
         const uint64_t cnt = in->bufs[li].count;
-        Ls[li] = red_layout(m, D, red_grid(m, s, cnt), 0);
+        TRY(set_smem_attr(ctx, m, s));  // before the occupancy query in red_grid
+        Ls[li] = red_layout(m, D, red_parts(m, s, cnt), 0);
         TRY(ensure_ws(ctx, s, Ls[li].total));
-        TRY(set_smem_attr(ctx, m, s));
         pack_args(m, args, nargs, li, abuf);
         char *dst = cross ? s.ws + Ls[li].o_res : (direct && D == 1 ? static_cast<char *>(direct) : s.ws + Ls[li].o_fold);
         if (cnt) TRY(launch_reduce(ctx, m, s, in->bufs[li].ptr(in->es), cnt, Ls[li], abuf, dst));
@@ -1848,7 +1888,7 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
     for (size_t li = 0; li < ctx->slots.size(); ++li) {
         Slot &s = ctx->slots[li];
         const uint64_t cnt = in->bufs[li].count;
-        Ls[li] = red_layout(m, D, red_grid(m, s, cnt), scan_slots(s, cnt));
+        Ls[li] = red_layout(m, D, red_parts(m, s, cnt), scan_slots(s, cnt));
         TRY(ensure_ws(ctx, s, Ls[li].total));
     }
     if (cross) {

@@ -24,8 +24,21 @@
 //  * Element types whose size is not 4, 8 or 16 bytes, unaligned views and
 //    the ragged last tile use direct (LDG/STG) loads with the same ordering.
 
+// Reduce main loop: 1 = direct 128-bit loads, every warp folding its own
+// contiguous range (no barrier in the loop); 0 = TMA tiles through shared
+// memory with one ordered block fold per tile (K3)
+#ifndef SKEL_RED_DIRECT
+#define SKEL_RED_DIRECT 0
+#endif
 #ifndef SKEL_RBLOCK
+#if SKEL_RED_DIRECT
+#define SKEL_RBLOCK 256
+#else
 #define SKEL_RBLOCK 512
+#endif
+#endif
+#ifndef SKEL_RED_U
+#define SKEL_RED_U 4  // direct Reduce: 16-byte loads in flight per lane
 #endif
 #ifndef SKEL_STAGES
 #define SKEL_STAGES 3
@@ -49,10 +62,21 @@ constexpr int RB = SKEL_RBLOCK;
 constexpr int NW = RB / 32;
 constexpr bool TMA_OK = sizeof(skel_T) == 4 || sizeof(skel_T) == 8 || sizeof(skel_T) == 16;
 constexpr int K = TMA_OK ? (int)(128 / sizeof(skel_T)) : (int)skel::cmax<skel_u64>(1, 128 / sizeof(skel_T));
-constexpr skel_u64 TILE = (skel_u64)RB * K;
-constexpr unsigned TILE_BYTES = (unsigned)(TILE * sizeof(skel_T));
+constexpr bool RDIRECT = SKEL_RED_DIRECT != 0;
+constexpr int RU = SKEL_RED_U;
+constexpr int PERV = TMA_OK ? (int)(16 / sizeof(skel_T)) : 1;  // elements per 16-byte lane load
+// Reduce work unit (elements): a TMA tile, or one round of RU loads of every warp
+constexpr skel_u64 TILE = RDIRECT ? (skel_u64)RB * PERV * RU : (skel_u64)RB * K;
+constexpr unsigned TILE_BYTES = (unsigned)((skel_u64)RB * K * sizeof(skel_T));
 constexpr int STAGES = SKEL_STAGES;
-constexpr unsigned DSMEM = TMA_OK ? STAGES * TILE_BYTES + 1024 : 0;
+// Reduce tile order: 0 = static contiguous tile ranges per CTA (one partial per
+// CTA); 1 = tile i on CTA i mod G (all CTAs stream adjacent tiles, like a
+// grid-stride loop), one partial per tile, folded in index order at the end
+#ifndef SKEL_RED_INTERLEAVE
+#define SKEL_RED_INTERLEAVE 0
+#endif
+constexpr bool RIL = SKEL_RED_INTERLEAVE != 0;
+constexpr unsigned DSMEM = (TMA_OK && !RDIRECT) ? STAGES * TILE_BYTES + 1024 : 0;
 // Scan: tiles per CTA per slice (see the Scan section)
 #ifndef SKEL_SCAN_CH
 #define SKEL_SCAN_CH 1
@@ -100,7 +124,9 @@ constexpr skel_sig_t skel_make_sig() {
     s.v[12] = SDSMEM;
     s.v[13] = PACKED;
     s.v[14] = SRB + 64 + 32 * PW;  // scan block size (consumers, producer, store and window warps); tile = SRB * K
-    s.v[15] = (skel_u64)SRB | ((skel_u64)SCAN_CH << 16) | ((skel_u64)REPL << 32);  // scan rows/tile | tiles/CTA/slice | status copies
+    s.v[15] = (skel_u64)SRB | ((skel_u64)SCAN_CH << 16) | ((skel_u64)REPL << 32) |
+              ((skel_u64)RIL << 48) | ((skel_u64)RDIRECT << 49);  // scan rows/tile | tiles/CTA/slice | status
+                                                                  // copies | reduce tile order | direct reduce
     for (int i = 0; i < skel_Lay::n && i < 32; ++i) {
         s.v[16 + 4 * i] = skel_Lay::size(i);
         s.v[17 + 4 * i] = skel_Lay::align(i);
@@ -272,7 +298,126 @@ extern __shared__ __align__(16) unsigned char skel_dsmem[];
 // ============================================================================
 // Reduce
 // ============================================================================
-extern "C" __global__ void __launch_bounds__(RB, 1)
+#ifndef SKEL_RED_MINB
+#if SKEL_RED_DIRECT
+#define SKEL_RED_MINB 4
+#else
+#define SKEL_RED_MINB 1
+#endif
+#endif
+// ordered warp fold of 32 valid values: lane 0 receives x_0 (+) ... (+) x_31
+template <class Tup> __device__ __forceinline__ skel_T warp_fold_full(skel_T x, int lane, Tup &t) {
+#pragma unroll
+    for (int d = 1; d < 32; d <<= 1) {
+        const skel_T o = skel::shfl_down(x, d);
+        if ((lane & (2 * d - 1)) == 0) x = opf(x, o, t);
+    }
+    return x;
+}
+__device__ __forceinline__ uint4 ld_stream16(const void *p) {
+    uint4 q;
+    asm volatile("ld.global.nc.L1::no_allocate.v4.u32 {%0,%1,%2,%3}, [%4];"
+                 : "=r"(q.x), "=r"(q.y), "=r"(q.z), "=r"(q.w)
+                 : "l"(p));
+    return q;
+}
+// in-order fold of the PERV elements of one 16-byte lane load
+template <bool OK = TMA_OK, class Tup> __device__ __forceinline__ skel_T fold16(const uint4 &q, Tup &t) {
+    if constexpr (OK) {
+        const auto e = skel::bit_cast<skel::arr<skel_T, PERV>>(q);
+        skel_T a = e.v[0];
+#pragma unroll
+        for (int k = 1; k < PERV; ++k) a = opf(a, e.v[k], t);
+        return a;
+    } else {
+        return skel_T{};
+    }
+}
+__device__ __forceinline__ VT vt_make(const skel_T &v) {
+    VT r;
+    r.v = v;
+    r.ok = true;
+    return r;
+}
+// Direct Reduce of this CTA's range, valid in thread 0 (RDIRECT).  The n
+// elements form warp-chunks of 32 consecutive lane loads (16 bytes each when
+// `vec`, else one element); the G*NW warps of the grid own contiguous chunk
+// ranges, each folds its range in order (lane fold, ordered shuffle tree per
+// chunk, running aggregate in lane 0) with RU loads in flight per lane; the
+// ragged tail (< one chunk) goes to the last warp; the CTA folds its warps in
+// order.  No barrier inside the loop.
+template <class Tup>
+__device__ __forceinline__ VT reduce_direct(const skel_T *__restrict__ in, skel_u64 n, bool vec, VT *wpart, Tup &tup) {
+    const int t = threadIdx.x, lane = t & 31, w = t >> 5;
+    const skel_u64 G = gridDim.x, c = blockIdx.x;
+    const skel_u64 per_chunk = (TMA_OK && vec) ? 32ull * PERV : 32ull;
+    const skel_u64 nch = n / per_chunk;
+    const skel_u64 NWT = G * NW, gw = c * NW + w;
+    const skel_u64 k0 = nch * gw / NWT, k1 = nch * (gw + 1) / NWT;
+    VT wrun;
+    wrun.ok = false;
+    skel_u64 k = k0;
+    if (TMA_OK && vec) {
+        const uint4 *base = reinterpret_cast<const uint4 *>(in) + lane;
+        for (; k + RU <= k1; k += RU) {
+            uint4 q[RU];
+#pragma unroll
+            for (int u = 0; u < RU; ++u) q[u] = ld_stream16(base + (k + u) * 32);
+#pragma unroll
+            for (int u = 0; u < RU; ++u) {
+                const skel_T a = warp_fold_full(fold16(q[u], tup), lane, tup);
+                if (lane == 0) wrun = comb(wrun, vt_make(a), tup);
+            }
+        }
+        for (; k < k1; ++k) {
+            const skel_T a = warp_fold_full(fold16(ld_stream16(base + k * 32), tup), lane, tup);
+            if (lane == 0) wrun = comb(wrun, vt_make(a), tup);
+        }
+    } else {
+        const skel_T *base = in + lane;
+        for (; k + RU <= k1; k += RU) {
+            skel_T q[RU];
+#pragma unroll
+            for (int u = 0; u < RU; ++u) q[u] = base[(k + u) * 32];
+#pragma unroll
+            for (int u = 0; u < RU; ++u) {
+                const skel_T a = warp_fold_full(q[u], lane, tup);
+                if (lane == 0) wrun = comb(wrun, vt_make(a), tup);
+            }
+        }
+        for (; k < k1; ++k) {
+            const skel_T a = warp_fold_full(base[k * 32], lane, tup);
+            if (lane == 0) wrun = comb(wrun, vt_make(a), tup);
+        }
+    }
+    if (gw == NWT - 1) {  // ragged tail, in order after the last chunk
+        const skel_u64 b0 = nch * per_chunk, rem = n - b0;
+        if (rem) {
+            const skel_u64 kt = (rem + 31) / 32;
+            VT a;
+            a.ok = false;
+            for (skel_u64 j2 = 0; j2 < kt; ++j2) {
+                const skel_u64 j = (skel_u64)lane * kt + j2;
+                if (j < rem) a = comb(a, vt_make(in[b0 + j]), tup);
+            }
+            a = warp_fold(a, lane, tup);
+            if (lane == 0) wrun = comb(wrun, a, tup);
+        }
+    }
+    if (lane == 0) wpart[w] = wrun;
+    __syncthreads();
+    VT r;
+    r.ok = false;
+    if (w == 0) {
+        VT y;
+        y.ok = false;
+        if (lane < NW) y = wpart[lane];
+        r = warp_fold(y, lane, tup);
+    }
+    return r;
+}
+
+extern "C" __global__ void __launch_bounds__(RB, SKEL_RED_MINB)
     skel_reduce_kernel(const __grid_constant__ skel_tmap tin, const skel_T *__restrict__ in, skel_u64 n, int use_tma,
                        skel_S *partials, unsigned *pvalid, unsigned *counter, skel_S *result, const skel_Buf args) {
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
@@ -282,11 +427,23 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
     const int t = threadIdx.x;
     const skel_u64 nft = n / TILE;
     const skel_u64 G = gridDim.x, c = blockIdx.x;
-    const skel_u64 t0 = nft * c / G, t1 = nft * (c + 1) / G, my = t1 - t0;
+    const skel_u64 t0 = nft * c / G, t1 = nft * (c + 1) / G;
+    const skel_u64 my = RIL ? (nft > c ? (nft - c + G - 1) / G : 0) : t1 - t0;
+    auto tile_at = [&](skel_u64 i) -> skel_u64 { return RIL ? c + i * G : t0 + i; };
     VT run;
     run.ok = false;
+    // RIL: every tile's fold is a partial of its own (index = tile)
+    auto take = [&](VT tv, skel_u64 tile) {
+        if (RIL) {
+            skel::st_value(&partials[tile], skel_S{tv.v});
+        } else {
+            run = comb(run, tv, tup);
+        }
+    };
 
-    if (TMA_OK && use_tma) {
+    if (RDIRECT) {
+        run = reduce_direct(in, n, use_tma != 0, wpart, tup);
+    } else if (TMA_OK && use_tma) {
         unsigned char *stages = aligned_stages(skel_dsmem);
         if (t == 0) {
             for (int s = 0; s < STAGES; ++s) skel::mbar_init(&bars[s], 1);
@@ -295,7 +452,7 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
         }
         __syncthreads();
         if (t == 0)
-            for (skel_u64 s = 0; s < STAGES && s < my; ++s) issue_tile(stages + s * TILE_BYTES, &tin, t0 + s, &bars[s]);
+            for (skel_u64 s = 0; s < STAGES && s < my; ++s) issue_tile(stages + s * TILE_BYTES, &tin, tile_at(s), &bars[s]);
         for (skel_u64 i = 0; i < my; ++i) {
             const int s = (int)(i % STAGES);
             skel::mbar_wait(&bars[s], (unsigned)((i / STAGES) & 1));
@@ -307,13 +464,13 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
 #pragma unroll
             for (int k = 1; k < K; ++k) a.v = opf(a.v, x[k], tup);
             __syncthreads();  // stage s fully consumed
-            if (t == 0 && i + STAGES < my) issue_tile(stages + s * TILE_BYTES, &tin, t0 + i + STAGES, &bars[s]);
+            if (t == 0 && i + STAGES < my) issue_tile(stages + s * TILE_BYTES, &tin, tile_at(i + STAGES), &bars[s]);
             VT tv = block_fold(a, wpart, tup);
-            if (t == 0) run = comb(run, tv, tup);
+            if (t == 0) take(tv, tile_at(i));
         }
     } else {
         for (skel_u64 i = 0; i < my; ++i) {
-            const skel_T *p = in + (t0 + i) * TILE + (skel_u64)t * K;
+            const skel_T *p = in + tile_at(i) * TILE + (skel_u64)t * K;
             VT a;
             a.v = p[0];
             a.ok = true;
@@ -321,11 +478,11 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
             for (int k = 1; k < K; ++k) a.v = opf(a.v, p[k], tup);
             __syncthreads();
             VT tv = block_fold(a, wpart, tup);
-            if (t == 0) run = comb(run, tv, tup);
+            if (t == 0) take(tv, tile_at(i));
         }
     }
     // ragged last tile: direct loads, owned by the last CTA (keeps index order)
-    if (c == G - 1 && nft * TILE < n) {
+    if (!RDIRECT && c == G - 1 && nft * TILE < n) {
         const skel_u64 base = nft * TILE, rem = n - base;
         const skel_u64 kt = (rem + RB - 1) / RB;
         VT a;
@@ -341,12 +498,16 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
         }
         __syncthreads();
         VT tv = block_fold(a, wpart, tup);
-        if (t == 0) run = comb(run, tv, tup);
+        if (t == 0) take(tv, nft);
     }
-    // publish this CTA's partial; the last CTA to finish folds them in order
+    // publish this CTA's partial (RIL: the tile partials are already out); the
+    // last CTA to finish folds them in order
+    const skel_u64 NP = (RIL && !RDIRECT) ? nft + (nft * TILE < n ? 1 : 0) : G;  // partials
     if (t == 0) {
-        skel::st_value(&partials[c], skel_S{run.v});
-        skel::st_relaxed_u32(&pvalid[c], run.ok ? 1u : 0u);
+        if (!RIL || RDIRECT) {
+            skel::st_value(&partials[c], skel_S{run.v});
+            skel::st_relaxed_u32(&pvalid[c], run.ok ? 1u : 0u);
+        }
         __threadfence();
         const unsigned prev = atomicAdd(counter, 1u);
         s_last = (prev == (unsigned)(G - 1));
@@ -354,17 +515,20 @@ extern "C" __global__ void __launch_bounds__(RB, 1)
     __syncthreads();
     if (s_last) {
         __threadfence();
-        const skel_u64 per = (G + RB - 1) / RB;
+        const skel_u64 per = (NP + RB - 1) / RB;
         VT a;
         a.ok = false;
-        for (skel_u64 k = 0; k < per; ++k) {
-            const skel_u64 j = (skel_u64)t * per + k;
-            if (j < G && skel::ld_relaxed_u32(&pvalid[j])) {
-                VT e;
-                e.v = skel::ld_value(&partials[j]).v;
-                e.ok = true;
-                a = comb(a, e, tup);
+        // loads in batches of 8 (independent L2 round trips), folded in order
+        for (skel_u64 k0 = 0; k0 < per; k0 += 8) {
+            VT e[8];
+#pragma unroll
+            for (int u = 0; u < 8; ++u) {
+                const skel_u64 j = (skel_u64)t * per + k0 + u;
+                e[u].ok = k0 + u < per && j < NP && ((RIL && !RDIRECT) || skel::ld_relaxed_u32(&pvalid[j]));
+                if (e[u].ok) e[u].v = skel::ld_value(&partials[j]).v;
             }
+#pragma unroll
+            for (int u = 0; u < 8; ++u) a = comb(a, e[u], tup);
         }
         VT r = block_fold(a, wpart, tup);
         if (t == 0) {
