@@ -562,7 +562,39 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
     ctx.sync()
     res["index_map_ms"] = max_over_ranks(e0.elapsed_time(e1) / reps)
     oi.destroy()
+    # NEXT-4: the blocked user function (same counts, loop control per 8 updates)
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_BLOCKED
+    ob = ctx.vector(n=pos.size, dtype=np.int32)
+    for _ in range(3):
+        ctx.map(MANDELBROT_BLOCKED, vin, ob, args=[capv])
+    barrier()
+    torch.cuda.synchronize()
+    e0.record(stream)
+    for _ in range(reps):
+        ctx.map(MANDELBROT_BLOCKED, vin, ob, args=[capv])
+    e1.record(stream)
+    ctx.sync()
+    ms_blk = max_over_ranks(e0.elapsed_time(e1) / reps)
+    res["blocked_ms"] = ms_blk
+    same = ob.download()
     counts = out.download()  # collective in rank mode: every rank takes part
+    # heavy variant ("also report the cap-4096 variant")
+    heavy = {}
+    for name, fn in (("paper", MANDELBROT), ("blocked", MANDELBROT_BLOCKED)):
+        c4 = np.int32(4096)
+        ctx.map(fn, vin, ob, args=[c4])
+        barrier()
+        torch.cuda.synchronize()
+        e0.record(stream)
+        for _ in range(3):
+            ctx.map(fn, vin, ob, args=[c4])
+        e1.record(stream)
+        ctx.sync()
+        heavy[name] = max_over_ranks(e0.elapsed_time(e1) / 3)
+    it4096 = int(ob.download().astype(np.int64).sum())
+    ob.destroy()
+    if rank == 0:
+        res["blocked_bit_identical"] = bool(np.array_equal(same, counts))
     if rank == 0:
         iters = int(counts.astype(np.int64).sum())
         res["sum_iter"] = iters
@@ -571,6 +603,10 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
         # vs 148 SM x 128 lanes x 1.965 GHz = 37.2 T FP32 instr/s
         peak_ops = 148 * 128 * 1.965e9
         res["fp32_frac"] = 8 * iters / (ms * 1e-3) / peak_ops
+        res["blocked_fp32_frac"] = 8 * iters / (ms_blk * 1e-3) / peak_ops
+        res["cap4096"] = {"sum_iter": it4096, "ms": heavy["paper"], "blocked_ms": heavy["blocked"],
+                          "fp32_frac": 8 * it4096 / (heavy["paper"] * 1e-3) / peak_ops,
+                          "blocked_fp32_frac": 8 * it4096 / (heavy["blocked"] * 1e-3) / peak_ops}
     vin.destroy()
     out.destroy()
     return res
@@ -620,10 +656,40 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         ms_graph = ms
     roof = lmosem_roofline(ctx, skel, rec, evv, timed, world)
     evv.destroy()
+    # configs[4]: the full reconstruction -- 10 subsets of 10^6 events (10^7,
+    # P:L603-605), each subset a different synthetic draw, all events staged on
+    # the devices beforehand (240 MB); one pass over the subsets from f0 = 1
+    nsub = 10
+    subs = []
+    for l in range(nsub):
+        evl = si.lmosem_events(nev, subset=l)
+        v = ctx.vector(n=nev, dtype=evl.dtype)
+        if world > 1:
+            v.set_distribution(skel.BLOCK)
+        v.upload_part(lo, evl[lo:hi])
+        subs.append(v)
+    rec2 = LMOSEM(ctx)
+    for v in subs:  # stage every subset (lazy H2D) and warm up
+        rec2.subset(v)
+    ctx.sync()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    barrier()
+    torch.cuda.synchronize()
+    e0.record(stream)
+    rec2.f.fill_dist(skel.BLOCK, np.float32(1))
+    for v in subs:
+        rec2.subset(v)
+    e1.record(stream)
+    ctx.sync()
+    ms_full = max_over_ranks(e0.elapsed_time(e1))
+    for v in subs:
+        v.destroy()
     return {"config": "configs[3]/[4]: one subset, 10^6 events, 150x150x280, events block over GPUs",
             "subset_s": ms * 1e-3, "subset_s_graph": ms_graph * 1e-3, "subset_s_fused": ms_fused * 1e-3,
             "roofline": roof,
             "events_per_s": nev / (min(ms_graph, ms_fused) * 1e-3),
+            "full_recon_s": ms_full * 1e-3, "full_recon": "10 subsets x 10^6 events (configs[4]), f0 = 1, "
+                                                          "events resident on the devices",
             "note": "includes f all-gather, c zero-fill, Siddon Map, c reduce-scatter and update Zip; "
                     "subset_s = eager calls, subset_s_graph = the same subset replayed as a CUDA graph, "
                     "subset_s_fused = the tail as one peer-memory kernel (skel_zip_combine, NEXT-1)"}

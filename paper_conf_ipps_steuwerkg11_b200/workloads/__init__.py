@@ -13,6 +13,7 @@ def source(name: str) -> str:
 
 MANDELBROT = source("mandelbrot")
 MANDELBROT_INDEX = source("mandelbrot_index")  # index Map variant (NEXT-4)
+MANDELBROT_BLOCKED = source("mandelbrot_blocked")  # loop control per block of updates (NEXT-4)
 LMOSEM_ERROR = source("lmosem_error")
 LMOSEM_UPDATE = source("lmosem_update")
 # voxel visits of one event's path (measurement only: the LM OSEM roofline

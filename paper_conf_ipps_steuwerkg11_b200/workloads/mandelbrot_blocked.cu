@@ -1,0 +1,45 @@
+// Mandelbrot customizing function, blocked form: the
+// same iteration as mandelbrot.cu (eq. (5); reading R4) with the
+// loop control paid once per block of MANDEL_B updates instead of per update.
+// Inside a block every update still evaluates the paper's escape test
+// x*x + y*y <= 4 on the current z, but only ORs it into a flag; a block in
+// which z escaped is rolled back to its start and replayed one update at a
+// time by the plain loop.  Every update that counts is therefore computed by
+// exactly the operations of mandelbrot.cu in the same order (FMA contraction
+// off), so the counts are bit-identical -- tested against the oracle and the
+// golden image CRCs.  What changes is the instruction mix: per update 8 FP32
+// operations + 1 compare instead of + 1 compare, 1 counter add, 1 counter
+// compare and 1 branch.
+#ifndef MANDEL_B
+#define MANDEL_B 8
+#endif
+struct Pos { float re, im; };
+int mandelbrot_blocked(Pos c, int cap) {
+    float x = 0.0f, y = 0.0f;
+    int n = 0;
+    while (n + MANDEL_B <= cap) {
+        const float x0 = x, y0 = y;
+        bool out = false;
+#pragma unroll
+        for (int k = 0; k < MANDEL_B; ++k) {
+            const float xx = x * x, yy = y * y;
+            out = out | !(xx + yy <= 4.0f);
+            const float xt = (xx - yy) + c.re;
+            y = (2.0f * x) * y + c.im;
+            x = xt;
+        }
+        if (out) {  // escaped inside this block: replay it update by update
+            x = x0;
+            y = y0;
+            break;
+        }
+        n += MANDEL_B;
+    }
+    while (n < cap && x * x + y * y <= 4.0f) {
+        float xt = (x * x - y * y) + c.re;
+        y = (2.0f * x) * y + c.im;
+        x = xt;
+        ++n;
+    }
+    return n;
+}

@@ -16,12 +16,12 @@ from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT
 pytestmark = pytest.mark.gpu
 
 
-def run(ctx, pos, cap, dist=None):
+def run(ctx, pos, cap, dist=None, fn=MANDELBROT):
     vin = ctx.vector(pos)
     if dist is not None:
         vin.set_distribution(dist)
     out = ctx.vector(n=pos.size, dtype=np.int32)
-    ctx.map(MANDELBROT, vin, out, args=[np.int32(cap)])
+    ctx.map(fn, vin, out, args=[np.int32(cap)])
     return out.download()
 
 
@@ -70,3 +70,22 @@ def test_index_map_variant_matches_the_golden_image(golden_dir, w, h, cap, D):
     with open(os.path.join(golden_dir, "mandelbrot.json")) as fh:
         case = [c for c in json.load(fh)["cases"] if (c["width"], c["height"], c["cap"]) == (w, h, cap)][0]
     assert zlib.crc32(got.tobytes()) == int(case["crc32"], 16)
+
+
+@pytest.mark.parametrize("w,h,cap,D", [(1024, 768, 256, 1), (4096, 3072, 256, 1), (1024, 768, 4096, 1),
+                                       (1024, 768, 256, 4), (257, 3, 9, 1)])
+def test_blocked_variant_bit_exact(golden_dir, w, h, cap, D):
+    """NEXT-4: the blocked user function (loop control per 8 updates, roll back
+    on escape) gives the same counts as eq. (5) as written: golden CRCs and the
+    oracle, on one device and block-distributed rows; a ragged 257x3 image with
+    a cap that is not a multiple of the block."""
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_BLOCKED
+    pos = si.mandelbrot_positions(w, h)
+    with skel.Context(D) as ctx:
+        got = run(ctx, pos, cap, skel.BLOCK if D > 1 else None, fn=MANDELBROT_BLOCKED)
+    cases = json.load(open(os.path.join(golden_dir, "mandelbrot.json")))["cases"]
+    case = [c for c in cases if (c["width"], c["height"], c["cap"]) == (w, h, cap)]
+    if case:
+        assert zlib.crc32(got.tobytes()) == int(case[0]["crc32"], 16)
+    if w * h <= 1 << 20:
+        assert np.array_equal(got, oracle.mandelbrot(pos, cap))

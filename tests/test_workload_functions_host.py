@@ -73,3 +73,49 @@ def test_paper_volume_no_flips(walk):
     want, _ = oracle.lmosem_error_image(ev, np.ones(int(np.prod(dims))), dims)
     assert np.array_equal(c > 0, want > 0)
     assert np.linalg.norm(c - want) <= 1e-6 * np.linalg.norm(want)
+
+
+MANDEL_SHIM = r'''
+#include "SRC"
+extern "C" void run(const float* pos, long n, int cap, int* out) {
+    for (long i = 0; i < n; ++i) out[i] = mandelbrot_blocked(Pos{pos[2*i], pos[2*i+1]}, cap);
+}
+'''
+
+
+@pytest.fixture(scope="module")
+def mandel_blocked(tmp_path_factory):
+    d = tmp_path_factory.mktemp("mandel")
+    src = d / "shim.cpp"
+    src.write_text(MANDEL_SHIM.replace(
+        "SRC", str(ROOT / "paper_conf_ipps_steuwerkg11_b200" / "workloads" / "mandelbrot_blocked.cu")))
+    so = d / "mandel.so"
+    subprocess.run(["g++", "-O2", "-std=c++17", "-ffp-contract=off", "-shared", "-fPIC", str(src), "-o", str(so)],
+                   check=True)
+    lib = ctypes.CDLL(str(so))
+    lib.run.argtypes = [ctypes.c_void_p, ctypes.c_long, ctypes.c_int, ctypes.c_void_p]
+
+    def run(pos, cap):
+        pos = np.ascontiguousarray(pos)
+        out = np.zeros(pos.size, np.int32)
+        lib.run(pos.ctypes.data, pos.size, cap, out.ctypes.data)
+        return out
+    return run
+
+
+@pytest.mark.parametrize("cap", [1, 7, 8, 9, 256])
+def test_blocked_mandelbrot_equals_the_plain_iteration(mandel_blocked, golden_dir, cap):
+    """mandelbrot_blocked.cu (loop control per block of 8 updates, roll back on
+    escape) counts exactly what eq. (5) as written counts: bit-identical to
+    the oracle on the whole 1024x768 image, for caps below, at and above the
+    block size, and to the golden CRC at cap 256."""
+    import json
+    import os
+    import zlib
+    pos = si.mandelbrot_positions(1024, 768)
+    got = mandel_blocked(pos, cap)
+    assert np.array_equal(got, oracle.mandelbrot(pos, cap))
+    if cap == 256:
+        with open(os.path.join(golden_dir, "mandelbrot.json")) as fh:
+            case = [c for c in json.load(fh)["cases"] if (c["width"], c["height"], c["cap"]) == (1024, 768, 256)][0]
+        assert zlib.crc32(got.tobytes()) == int(case["crc32"], 16)
