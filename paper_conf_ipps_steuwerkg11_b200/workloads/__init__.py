@@ -22,42 +22,30 @@ LMOSEM_VISITS = LMOSEM_ERROR + """
 int lmosem_visits(Event e, int nx, int ny, int nz) {
     Walk w;
     if (!walk_init(e, nx, ny, nz, w)) return 0;
-    double an0 = w.an[0], an1 = w.an[1], an2 = w.an[2], ac = w.amin;
-    const double aend = w.amax - 1.0e-12;
-    int n = 0;
-    for (int it = 0; it < w.n_steps && ac < aend; ++it) {
-        const double a1 = dmin(dmin(dmin(an0, an1), an2), w.amax);
-        an0 = an0 == a1 ? an0 + w.da[0] : an0;
-        an1 = an1 == a1 ? an1 + w.da[1] : an1;
-        an2 = an2 == a1 ? an2 + w.da[2] : an2;
-        ac = a1;
-        ++n;
-    }
-    return n;
+    return w.n_cross + 1;  // one segment per crossing, then the last one
 }
 """
 # 4-float groups the back projection reduces into (one red.global.add.v4.f32 each)
 LMOSEM_GROUPS = LMOSEM_ERROR + """
+static __forceinline__ void count_group(int v, float len, unsigned nvox, int &g, int &n) {
+    if (len > 0.0f && (unsigned)v < nvox && (v >> 2) != g) {
+        g = v >> 2;
+        ++n;
+    }
+}
 int lmosem_groups(Event e, int nx, int ny, int nz) {
     Walk w;
     if (!walk_init(e, nx, ny, nz, w)) return 0;
-    double an0 = w.an[0], an1 = w.an[1], an2 = w.an[2], ac = w.amin;
-    const double aend = w.amax - 1.0e-12;
-    int v = w.v, g = -1, n = 0;
-    for (int it = 0; it < w.n_steps && ac < aend; ++it) {
-        const double a1 = dmin(dmin(dmin(an0, an1), an2), w.amax);
-        const float len = (float)((a1 - ac) * w.len_scale);
-        if (len > 0.0f && (unsigned)v < w.nvox && (v >> 2) != g) {
-            g = v >> 2;
-            ++n;
-        }
-        const bool cx = an0 == a1, cy = an1 == a1, cz = an2 == a1;
-        v += (cx ? w.dv[0] : 0) + (cy ? w.dv[1] : 0) + (cz ? w.dv[2] : 0);
-        an0 = cx ? an0 + w.da[0] : an0;
-        an1 = cy ? an1 + w.da[1] : an1;
-        an2 = cz ? an2 + w.da[2] : an2;
-        ac = a1;
+    Cursor cur;
+    cursor_init(w, cur);
+    int g = -1, n = 0;
+    for (int it = 0; it < w.n_cross; ++it) {
+        int vs;
+        const double a1 = cross_step(w, cur, vs, true);
+        count_group(vs, (float)((a1 - cur.ac) * w.len_scale), w.nvox, g, n);
+        cur.ac = a1;
     }
+    count_group(cur.v, (float)((w.amax - cur.ac) * w.len_scale), w.nvox, g, n);
     return n;
 }
 """

@@ -12,6 +12,9 @@ import skel_inputs as si
 from paper_conf_ipps_steuwerkg11_b200 import skel
 from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_ERROR
 
+if os.environ.get("LM_SRC"):  # A/B: an alternative error-image function text
+    LMOSEM_ERROR = open(os.environ["LM_SRC"]).read()
+
 ev = si.lmosem_events(1_000_000, subset=0)
 with skel.Context(1) as ctx:
     stream = torch.cuda.ExternalStream(ctx.stream(0))
