@@ -654,6 +654,27 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         g.destroy()
     except skel.SkelError:  # a collective backend that cannot be captured
         ms_graph = ms
+    coll = None
+    if world > 1:  # the exchange steps alone, bus GB/s vs NVLink
+        S = rec.nvox * 4
+        c, f = rec.c, rec.f
+
+        def fill_rs():
+            c.fill_dist(skel.COPY, np.float32(0))
+            c.set_distribution(skel.BLOCK, skel.COMBINE_ADD)  # copy -> block + add: reduce-scatter
+
+        def ag():
+            f.set_distribution(skel.BLOCK)  # copy -> block: local slice (no data movement)
+            f.set_distribution(skel.COPY)   # block -> copy: all-gather
+        ms_fill = timed(lambda: c.fill_dist(skel.COPY, np.float32(0)))
+        ms_rs = max(timed(fill_rs) - ms_fill, 1e-6)
+        ms_ag = timed(ag)
+        busf = (world - 1) / world
+        coll = {"bytes": S, "reduce_scatter_ms": ms_rs, "all_gather_ms": ms_ag,
+                "reduce_scatter_busbw_GBps": S * busf / (ms_rs * 1e-3) / 1e9,
+                "all_gather_busbw_GBps": S * busf / (ms_ag * 1e-3) / 1e9,
+                "peak_GBps": 770.0, "peak_source": "B200_PROFILING.md measured peer copy per direction "
+                                                  "(900 nominal)"}
     roof = lmosem_roofline(ctx, skel, rec, evv, timed, world)
     evv.destroy()
     # configs[4]: the full reconstruction -- 10 subsets of 10^6 events (10^7,
@@ -686,7 +707,7 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         v.destroy()
     return {"config": "configs[3]/[4]: one subset, 10^6 events, 150x150x280, events block over GPUs",
             "subset_s": ms * 1e-3, "subset_s_graph": ms_graph * 1e-3, "subset_s_fused": ms_fused * 1e-3,
-            "roofline": roof,
+            "roofline": roof, "exchange": coll,
             "events_per_s": nev / (min(ms_graph, ms_fused) * 1e-3),
             "full_recon_s": ms_full * 1e-3, "full_recon": "10 subsets x 10^6 events (configs[4]), f0 = 1, "
                                                           "events resident on the devices",

@@ -90,6 +90,16 @@ constexpr skel_sig_t skel_make_sig() {
 }
 extern "C" __device__ skel_sig_t skel_sig = skel_make_sig();
 
+// Minimum resident CTAs per SM the element-wise kernels are compiled for (a
+// register cap of 65536 / (SKEL_BLOCK * SKEL_MINB) per thread).  A user
+// function may set it by defining SKEL_MINB in its text (the text precedes
+// this template), e.g. a latency-bound function that wants more warps.
+#ifdef SKEL_MINB
+#define SKEL_EW_BOUNDS __launch_bounds__(SKEL_BLOCK, SKEL_MINB)
+#else
+#define SKEL_EW_BOUNDS __launch_bounds__(SKEL_BLOCK)
+#endif
+
 // ---- streaming loads / stores of one chunk ---------------------------------
 #ifndef SKEL_LD_HINT
 #define SKEL_LD_HINT ".nc.L1::no_allocate"
@@ -189,6 +199,7 @@ __device__ __forceinline__ skel_u64 skel_idx_chunks(skel_O *out, skel_u64 n, ske
     using I = skel::decay_t<skel_A>;
     if constexpr (SKEL_E > 1 && !V) {
         const skel_u64 nch = n / SKEL_E;
+#pragma unroll 1
         for (skel_u64 c = tid; c < nch; c += stride) {
             skel::arr<skel_O, SKEL_E> yo;
 #pragma unroll
@@ -209,16 +220,17 @@ __device__ __forceinline__ void skel_idx_one(skel_O *out, skel_u64 i, skel_u64 b
         out[i] = skel::caller<skel_Seq>::call(&SKEL_FN, t, (I)(base + i));
     }
 }
-extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
+extern "C" __global__ void SKEL_EW_BOUNDS
     skel_ew_kernel(skel_O *__restrict__ out, skel_u64 n, skel_u64 base, int vec_ok, const skel_Buf args) {
     auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
     const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;
     const skel_u64 done = vec_ok ? skel_idx_chunks(out, n, base, tid, stride, t) : 0;
+#pragma unroll 1
     for (skel_u64 i = done + tid; i < n; i += stride) skel_idx_one(out, i, base, t);
 }
 #else
-extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
+extern "C" __global__ void SKEL_EW_BOUNDS
     skel_ew_kernel(const skel_A *__restrict__ a, const skel_B *__restrict__ b, skel_O *__restrict__ out, skel_u64 n,
                    int vec_ok, const skel_Buf args) {
     auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
@@ -233,6 +245,20 @@ extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
         const char *pb = reinterpret_cast<const char *>(b);
         char *po = reinterpret_cast<char *>(out);
         skel_u64 c = tid;
+        // `unroll 1` on the grid-stride loops: unrolling them makes the compiler
+        // compute trip counts with a 64-bit division before the first load
+        // -- measured better for Map at every size; a Zip streams more bytes per
+        // chunk and gains from the compiler's 2x unroll above 2^24 (1.92 -> 1.87 ms
+        // at 2^30) more than the prologue costs it (tools/ew_unroll_variants.sh).
+        // SKEL_MAIN_UNROLL: the main loop's pragma (tuning hook).
+#ifndef SKEL_MAIN_UNROLL
+#if SKEL_NIN == 2
+#define SKEL_MAIN_UNROLL
+#else
+#define SKEL_MAIN_UNROLL _Pragma("unroll 1")
+#endif
+#endif
+        SKEL_MAIN_UNROLL
         for (; c + (SKEL_UNROLL - 1) * stride < nch; c += SKEL_UNROLL * stride) {
             skel::chunk<skel_CA> ca[SKEL_UNROLL];
             skel::chunk<skel_CB> cb[SKEL_UNROLL];
@@ -246,6 +272,7 @@ extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
                 skel_chunk_op(ca[u], cb[u], po + (c + u * stride) * skel_CO, t);
             }
         }
+#pragma unroll 1
         for (; c < nch; c += stride) {
             skel::chunk<skel_CA> ca = skel_ld<skel_CA>(pa + c * skel_CA);
             skel::chunk<skel_CB> cb;
@@ -254,6 +281,7 @@ extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
         }
     }
     // scalar path: the tail, or everything for non-vectorisable element types
+#pragma unroll 1
     for (skel_u64 i = done + tid; i < n; i += stride) skel_one(a, b, out, i, t);
 }
 #endif  // SKEL_NIN == 0
@@ -295,7 +323,7 @@ __device__ __forceinline__ void skel_zipcomb_elem(const skel_A &xa, const skel_p
     }
 }
 
-extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
+extern "C" __global__ void SKEL_EW_BOUNDS
     skel_zipcomb_kernel(const skel_A *__restrict__ a, const skel_ptrs bsrc, int nsrc, skel_B *bown,
                         const skel_ptrs odst, int ndst, skel_u64 n, int op, int vec_ok, const skel_Buf args) {
     auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
@@ -306,6 +334,7 @@ extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
         if (vec_ok) {
             const skel_u64 nch = n / SKEL_E;
             done = nch * SKEL_E;
+#pragma unroll 1
             for (skel_u64 c = tid; c < nch; c += stride) {
                 const auto xa = skel::bit_cast<skel::arr<skel_A, SKEL_E>>(
                     skel_ld<skel_CA>(reinterpret_cast<const char *>(a) + c * skel_CA));
@@ -325,6 +354,7 @@ extern "C" __global__ void __launch_bounds__(SKEL_BLOCK)
             }
         }
     }
+#pragma unroll 1
     for (skel_u64 i = done + tid; i < n; i += stride) skel_zipcomb_elem(a[i], bsrc, nsrc, bown, odst, ndst, i, op, t);
 }
 #endif

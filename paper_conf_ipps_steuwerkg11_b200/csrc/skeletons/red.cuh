@@ -305,6 +305,12 @@ extern __shared__ __align__(16) unsigned char skel_dsmem[];
 #define SKEL_RED_MINB 1
 #endif
 #endif
+// a / b in 32-bit arithmetic when both fit (the 64-bit division is a
+// subroutine call of ~100 instructions ahead of the first load)
+__device__ __forceinline__ skel_u64 udiv(skel_u64 a, skel_u64 b) {
+    if (((a | b) >> 32) == 0) return (unsigned)a / (unsigned)b;
+    return a / b;
+}
 // ordered warp fold of 32 valid values: lane 0 receives x_0 (+) ... (+) x_31
 template <class Tup> __device__ __forceinline__ skel_T warp_fold_full(skel_T x, int lane, Tup &t) {
 #pragma unroll
@@ -353,7 +359,7 @@ __device__ __forceinline__ VT reduce_direct(const skel_T *__restrict__ in, skel_
     const skel_u64 per_chunk = (TMA_OK && vec) ? 32ull * PERV : 32ull;
     const skel_u64 nch = n / per_chunk;
     const skel_u64 NWT = G * NW, gw = c * NW + w;
-    const skel_u64 k0 = nch * gw / NWT, k1 = nch * (gw + 1) / NWT;
+    const skel_u64 k0 = udiv(nch * gw, NWT), k1 = udiv(nch * (gw + 1), NWT);
     VT wrun;
     wrun.ok = false;
     skel_u64 k = k0;
@@ -427,7 +433,7 @@ extern "C" __global__ void __launch_bounds__(RB, SKEL_RED_MINB)
     const int t = threadIdx.x;
     const skel_u64 nft = n / TILE;
     const skel_u64 G = gridDim.x, c = blockIdx.x;
-    const skel_u64 t0 = nft * c / G, t1 = nft * (c + 1) / G;
+    const skel_u64 t0 = udiv(nft * c, G), t1 = udiv(nft * (c + 1), G);
     const skel_u64 my = RIL ? (nft > c ? (nft - c + G - 1) / G : 0) : t1 - t0;
     auto tile_at = [&](skel_u64 i) -> skel_u64 { return RIL ? c + i * G : t0 + i; };
     VT run;
@@ -845,7 +851,7 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
     const skel_u64 G = gridDim.x, c = blockIdx.x;
     const skel_u64 nft = n / STILE;  // full tiles
     const skel_u64 per_slice = G * SCAN_CH;
-    const skel_u64 nslices = (nft + per_slice - 1) / per_slice;
+    const skel_u64 nslices = udiv(nft + per_slice - 1, per_slice);
     const skel_u64 rstride = (nslices * G + 63) / 64 * 64;  // status words per copy
     const bool tma = TMA_OK && use_tma;
     unsigned char *stages = aligned_stages(skel_dsmem);

@@ -17,7 +17,7 @@ import numpy as np  # noqa: E402
 import torch  # noqa: E402
 
 from paper_conf_ipps_steuwerkg11_b200 import skel  # noqa: E402
-from paper_conf_ipps_steuwerkg11_b200.workloads import MAP_F32, SUM_F32  # noqa: E402
+from paper_conf_ipps_steuwerkg11_b200.workloads import MAP_F32, SAXPY_F32, SUM_F32  # noqa: E402
 
 
 def main():
@@ -25,6 +25,7 @@ def main():
     hw = ctypes.CDLL(os.path.join(ROOT, "paper_conf_ipps_steuwerkg11_b200", "libhandwritten.so"))
     P, S = ctypes.c_void_p, ctypes.c_size_t
     hw.hw_map_f32.argtypes = [P, P, S, P]
+    hw.hw_saxpy_f32.argtypes = [P, P, P, ctypes.c_float, S, P]
     hw.hw_sum_f32.argtypes = [P, S, P, P]
     hw.hw_cubsum_f32.argtypes = [P, S, P, P]
     hw.hw_exscan_f32.argtypes = [P, P, S, P]
@@ -45,6 +46,8 @@ def main():
                 sets.append((x, o, r, x.device_ptr()[0], o.device_ptr()[0], r.device_ptr()[0]))
             ops = {
                 "map_skel": lambda st: ctx.map(MAP_F32, st[0], st[1]),
+                "zip_skel": lambda st: ctx.zip(SAXPY_F32, st[0], st[1], st[1], args=[np.float32(2.5)]),
+                "zip_hw": lambda st: hw.hw_saxpy_f32(st[3], st[4], st[4], 2.5, n, sp),
                 "map_hw": lambda st: hw.hw_map_f32(st[3], st[4], n, sp),
                 "reduce_skel": lambda st: ctx.reduce_to(SUM_F32, st[0], st[2]),
                 "reduce_cub": lambda st: hw.hw_cubsum_f32(st[3], n, st[5], sp),
