@@ -261,6 +261,7 @@ __device__ __forceinline__ void st_relaxed_u32(unsigned *p, unsigned v) {
     asm volatile("st.relaxed.gpu.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
 }
 // element values published through the flags: word-wise relaxed accesses
+__device__ __forceinline__ void fence_acq_rel_gpu() { asm volatile("fence.acq_rel.gpu;" ::: "memory"); }
 template <class T> __device__ __forceinline__ void st_value(T *p, const T &v) {
     constexpr int W = (int)((sizeof(T) + 3) / 4);
     union U { T t; unsigned w[W]; U() {} } a;

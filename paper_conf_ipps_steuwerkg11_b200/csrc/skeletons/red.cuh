@@ -514,13 +514,18 @@ extern "C" __global__ void __launch_bounds__(RB, SKEL_RED_MINB)
             skel::st_value(&partials[c], skel_S{run.v});
             skel::st_relaxed_u32(&pvalid[c], run.ok ? 1u : 0u);
         }
-        __threadfence();
+        // message passing through the counter: release fence before the
+        // increment, acquire fence in the CTA that sees the last count (an
+        // acq_rel fence, not the sequentially consistent __threadfence); the
+        // barrier then orders the other threads' loads after it
+        skel::fence_acq_rel_gpu();
         const unsigned prev = atomicAdd(counter, 1u);
-        s_last = (prev == (unsigned)(G - 1));
+        const bool last = prev == (unsigned)(G - 1);
+        if (last) skel::fence_acq_rel_gpu();
+        s_last = last;
     }
     __syncthreads();
     if (s_last) {
-        __threadfence();
         const skel_u64 per = (NP + RB - 1) / RB;
         VT a;
         a.ok = false;
