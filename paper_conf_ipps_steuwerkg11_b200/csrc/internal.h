@@ -43,11 +43,14 @@ struct Module {
     std::set<int> attr_set_on;  // devices on which smem attributes were set
     // element-wise grid policy per size class (log2 of the chunk count), chosen
     // by measurement: 0 = UNROLL chunks in flight per thread (bandwidth-bound
-    // user functions), 1 = one chunk per thread (compute-bound, divergent ones)
+    // user functions), 1 = one chunk per thread, 2 = one element per thread
+    // through the scalar path (compute-bound, divergent ones: finer work items
+    // even out the lanes of a warp)
+    static constexpr int kPolicies = 3, kRounds = 2;
     struct EwTune {
-        int trial = 0;   // launches timed so far (policies alternate 0,1,0,1)
+        int trial = 0;   // launches timed so far (policies in turn: 0,1,2,0,1,2)
         int best = -1;   // decided policy, -1 while measuring
-        cudaEvent_t ev[8] = {};
+        cudaEvent_t ev[2 * kPolicies * kRounds] = {};
     };
     std::map<int, EwTune> ew_tune;
     int red_occ = 0;  // resident Reduce CTAs per SM (0 = not yet queried)

@@ -370,8 +370,9 @@ def test_double_reduce_scan(ctx, n):
 @pytest.mark.parametrize("n", [(1 << 22) + 5, 1 << 24])
 def test_map_zip_grid_policy_trials_bit_identical(n):
     """The element-wise grid policy is chosen per module and size class by timing
-    both candidates on the first launches (K1/K2): every launch --
-    trials of either policy and the decided one -- must give the same bits."""
+    the three candidates on the first launches (K1/K2): every
+    launch -- trials of each policy (incl. the scalar one-element-per-thread
+    path) and the decided one -- must give the same bits."""
     with skel.Context(1) as c:
         x, y = si.uniform_f32(n, 11), si.uniform_f32(n, 12)
         vx, vy = c.vector(x), c.vector(y)

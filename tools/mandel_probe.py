@@ -16,7 +16,7 @@ with skel.Context(1) as ctx:
         outs = {}
         for name, fn in (("paper", MANDELBROT), ("blocked", MANDELBROT_BLOCKED)):
             out = ctx.vector(n=pos.size, dtype=np.int32)
-            for _ in range(3):
+            for _ in range(7):  # grid-policy trials (6) + one decided launch
                 ctx.map(fn, vin, out, args=[np.int32(cap)])
             ctx.sync()
             e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
