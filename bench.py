@@ -649,6 +649,20 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         return max_over_ranks(e0.elapsed_time(e1) / reps)
 
     ms = timed(lambda: rec.subset(evv))
+    # the same subset with its events ordered longest path first (host
+    # preprocessing per subset, lmosem.order_by_path; each rank orders its part)
+    from paper_conf_ipps_steuwerkg11_b200.lmosem import order_by_path
+    t0 = time.perf_counter()
+    ev_ord = order_by_path(ev[lo:hi])
+    order_host_s = time.perf_counter() - t0
+    evo = ctx.vector(n=nev, dtype=ev.dtype)
+    if world > 1:
+        evo.set_distribution(skel.BLOCK)
+    evo.upload_part(lo, ev_ord)
+    for _ in range(TUNE):
+        rec.subset(evo)
+    ms_ord = timed(lambda: rec.subset(evo))
+    evo.destroy()
     for _ in range(TUNE):
         rec.subset(evv, fused=True)
     ms_fused = timed(lambda: rec.subset(evv, fused=True))
@@ -687,36 +701,46 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
     # P:L603-605), each subset a different synthetic draw, all events staged on
     # the devices beforehand (240 MB); one pass over the subsets from f0 = 1
     nsub = 10
-    subs = []
-    for l in range(nsub):
-        evl = si.lmosem_events(nev, subset=l)
-        v = ctx.vector(n=nev, dtype=evl.dtype)
-        if world > 1:
-            v.set_distribution(skel.BLOCK)
-        v.upload_part(lo, evl[lo:hi])
-        subs.append(v)
-    rec2 = LMOSEM(ctx)
-    for v in subs:  # stage every subset (lazy H2D) and warm up
-        rec2.subset(v)
-    ctx.sync()
-    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-    barrier()
-    torch.cuda.synchronize()
-    e0.record(stream)
-    rec2.f.fill_dist(skel.BLOCK, np.float32(1))
-    for v in subs:
-        rec2.subset(v)
-    e1.record(stream)
-    ctx.sync()
-    ms_full = max_over_ranks(e0.elapsed_time(e1))
-    for v in subs:
-        v.destroy()
+    full = {}
+    for mode in ("given", "ordered"):
+        subs = []
+        for l in range(nsub):
+            evl = si.lmosem_events(nev, subset=l)[lo:hi]
+            if mode == "ordered":
+                evl = order_by_path(evl)
+            v = ctx.vector(n=nev, dtype=evl.dtype)
+            if world > 1:
+                v.set_distribution(skel.BLOCK)
+            v.upload_part(lo, evl)
+            subs.append(v)
+        rec2 = LMOSEM(ctx)
+        for v in subs:  # stage every subset (lazy H2D) and warm up
+            rec2.subset(v)
+        ctx.sync()
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        barrier()
+        torch.cuda.synchronize()
+        e0.record(stream)
+        rec2.f.fill_dist(skel.BLOCK, np.float32(1))
+        for v in subs:
+            rec2.subset(v)
+        e1.record(stream)
+        ctx.sync()
+        full[mode] = max_over_ranks(e0.elapsed_time(e1))
+        for v in subs:
+            v.destroy()
+    ms_full = full["given"]
     return {"config": "configs[3]/[4]: one subset, 10^6 events, 150x150x280, events block over GPUs",
             "subset_s": ms * 1e-3, "subset_s_graph": ms_graph * 1e-3, "subset_s_fused": ms_fused * 1e-3,
             "roofline": roof, "exchange": coll,
             "events_per_s": nev / (min(ms_graph, ms_fused) * 1e-3),
             "full_recon_s": ms_full * 1e-3, "full_recon": "10 subsets x 10^6 events (configs[4]), f0 = 1, "
                                                           "events resident on the devices",
+            "ordered": {"subset_s": ms_ord * 1e-3, "full_recon_s": full["ordered"] * 1e-3,
+                        "order_host_s_per_subset": order_host_s,
+                        "note": "events of each subset ordered longest path first on the host before upload "
+                                "(lmosem.order_by_path: list-mode events carry no order; same image up to "
+                                "float rounding)"},
             "note": "includes f all-gather, c zero-fill, Siddon Map, c reduce-scatter and update Zip; "
                     "subset_s = eager calls, subset_s_graph = the same subset replayed as a CUDA graph, "
                     "subset_s_fused = the tail as one peer-memory kernel (skel_zip_combine, NEXT-1)"}

@@ -17,6 +17,31 @@ from .workloads import LMOSEM_ERROR, LMOSEM_UPDATE
 DIMS = (150, 150, 280)
 
 
+def order_by_path(ev: np.ndarray, dims=DIMS) -> np.ndarray:
+    """The events of a subset reordered longest path first (host preprocessing,
+    like reading the subset from file).  List-mode events carry no
+    order, and the error image is a sum over them, so any order gives the same
+    image up to float rounding (R10(x)).  With similar path lengths next to each
+    other, the 32 rays of a warp finish together (thread efficiency) and the
+    longest rays start first (shorter launch tail): DESIGN.md §4.2.
+    Key: the L1 length |dx|+|dy|+|dz| of the segment clipped to the volume
+    (slab clipping, float64) -- proportional to the voxel steps of the walk."""
+    p = np.stack([ev["x1"], ev["y1"], ev["z1"]]).astype(np.float64)
+    d = np.stack([ev["x2"], ev["y2"], ev["z2"]]).astype(np.float64) - p
+    amin = np.zeros(len(ev))
+    amax = np.ones(len(ev))
+    for a, n in enumerate(dims):
+        nz = d[a] != 0
+        with np.errstate(divide="ignore", invalid="ignore"):
+            a0 = np.where(nz, (0.0 - p[a]) / d[a], -np.inf)
+            a1 = np.where(nz, (float(n) - p[a]) / d[a], np.inf)
+        inside = (p[a] >= 0) & (p[a] < n)
+        amin = np.maximum(amin, np.where(nz, np.minimum(a0, a1), np.where(inside, -np.inf, np.inf)))
+        amax = np.minimum(amax, np.where(nz, np.maximum(a0, a1), np.inf))
+    key = np.where(amax > amin, (amax - amin) * np.abs(d).sum(axis=0), 0.0)
+    return ev[np.argsort(-key, kind="stable")]
+
+
 class LMOSEM:
     def __init__(self, ctx: skel.Context, dims=DIMS, f0: float = 1.0):
         self.ctx = ctx

@@ -106,3 +106,19 @@ def test_full_size_subset_matches_oracle():
     want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
     assert rel_l2(f, want) <= 1e-4
     assert abs(float(f[c > 0].astype(np.float64).sum()) - nv) <= 1e-4 * nv
+
+
+@pytest.mark.parametrize("n,D", [(1_000_000, 1), (40_000, 4)])
+def test_path_ordered_events_match_oracle_in_given_order(n, D):
+    """The events reordered longest path first (lmosem.order_by_path, host
+    preprocessing) give the oracle's image for the events in
+    their given order: the error image is a sum over events (R10(x))."""
+    from paper_conf_ipps_steuwerkg11_b200.lmosem import order_by_path
+    events = si.lmosem_events(n, subset=3)
+    with skel.Context(D) as ctx:
+        rec = LMOSEM(ctx)
+        rec.subset(rec.events(order_by_path(events)))
+        f = rec.image()
+    want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
+    assert rel_l2(f, want) <= 1e-4
+    assert abs(float(f[c > 0].astype(np.float64).sum()) - nv) <= 1e-4 * nv

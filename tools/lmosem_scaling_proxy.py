@@ -22,7 +22,11 @@ with skel.Context(1) as ctx:
     c = ctx.vector(n=150 * 150 * 280, dtype=np.float32)
     dims = [np.int32(150), np.int32(150), np.int32(280)]
     for D in (1, 2, 4, 8):
-        e = ctx.vector(ev[: 1_000_000 // D])
+        part = ev[: 1_000_000 // D]
+        if os.environ.get("LM_ORDER"):  # each GPU orders its part longest path first
+            from paper_conf_ipps_steuwerkg11_b200.lmosem import order_by_path
+            part = order_by_path(part)
+        e = ctx.vector(part)
         for _ in range(3):
             ctx.map(LMOSEM_ERROR, e, None, args=[f, c, *dims])
         ctx.sync()
