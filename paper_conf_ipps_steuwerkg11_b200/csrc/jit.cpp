@@ -351,7 +351,9 @@ int get_module_slow(skel_ctx_s *ctx, Kind kind, const char *src, Module **out) {
     };
     if (kind == Kind::Red) {
         if (!getk("skel_reduce_kernel", &m->k_main) || !getk("skel_scan_kernel", &m->k_scan) ||
-            !getk("skel_fold_kernel", &m->k_fold) || !getk("skel_seed_kernel", &m->k_seed))
+            !getk("skel_fold_kernel", &m->k_fold) || !getk("skel_seed_kernel", &m->k_seed) ||
+            !getk("skel_scan_agg_kernel", &m->k_scan_agg) || !getk("skel_scan_small_kernel", &m->k_scan_small) ||
+            !getk("skel_fold_aggs_kernel", &m->k_fold_aggs))
             return SKEL_ERR_CUDA;
     } else {
         if (!getk("skel_ew_kernel", &m->k_main)) return SKEL_ERR_CUDA;

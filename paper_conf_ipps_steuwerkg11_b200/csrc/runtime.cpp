@@ -1072,9 +1072,36 @@ size_t red_parts(Module *m, const Slot &s, uint64_t cnt) {
     return std::max<size_t>(G, (size_t)(cnt / m->sig[10]) + 1);
 }
 
+// small vectors: tile aggregates + a one-CTA ordered fold (two short launches)
+// up to SKEL_RED_SMALL_MAX elements (tuning hook; default 32 MiB of elements:
+// measured crossover with the TMA kernel between 2^23 and 2^24 floats)
+uint64_t red_small_tile(const Module *m) { return m->sig[9] * ((m->sig[15] >> 50) & 0xff); }
+bool red_small(const Module *m, uint64_t cnt) {
+    static const uint64_t env = [] {
+        const char *e = getenv("SKEL_RED_SMALL_MAX");
+        return e ? (uint64_t)strtoull(e, nullptr, 10) : ~0ull;
+    }();
+    const uint64_t mx = env != ~0ull ? env : (uint64_t)(32u << 20) / m->sig[3];
+    return m->k_fold_aggs && red_small_tile(m) > 0 && cnt <= mx;
+}
+
 // local reduce of the slot's data into dst
 int launch_reduce(skel_ctx_s *ctx, Module *m, Slot &s, const void *in, uint64_t cnt, const RedLayout &L,
                   std::vector<unsigned char> &abuf, void *dst) {
+    if (red_small(m, cnt)) {
+        const uint64_t ST = red_small_tile(m);
+        uint64_t nt = (cnt + ST - 1) / ST;
+        void *aggs = s.ws + L.total;  // room reserved by reduce_core
+        void *pa[] = {&in, &cnt, &aggs, abuf.data()};
+        DevGuard g(s.dev);
+        CK(ctx, cudaLaunchKernel((const void *)m->k_scan_agg, dim3((unsigned)nt), dim3((unsigned)m->sig[9]), pa, 0,
+                                 s.stream));
+        const void *caggs = aggs;
+        void *pf[] = {&caggs, &nt, &dst, abuf.data()};
+        CK(ctx, cudaLaunchKernel((const void *)m->k_fold_aggs, dim3(1), dim3((unsigned)m->sig[9]), pf, 0, s.stream));
+        ctx->stats.kernel_launches += 2;
+        return SKEL_OK;
+    }
     const uint64_t TILE = m->sig[10], RB = m->sig[9];
     const uint64_t nft = cnt / TILE;
     const size_t G = red_grid(m, s, cnt);
@@ -1107,7 +1134,8 @@ int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args
         const uint64_t cnt = in->bufs[li].count;
         TRY(set_smem_attr(ctx, m, s));  // before the occupancy query in red_grid
         Ls[li] = red_layout(m, D, red_parts(m, s, cnt), 0);
-        TRY(ensure_ws(ctx, s, Ls[li].total));
+        const size_t extra = red_small(m, cnt) ? (size_t)((cnt + red_small_tile(m) - 1) / red_small_tile(m)) * Ls[li].slot : 0;
+        TRY(ensure_ws(ctx, s, Ls[li].total + extra));
         pack_args(m, args, nargs, li, abuf);
         char *dst = cross ? s.ws + Ls[li].o_res : (direct && D == 1 ? static_cast<char *>(direct) : s.ws + Ls[li].o_fold);
         if (cnt) TRY(launch_reduce(ctx, m, s, in->bufs[li].ptr(in->es), cnt, Ls[li], abuf, dst));
@@ -1898,11 +1926,22 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         const uint64_t per_slice = scan_grid(s) * CH, nft = cnt / TILE;
         return std::max<uint64_t>(1, (nft + per_slice - 1) / per_slice) * scan_grid(s);
     };
+    // small vectors: two short launches (tile aggregates, seeded tile scans)
+    // instead of the persistent pipeline; SKEL_SCAN_SMALL_MAX
+    // (elements, a tuning hook) moves the switch point
+    static const uint64_t small_max_env = [] {
+        const char *e = getenv("SKEL_SCAN_SMALL_MAX");
+        return e ? (uint64_t)strtoull(e, nullptr, 10) : ~0ull;
+    }();
+    const uint64_t SM_TILE = m->sig[9] * ((m->sig[15] >> 50) & 0xff);  // reduce block x elements per thread
+    const uint64_t small_max = small_max_env != ~0ull ? small_max_env : (uint64_t)(4u << 20) * 4 / m->sig[3];
+    auto small_scan = [&](uint64_t cnt) { return m->k_scan_small && SM_TILE > 0 && cnt <= small_max; };
     for (size_t li = 0; li < ctx->slots.size(); ++li) {
         Slot &s = ctx->slots[li];
         const uint64_t cnt = in->bufs[li].count;
         Ls[li] = red_layout(m, D, red_parts(m, s, cnt), scan_slots(s, cnt));
-        TRY(ensure_ws(ctx, s, Ls[li].total));
+        const size_t extra = small_scan(cnt) ? (size_t)((cnt + SM_TILE - 1) / SM_TILE) * Ls[li].slot : 0;
+        TRY(ensure_ws(ctx, s, Ls[li].total + extra));
     }
     if (cross) {
         std::vector<RedLayout> Lr;
@@ -1933,6 +1972,18 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         }
         const void *pin = in->bufs[li].ptr(in->es);
         void *pout = out->bufs[li].ptr(out->es);
+        if (small_scan(cnt)) {
+            const unsigned nt = (unsigned)((cnt + SM_TILE - 1) / SM_TILE);
+            void *aggs = s.ws + L.total;
+            void *pa[] = {&pin, &cnt, &aggs, abuf.data()};
+            CK(ctx, cudaLaunchKernel((const void *)m->k_scan_agg, dim3(nt), dim3((unsigned)m->sig[9]), pa, 0, s.stream));
+            const void *caggs = aggs;
+            void *ps[] = {&pin, &pout, &cnt, &caggs, idbuf.data(), &seed, abuf.data()};
+            CK(ctx, cudaLaunchKernel((const void *)m->k_scan_small, dim3(nt), dim3((unsigned)m->sig[9]), ps, 0,
+                                     s.stream));
+            ctx->stats.kernel_launches += 2;
+            continue;
+        }
         CUtensorMap tin, tout;
         const uint64_t rows = (cnt / TILE) * SRB;
         int use_tma = m->sig[5] && make_tmap(&tin, pin, rows, (uint32_t)(SRB / 2)) &&

@@ -89,6 +89,9 @@ constexpr int PW = SKEL_SCAN_PW;  // Scan window warps (slices folded concurrent
 #ifndef SKEL_SCAN_RB
 #define SKEL_SCAN_RB 512
 #endif
+#ifndef SKEL_SCAN_SPER
+#define SKEL_SCAN_SPER 8  // small-vector Scan: elements per thread (tile = RB x SPER)
+#endif
 #ifndef SKEL_SCAN_STAGES
 #define SKEL_SCAN_STAGES 3
 #endif
@@ -125,7 +128,7 @@ constexpr skel_sig_t skel_make_sig() {
     s.v[13] = PACKED;
     s.v[14] = SRB + 64 + 32 * PW;  // scan block size (consumers, producer, store and window warps); tile = SRB * K
     s.v[15] = (skel_u64)SRB | ((skel_u64)SCAN_CH << 16) | ((skel_u64)REPL << 32) |
-              ((skel_u64)RIL << 48) | ((skel_u64)RDIRECT << 49);  // scan rows/tile | tiles/CTA/slice | status
+              ((skel_u64)RIL << 48) | ((skel_u64)RDIRECT << 49) | ((skel_u64)SKEL_SCAN_SPER << 50);  // scan rows/tile | tiles/CTA/slice | status
                                                                   // copies | reduce tile order | direct reduce
     for (int i = 0; i < skel_Lay::n && i < 32; ++i) {
         s.v[16 + 4 * i] = skel_Lay::size(i);
@@ -1090,4 +1093,146 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
             __threadfence();
         }
     }
+}
+
+// ============================================================================
+// Scan for small vectors: two short launches instead of the
+// persistent pipeline, whose fixed costs (per-CTA prologue, a 64 KB tile per
+// CTA, one status poll round trip per slice) dominate below a few MB.
+//   skel_scan_agg_kernel:   aggregate of every tile of RB x SPER elements
+//   skel_scan_small_kernel: per tile, prefix = carry (+) aggregates of the
+//                           tiles before it (ordered block fold), then an
+//                           ordered in-tile exclusive scan
+// The second read of the input hits L2 at these sizes (12 B/element of L2/HBM
+// traffic instead of 8); in-place is safe (a CTA reads its tile before any of
+// its threads writes).
+// ============================================================================
+constexpr int SPER = SKEL_SCAN_SPER;  // elements per thread
+constexpr skel_u64 SM_TILE = (skel_u64)RB * SPER;
+constexpr bool SVEC = TMA_OK && (SPER * sizeof(skel_T)) % 16 == 0;
+
+// this thread's SPER contiguous elements from index i0 (valid: i0 + k < n)
+__device__ __forceinline__ int small_load(const skel_T *in, skel_u64 n, skel_u64 i0, skel_T *x) {
+    if (i0 >= n) return 0;
+    const skel_u64 left = n - i0;
+    if constexpr (SVEC) {
+        if (left >= (skel_u64)SPER && ((reinterpret_cast<unsigned long long>(in + i0) & 15ull) == 0)) {
+            constexpr int NQ = skel::cmax<int>(1, (int)(SPER * sizeof(skel_T) / 16));
+            skel::arr<uint4, NQ> q;
+            const uint4 *p = reinterpret_cast<const uint4 *>(in + i0);
+#pragma unroll
+            for (int j = 0; j < NQ; ++j) q.v[j] = __ldg(p + j);
+            const auto e = skel::bit_cast<skel::arr<skel_T, SPER>>(q);
+#pragma unroll
+            for (int k = 0; k < SPER; ++k) x[k] = e.v[k];
+            return SPER;
+        }
+    }
+    const int m = left < (skel_u64)SPER ? (int)left : SPER;
+#pragma unroll
+    for (int k = 0; k < SPER; ++k)
+        if (k < m) x[k] = in[i0 + k];
+    return m;
+}
+
+extern "C" __global__ void __launch_bounds__(RB)
+    skel_scan_agg_kernel(const skel_T *__restrict__ in, skel_u64 n, skel_S *aggs, const skel_Buf args) {
+    auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    __shared__ VT wpart[NW];
+    const int t = threadIdx.x;
+    skel_T x[SPER];
+    const int m = small_load(in, n, blockIdx.x * SM_TILE + (skel_u64)t * SPER, x);
+    VT a;
+    a.ok = false;
+#pragma unroll
+    for (int k = 0; k < SPER; ++k)
+        if (k < m) a = comb(a, vt_make(x[k]), tup);
+    const VT r = block_fold(a, wpart, tup);
+    if (t == 0) aggs[blockIdx.x].v = r.v;  // every tile holds >= 1 element
+}
+
+extern "C" __global__ void __launch_bounds__(RB)
+    skel_scan_small_kernel(const skel_T *in, skel_T *out, skel_u64 n, const skel_S *aggs, const skel_S identity,
+                           const skel_S *seed, const skel_Buf args) {
+    auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    __shared__ VT wpart[NW];
+    __shared__ VT wsc[NW];
+    __shared__ VT s_pre;
+    const int t = threadIdx.x;
+    const skel_u64 b = blockIdx.x;
+    skel_T x[SPER];  // loaded first: its latency overlaps the prefix fold
+    const int m = small_load(in, n, b * SM_TILE + (skel_u64)t * SPER, x);
+    // prefix of the tiles before this one, folded in order
+    const skel_u64 per = (b + RB - 1) / RB;
+    VT a;
+    a.ok = false;
+    for (skel_u64 k = 0; k < per; ++k) {
+        const skel_u64 j = (skel_u64)t * per + k;
+        if (j < b) a = comb(a, vt_make(aggs[j].v), tup);
+    }
+    const VT tiles = block_fold(a, wpart, tup);
+    if (t == 0) {
+        VT carry;
+        carry.v = seed ? seed->v : identity.v;  // as the persistent Scan: out[0] = seed or identity
+        carry.ok = true;
+        s_pre = comb(carry, tiles, tup);
+    }
+    VT mine;
+    mine.ok = false;
+#pragma unroll
+    for (int k = 0; k < SPER; ++k)
+        if (k < m) mine = comb(mine, vt_make(x[k]), tup);
+    VT tot;
+    const VT excl = block_exscan(mine, wsc, &tot, tup);  // its barriers also publish s_pre
+    skel_T r = comb(s_pre, excl, tup).v;
+    skel_T *o = out + b * SM_TILE + (skel_u64)t * SPER;
+    if constexpr (SVEC) {
+        if (m == SPER && ((reinterpret_cast<unsigned long long>(o) & 15ull) == 0)) {  // 128-bit stores
+            skel::arr<skel_T, SPER> y;
+#pragma unroll
+            for (int k = 0; k < SPER; ++k) {
+                y.v[k] = r;
+                r = opf(r, x[k], tup);
+            }
+            constexpr int NQ = skel::cmax<int>(1, (int)(SPER * sizeof(skel_T) / 16));
+            const auto q = skel::bit_cast<skel::arr<uint4, NQ>>(y);
+#pragma unroll
+            for (int j = 0; j < NQ; ++j) reinterpret_cast<uint4 *>(o)[j] = q.v[j];
+            return;
+        }
+    }
+#pragma unroll
+    for (int k = 0; k < SPER; ++k) {
+        if (k < m) {
+            const skel_T e = x[k];
+            o[k] = r;
+            r = opf(r, e, tup);
+        }
+    }
+}
+
+// Reduce for small vectors: skel_scan_agg_kernel's tile aggregates, then this
+// one-CTA ordered fold of them (two short launches instead of the TMA ring
+// and the last-CTA handshake)
+extern "C" __global__ void __launch_bounds__(RB)
+    skel_fold_aggs_kernel(const skel_S *aggs, skel_u64 count, skel_S *out, const skel_Buf args) {
+    auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    __shared__ VT wpart[NW];
+    const int t = threadIdx.x;
+    const skel_u64 per = (count + RB - 1) / RB;
+    VT a;
+    a.ok = false;
+    for (skel_u64 k0 = 0; k0 < per; k0 += 8) {  // loads in batches of 8, folded in order
+        VT e[8];
+#pragma unroll
+        for (int u = 0; u < 8; ++u) {
+            const skel_u64 j = (skel_u64)t * per + k0 + u;
+            e[u].ok = k0 + u < per && j < count;
+            if (e[u].ok) e[u].v = aggs[j].v;
+        }
+#pragma unroll
+        for (int u = 0; u < 8; ++u) a = comb(a, e[u], tup);
+    }
+    const VT r = block_fold(a, wpart, tup);
+    if (t == 0) out->v = r.v;
 }
