@@ -662,7 +662,6 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
     for _ in range(TUNE):
         rec.subset(evo)
     ms_ord = timed(lambda: rec.subset(evo))
-    evo.destroy()
     for _ in range(TUNE):
         rec.subset(evv, fused=True)
     ms_fused = timed(lambda: rec.subset(evv, fused=True))
@@ -695,7 +694,8 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
                 "all_gather_busbw_GBps": S * busf / (ms_ag * 1e-3) / 1e9,
                 "peak_GBps": 770.0, "peak_source": "B200_PROFILING.md measured peer copy per direction "
                                                   "(900 nominal)"}
-    roof = lmosem_roofline(ctx, skel, rec, evv, timed, world)
+    roof = lmosem_roofline(ctx, skel, rec, evv, timed, world, evo)
+    evo.destroy()
     evv.destroy()
     # configs[4]: the full reconstruction -- 10 subsets of 10^6 events (10^7,
     # P:L603-605), each subset a different synthetic draw, all events staged on
@@ -746,7 +746,7 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
                     "subset_s_fused = the tail as one peer-memory kernel (skel_zip_combine, NEXT-1)"}
 
 
-def lmosem_roofline(ctx, skel, rec, evv, timed, nd):
+def lmosem_roofline(ctx, skel, rec, evv, timed, nd, evo=None):
     """Roofline of the error-image Map.  Every voxel visit of a
     path is one scattered 4-byte request in each walk (a gather of f forward,
     a red.add into c backward) and the lanes of a warp are on different rays,
@@ -773,6 +773,7 @@ def lmosem_roofline(ctx, skel, rec, evv, timed, nd):
     c.fill_dist(skel.COPY, np.float32(0))
     ctx.map(LMOSEM_ERROR, evv, None, args=[f, c, *dims])
     ms_map = timed(lambda: ctx.map(LMOSEM_ERROR, evv, None, args=[f, c, *dims]))
+    ms_map_ord = timed(lambda: ctx.map(LMOSEM_ERROR, evo, None, args=[f, c, *dims])) if evo is not None else None
     c.mark_device_modified()
     # probes: 2^20 elements x PROBE_K scattered requests each (per GPU), into (a) an
     # image-sized 25 MB buffer (random lines: L2 hit/miss and far-partition traffic
@@ -810,6 +811,10 @@ def lmosem_roofline(ctx, skel, rec, evv, timed, nd):
     return {"kernel": "LM OSEM error-image Map (skel_ew_kernel + lmosem_error)", "bound": "l1tex",
             "achieved": achieved, "peak": peak, "unit": "G scattered requests/s per GPU",
             "frac": ideal_ms / ms_map, "map_ms": ms_map, "ideal_ms": ideal_ms, "visits_per_subset": visits,
+            "ordered": None if ms_map_ord is None else {
+                "map_ms": ms_map_ord, "frac": ideal_ms / ms_map_ord,
+                "achieved": reqs / (ms_map_ord * 1e-3) / 1e9,
+                "note": "the same Map over the subset ordered longest path first (lmosem.order_by_path)"},
             "vector_reductions_per_subset": groups, "peak_gather": peak_g, "peak_red_v4": peak_r4,
             "peak_red": peak_r,
             "probes_Greq_per_s": {k: {"gather": v[0], "red": v[1], "red_v4": v[2]} for k, v in probes.items()},
