@@ -651,10 +651,11 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
     ms = timed(lambda: rec.subset(evv))
     # the same subset with its events ordered longest path first (host
     # preprocessing per subset, lmosem.order_by_path; each rank orders its part)
-    from paper_conf_ipps_steuwerkg11_b200.lmosem import order_by_path
+    from paper_conf_ipps_steuwerkg11_b200.lmosem import prepare_part
     t0 = time.perf_counter()
-    ev_ord = order_by_path(ev[lo:hi])
+    ev_ord, ord_block = prepare_part(ev[lo:hi])
     order_host_s = time.perf_counter() - t0
+    rec.map_block = ord_block
     evo = ctx.vector(n=nev, dtype=ev.dtype)
     if world > 1:
         evo.set_distribution(skel.BLOCK)
@@ -662,6 +663,7 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
     for _ in range(TUNE):
         rec.subset(evo)
     ms_ord = timed(lambda: rec.subset(evo))
+    rec.map_block = 0
     for _ in range(TUNE):
         rec.subset(evv, fused=True)
     ms_fused = timed(lambda: rec.subset(evv, fused=True))
@@ -694,7 +696,7 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
                 "all_gather_busbw_GBps": S * busf / (ms_ag * 1e-3) / 1e9,
                 "peak_GBps": 770.0, "peak_source": "B200_PROFILING.md measured peer copy per direction "
                                                   "(900 nominal)"}
-    roof = lmosem_roofline(ctx, skel, rec, evv, timed, world, evo)
+    roof = lmosem_roofline(ctx, skel, rec, evv, timed, world, evo, ord_block)
     evo.destroy()
     evv.destroy()
     # configs[4]: the full reconstruction -- 10 subsets of 10^6 events (10^7,
@@ -707,13 +709,14 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         for l in range(nsub):
             evl = si.lmosem_events(nev, subset=l)[lo:hi]
             if mode == "ordered":
-                evl = order_by_path(evl)
+                evl, _ = prepare_part(evl)
             v = ctx.vector(n=nev, dtype=evl.dtype)
             if world > 1:
                 v.set_distribution(skel.BLOCK)
             v.upload_part(lo, evl)
             subs.append(v)
         rec2 = LMOSEM(ctx)
+        rec2.map_block = ord_block if mode == "ordered" else 0
         for v in subs:  # stage every subset (lazy H2D) and warm up
             rec2.subset(v)
         ctx.sync()
@@ -737,16 +740,16 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
             "full_recon_s": ms_full * 1e-3, "full_recon": "10 subsets x 10^6 events (configs[4]), f0 = 1, "
                                                           "events resident on the devices",
             "ordered": {"subset_s": ms_ord * 1e-3, "full_recon_s": full["ordered"] * 1e-3,
-                        "order_host_s_per_subset": order_host_s,
-                        "note": "events of each subset ordered longest path first on the host before upload "
-                                "(lmosem.order_by_path: list-mode events carry no order; same image up to "
-                                "float rounding)"},
+                        "order_host_s_per_subset": order_host_s, "map_cta_threads": ord_block or 256,
+                        "note": "events of each device's part ordered on the host before upload (lmosem.prepare_part: "
+                                "longest path first, or below 3e5 events per device warp groups dealt over "
+                                "128-thread CTAs; list-mode events carry no order, same image up to float rounding)"},
             "note": "includes f all-gather, c zero-fill, Siddon Map, c reduce-scatter and update Zip; "
                     "subset_s = eager calls, subset_s_graph = the same subset replayed as a CUDA graph, "
                     "subset_s_fused = the tail as one peer-memory kernel (skel_zip_combine, NEXT-1)"}
 
 
-def lmosem_roofline(ctx, skel, rec, evv, timed, nd, evo=None):
+def lmosem_roofline(ctx, skel, rec, evv, timed, nd, evo=None, evo_block=0):
     """Roofline of the error-image Map.  Every voxel visit of a
     path is one scattered 4-byte request in each walk (a gather of f forward,
     a red.add into c backward) and the lanes of a warp are on different rays,
@@ -773,7 +776,13 @@ def lmosem_roofline(ctx, skel, rec, evv, timed, nd, evo=None):
     c.fill_dist(skel.COPY, np.float32(0))
     ctx.map(LMOSEM_ERROR, evv, None, args=[f, c, *dims])
     ms_map = timed(lambda: ctx.map(LMOSEM_ERROR, evv, None, args=[f, c, *dims]))
-    ms_map_ord = timed(lambda: ctx.map(LMOSEM_ERROR, evo, None, args=[f, c, *dims])) if evo is not None else None
+    ms_map_ord = None
+    if evo is not None:  # the prepared part, at its CTA size (lmosem.prepare_part)
+        ctx.set_block_size(evo_block)
+        for _ in range(TUNE):
+            ctx.map(LMOSEM_ERROR, evo, None, args=[f, c, *dims])
+        ms_map_ord = timed(lambda: ctx.map(LMOSEM_ERROR, evo, None, args=[f, c, *dims]))
+        ctx.set_block_size(0)
     c.mark_device_modified()
     # probes: 2^20 elements x PROBE_K scattered requests each (per GPU), into (a) an
     # image-sized 25 MB buffer (random lines: L2 hit/miss and far-partition traffic

@@ -42,6 +42,43 @@ def order_by_path(ev: np.ndarray, dims=DIMS) -> np.ndarray:
     return ev[np.argsort(-key, kind="stable")]
 
 
+def deal_warps(ev: np.ndarray, block: int = 256, warp: int = 32) -> np.ndarray:
+    """Events ordered longest path first (order_by_path), then their groups of
+    `warp` consecutive events dealt round-robin to the `block`-thread CTAs of a
+    one-event-per-thread launch (snake order): a warp keeps rays of similar
+    length, and every CTA gets one group from each length range, so the CTAs
+    (and the SMs that host them) carry equal work."""
+    o = order_by_path(ev)
+    n = len(o)
+    ng = -(-n // warp)
+    per_cta = block // warp
+    ncta = -(-ng // per_cta)
+    # group g (in length order) goes to slot g // ncta of a CTA dealt in snake
+    # order (0..ncta-1, then ncta-1..0, ...), which evens out the CTAs' sums
+    gid = np.arange(ng)
+    rnd, pos = gid // ncta, gid % ncta
+    cta = np.where(rnd % 2 == 0, pos, ncta - 1 - pos)
+    dest = cta * per_cta + rnd
+    order = np.argsort(dest, kind="stable")
+    idx = (order[:, None] * warp + np.arange(warp)[None, :]).ravel()
+    return o[idx[idx < n]]
+
+
+# events per device below which one launch holds less than about one wave of
+# the GPU (148 SMs x 2048 threads); there 128-thread CTAs and warp-dealt order
+# balance the SMs better (DESIGN.md §4.2)
+SMALL_PART = 300_000
+
+
+def prepare_part(ev: np.ndarray, dims=DIMS) -> tuple[np.ndarray, int]:
+    """(events, CTA size for the error-image Map) for one device's part of a
+    subset: longest path first at the default CTA size, or -- for parts below
+    SMALL_PART events -- warp groups dealt over 128-thread CTAs."""
+    if len(ev) <= SMALL_PART:
+        return deal_warps(ev, block=128), 128
+    return order_by_path(ev, dims), 0
+
+
 class LMOSEM:
     def __init__(self, ctx: skel.Context, dims=DIMS, f0: float = 1.0):
         self.ctx = ctx
@@ -51,9 +88,14 @@ class LMOSEM:
         self.c = ctx.vector(n=self.nvox, dtype=np.float32)
         self.f.fill_dist(skel.BLOCK, np.float32(f0))  # f0 = 1 everywhere (reading R10(ii))
         self.dims_args = [np.int32(d) for d in self.dims]
+        self.map_block = 0  # CTA size of the error-image Map (0 = the context's default)
 
     def prepare(self):
+        if self.map_block:
+            self.ctx.set_block_size(self.map_block)
         self.ctx.prepare("map", LMOSEM_ERROR)
+        if self.map_block:
+            self.ctx.set_block_size(0)
         self.ctx.prepare("zip", LMOSEM_UPDATE)
 
     def events(self, ev: np.ndarray) -> skel.Vector:
@@ -68,7 +110,11 @@ class LMOSEM:
         ctx, f, c = self.ctx, self.f, self.c
         f.set_distribution(skel.COPY)                     # block -> copy: all-gather (no-op after a fused tail)
         c.fill_dist(skel.COPY, np.float32(0))             # fresh zero copy on every device
+        if self.map_block:
+            ctx.set_block_size(self.map_block)
         ctx.map(LMOSEM_ERROR, events, None, args=[f, c, *self.dims_args])
+        if self.map_block:
+            ctx.set_block_size(0)
         c.mark_device_modified()                          # dataOnDevicesModified()
         if fused:
             ctx.zip_combine(LMOSEM_UPDATE, f, c, skel.COMBINE_ADD, f)

@@ -122,3 +122,22 @@ def test_path_ordered_events_match_oracle_in_given_order(n, D):
     want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
     assert rel_l2(f, want) <= 1e-4
     assert abs(float(f[c > 0].astype(np.float64).sum()) - nv) <= 1e-4 * nv
+
+
+@pytest.mark.parametrize("D", [1, 3])
+def test_dealt_parts_on_128_thread_ctas_match_oracle(D):
+    """lmosem.prepare_part for a small part (warp groups of similar length dealt
+    over 128-thread CTAs, the error-image Map compiled for that CTA size): the
+    same image as the oracle's for the events in their given order."""
+    from paper_conf_ipps_steuwerkg11_b200.lmosem import prepare_part
+    events = si.lmosem_events(30_000, subset=6)
+    prepared, block = prepare_part(events)
+    assert block == 128 and len(prepared) == len(events)
+    with skel.Context(D) as ctx:
+        rec = LMOSEM(ctx)
+        rec.map_block = block
+        rec.subset(rec.events(prepared))
+        f = rec.image()
+    want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
+    assert rel_l2(f, want) <= 1e-4
+    assert abs(float(f[c > 0].astype(np.float64).sum()) - nv) <= 1e-4 * nv

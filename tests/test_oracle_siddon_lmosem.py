@@ -217,3 +217,21 @@ def test_order_by_path_is_a_permutation_longest_first():
     r = np.corrcoef(np.argsort(np.argsort(nvox)), np.arange(len(o)))[0, 1]
     assert r < -0.97, r
     assert nvox[: len(o) // 10].mean() > 1.5 * nvox[-len(o) // 10:].mean()
+
+
+def test_deal_warps_balances_ctas():
+    """lmosem.deal_warps: a permutation; every 128-thread CTA receives one warp
+    group from each length range, so the CTAs' summed path lengths (the oracle's
+    exact voxel counts) are nearly equal while a warp's lengths stay close."""
+    import skel_inputs as si
+    from paper_conf_ipps_steuwerkg11_b200.lmosem import deal_warps
+    ev = si.lmosem_events(4096, subset=7)
+    d = deal_warps(ev, block=128)
+    rows = lambda a: sorted(map(bytes, a.view(np.uint8).reshape(len(a), -1)))  # noqa: E731
+    assert rows(d) == rows(ev)
+    nvox = np.array([len(oracle.compute_path((e["x1"], e["y1"], e["z1"]), (e["x2"], e["y2"], e["z2"]))[0])
+                     for e in d], dtype=np.float64)
+    per_cta = nvox.reshape(-1, 128).sum(axis=1)
+    assert per_cta.std() / per_cta.mean() < 0.03
+    per_warp_spread = (nvox.reshape(-1, 32).max(axis=1) - nvox.reshape(-1, 32).min(axis=1)).mean()
+    assert per_warp_spread < 0.25 * nvox.mean()

@@ -23,7 +23,10 @@ with skel.Context(1) as ctx:
     dims = [np.int32(150), np.int32(150), np.int32(280)]
     for D in (1, 2, 4, 8):
         part = ev[: 1_000_000 // D]
-        if os.environ.get("LM_ORDER"):  # each GPU orders its part longest path first
+        if os.environ.get("LM_ORDER") == "dealt":  # longest first, warp groups dealt to the CTAs
+            from paper_conf_ipps_steuwerkg11_b200.lmosem import deal_warps
+            part = deal_warps(part, block=int(os.environ.get("SKEL_BLOCK_SIZE", "256")))
+        elif os.environ.get("LM_ORDER"):  # each GPU orders its part longest path first
             from paper_conf_ipps_steuwerkg11_b200.lmosem import order_by_path
             part = order_by_path(part)
         e = ctx.vector(part)
