@@ -41,6 +41,7 @@ struct Module {
     cudaKernel_t k_scan_agg = nullptr;    // small-vector Scan: tile aggregates
     cudaKernel_t k_scan_small = nullptr;  // small-vector Scan: seeded tile scans
     cudaKernel_t k_fold_aggs = nullptr;   // small-vector Reduce: ordered fold of the tile aggregates
+    cudaKernel_t k_red_agg2 = nullptr;    // small-vector Reduce: aggregates of double-size tiles
     cudaKernel_t k_zipcomb = nullptr;  // Zip modules: fused combine + zip + broadcast
     uint64_t sig[16 + 4 * 32] = {0};
     std::set<int> attr_set_on;  // devices on which smem attributes were set

@@ -353,7 +353,7 @@ int get_module_slow(skel_ctx_s *ctx, Kind kind, const char *src, Module **out) {
         if (!getk("skel_reduce_kernel", &m->k_main) || !getk("skel_scan_kernel", &m->k_scan) ||
             !getk("skel_fold_kernel", &m->k_fold) || !getk("skel_seed_kernel", &m->k_seed) ||
             !getk("skel_scan_agg_kernel", &m->k_scan_agg) || !getk("skel_scan_small_kernel", &m->k_scan_small) ||
-            !getk("skel_fold_aggs_kernel", &m->k_fold_aggs))
+            !getk("skel_fold_aggs_kernel", &m->k_fold_aggs) || !getk("skel_red_agg2_kernel", &m->k_red_agg2))
             return SKEL_ERR_CUDA;
     } else {
         if (!getk("skel_ew_kernel", &m->k_main)) return SKEL_ERR_CUDA;

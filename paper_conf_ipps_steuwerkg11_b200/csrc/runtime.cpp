@@ -1073,29 +1073,33 @@ size_t red_parts(Module *m, const Slot &s, uint64_t cnt) {
 }
 
 // small vectors: tile aggregates + a one-CTA ordered fold (two short launches)
-// up to SKEL_RED_SMALL_MAX elements (tuning hook; default 32 MiB of elements:
-// measured crossover with the TMA kernel between 2^23 and 2^24 floats)
-uint64_t red_small_tile(const Module *m) { return m->sig[9] * ((m->sig[15] >> 50) & 0xff); }
+// up to SKEL_RED_SMALL_MAX elements (tuning hook; default 64 MiB of elements:
+// measured crossover with the TMA kernel between 2^24 and 2^25 floats).  Above
+// 8 MiB the tiles are twice as large (16 elements per thread for floats).
+bool red_small_big_tiles(const Module *m, uint64_t cnt) { return cnt * m->sig[3] > (8ull << 20); }
+uint64_t red_small_tile(const Module *m, uint64_t cnt) {
+    return m->sig[9] * ((m->sig[15] >> 50) & 0xff) * (red_small_big_tiles(m, cnt) ? 2 : 1);
+}
 bool red_small(const Module *m, uint64_t cnt) {
     static const uint64_t env = [] {
         const char *e = getenv("SKEL_RED_SMALL_MAX");
         return e ? (uint64_t)strtoull(e, nullptr, 10) : ~0ull;
     }();
-    const uint64_t mx = env != ~0ull ? env : (uint64_t)(32u << 20) / m->sig[3];
-    return m->k_fold_aggs && red_small_tile(m) > 0 && cnt <= mx;
+    const uint64_t mx = env != ~0ull ? env : (uint64_t)(64u << 20) / m->sig[3];
+    return m->k_fold_aggs && m->k_red_agg2 && red_small_tile(m, cnt) > 0 && cnt <= mx;
 }
 
 // local reduce of the slot's data into dst
 int launch_reduce(skel_ctx_s *ctx, Module *m, Slot &s, const void *in, uint64_t cnt, const RedLayout &L,
                   std::vector<unsigned char> &abuf, void *dst) {
     if (red_small(m, cnt)) {
-        const uint64_t ST = red_small_tile(m);
+        const uint64_t ST = red_small_tile(m, cnt);
         uint64_t nt = (cnt + ST - 1) / ST;
         void *aggs = s.ws + L.total;  // room reserved by reduce_core
         void *pa[] = {&in, &cnt, &aggs, abuf.data()};
         DevGuard g(s.dev);
-        CK(ctx, cudaLaunchKernel((const void *)m->k_scan_agg, dim3((unsigned)nt), dim3((unsigned)m->sig[9]), pa, 0,
-                                 s.stream));
+        const void *kagg = red_small_big_tiles(m, cnt) ? (const void *)m->k_red_agg2 : (const void *)m->k_scan_agg;
+        CK(ctx, cudaLaunchKernel(kagg, dim3((unsigned)nt), dim3((unsigned)m->sig[9]), pa, 0, s.stream));
         const void *caggs = aggs;
         void *pf[] = {&caggs, &nt, &dst, abuf.data()};
         CK(ctx, cudaLaunchKernel((const void *)m->k_fold_aggs, dim3(1), dim3((unsigned)m->sig[9]), pf, 0, s.stream));
@@ -1134,7 +1138,8 @@ int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args
         const uint64_t cnt = in->bufs[li].count;
         TRY(set_smem_attr(ctx, m, s));  // before the occupancy query in red_grid
         Ls[li] = red_layout(m, D, red_parts(m, s, cnt), 0);
-        const size_t extra = red_small(m, cnt) ? (size_t)((cnt + red_small_tile(m) - 1) / red_small_tile(m)) * Ls[li].slot : 0;
+        const size_t extra =
+            red_small(m, cnt) ? (size_t)((cnt + red_small_tile(m, cnt) - 1) / red_small_tile(m, cnt)) * Ls[li].slot : 0;
         TRY(ensure_ws(ctx, s, Ls[li].total + extra));
         pack_args(m, args, nargs, li, abuf);
         char *dst = cross ? s.ws + Ls[li].o_res : (direct && D == 1 ? static_cast<char *>(direct) : s.ws + Ls[li].o_fold);

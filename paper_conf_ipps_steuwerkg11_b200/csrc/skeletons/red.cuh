@@ -1112,43 +1112,59 @@ constexpr skel_u64 SM_TILE = (skel_u64)RB * SPER;
 constexpr bool SVEC = TMA_OK && (SPER * sizeof(skel_T)) % 16 == 0;
 
 // this thread's SPER contiguous elements from index i0 (valid: i0 + k < n)
+template <int PER = SPER>
 __device__ __forceinline__ int small_load(const skel_T *in, skel_u64 n, skel_u64 i0, skel_T *x) {
+    constexpr bool VEC = TMA_OK && (PER * sizeof(skel_T)) % 16 == 0;
     if (i0 >= n) return 0;
     const skel_u64 left = n - i0;
-    if constexpr (SVEC) {
-        if (left >= (skel_u64)SPER && ((reinterpret_cast<unsigned long long>(in + i0) & 15ull) == 0)) {
-            constexpr int NQ = skel::cmax<int>(1, (int)(SPER * sizeof(skel_T) / 16));
+    if constexpr (VEC) {
+        if (left >= (skel_u64)PER && ((reinterpret_cast<unsigned long long>(in + i0) & 15ull) == 0)) {
+            constexpr int NQ = skel::cmax<int>(1, (int)(PER * sizeof(skel_T) / 16));
             skel::arr<uint4, NQ> q;
             const uint4 *p = reinterpret_cast<const uint4 *>(in + i0);
 #pragma unroll
             for (int j = 0; j < NQ; ++j) q.v[j] = __ldg(p + j);
-            const auto e = skel::bit_cast<skel::arr<skel_T, SPER>>(q);
+            const auto e = skel::bit_cast<skel::arr<skel_T, PER>>(q);
 #pragma unroll
-            for (int k = 0; k < SPER; ++k) x[k] = e.v[k];
-            return SPER;
+            for (int k = 0; k < PER; ++k) x[k] = e.v[k];
+            return PER;
         }
     }
-    const int m = left < (skel_u64)SPER ? (int)left : SPER;
+    const int m = left < (skel_u64)PER ? (int)left : PER;
 #pragma unroll
-    for (int k = 0; k < SPER; ++k)
+    for (int k = 0; k < PER; ++k)
         if (k < m) x[k] = in[i0 + k];
     return m;
+}
+
+// ordered fold of one tile of RB x PER elements into aggs[blockIdx.x]
+template <int PER, class Tup>
+__device__ __forceinline__ void tile_aggregate(const skel_T *in, skel_u64 n, skel_S *aggs, VT *wpart, Tup &tup) {
+    const int t = threadIdx.x;
+    skel_T x[PER];
+    const int m = small_load<PER>(in, n, blockIdx.x * ((skel_u64)RB * PER) + (skel_u64)t * PER, x);
+    VT a;
+    a.ok = false;
+#pragma unroll
+    for (int k = 0; k < PER; ++k)
+        if (k < m) a = comb(a, vt_make(x[k]), tup);
+    const VT r = block_fold(a, wpart, tup);
+    if (t == 0) aggs[blockIdx.x].v = r.v;  // every tile holds >= 1 element
 }
 
 extern "C" __global__ void __launch_bounds__(RB)
     skel_scan_agg_kernel(const skel_T *__restrict__ in, skel_u64 n, skel_S *aggs, const skel_Buf args) {
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     __shared__ VT wpart[NW];
-    const int t = threadIdx.x;
-    skel_T x[SPER];
-    const int m = small_load(in, n, blockIdx.x * SM_TILE + (skel_u64)t * SPER, x);
-    VT a;
-    a.ok = false;
-#pragma unroll
-    for (int k = 0; k < SPER; ++k)
-        if (k < m) a = comb(a, vt_make(x[k]), tup);
-    const VT r = block_fold(a, wpart, tup);
-    if (t == 0) aggs[blockIdx.x].v = r.v;  // every tile holds >= 1 element
+    tile_aggregate<SPER>(in, n, aggs, wpart, tup);
+}
+// the same with tiles of twice the size: the small-vector Reduce above 2^21
+// 4-byte elements (more bytes in flight per thread)
+extern "C" __global__ void __launch_bounds__(RB)
+    skel_red_agg2_kernel(const skel_T *__restrict__ in, skel_u64 n, skel_S *aggs, const skel_Buf args) {
+    auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    __shared__ VT wpart[NW];
+    tile_aggregate<2 * SPER>(in, n, aggs, wpart, tup);
 }
 
 extern "C" __global__ void __launch_bounds__(RB)
