@@ -272,12 +272,23 @@ extern "C" __global__ void SKEL_EW_BOUNDS
                 skel_chunk_op(ca[u], cb[u], po + (c + u * stride) * skel_CO, t);
             }
         }
-#pragma unroll 1
-        for (; c < nch; c += stride) {
-            skel::chunk<skel_CA> ca = skel_ld<skel_CA>(pa + c * skel_CA);
-            skel::chunk<skel_CB> cb;
-            if constexpr (SKEL_NIN == 2) cb = skel_ld<skel_CB>(pb + c * skel_CB);
-            skel_chunk_op(ca, cb, po + c * skel_CO, t);
+        // the < SKEL_UNROLL chunks left to this thread: one predicated round, so
+        // their loads are in flight together (a loop would pay one memory round
+        // trip per chunk -- what bounded vectors of 2^21..2^23 elements, where a
+        // thread holds 2-4 chunks)
+        if (c < nch) {
+            skel::chunk<skel_CA> ca[SKEL_UNROLL];
+            skel::chunk<skel_CB> cb[SKEL_UNROLL];
+#pragma unroll
+            for (int u = 0; u < SKEL_UNROLL; ++u) {
+                if (c + u * stride < nch) {
+                    ca[u] = skel_ld<skel_CA>(pa + (c + u * stride) * skel_CA);
+                    if constexpr (SKEL_NIN == 2) cb[u] = skel_ld<skel_CB>(pb + (c + u * stride) * skel_CB);
+                }
+            }
+#pragma unroll
+            for (int u = 0; u < SKEL_UNROLL; ++u)
+                if (c + u * stride < nch) skel_chunk_op(ca[u], cb[u], po + (c + u * stride) * skel_CO, t);
         }
     }
     // scalar path: the tail, or everything for non-vectorisable element types
