@@ -415,3 +415,27 @@ def test_void_index_map_side_effects():
         acc.mark_device_modified()
         acc.set_distribution(skel.BLOCK, skel.COMBINE_ADD)
         assert np.array_equal(acc.download(), (np.arange(n) % 5 + 1).astype(np.int32))
+
+
+@pytest.mark.parametrize("n", [(1 << 21) + 5, 3_000_017])
+def test_small_paths_with_double_tiles_i32(ctx, n):
+    """Between 8 and 16 MiB the Reduce takes its small-vector path with
+    double-size tiles and the Scan its small-vector path:
+    integer results bit-exact."""
+    x = si.uniform_int01(n, 21)
+    vx = ctx.vector(x)
+    assert int(ctx.reduce(SUM_I32, vx)) == int(x.astype(np.int64).sum())
+    out = ctx.vector(n=n, dtype=np.int32)
+    ctx.scan(SUM_I32, vx, out, np.int32(0))
+    assert np.array_equal(out.download(), oracle.skel_scan(SUM_I32, x, 0))
+
+
+def test_small_paths_with_double_tiles_noncommutative_16B(ctx):
+    n = 700_001  # 11.2 MB of 16-byte elements
+    m = rand_struct(M2, n, 77)
+    assert ctx.reduce(MAT_U, ctx.vector(m)).tobytes() == oracle.skel_reduce(MAT_U, m).tobytes()
+    ident = np.zeros(1, M2)
+    ident["a"], ident["d"] = 1, 1
+    out = ctx.vector(n=n, dtype=M2)
+    ctx.scan(MAT_U, ctx.vector(m), out, ident[0])
+    assert out.download().tobytes() == oracle.skel_scan(MAT_U, m, ident[0]).tobytes()
