@@ -103,7 +103,7 @@ def mandel_blocked(tmp_path_factory):
     return run
 
 
-@pytest.mark.parametrize("cap", [1, 7, 8, 9, 256])
+@pytest.mark.parametrize("cap", [1, 7, 8, 9, 256, 1024, 1500])
 def test_blocked_mandelbrot_equals_the_plain_iteration(mandel_blocked, golden_dir, cap):
     """mandelbrot_blocked.cu (loop control per block of 8 updates, roll back on
     escape) counts exactly what eq. (5) as written counts: bit-identical to
