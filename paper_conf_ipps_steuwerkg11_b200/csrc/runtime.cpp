@@ -786,6 +786,54 @@ int ew_grid(const Slot &s, size_t chunks, int block, int per_thread) {
     return (int)std::max<size_t>(g, 1);
 }
 
+// element-wise grid policy for a module and size class (log2 of the chunk
+// count), chosen by measurement among the policies in `mask` (bit p = policy
+// p; the lowest one is the default another must beat by 3%): the first
+// launches on the first device time each in turn, twice (events around the
+// launch, outside graph captures); later launches use the fastest
+struct EwChoice {
+    int policy = 0, tslot = -1;
+    Module::EwTune *tu = nullptr;
+};
+int ew_choose(skel_ctx_s *ctx, Module *m, Slot &s, size_t li, uint64_t chunks, unsigned mask, EwChoice &ch) {
+    int pol[Module::kPolicies], P = 0;
+    for (int p = 0; p < Module::kPolicies; ++p)
+        if (mask & (1u << p)) pol[P++] = p;
+    ch.policy = pol[0];
+    Module::EwTune *tu = &m->ew_tune[64 - __builtin_clzll((unsigned long long)std::max<uint64_t>(chunks, 1))];
+    ch.tu = tu;
+    cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
+    cudaStreamIsCapturing(s.stream, &cs);
+    const int NT = P * Module::kRounds;
+    if (tu->best < 0 && li == 0 && cs == cudaStreamCaptureStatusNone) {
+        if (tu->trial == NT) {  // all samples recorded: decide (one wait, once per class)
+            CK(ctx, cudaEventSynchronize(tu->ev[2 * NT - 1]));
+            float best_t[Module::kPolicies];
+            for (int p = 0; p < P; ++p) best_t[p] = 3.0e38f;
+            for (int k = 0; k < NT; ++k) {
+                float t = 0;
+                CK(ctx, cudaEventElapsedTime(&t, tu->ev[2 * k], tu->ev[2 * k + 1]));
+                best_t[k % P] = std::min(best_t[k % P], t);
+            }
+            int b = 0;
+            for (int p = 1; p < P; ++p)
+                if (best_t[p] < 0.97f * best_t[0] && best_t[p] < best_t[b]) b = p;
+            tu->best = pol[b];
+            for (cudaEvent_t &e : tu->ev) {
+                if (e) cudaEventDestroy(e);
+                e = nullptr;
+            }
+        } else {
+            ch.tslot = tu->trial++;
+            ch.policy = pol[ch.tslot % P];
+            for (int k = 0; k < 2; ++k)
+                if (!tu->ev[2 * ch.tslot + k]) CK(ctx, cudaEventCreate(&tu->ev[2 * ch.tslot + k]));
+        }
+    }
+    if (tu->best >= 0) ch.policy = tu->best;
+    return SKEL_OK;
+}
+
 int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_s *b, skel_vec_s *out,
            const skel_arg *args, int nargs) {
     Module *m = nullptr;
@@ -823,43 +871,11 @@ int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_
         const size_t chunks = vec_ok ? std::max<uint64_t>(cnt / E, 1) : cnt;
         const int unroll = std::max<int>(1, (int)m->sig[10]);
         DevGuard g(s.dev);
-        // grid policy (Module::EwTune): the first launches of a size class time
-        // both policies alternately on the first device; later ones use the faster
-        Module::EwTune *tu = nullptr;
-        int policy = 0, tslot = -1;
-        if (vec_ok && E > 1 && unroll > 1) {
-            tu = &m->ew_tune[64 - __builtin_clzll((unsigned long long)chunks)];
-            cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
-            cudaStreamIsCapturing(s.stream, &cs);
-            if (tu->best < 0 && li == 0 && cs == cudaStreamCaptureStatusNone) {
-                constexpr int P = Module::kPolicies, NT = Module::kPolicies * Module::kRounds;
-                if (tu->trial == NT) {  // all samples recorded: decide (one wait, once per class)
-                    CK(ctx, cudaEventSynchronize(tu->ev[2 * NT - 1]));
-                    float best_t[P];
-                    for (int p = 0; p < P; ++p) best_t[p] = 3.0e38f;
-                    for (int k = 0; k < NT; ++k) {
-                        float t = 0;
-                        CK(ctx, cudaEventElapsedTime(&t, tu->ev[2 * k], tu->ev[2 * k + 1]));
-                        best_t[k % P] = std::min(best_t[k % P], t);
-                    }
-                    // another policy must beat the default by 3% (timer noise)
-                    int b = 0;
-                    for (int p = 1; p < P; ++p)
-                        if (best_t[p] < 0.97f * best_t[0] && best_t[p] < best_t[b]) b = p;
-                    tu->best = b;
-                    for (cudaEvent_t &e : tu->ev) {
-                        cudaEventDestroy(e);
-                        e = nullptr;
-                    }
-                } else {
-                    tslot = tu->trial++;
-                    policy = tslot % P;
-                    for (int k = 0; k < 2; ++k)
-                        if (!tu->ev[2 * tslot + k]) CK(ctx, cudaEventCreate(&tu->ev[2 * tslot + k]));
-                }
-            }
-            if (tu->best >= 0) policy = tu->best;
-        }
+        // grid policy (Module::EwTune): measured among policies 0/1/2
+        EwChoice ch;
+        if (vec_ok && E > 1 && unroll > 1) TRY(ew_choose(ctx, m, s, li, chunks, 0x7u, ch));
+        const int policy = ch.policy, tslot = ch.tslot;
+        Module::EwTune *tu = ch.tu;
         // policy 2: the scalar path, one element per thread
         int vk = policy == 2 ? 0 : vec_ok;
         const int grid = policy == 2 ? ew_grid(s, cnt, block, 1)
@@ -1695,10 +1711,19 @@ int skel_map_index(skel_ctx_t ctx, const char *src, size_t n, skel_vec_t out, co
         int vec_ok = !po || al16(po);
         pack_args(m, args, nargs, li, abuf);
         const size_t chunks = vec_ok && rsz != 0 ? std::max<uint64_t>(cnt / E, 1) : cnt;
-        const int grid = ew_grid(s, chunks, block, 1);
-        void *params[] = {&po, &cnt, &base, &vec_ok, abuf.data()};
         DevGuard g(s.dev);
+        // measured choice between one chunk of E outputs per thread (policy 1) and
+        // one element per thread through the scalar path (policy 2): a divergent,
+        // compute-bound function (Mandelbrot) balances better with the second
+        EwChoice ch;
+        ch.policy = 1;
+        if (vec_ok && rsz != 0 && E > 1) TRY(ew_choose(ctx, m, s, li, chunks, 0x6u, ch));
+        int vk = ch.policy == 2 ? 0 : vec_ok;
+        const int grid = ew_grid(s, ch.policy == 2 ? cnt : chunks, block, 1);
+        void *params[] = {&po, &cnt, &base, &vk, abuf.data()};
+        if (ch.tslot >= 0) CK(ctx, cudaEventRecord(ch.tu->ev[2 * ch.tslot], s.stream));
         CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+        if (ch.tslot >= 0) CK(ctx, cudaEventRecord(ch.tu->ev[2 * ch.tslot + 1], s.stream));
         ctx->stats.kernel_launches++;
     }
     if (rsz != 0) {
