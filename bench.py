@@ -615,6 +615,29 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
                           "blocked_fp32_frac": 8 * it4096 / (heavy["blocked"] * 1e-3) / peak_ops}
     vin.destroy()
     out.destroy()
+    # configs[0]: 1024x768, cap 256, single distribution (device 0 / rank 0)
+    ps = si.mandelbrot_positions(1024, 768)
+    vs = ctx.vector(n=ps.size, dtype=ps.dtype)
+    vs.set_distribution(skel.SINGLE)
+    vs.upload(ps)
+    os_ = ctx.vector(n=ps.size, dtype=np.int32)
+    os_.set_distribution(skel.SINGLE)
+    for _ in range(TUNE):
+        ctx.map(MANDELBROT, vs, os_, args=[capv])
+    barrier()
+    torch.cuda.synchronize()
+    e0.record(stream)
+    for _ in range(reps):
+        ctx.map(MANDELBROT, vs, os_, args=[capv])
+    e1.record(stream)
+    ctx.sync()
+    ms_s = max_over_ranks(e0.elapsed_time(e1) / reps)
+    res["configs0_1024x768"] = {"ms": ms_s, "Mpix_per_s": ps.size / (ms_s * 1e-3) / 1e6,
+                                "sum_iter": 28347768,
+                                "fp32_frac": 8 * 28347768 / (ms_s * 1e-3) / (148 * 128 * 1.965e9),
+                                "note": "single distribution: one GPU computes, 2.6 waves (latency-sized)"}
+    vs.destroy()
+    os_.destroy()
     return res
 
 
