@@ -1089,8 +1089,8 @@ size_t red_parts(Module *m, const Slot &s, uint64_t cnt) {
 }
 
 // small vectors: tile aggregates + a one-CTA ordered fold (two short launches)
-// up to SKEL_RED_SMALL_MAX elements (tuning hook; default 64 MiB of elements:
-// measured crossover with the TMA kernel between 2^24 and 2^25 floats).  Above
+// up to SKEL_RED_SMALL_MAX elements (tuning hook; default 128 MiB of elements:
+// measured crossover with the TMA kernel between 2^25 and 2^26 floats).  Above
 // 8 MiB the tiles are twice as large (16 elements per thread for floats).
 bool red_small_big_tiles(const Module *m, uint64_t cnt) { return cnt * m->sig[3] > (8ull << 20); }
 uint64_t red_small_tile(const Module *m, uint64_t cnt) {
@@ -1101,7 +1101,7 @@ bool red_small(const Module *m, uint64_t cnt) {
         const char *e = getenv("SKEL_RED_SMALL_MAX");
         return e ? (uint64_t)strtoull(e, nullptr, 10) : ~0ull;
     }();
-    const uint64_t mx = env != ~0ull ? env : (uint64_t)(64u << 20) / m->sig[3];
+    const uint64_t mx = env != ~0ull ? env : (uint64_t)(128u << 20) / m->sig[3];
     return m->k_fold_aggs && m->k_red_agg2 && red_small_tile(m, cnt) > 0 && cnt <= mx;
 }
 
