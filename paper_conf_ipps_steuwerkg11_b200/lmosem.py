@@ -98,8 +98,21 @@ class LMOSEM:
             self.ctx.set_block_size(0)
         self.ctx.prepare("zip", LMOSEM_UPDATE)
 
-    def events(self, ev: np.ndarray) -> skel.Vector:
-        """Vector<Event> of one subset, block-distributed (Listing 4)."""
+    def events(self, ev: np.ndarray, prepare: bool = False) -> skel.Vector:
+        """Vector<Event> of one subset, block-distributed (Listing 4).
+        prepare=True: each device's part [k*ceil(n/D), ...) reordered by
+        prepare_part (the error-image Map then uses the CTA size it picks).
+        In rank mode pass the whole subset on every rank, as for a plain upload."""
+        if prepare and len(ev):
+            D = self.ctx.D
+            ps = -(-len(ev) // D)
+            parts = []
+            for k in range(D):
+                part, blk = prepare_part(ev[k * ps:(k + 1) * ps], self.dims)
+                parts.append(part)
+                if k == 0:
+                    self.map_block = blk
+            ev = np.concatenate(parts)
         v = self.ctx.vector(ev)
         v.set_distribution(skel.BLOCK)
         return v

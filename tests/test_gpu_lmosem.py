@@ -141,3 +141,17 @@ def test_dealt_parts_on_128_thread_ctas_match_oracle(D):
     want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
     assert rel_l2(f, want) <= 1e-4
     assert abs(float(f[c > 0].astype(np.float64).sum()) - nv) <= 1e-4 * nv
+
+
+@pytest.mark.parametrize("D", [1, 4])
+def test_events_prepare_option(D):
+    """LMOSEM.events(ev, prepare=True): each device's part reordered (and the
+    Map's CTA size picked) by prepare_part; the image is the oracle's."""
+    events = si.lmosem_events(24_000, subset=8)
+    with skel.Context(D) as ctx:
+        rec = LMOSEM(ctx)
+        rec.subset(rec.events(events, prepare=True))
+        assert rec.map_block == 128
+        f = rec.image()
+    want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
+    assert rel_l2(f, want) <= 1e-4
