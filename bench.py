@@ -518,7 +518,68 @@ def bench_overhead(ctx, skel, stream, args):
     res["kernel_cache"] = {"nvrtc_build_ms": round(st1["compile_ms"], 1), "disk_load_ms": round(st2["disk_load_ms"], 2),
                            "load_speedup": round(st1["compile_ms"] / max(st2["disk_load_ms"], 1e-6), 1),
                            "kernels": [k for k, _ in srcs], "paper": "loading is at least 5x faster (P:L248-250)"}
+    res["small"] = bench_overhead_small(ctx, hw, stream)
     return res
+
+
+def bench_overhead_small(ctx, hw, stream):
+    """Latency-sized vectors: us per launch of each skeleton
+    and of the same operation hand-written / from CUB, every launch replayed in
+    a CUDA graph over rotating operand sets (>= 4x L2 of operands, so every
+    launch reads from HBM), float32."""
+    import math
+
+    import torch
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MAP_F32, SAXPY_F32, SUM_F32
+    import ctypes
+    hw.hw_cubsum_f32.argtypes = [ctypes.c_void_p, ctypes.c_size_t, ctypes.c_void_p, ctypes.c_void_p]
+    sp = ctx.stream(0)
+    out = {}
+    for k in (20, 22, 24):
+        n = 1 << k
+        R = max(2, min(64, math.ceil(4 * 126e6 / (2 * n * 4))))
+        sets = []
+        for _ in range(R):
+            x, o, r = (ctx.vector(n=n if i < 2 else 1, dtype=np.float32) for i in range(3))
+            x.fill(np.float32(1))
+            sets.append((x, o, r, x.device_ptr()[0], o.device_ptr()[0], r.device_ptr()[0]))
+        ops = {
+            "map": (lambda st: ctx.map(MAP_F32, st[0], st[1]), lambda st: hw.hw_map_f32(st[3], st[4], n, sp)),
+            "zip": (lambda st: ctx.zip(SAXPY_F32, st[0], st[1], st[1], args=[np.float32(2.5)]),
+                    lambda st: hw.hw_saxpy_f32(st[3], st[4], st[4], 2.5, n, sp)),
+            "reduce": (lambda st: ctx.reduce_to(SUM_F32, st[0], st[2]), lambda st: hw.hw_cubsum_f32(st[3], n, st[5], sp)),
+            "scan": (lambda st: ctx.scan(SUM_F32, st[0], st[1], np.float32(0)),
+                     lambda st: hw.hw_exscan_f32(st[3], st[4], n, sp)),
+        }
+        row = {}
+        for name, pair in ops.items():
+            us = []
+            for op in pair:
+                def fn(op=op):
+                    for st in sets:
+                        op(st)
+                for _ in range(TUNE):
+                    fn()
+                ctx.sync()
+                g = ctx.capture(fn)
+                g.launch()
+                ctx.sync()
+                e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                e0.record(stream)
+                for _ in range(10):
+                    g.launch()
+                e1.record(stream)
+                ctx.sync()
+                g.destroy()
+                us.append(round(e0.elapsed_time(e1) * 1e3 / (10 * R), 2))
+            row[name] = {"skeleton_us": us[0], "reference_us": us[1]}
+        out[f"2^{k}"] = row
+        for st in sets:
+            for v in st[:3]:
+                v.destroy()
+    out["reference"] = "map/zip: hand-written float4 nvcc kernels; reduce: CUB DeviceReduce::Sum (two kernels, " \
+                       "commutative only); scan: CUB DeviceScan::ExclusiveSum"
+    return out
 
 
 def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
