@@ -12,7 +12,7 @@ from __future__ import annotations
 import numpy as np
 
 from . import skel
-from .workloads import LMOSEM_ERROR, LMOSEM_UPDATE
+from .workloads import LMOSEM_ERROR, LMOSEM_ERROR_PREPARED, LMOSEM_UPDATE
 
 DIMS = (150, 150, 280)
 
@@ -89,11 +89,12 @@ class LMOSEM:
         self.f.fill_dist(skel.BLOCK, np.float32(f0))  # f0 = 1 everywhere (reading R10(ii))
         self.dims_args = [np.int32(d) for d in self.dims]
         self.map_block = 0  # CTA size of the error-image Map (0 = the context's default)
+        self.error_src = LMOSEM_ERROR  # LMOSEM_ERROR_PREPARED for prepared event order
 
     def prepare(self):
         if self.map_block:
             self.ctx.set_block_size(self.map_block)
-        self.ctx.prepare("map", LMOSEM_ERROR)
+        self.ctx.prepare("map", self.error_src)
         if self.map_block:
             self.ctx.set_block_size(0)
         self.ctx.prepare("zip", LMOSEM_UPDATE)
@@ -112,6 +113,7 @@ class LMOSEM:
                 parts.append(part)
                 if k == 0:
                     self.map_block = blk
+            self.error_src = LMOSEM_ERROR_PREPARED
             ev = np.concatenate(parts)
         v = self.ctx.vector(ev)
         v.set_distribution(skel.BLOCK)
@@ -125,7 +127,7 @@ class LMOSEM:
         c.fill_dist(skel.COPY, np.float32(0))             # fresh zero copy on every device
         if self.map_block:
             ctx.set_block_size(self.map_block)
-        ctx.map(LMOSEM_ERROR, events, None, args=[f, c, *self.dims_args])
+        ctx.map(self.error_src, events, None, args=[f, c, *self.dims_args])
         if self.map_block:
             ctx.set_block_size(0)
         c.mark_device_modified()                          # dataOnDevicesModified()

@@ -15,6 +15,10 @@ MANDELBROT = source("mandelbrot")
 MANDELBROT_INDEX = source("mandelbrot_index")  # index Map variant (NEXT-4)
 MANDELBROT_BLOCKED = source("mandelbrot_blocked")  # loop control per block of updates (NEXT-4)
 LMOSEM_ERROR = source("lmosem_error")
+# the same function for prepared (longest-path-first) event order, where the
+# Map is bound by L1TEX requests: 16-byte gathers per 4-float group in the
+# forward projection too; in the given order they are slower
+LMOSEM_ERROR_PREPARED = "#define LMOSEM_VEC_FWD 1\n" + LMOSEM_ERROR
 LMOSEM_UPDATE = source("lmosem_update")
 # voxel visits of one event's path (measurement only: the LM OSEM roofline
 # counts one scattered request per visit in each of the two walks)

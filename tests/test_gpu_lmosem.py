@@ -108,15 +108,20 @@ def test_full_size_subset_matches_oracle():
     assert abs(float(f[c > 0].astype(np.float64).sum()) - nv) <= 1e-4 * nv
 
 
-@pytest.mark.parametrize("n,D", [(1_000_000, 1), (40_000, 4)])
-def test_path_ordered_events_match_oracle_in_given_order(n, D):
+@pytest.mark.parametrize("n,D,prepared_fn", [(1_000_000, 1, False), (1_000_000, 1, True), (40_000, 4, True)])
+def test_path_ordered_events_match_oracle_in_given_order(n, D, prepared_fn):
     """The events reordered longest path first (lmosem.order_by_path, host
-    preprocessing) give the oracle's image for the events in
-    their given order: the error image is a sum over events (R10(x))."""
+    preprocessing) -- with the plain error function or the one
+    for prepared order (16-byte forward gathers) -- give the oracle's image for
+    the events in their given order: the error image is a sum over events
+    (R10(x))."""
     from paper_conf_ipps_steuwerkg11_b200.lmosem import order_by_path
+    from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_ERROR_PREPARED
     events = si.lmosem_events(n, subset=3)
     with skel.Context(D) as ctx:
         rec = LMOSEM(ctx)
+        if prepared_fn:
+            rec.error_src = LMOSEM_ERROR_PREPARED
         rec.subset(rec.events(order_by_path(events)))
         f = rec.image()
     want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
