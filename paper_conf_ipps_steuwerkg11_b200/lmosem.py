@@ -64,10 +64,11 @@ def deal_warps(ev: np.ndarray, block: int = 256, warp: int = 32) -> np.ndarray:
     return o[idx[idx < n]]
 
 
-# events per device below which one launch holds less than about one wave of
-# the GPU (148 SMs x 2048 threads); there 128-thread CTAs and warp-dealt order
-# balance the SMs better
-SMALL_PART = 300_000
+# events per device below which a launch is well under one wave of the GPU
+# (148 SMs x 2048 threads); there 128-thread CTAs and warp-dealt order balance
+# the SMs better (measured: better at 1.25e5 events per GPU,
+# worse at 2.5e5)
+SMALL_PART = 150_000
 
 
 def prepare_part(ev: np.ndarray, dims=DIMS) -> tuple[np.ndarray, int]:
