@@ -830,7 +830,7 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
             "ordered": {"subset_s": ms_ord * 1e-3, "full_recon_s": full["ordered"] * 1e-3,
                         "order_host_s_per_subset": order_host_s, "map_cta_threads": ord_block or 256,
                         "note": "events of each device's part ordered on the host before upload (lmosem.prepare_part: "
-                                "longest path first, or below 3e5 events per device warp groups dealt over "
+                                "longest path first, or below 1.5e5 events per device warp groups dealt over "
                                 "128-thread CTAs; list-mode events carry no order, same image up to float rounding)"},
             "note": "includes f all-gather, c zero-fill, Siddon Map, c reduce-scatter and update Zip; "
                     "subset_s = eager calls, subset_s_graph = the same subset replayed as a CUDA graph, "
