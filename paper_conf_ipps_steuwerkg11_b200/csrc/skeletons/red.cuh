@@ -733,6 +733,60 @@ __device__ __forceinline__ VT warp_fold_aggs(const skel_u64 *st64, const unsigne
     return vt_shfl_idx(a, 0);
 }
 
+#ifndef SKEL_SCAN_CPOLL
+#define SKEL_SCAN_CPOLL 1
+#endif
+// the same ordered fold with coalesced probes (packed status words only): probe
+// round k reads words base + 32k + lane, so one round touches 2 L2 lines instead
+// of `per` rounds each spanning 32 lines (4x fewer sector requests per poll on
+// the hot status lines); the words are transposed through shared memory so each
+// lane folds `per` consecutive aggregates in order before the warp fold
+template <class Tup>
+__device__ __forceinline__ VT warp_fold_aggs_coalesced(const skel_u64 *st64, skel_u64 *sbuf, skel_u64 base, int cnt,
+                                                       unsigned epoch, int lane, Tup &t) {
+    const int rounds = (cnt + 31) / 32;
+    unsigned pending = 0;  // bit k: word base + 32k + lane still unpublished
+#pragma unroll
+    for (int k = 0; k < AGG_PER; ++k)
+        if (k < rounds && 32 * k + lane < cnt) pending |= 1u << k;
+    for (unsigned ns = SKEL_SCAN_BACKOFF_MIN;; ns = ns < SKEL_SCAN_BACKOFF_MAX ? 2 * ns : ns) {
+        skel_u64 word[AGG_PER];
+#pragma unroll
+        for (int k = 0; k < AGG_PER; ++k)
+            if (pending >> k & 1u)
+                asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];"
+                             : "=l"(word[k])
+                             : "l"(st64 + base + 32 * k + lane)
+                             : "memory");
+#pragma unroll
+        for (int k = 0; k < AGG_PER; ++k)
+            if ((pending >> k & 1u) && ((unsigned)word[k] >> 2) == epoch) {
+                sbuf[32 * k + lane] = word[k];
+                pending &= ~(1u << k);
+            }
+        if (__all_sync(0xffffffffu, pending == 0)) break;
+        __nanosleep(ns);
+    }
+    __syncwarp();
+    const int per = (cnt + 31) / 32;
+    VT a;
+    a.ok = false;
+#pragma unroll
+    for (int k = 0; k < AGG_PER; ++k) {
+        const int i = lane * per + k;
+        if (k < per && i < cnt) {
+            const skel_u64 w = sbuf[i];
+            VT x;
+            x.ok = ((unsigned)w & 3u) == 1u;
+            x.v = skel::bit_cast<skel_S>((unsigned)(w >> 32)).v;
+            a = comb(a, x, t);
+        }
+    }
+    __syncwarp();  // sbuf is reused by the next window
+    a = warp_fold(a, lane, t);
+    return vt_shfl_idx(a, 0);
+}
+
 
 // work item q of a CTA's sequence: P1 of slices 0..LAG-1, then per slice s:
 // P1(s+LAG) x CH (if that slice exists), P2(s) x CH.  Returns false past the
@@ -855,6 +909,7 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
     __shared__ skel_u64 full_bar[SSTAGES], empty_bar[SSTAGES], outs_bar[SSTAGES], pre_full[NPRE], pre_empty[NPRE];
     __shared__ VT wsc[2][SNW];  // warp partials, alternated between consecutive tiles
     __shared__ VT s_pre[NPRE];
+    __shared__ skel_u64 s_win[(PACKED && SKEL_SCAN_CPOLL) ? PW * 32 * AGG_PER : 1];  // coalesced-poll transpose
     const int t = threadIdx.x, lane = t & 31, w = t >> 5;
     const skel_u64 G = gridDim.x, c = blockIdx.x;
     const skel_u64 nft = n / STILE;  // full tiles
@@ -960,7 +1015,13 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
             const int cnt = s == 0 ? (int)c : (int)G - 1;
             VT win;
             win.ok = false;
-            if (cnt > 0) win = warp_fold_aggs(status + (c % REPL) * rstride, flags, aggv, base, cnt, epoch, lane, tup);
+            if (cnt > 0) {
+                if constexpr (PACKED && SKEL_SCAN_CPOLL)
+                    win = warp_fold_aggs_coalesced(status + (c % REPL) * rstride, s_win + k * 32 * AGG_PER, base, cnt,
+                                                   epoch, lane, tup);
+                else
+                    win = warp_fold_aggs(status + (c % REPL) * rstride, flags, aggv, base, cnt, epoch, lane, tup);
+            }
             if (lane == 0) {
                 SKEL_STAMP(1, s, c);
                 s_pre[slot] = win;
