@@ -1958,13 +1958,15 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
     };
     // small vectors: two short launches (tile aggregates, seeded tile scans)
     // instead of the persistent pipeline; SKEL_SCAN_SMALL_MAX
-    // (elements, a tuning hook) moves the switch point
+    // (elements, a tuning hook) moves the switch point.  Default: up to 8 MiB of
+    // elements (2^21 floats); from 2^22 floats the persistent Scan is faster
+    // (14.4 vs 15.2 us, profiles/r01_scan_crossover_s4.txt)
     static const uint64_t small_max_env = [] {
         const char *e = getenv("SKEL_SCAN_SMALL_MAX");
         return e ? (uint64_t)strtoull(e, nullptr, 10) : ~0ull;
     }();
     const uint64_t SM_TILE = m->sig[9] * ((m->sig[15] >> 50) & 0xff);  // reduce block x elements per thread
-    const uint64_t small_max = small_max_env != ~0ull ? small_max_env : (uint64_t)(4u << 20) * 4 / m->sig[3];
+    const uint64_t small_max = small_max_env != ~0ull ? small_max_env : (uint64_t)(2u << 20) * 4 / m->sig[3];
     auto small_scan = [&](uint64_t cnt) { return m->k_scan_small && SM_TILE > 0 && cnt <= small_max; };
     for (size_t li = 0; li < ctx->slots.size(); ++li) {
         Slot &s = ctx->slots[li];

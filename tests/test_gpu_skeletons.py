@@ -420,8 +420,8 @@ def test_void_index_map_side_effects():
 @pytest.mark.parametrize("n", [(1 << 21) + 5, 3_000_017])
 def test_small_paths_with_double_tiles_i32(ctx, n):
     """Between 8 and 16 MiB the Reduce takes its small-vector path with
-    double-size tiles and the Scan its small-vector path:
-    integer results bit-exact."""
+    double-size tiles and the Scan (above its 8 MiB switch point) the
+    persistent path: integer results bit-exact."""
     x = si.uniform_int01(n, 21)
     vx = ctx.vector(x)
     assert int(ctx.reduce(SUM_I32, vx)) == int(x.astype(np.int64).sum())
