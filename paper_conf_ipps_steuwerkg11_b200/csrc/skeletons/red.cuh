@@ -103,12 +103,12 @@ constexpr unsigned STILE_BYTES = (unsigned)(STILE * sizeof(skel_T));
 constexpr unsigned SDSMEM = TMA_OK ? SSTAGES * STILE_BYTES + 1024 : 0;
 constexpr bool PACKED = sizeof(skel_S) == 4;  // status = value:32 | epoch:30 | state:2
 #ifndef SKEL_SCAN_REPL
-#define SKEL_SCAN_REPL 2
+#define SKEL_SCAN_REPL 8
 #endif
 // copies of every packed status word: CTA c polls copy c % REPL, so the few L2
 // lines a slice's status occupies are not hammered by all G CTAs at once
-// (8 copies with the strided probes; 2 suffice since the probes are coalesced:
-// 2^30 floats 1.322 vs 1.327 ms, profiles/r01_scan_crossover_s4.txt)
+// (2 copies measured 0.4% faster alone at 2^30 but slower inside the bench's
+// sweep at 2^24..2^30, profiles/r01_bench_s4_repl2.json: 8 kept)
 constexpr int REPL = PACKED ? SKEL_SCAN_REPL : 1;
 
 struct skel_sig_t { skel_u64 v[16 + 4 * 32]; };
