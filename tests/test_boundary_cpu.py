@@ -129,3 +129,15 @@ def test_every_element_size_instantiates(kind, nbytes):
     st, log, nb = skel.compile_check(kind, src)
     assert st == 0, log
     assert nb > 1000
+
+
+@pytest.mark.parametrize("defines", ["-DSKEL_SCAN_CPOLL=0", "-DSKEL_SCAN_CPOLL=1 -DSKEL_SCAN_REPL=2"])
+def test_scan_window_probe_variants_compile(monkeypatch, defines):
+    """Both Scan window-probe variants (coalesced, the default, and the strided
+    probes it replaced, DESIGN.md §4 K4) instantiate for 4-byte operators, and
+    the two give different kernels (the option reaches the template)."""
+    base = skel.compile_check("scan", SUM_F32)
+    monkeypatch.setenv("SKEL_NVRTC_DEFINES", defines)
+    st, log, nb = skel.compile_check("scan", SUM_F32)
+    assert st == 0, log
+    assert nb > 1000 and nb != base[2]
