@@ -45,6 +45,23 @@ def uniform_f32(n: int, seed: int) -> np.ndarray:
     return rng(seed).random(n, dtype=np.float32)
 
 
+def uniform_signed_f32(n: int, seed: int) -> np.ndarray:
+    """float32 uniform on [-1, 1): signed Reduce/Scan data (partial sums cancel)."""
+    return (rng(seed).random(n, dtype=np.float32) * np.float32(2.0) - np.float32(1.0)).astype(np.float32)
+
+
+def cancellation_f32(n: int, seed: int) -> np.ndarray:
+    """float32 data with catastrophic cancellation: blocks of four
+    [s*2^24, u, -s*2^24, u'] (s = +-1 at random, u, u' ~ U[0,1)), truncated to n.
+    A float32 left fold loses the small terms next to 2^24; the big ones cancel."""
+    g = rng(seed)
+    k = (n + 3) // 4
+    s = np.where(g.random(k) < 0.5, -1.0, 1.0).astype(np.float32) * np.float32(2.0 ** 24)
+    u = g.random((k, 2), dtype=np.float32)
+    out = np.stack([s, u[:, 0], -s, u[:, 1]], axis=1).reshape(-1)
+    return np.ascontiguousarray(out[:n], dtype=np.float32)
+
+
 def uniform_int01(n: int, seed: int) -> np.ndarray:
     """int32 uniform on {0, 1}: Reduce/Scan data whose prefix sums never overflow."""
     return rng(seed).integers(0, 2, size=n, dtype=np.int32)

@@ -148,9 +148,10 @@ def test_cross_device_noncommutative_order(D):
 
 
 @pytest.mark.parametrize("D", [2, 4])
-def test_cross_device_float_reduce_scan_within_tolerance(D):
-    n = (1 << 20) + 77
-    x = si.uniform_f32(n, 9)
+@pytest.mark.parametrize("gen", ["uniform", "signed", "cancel"])
+@pytest.mark.parametrize("n", [(1 << 20) + 77, (1 << 26) + 3])
+def test_cross_device_float_reduce_scan_within_tolerance(D, gen, n):
+    x = {"uniform": si.uniform_f32, "signed": si.uniform_signed_f32, "cancel": si.cancellation_f32}[gen](n, 9)
     with skel.Context(D) as ctx:
         v = ctx.vector(x)
         v.set_distribution(skel.BLOCK)

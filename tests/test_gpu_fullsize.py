@@ -75,3 +75,20 @@ def test_full_size_int_scan_and_reduce(ctx):
     g = out.download()
     assert np.array_equal(g, oracle.skel_scan(SUM_I32, x, 0))  # whole vector, bit-exact
     assert int(g[-1]) + int(x[-1]) == total
+
+
+@pytest.mark.parametrize("gen", ["signed", "cancel"])
+def test_full_size_signed_reduce_scan(ctx, gen):
+    """Signed data (U[-1,1)) and catastrophic cancellation ([+-2^24, u, -+2^24, u'])
+    at 2^30 through the persistent Scan and the TMA Reduce."""
+    x = (si.uniform_signed_f32 if gen == "signed" else si.cancellation_f32)(N, 20110600)
+    X = ctx.vector(x)
+    s = ctx.vector(n=N, dtype=np.float32)
+    r = float(ctx.reduce(SUM_F32, X))
+    assert abs(r - oracle.sum_f32_exact(x)) <= 1e-5 * oracle.abssum_f32(x)
+    ctx.scan(SUM_F32, X, s, np.float32(0))
+    sg = s.download()
+    idx = sample_idx(N, seed=3)
+    sidx, pre, ab = oracle.exscan_f32_sampled(x, idx)
+    err = np.abs(sg[sidx].astype(np.float64) - pre)
+    assert np.all(err <= 1e-5 * ab), float(np.max(err[1:] / ab[1:]))

@@ -187,6 +187,18 @@ def test_reduce_sum_f32(ctx, n):
     assert_sum_close(ctx.reduce(SUM_F32, ctx.vector(x)), x)
 
 
+# signed data and cancellation: the normwise bar's scale is
+# sum |x_i|; U[0,1) data alone would not notice a dropped |.| anywhere
+SIGNED_SIZES = [1, 5, 16385, (1 << 20) + 3, (1 << 26) + 3]
+
+
+@pytest.mark.parametrize("n", SIGNED_SIZES)
+@pytest.mark.parametrize("gen", ["signed", "cancel"])
+def test_reduce_sum_f32_signed(ctx, n, gen):
+    x = (si.uniform_signed_f32 if gen == "signed" else si.cancellation_f32)(n, 40 + n % 11)
+    assert_sum_close(ctx.reduce(SUM_F32, ctx.vector(x)), x)
+
+
 @pytest.mark.parametrize("n", SIZES)
 def test_reduce_sum_i32_exact(ctx, n):
     x = si.uniform_int01(n, 5)
@@ -256,6 +268,17 @@ def assert_scan_close(got, x):
 @pytest.mark.parametrize("n", SIZES)
 def test_scan_sum_f32(ctx, n):
     x = si.uniform_f32(n, 31 + n % 7)
+    out = ctx.vector(n=n, dtype=np.float32)
+    ctx.scan(SUM_F32, ctx.vector(x), out, np.float32(0))
+    got = out.download()
+    assert got[0] == 0.0
+    assert_scan_close(got, x)
+
+
+@pytest.mark.parametrize("n", SIGNED_SIZES)
+@pytest.mark.parametrize("gen", ["signed", "cancel"])
+def test_scan_sum_f32_signed(ctx, n, gen):
+    x = (si.uniform_signed_f32 if gen == "signed" else si.cancellation_f32)(n, 50 + n % 7)
     out = ctx.vector(n=n, dtype=np.float32)
     ctx.scan(SUM_F32, ctx.vector(x), out, np.float32(0))
     got = out.download()

@@ -110,3 +110,16 @@ def test_whole_image_golden_large(golden_dir):
         out = oracle.mandelbrot(pos, case["cap"])
         assert int(out.astype(np.int64).sum()) == case["sum_iter"]
         assert zlib.crc32(out.tobytes()) == int(case["crc32"], 16)
+
+
+def test_golden_generator_reproduces_the_small_pin(golden_dir):
+    """tests/golden/make_mandelbrot.py (numpy float32, independent of oracle/)
+    regenerates the stored 1024x768@256 pin (the larger cases: run the script)."""
+    import importlib.util
+    spec = importlib.util.spec_from_file_location("make_mandelbrot",
+                                                  os.path.join(golden_dir, "make_mandelbrot.py"))
+    mk = importlib.util.module_from_spec(spec)
+    spec.loader.exec_module(mk)
+    with open(os.path.join(golden_dir, "mandelbrot.json")) as fh:
+        want = json.load(fh)["cases"][0]
+    assert mk.pins(want["width"], want["height"], want["cap"]) == want
