@@ -161,6 +161,139 @@ def cpu_baseline(total_log2=30, chunk_log2=26):
             "host_cpus": os.cpu_count()}
 
 
+def host_info() -> dict:
+    """The host the oracle runs on: logical CPUs, the ones this process may
+    use, and lscpu's model name."""
+    model = None
+    try:
+        out = subprocess.run(["lscpu"], capture_output=True, text=True, timeout=10).stdout
+        for ln in out.splitlines():
+            if ln.lower().startswith("model name"):
+                model = ln.split(":", 1)[1].strip()
+                break
+    except Exception:
+        pass
+    try:
+        usable = len(os.sched_getaffinity(0))
+    except Exception:
+        usable = os.cpu_count()
+    return {"host_cpus": os.cpu_count(), "usable_cpus": usable, "cpu_model": model}
+
+
+def _threads() -> int:
+    return max(1, host_info()["usable_cpus"] or 1)
+
+
+def _par(fn, items, threads):
+    """Run fn over items on `threads` host threads (the oracle's C loops release
+    the GIL, so disjoint chunks run side by side)."""
+    from concurrent.futures import ThreadPoolExecutor
+    if threads <= 1:
+        return [fn(it) for it in items]
+    with ThreadPoolExecutor(max_workers=threads) as ex:
+        return list(ex.map(fn, items))
+
+
+def oracle_step_allcores(x, y, threads):
+    """oracle_step on all host cores: Map/Zip/Reduce on disjoint chunks; Scan as
+    chunk sums (float64) then seeded chunk scans (oracle_exscan_f32_seeded)."""
+    import oracle
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MAP_F32, SAXPY_F32
+    n = x.size
+    cuts = np.linspace(0, n, threads + 1).astype(np.int64)
+    rng = list(zip(cuts[:-1], cuts[1:]))
+    m, z, s = np.empty_like(x), np.empty_like(x), np.empty_like(x)
+
+    def mz(r):
+        a, b = r
+        m[a:b] = oracle.skel_map(MAP_F32, x[a:b], np.float32)
+        z[a:b] = oracle.skel_zip(SAXPY_F32, x[a:b], y[a:b], np.float32, args=[np.float32(2.5)])
+    _par(mz, rng, threads)
+    sums = _par(lambda r: oracle.sum_f32_exact(x[r[0]:r[1]]), rng, threads)
+    pre = np.concatenate([[0.0], np.cumsum(sums)])
+    _par(lambda k: oracle.exscan_f32_seeded(x[rng[k][0]:rng[k][1]], pre[k], s[rng[k][0]:rng[k][1]]),
+         range(len(rng)), threads)
+    return float(pre[-1])
+
+
+def cpu_baseline_allcores(total_log2=30, chunk_log2=26):
+    """The skeleton step's oracle on every usable host core (same bounded sample
+    as cpu_baseline)."""
+    import skel_inputs as si
+    T = _threads()
+    chunks = 1 << (total_log2 - chunk_log2)
+    n = 1 << chunk_log2
+    oracle_step(si.uniform_f32(1024, 1), si.uniform_f32(1024, 2))
+    t = 0.0
+    for c in range(chunks):
+        x, y = si.uniform_f32(n, SEED + 2 * c), si.uniform_f32(n, SEED + 2 * c + 1)
+        t0 = time.perf_counter()
+        oracle_step_allcores(x, y, T)
+        t += time.perf_counter() - t0
+    return {"value": STEP_BYTES * chunks * n / t / 1e9, "unit": "GB/s", "cores": T, "kind": "oracle (all cores)",
+            "sample": f"the same 2^{total_log2} elements in {chunks} chunks of 2^{chunk_log2}, each split over {T} "
+                      f"threads (scan: chunk sums, then seeded chunk scans), {t:.1f} s"}
+
+
+def cpu_baseline_mandelbrot():
+    """Oracle (eq. (5), oracle_mandelbrot) for configs[0] and configs[2]: one
+    thread, and every usable core over row bands."""
+    import oracle
+    import skel_inputs as si
+    T = _threads()
+    res = {}
+    for tag, (w, h) in (("configs0_1024x768", (1024, 768)), ("configs2_4096x3072", (4096, 3072))):
+        pos = si.mandelbrot_positions(w, h)
+        t0 = time.perf_counter()
+        oracle.mandelbrot(pos, 256)
+        t1 = time.perf_counter() - t0
+        cuts = np.linspace(0, pos.size, 4 * T + 1).astype(np.int64)
+        t0 = time.perf_counter()
+        _par(lambda k: oracle.mandelbrot(pos[cuts[k]:cuts[k + 1]], 256), range(4 * T), T)
+        tT = time.perf_counter() - t0
+        res[tag] = {"ms_1core": t1 * 1e3, "Mpix_per_s_1core": pos.size / t1 / 1e6,
+                    "ms_allcores": tT * 1e3, "Mpix_per_s_allcores": pos.size / tT / 1e6}
+    return {"kind": "oracle", "unit": "Mpix/s", "cores": T, "value": res["configs2_4096x3072"]["Mpix_per_s_1core"],
+            "sample": "whole images, cap 256 (value: configs[2] on 1 core)", **res}
+
+
+def _lm_allcores(ev, f, T):
+    """Listing 3 for one subset on T threads: each thread's chunk of events
+    into a private error image (oracle_lmosem_error_image), the images summed,
+    then the update (oracle_lmosem_update)."""
+    import oracle
+    cuts = np.linspace(0, ev.size, T + 1).astype(np.int64)
+    parts = _par(lambda k: oracle.lmosem_error_image(ev[cuts[k]:cuts[k + 1]], f)[0], range(T), T)
+    c = parts[0]
+    for p in parts[1:]:
+        c += p
+    return oracle.lmosem_update(f, c)
+
+
+def cpu_baseline_lmosem(subsets):
+    """Oracle LM OSEM (Listing 3): one subset on one core, the same subset and
+    the full 10-subset reconstruction (configs[4], once per job) on all cores."""
+    import oracle
+    T = _threads()
+    nvox = 150 * 150 * 280
+    f0 = np.ones(nvox, np.float64)
+    t0 = time.perf_counter()
+    oracle.lmosem_subset(subsets[0], f0)
+    t1 = time.perf_counter() - t0
+    t0 = time.perf_counter()
+    _lm_allcores(subsets[0], f0, T)
+    tT = time.perf_counter() - t0
+    t0 = time.perf_counter()
+    f = f0.copy()
+    for ev in subsets:
+        f = _lm_allcores(ev, f, T)
+    tR = time.perf_counter() - t0
+    return {"kind": "oracle", "unit": "s", "cores": T, "value": t1,
+            "sample": f"one subset of {subsets[0].size} events on 1 core (value), on {T} cores, and the "
+                      f"{len(subsets)}-subset reconstruction on {T} cores",
+            "subset_s_1core": t1, "subset_s_allcores": tT, "full_recon_s_allcores": tR}
+
+
 def run_reference(args):
     world, rank, _ = env_world()
     if rank != 0:
@@ -320,9 +453,10 @@ def main():
                 "algorithmic_bytes_per_launch": BYTES_PER_ELEM[dom] * nloc,
                 "traffic": traffic, "traffic_source": "profiles/traffic.json (ncu --set full)" if traffic else None}
 
-    # ---- end to end through the C-ABI: pinned host inputs -> result scalar
+    # ---- end to end through the C-ABI: pinned host inputs -> every result on the host
     e2e = None
     if args.e2e_steps > 0:
+        hbuf = torch.empty(nloc, dtype=torch.float32, pin_memory=True).numpy()  # the user's result buffer
         ctx.sync()
         barrier()
         st0 = ctx.stats()
@@ -334,15 +468,19 @@ def main():
             ctx.map(MAP_F32, x, m)
             ctx.zip(SAXPY_F32, x, y, z, args=[a])
             ctx.scan(SUM_F32, x, s, np.float32(0))
-            ctx.reduce(SUM_F32, x)  # blocking: the step's result on the host
+            ctx.reduce(SUM_F32, x)  # blocking: the scalar on the host
+            for v in (m, z, s):     # this rank's block of every output vector on the host
+                v.download_part(lo, hbuf)
         ctx.sync()
         dt = max_over_ranks(time.perf_counter() - t0) / args.e2e_steps
         st1 = ctx.stats()
         e2e = {"value": STEP_BYTES * N / dt / 1e9, "unit": "GB/s", "ms_per_step": dt * 1e3,
                "h2d_bytes_per_step": (st1["h2d_bytes"] - st0["h2d_bytes"]) // args.e2e_steps,
                "d2h_bytes_per_step": (st1["d2h_bytes"] - st0["d2h_bytes"]) // args.e2e_steps,
-               "path": "skel_vector_mark_host_modified on pinned host mirrors, then map/zip/scan/reduce "
-                       "(lazy H2D inside) and skel_reduce's blocking D2H of the scalar"}
+               "path": "skel_vector_mark_host_modified on pinned host mirrors of x, y, then map/zip/scan/reduce "
+                       "(lazy H2D inside), skel_reduce's blocking D2H of the scalar, and skel_vector_download_part "
+                       "of the Map, Zip and Scan outputs into a pinned host buffer"}
+        del hbuf
 
     # free the big vectors before the side measurements
     for v in (x, y, m, z, s):
@@ -359,6 +497,12 @@ def main():
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu:
         cpu = cpu_baseline()
+        cpu.update(host_info())
+        cpu["allcores"] = cpu_baseline_allcores()
+        if "mandelbrot" in extras:
+            extras["mandelbrot"]["cpu_baseline"] = cpu_baseline_mandelbrot()
+        if "lmosem" in extras:
+            extras["lmosem"]["cpu_baseline"] = cpu_baseline_lmosem(lm_subsets(1_000_000, 10, 0, 1_000_000))
 
     if rank == 0:
         line = {"metric": METRIC, "value": value, "unit": "GB/s", "n_gpus": world, "steps": args.steps,
@@ -702,13 +846,27 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
     return res
 
 
+_LM_CACHE: dict = {}
+
+
+def lm_subsets(nev, nsub, lo, hi):
+    """Events [lo, hi) of subsets 0..nsub-1 of nev events each (generated once per job)."""
+    import skel_inputs as si
+    out = []
+    for l in range(nsub):
+        if (nev, l) not in _LM_CACHE:
+            _LM_CACHE[(nev, l)] = si.lmosem_events(nev, subset=l)
+        out.append(_LM_CACHE[(nev, l)][lo:hi])
+    return out
+
+
 def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
     """configs[3]/[4]: one subset of 10^6 events into 150x150x280, events block-distributed."""
     import torch
     import skel_inputs as si
     from paper_conf_ipps_steuwerkg11_b200.lmosem import LMOSEM
     nev = 1_000_000
-    ev = si.lmosem_events(nev, subset=0)
+    ev = lm_subsets(nev, 1, 0, nev)[0]
     rec = LMOSEM(ctx)
     rec.prepare()
     evv = ctx.vector(n=nev, dtype=ev.dtype)
@@ -793,8 +951,7 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
     full = {}
     for mode in ("given", "ordered"):
         subs = []
-        for l in range(nsub):
-            evl = si.lmosem_events(nev, subset=l)[lo:hi]
+        for evl in lm_subsets(nev, nsub, lo, hi):
             if mode == "ordered":
                 evl, _ = prepare_part(evl)
             v = ctx.vector(n=nev, dtype=evl.dtype)

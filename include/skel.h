@@ -96,6 +96,8 @@ typedef struct {
     uint64_t compile_mem_hits, compile_disk_hits, compile_misses;
     double compile_ms;   /* total NVRTC time                                          */
     double disk_load_ms; /* total time loading cubins from the disk cache */
+    uint64_t scan_coop_fallbacks; /* persistent Scans that could not be made co-resident
+                                     (cooperative launch refused) and ran as two launches */
 } skel_stats;
 
 /* ---- context ------------------------------------------------------------
@@ -160,6 +162,15 @@ int skel_vector_upload(skel_vec_t v, const void *src, size_t n);
  * the range is written into the full host copy. */
 int skel_vector_upload_part(skel_vec_t v, size_t lo, const void *src, size_t count);
 int skel_vector_download(skel_vec_t v, void *dst, size_t n);
+/* Download elements [lo, lo + count) into dst (the counterpart of
+ * upload_part).  If the host copy is valid and covers the range it is copied
+ * from there; otherwise the range is read straight from the device storage
+ * that holds it (one D2H per overlapping part; a pinned dst gives the full
+ * PCIe/C2C rate) without touching the host mirror.  In rank mode the range
+ * must lie in this rank's block part (or the vector must be copy-distributed
+ * and not diverged, or single on rank 0), else SKEL_ERR_STATE.  Blocks.
+ * SKEL_ERR_SIZE if the range is outside the vector. */
+int skel_vector_download_part(skel_vec_t v, size_t lo, void *dst, size_t count);
 int skel_vector_host_ptr(skel_vec_t v, void **host);
 int skel_vector_mark_host_modified(skel_vec_t v);
 int skel_vector_fill(skel_vec_t v, const void *value);

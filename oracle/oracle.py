@@ -64,6 +64,7 @@ def core() -> ctypes.CDLL:
         lib.oracle_abssum_f32.argtypes = [P, ctypes.c_size_t]
         lib.oracle_abssum_f32.restype = ctypes.c_double
         lib.oracle_exscan_f32_exact.argtypes = [P, P, P, ctypes.c_size_t]
+        lib.oracle_exscan_f32_seeded.argtypes = [P, P, ctypes.c_size_t, ctypes.c_double]
         lib.oracle_exscan_f32_sampled.argtypes = [P, ctypes.c_size_t, P, ctypes.c_size_t, P, P]
         _core = lib
     return _core
@@ -272,6 +273,16 @@ def exscan_f32_exact(x: np.ndarray):
     if x.size:
         core().oracle_exscan_f32_exact(_ptr(x), _ptr(out), _ptr(ab), x.size)
     return out, ab
+
+
+def exscan_f32_seeded(x: np.ndarray, s0: float, out: np.ndarray | None = None) -> np.ndarray:
+    """Exclusive float '+' scan of a chunk whose preceding elements sum to s0."""
+    x = np.ascontiguousarray(x, dtype=np.float32)
+    if out is None:
+        out = np.empty(x.size, np.float32)
+    if x.size:
+        core().oracle_exscan_f32_seeded(_ptr(x), _ptr(out), x.size, float(s0))
+    return out
 
 
 def exscan_f32_sampled(x: np.ndarray, idx: np.ndarray):

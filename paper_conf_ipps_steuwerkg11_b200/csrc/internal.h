@@ -74,6 +74,8 @@ struct Slot {
     int sms = 148;  // multiprocessor count
     cudaStream_t stream = nullptr;
     cudaEvent_t ev = nullptr;  // join event
+    cudaEvent_t ev_scan = nullptr;  // after this slot's persistent Scan (chains slots sharing a GPU)
+    bool ev_scan_live = false;      // ev_scan has been recorded at least once
     // grow-only workspace for reduce/scan partials, look-back status, seeds
     char *ws = nullptr;
     size_t ws_cap = 0;
@@ -113,6 +115,9 @@ struct skel_ctx_s {
     std::string cache_dir;
     bool disk_cache = true;
     bool fmad = false;
+    // every pair of distinct physical devices has peer access enabled (in-process
+    // mode); the fused peer-memory paths need it, else they take the unfused one
+    bool peer_all = true;
     skel_stats stats{};
     std::string last_error;
     std::map<std::string, std::unique_ptr<skelrt::Module>> modules;

@@ -344,6 +344,30 @@ int plan_exchange(skel_dist from, skel_dist to, skel_combine combine) {
     return to == SKEL_BLOCK ? SKEL_XCHG_LOCAL_SLICE : SKEL_XCHG_KEEP_ROOT;
 }
 
+// Kernels that read other devices' buffers (combine, gather) need peer access.
+// Without it between some pair of GPUs (ctx->peer_all false), every operand on
+// another physical device is first copied into slot s's scratch (cudaMemcpy
+// stages through the host when P2P is unavailable) and read from there.
+int stage_remote(skel_ctx_s *ctx, Slot &s, std::vector<const void *> &src, const std::vector<int> &src_dev,
+                 size_t bytes) {
+    if (ctx->peer_all) return SKEL_OK;
+    size_t remote = 0;
+    for (size_t j = 0; j < src.size(); ++j) remote += src_dev[j] != s.dev;
+    if (!remote) return SKEL_OK;
+    const size_t stride = align_up(std::max<size_t>(bytes, 1), 256);
+    TRY(scratch(ctx, s, stride * remote));
+    DevGuard g(s.dev);
+    size_t k = 0;
+    for (size_t j = 0; j < src.size(); ++j) {
+        if (src_dev[j] == s.dev) continue;
+        char *dst = s.scratch + stride * k++;
+        if (bytes) CK(ctx, cudaMemcpyAsync(dst, src[j], bytes, cudaMemcpyDefault, s.stream));
+        ctx->stats.d2d_bytes += bytes;
+        src[j] = dst;
+    }
+    return SKEL_OK;
+}
+
 // ---- the exchanges (DESIGN.md §5 table T1) -----------------------------------
 // Local mode: every logical device is in this process; data moves with
 // cudaMemcpyAsync (peer or same GPU) and the combine kernel.
@@ -441,7 +465,9 @@ int xchg_local(skel_vec_s *v, int x, skel_combine combine) {
                 B[d].count = cnt;
                 if (!cnt) continue;
                 std::vector<const void *> src(D);
-                for (int j = 0; j < D; ++j) src[j] = B[j].base + lo * es;
+                std::vector<int> sdev(D);
+                for (int j = 0; j < D; ++j) src[j] = B[j].base + lo * es, sdev[j] = S[j].dev;
+                TRY(stage_remote(ctx, S[d], src, sdev, cnt * es));
                 DevGuard g(S[d].dev);
                 CK(ctx, launch_combine(B[d].base + lo * es, src.data(), D, cnt, v->dt, combine, S[d].stream));
                 ctx->stats.kernel_launches++;
@@ -455,7 +481,9 @@ int xchg_local(skel_vec_s *v, int x, skel_combine combine) {
         }
         case SKEL_XCHG_REDUCE: {
             std::vector<const void *> src(D);
-            for (int j = 0; j < D; ++j) src[j] = B[j].base;
+            std::vector<int> sdev(D);
+            for (int j = 0; j < D; ++j) src[j] = B[j].base, sdev[j] = S[j].dev;
+            TRY(stage_remote(ctx, S[0], src, sdev, n * es));
             DevGuard g(S[0].dev);
             CK(ctx, launch_combine(B[0].base, src.data(), D, n, v->dt, combine, S[0].stream));
             ctx->stats.kernel_launches++;
@@ -631,9 +659,19 @@ int set_distribution_fn(skel_vec_s *v, skel_dist dist, const char *src) {
         auto &S = ctx->slots;
         auto &B = v->bufs;
         TRY(join(ctx));
+        // operands of device d's fold, staged locally when P2P is missing
+        auto operands = [&](int d, size_t lo, size_t cnt, std::vector<const char *> &srcs) -> int {
+            std::vector<const void *> src(D);
+            std::vector<int> sdev(D);
+            for (int j = 0; j < D; ++j) src[j] = B[j].base + lo * es, sdev[j] = S[j].dev;
+            TRY(stage_remote(ctx, S[d], src, sdev, cnt * es));
+            srcs.resize(D);
+            for (int j = 0; j < D; ++j) srcs[j] = static_cast<const char *>(src[j]);
+            return SKEL_OK;
+        };
         if (dist == SKEL_SINGLE) {
-            std::vector<const char *> srcs(D);
-            for (int j = 0; j < D; ++j) srcs[j] = B[j].base;
+            std::vector<const char *> srcs;
+            TRY(operands(0, 0, n, srcs));
             TRY(fold_raw(ctx, m, S[0], srcs, B[0].base, n));
             ctx->stats.d2d_bytes += (D - 1) * n * es;
             TRY(join(ctx));
@@ -647,8 +685,8 @@ int set_distribution_fn(skel_vec_s *v, skel_dist dist, const char *src) {
             for (int d = 0; d < D; ++d) {
                 const size_t lo = part_lo(v, d), cnt = want_count(v, SKEL_BLOCK, d);
                 if (!cnt) continue;
-                std::vector<const char *> srcs(D);
-                for (int j = 0; j < D; ++j) srcs[j] = B[j].base + lo * es;
+                std::vector<const char *> srcs;
+                TRY(operands(d, lo, cnt, srcs));
                 char *own = B[d].base + lo * es;
                 if (d < 2) {
                     TRY(fold_raw(ctx, m, S[d], srcs, own, cnt));
@@ -1166,10 +1204,13 @@ int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args
     const int K = cross ? (int)((in->n + ps - 1) / ps) : 1;  // devices holding data
     if (cross && !ctx->rank_mode) {
         TRY(join(ctx));
-        std::vector<const void *> src(K);
-        for (int j = 0; j < K; ++j) src[j] = ctx->slots[j].ws + Ls[j].o_res;
+        std::vector<const void *> src0(K);
+        std::vector<int> sdev(K);
+        for (int j = 0; j < K; ++j) src0[j] = ctx->slots[j].ws + Ls[j].o_res, sdev[j] = ctx->slots[j].dev;
         for (size_t li = 0; li < ctx->slots.size(); ++li) {
             Slot &s = ctx->slots[li];
+            std::vector<const void *> src = src0;
+            TRY(stage_remote(ctx, s, src, sdev, es));
             DevGuard g(s.dev);
             CK(ctx, launch_gather(s.ws + Ls[li].o_gather, src.data(), K, es, s.stream));  // packed slot<T>[K]
             ctx->stats.kernel_launches++;
@@ -1260,6 +1301,7 @@ static int init_slot(skel_ctx_s *ctx, int d, int dev) {
     CK(ctx, cudaDeviceGetAttribute(&s.sms, cudaDevAttrMultiProcessorCount, dev));
     CK(ctx, cudaStreamCreateWithFlags(&s.stream, cudaStreamNonBlocking));
     CK(ctx, cudaEventCreateWithFlags(&s.ev, cudaEventDisableTiming));
+    CK(ctx, cudaEventCreateWithFlags(&s.ev_scan, cudaEventDisableTiming));
     void *p = nullptr;
     CK(ctx, cudaMalloc(&p, 256));
     CK(ctx, cudaMemsetAsync(p, 0, 256, s.stream));  // ordered with the epoch write below
@@ -1308,7 +1350,14 @@ int skel_init(int num_devices, skel_ctx_t *out) {
                 cudaDeviceCanAccessPeer(&can, a.dev, b.dev);
                 if (can) {
                     DevGuard g(a.dev);
-                    if (cudaDeviceEnablePeerAccess(b.dev, 0) != cudaSuccess) cudaGetLastError();
+                    cudaError_t pe = cudaDeviceEnablePeerAccess(b.dev, 0);
+                    if (pe == cudaErrorPeerAccessAlreadyEnabled) pe = cudaSuccess;
+                    if (pe != cudaSuccess) {
+                        cudaGetLastError();
+                        ctx->peer_all = false;
+                    }
+                } else {
+                    ctx->peer_all = false;
                 }
             }
     *out = ctx;
@@ -1378,6 +1427,7 @@ int skel_finalize(skel_ctx_t ctx) {
         cudaFree(s.st64);
         cudaFree(s.fl32);
         cudaEventDestroy(s.ev);
+        cudaEventDestroy(s.ev_scan);
         cudaStreamDestroy(s.stream);
     }
     delete ctx;
@@ -1572,6 +1622,63 @@ int skel_vector_download(skel_vec_t v, void *dst, size_t n) {
     return SKEL_OK;
 }
 
+int skel_vector_download_part(skel_vec_t v, size_t lo, void *dst, size_t count) {
+    if (!v || (!dst && count)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad download_part arguments");
+    skel_ctx_s *ctx = v->ctx;
+    if (lo > v->n || count > v->n - lo) return fail(ctx, SKEL_ERR_SIZE, "range outside the vector");
+    if (!count) return SKEL_OK;
+    const size_t es = v->es, hi = lo + count;
+    if (v->host_valid && v->host && lo >= v->host_lo && hi <= v->host_lo + v->host_n) {
+        TRY(sync_all(ctx));  // the mirror may still be the target of an in-flight D2H
+        memcpy(dst, v->host + (lo - v->host_lo) * es, count * es);
+        return SKEL_OK;
+    }
+    if (!v->dev_valid) TRY(ensure_device(v));
+    // which local slots hold [lo, hi) and where
+    struct Piece { size_t li, src_off, lo, cnt; };
+    std::vector<Piece> pieces;
+    bool covered = false;
+    if (v->dist == SKEL_BLOCK && ctx->D > 1) {
+        size_t got = 0;
+        for (size_t li = 0; li < ctx->slots.size(); ++li) {
+            size_t plo, phi;
+            part_range(v->n, ctx->D, ctx->slots[li].d, &plo, &phi);
+            const size_t a = std::max(lo, plo), b = std::min(hi, phi);
+            if (a < b) {
+                pieces.push_back({li, a - plo, a, b - a});
+                got += b - a;
+            }
+        }
+        covered = got == count;
+    } else if (v->dist == SKEL_COPY || ctx->D == 1) {
+        // device 0's copy (reading R6) -- or, in rank mode, the local copy if it cannot have diverged
+        if (!ctx->rank_mode || ctx->D == 1 || !v->diverged) {
+            pieces.push_back({0, lo, lo, count});
+            covered = true;
+        }
+    } else if (v->dist == SKEL_SINGLE && ctx->slots[0].d == 0) {
+        pieces.push_back({0, lo, lo, count});
+        covered = true;
+    }
+    if (!covered && ctx->rank_mode)  // a collective fallback would need every rank to take it
+        return fail(ctx, SKEL_ERR_STATE, "download_part in rank mode: the range is not held by this rank");
+    if (!covered) {  // in-process devices: the full download
+        TRY(ensure_host(v));
+        memcpy(dst, v->host + lo * es, count * es);
+        return SKEL_OK;
+    }
+    for (const Piece &p : pieces) {
+        Slot &s = ctx->slots[p.li];
+        const Buf &b = v->bufs[p.li];
+        DevGuard g(s.dev);
+        CK(ctx, cudaMemcpyAsync(static_cast<char *>(dst) + (p.lo - lo) * es, b.ptr(es) + p.src_off * es, p.cnt * es,
+                                cudaMemcpyDeviceToHost, s.stream));
+        ctx->stats.d2h_bytes += p.cnt * es;
+        ctx->stats.d2h_copies++;
+    }
+    return sync_all(ctx);
+}
+
 int skel_vector_host_ptr(skel_vec_t v, void **host) {
     if (!v || !host) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad arguments");
     TRY(ensure_host(v));
@@ -1752,8 +1859,11 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
     if (b->dist != SKEL_COPY && ctx->D > 1)
         return fail(ctx, SKEL_ERR_STATE, "a combine merges per-device copies: b must be SKEL_COPY");
     const int D = ctx->D;
+    // in-process mode loads and stores through the other devices' buffers: only
+    // with peer access between every pair of distinct GPUs (else the unfused
+    // reduce-scatter + Zip + all-gather, which moves data with copies)
     const bool fused = D > 1 && D <= 16 && (a->dist == SKEL_COPY || a->dist == SKEL_BLOCK) &&
-                       (out != a || a->dist == SKEL_COPY) && !ctx->capturing;
+                       (out != a || a->dist == SKEL_COPY) && !ctx->capturing && (ctx->rank_mode || ctx->peer_all);
     if (!fused) {  // the same result as the unfused sequence
         if (D > 1) TRY(set_distribution(b, SKEL_BLOCK, combine));
         if (a->dist != b->dist) TRY(set_distribution(a, b->dist, SKEL_COMBINE_NONE));
@@ -1950,7 +2060,12 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
             occ = 1;
         }
     }
-    auto scan_grid = [&](const Slot &s) -> uint64_t { return (uint64_t)s.sms * (uint64_t)occ; };
+    // A window folds G-1 aggregates with one warp, at most 32 x AGG_PER = 512 of
+    // them (red.cuh), so the grid is capped at 513 CTAs (the kernel traps above)
+    constexpr uint64_t kScanMaxGrid = 32 * 16 + 1;
+    auto scan_grid = [&](const Slot &s) -> uint64_t {
+        return std::min<uint64_t>((uint64_t)s.sms * (uint64_t)occ, kScanMaxGrid);
+    };
     // one aggregate status word per (slice, CTA)
     auto scan_slots = [&](const Slot &s, uint64_t cnt) -> uint64_t {
         const uint64_t per_slice = scan_grid(s) * CH, nft = cnt / TILE;
@@ -1972,7 +2087,10 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         Slot &s = ctx->slots[li];
         const uint64_t cnt = in->bufs[li].count;
         Ls[li] = red_layout(m, D, red_parts(m, s, cnt), scan_slots(s, cnt));
-        const size_t extra = small_scan(cnt) ? (size_t)((cnt + SM_TILE - 1) / SM_TILE) * Ls[li].slot : 0;
+        // room for the small path's tile aggregates also when the persistent
+        // kernel is chosen: it falls back to the small path if the cooperative
+        // launch cannot make its grid co-resident
+        const size_t extra = SM_TILE > 0 ? (size_t)((cnt + SM_TILE - 1) / SM_TILE) * Ls[li].slot : 0;
         TRY(ensure_ws(ctx, s, Ls[li].total + extra));
     }
     if (cross) {
@@ -2004,7 +2122,49 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         }
         const void *pin = in->bufs[li].ptr(in->es);
         void *pout = out->bufs[li].ptr(out->es);
-        if (small_scan(cnt)) {
+        bool small = small_scan(cnt);
+        if (!small) {
+            // The persistent Scan's windows wait on aggregates of higher-index
+            // CTAs, so the whole grid must be resident at once: launch it
+            // cooperatively (the driver guarantees co-residency or refuses).
+            // Persistent Scans of logical devices that share one GPU run one
+            // after another (event chain) so their grids never interleave.
+            for (size_t lj = 0; lj < li; ++lj)
+                if (ctx->slots[lj].dev == s.dev && ctx->slots[lj].ev_scan_live)
+                    CK(ctx, cudaStreamWaitEvent(s.stream, ctx->slots[lj].ev_scan, 0));
+            CUtensorMap tin, tout;
+            const uint64_t rows = (cnt / TILE) * SRB;
+            int use_tma = m->sig[5] && make_tmap(&tin, pin, rows, (uint32_t)(SRB / 2)) &&
+                          make_tmap(&tout, pout, rows, (uint32_t)(SRB / 2));
+            void *status = s.st64, *flags = s.fl32, *aggv = s.ws + L.o_aggv, *incv = s.ws + L.o_incv;
+            unsigned *counters = s.counters;
+            unsigned *epoch_ptr = s.counters + 3;  // device-resident scan epoch (graph-replay safe)
+            void *total = nullptr;
+            void *params[] = {&tin, &tout, &pin, &pout, &cnt, &use_tma, idbuf.data(), &seed, &status, &flags,
+                              &aggv, &incv, &counters, &epoch_ptr, &total, abuf.data()};
+            cudaLaunchConfig_t cfg = {};
+            cfg.gridDim = dim3((unsigned)G);
+            cfg.blockDim = dim3((unsigned)m->sig[14]);
+            cfg.dynamicSmemBytes = use_tma ? m->sig[12] : 0;
+            cfg.stream = s.stream;
+            cudaLaunchAttribute attr[1];
+            attr[0].id = cudaLaunchAttributeCooperative;
+            attr[0].val.cooperative = 1;
+            cfg.attrs = attr;
+            cfg.numAttrs = 1;
+            const cudaError_t le = cudaLaunchKernelExC(&cfg, (const void *)m->k_scan, params);
+            if (le == cudaErrorCooperativeLaunchTooLarge) {
+                cudaGetLastError();  // fewer SMs than queried (MPS / green context): two short launches
+                ctx->stats.scan_coop_fallbacks++;
+                small = true;
+            } else {
+                CK(ctx, le);
+                CK(ctx, cudaEventRecord(s.ev_scan, s.stream));
+                s.ev_scan_live = true;
+                ctx->stats.kernel_launches++;
+            }
+        }
+        if (small && SM_TILE > 0) {
             const unsigned nt = (unsigned)((cnt + SM_TILE - 1) / SM_TILE);
             void *aggs = s.ws + L.total;
             void *pa[] = {&pin, &cnt, &aggs, abuf.data()};
@@ -2014,21 +2174,10 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
             CK(ctx, cudaLaunchKernel((const void *)m->k_scan_small, dim3(nt), dim3((unsigned)m->sig[9]), ps, 0,
                                      s.stream));
             ctx->stats.kernel_launches += 2;
-            continue;
+        } else if (small) {
+            return fail(ctx, SKEL_ERR_CUDA, "persistent Scan grid cannot be co-resident and this module has no "
+                                            "small-vector path");
         }
-        CUtensorMap tin, tout;
-        const uint64_t rows = (cnt / TILE) * SRB;
-        int use_tma = m->sig[5] && make_tmap(&tin, pin, rows, (uint32_t)(SRB / 2)) &&
-                      make_tmap(&tout, pout, rows, (uint32_t)(SRB / 2));
-        void *status = s.st64, *flags = s.fl32, *aggv = s.ws + L.o_aggv, *incv = s.ws + L.o_incv;
-        unsigned *counters = s.counters;
-        unsigned *epoch_ptr = s.counters + 3;  // device-resident scan epoch (graph-replay safe)
-        void *total = nullptr;
-        void *params[] = {&tin, &tout, &pin, &pout, &cnt, &use_tma, idbuf.data(), &seed, &status, &flags,
-                          &aggv, &incv, &counters, &epoch_ptr, &total, abuf.data()};
-        CK(ctx, cudaLaunchKernel((const void *)m->k_scan, dim3((unsigned)G), dim3((unsigned)m->sig[14]), params,
-                                 use_tma ? m->sig[12] : 0, s.stream));
-        ctx->stats.kernel_launches++;
     }
     out->dev_valid = true;
     device_wrote(out);

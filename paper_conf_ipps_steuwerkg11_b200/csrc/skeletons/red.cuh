@@ -17,10 +17,14 @@
 //    reduction (in-thread fold, shuffle tree lower-lane-left, warps in
 //    order), a running CTA aggregate, and a last-CTA-done ordered fold of the
 //    CTA partials: a single pass over the input (4 B/element for float).
-//  * Scan: single-pass decoupled look-back (Merrill & Garland) over
-//    dynamically ticketed tiles; tile status words carry an epoch so no
-//    memset is needed between launches; outputs are staged in the same
-//    swizzled smem stage and written by TMA tensor stores (8 B/element).
+//  * Scan: a persistent grid (one CTA per SM, launched cooperatively so the
+//    whole grid is co-resident) walks the vector in slices of G tiles; a
+//    CTA publishes its tile aggregate A(s,c) and folds the window of G-1
+//    aggregates W(s) = A(s-1,c+1..G-1) (+) A(s,0..c-1) ahead of its consumers
+//    (the window waits on higher-index CTAs of the previous slice, hence the
+//    co-residency requirement).  Status words carry an epoch so no memset is
+//    needed between launches; outputs are staged in the same swizzled smem
+//    stage and written by TMA tensor stores (8 B/element).
 //  * Element types whose size is not 4, 8 or 16 bytes, unaligned views and
 //    the ragged last tile use direct (LDG/STG) loads with the same ordering.
 
@@ -927,6 +931,9 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
         const skel_u64 left = nft - first;
         return (int)(left < (skel_u64)SCAN_CH ? left : (skel_u64)SCAN_CH);
     };
+    // a window folds G-1 aggregates with one warp (<= 32 x AGG_PER); the host
+    // caps the grid at 513 CTAs -- a larger grid would fold silently wrong
+    if (G - 1 > (skel_u64)(32 * AGG_PER)) __trap();
     if (t == 0) {
         for (int st = 0; st < SSTAGES; ++st) {
             skel::mbar_init(&full_bar[st], 1);

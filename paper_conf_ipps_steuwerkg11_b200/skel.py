@@ -46,7 +46,8 @@ class Stats(ctypes.Structure):
                 ("d2d_bytes", ctypes.c_uint64), ("nccl_bytes", ctypes.c_uint64),
                 ("kernel_launches", ctypes.c_uint64), ("compile_mem_hits", ctypes.c_uint64),
                 ("compile_disk_hits", ctypes.c_uint64), ("compile_misses", ctypes.c_uint64),
-                ("compile_ms", ctypes.c_double), ("disk_load_ms", ctypes.c_double)]
+                ("compile_ms", ctypes.c_double), ("disk_load_ms", ctypes.c_double),
+                ("scan_coop_fallbacks", ctypes.c_uint64)]
 
     def asdict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}
@@ -77,7 +78,7 @@ def lib() -> ctypes.CDLL:
             "skel_reset_stats": [P],
             "skel_vector_create": [P, S, S, PP], "skel_vector_destroy": [P], "skel_vector_set_dtype": [P, I],
             "skel_vector_size": [P, ctypes.POINTER(S), ctypes.POINTER(S)], "skel_vector_upload": [P, P, S],
-            "skel_vector_download": [P, P, S], "skel_vector_upload_part": [P, S, P, S], "skel_vector_host_ptr": [P, PP],
+            "skel_vector_download": [P, P, S], "skel_vector_download_part": [P, S, P, S], "skel_vector_upload_part": [P, S, P, S], "skel_vector_host_ptr": [P, PP],
             "skel_vector_mark_host_modified": [P], "skel_vector_fill": [P, P], "skel_vector_fill_dist": [P, I, P],
             "skel_vector_set_distribution": [P, I, I], "skel_vector_get_distribution": [P, ctypes.POINTER(I)],
             "skel_vector_set_distribution_fn": [P, I, ctypes.c_char_p],
@@ -375,6 +376,13 @@ class Vector:
     def download(self) -> np.ndarray:
         out = np.empty(self.n, dtype=self.dtype)
         _check(lib().skel_vector_download(self._h, out.ctypes.data, out.size), self.ctx._h)
+        return out
+
+    def download_part(self, lo: int, out: np.ndarray) -> np.ndarray:
+        """Elements [lo, lo + out.size) into `out` (straight from the devices
+        holding them; pass pinned memory for full-rate copies)."""
+        assert out.dtype == self.dtype and out.flags["C_CONTIGUOUS"]
+        _check(lib().skel_vector_download_part(self._h, lo, out.ctypes.data, out.size), self.ctx._h)
         return out
 
     def host_view(self) -> np.ndarray:

@@ -102,3 +102,35 @@ def test_disk_kernel_cache_roundtrip(tmp_path):
         s = ctx.stats()
         assert s["compile_disk_hits"] == 1 and s["compile_misses"] == 0
         assert np.array_equal(out.download(), x + 7)
+
+
+@pytest.mark.parametrize("D", [1, 4])
+@pytest.mark.parametrize("dist", ["single", "block", "copy"])
+def test_download_part_reads_the_range_from_the_devices(D, dist):
+    """download_part (the counterpart of upload_part): a range comes
+    straight from the device storage that holds it -- exactly its bytes, no
+    full-vector D2H, the host mirror untouched -- and from the host mirror when
+    that is valid."""
+    n = 100_003
+    x = si.uniform_f32(n, 7)
+    with skel.Context(D) as ctx:
+        v = ctx.vector(x)
+        out = ctx.vector(n=n, dtype=np.float32)
+        v.set_distribution({"single": skel.SINGLE, "block": skel.BLOCK, "copy": skel.COPY}[dist])
+        ctx.map(MAP_F32, v, out)
+        want = oracle.skel_map(MAP_F32, x, np.float32)
+        ctx.sync()
+        ctx.reset_stats()
+        for lo, cnt in ((0, n), (0, 1), (n - 1, 1), (25_000, 50_001), (12_345, 0)):
+            got = out.download_part(lo, np.empty(cnt, np.float32))
+            assert np.array_equal(got, want[lo:lo + cnt])
+        st = ctx.stats()
+        assert st["d2h_bytes"] == 4 * (n + 1 + 1 + 50_001)  # only the ranges travelled
+        # a full download validates the mirror; a later part is a host memcpy
+        assert np.array_equal(out.download(), want)
+        ctx.reset_stats()
+        assert np.array_equal(out.download_part(3, np.empty(10, np.float32)), want[3:13])
+        assert ctx.stats()["d2h_bytes"] == 0
+        with pytest.raises(skel.SkelError) as e:
+            out.download_part(n - 2, np.empty(3, np.float32))
+        assert e.value.name == "SKEL_ERR_SIZE"
