@@ -228,6 +228,17 @@ int skel_map(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out,
  * n and keeps its distribution; out = NULL for a void f (side effects only),
  * which runs over a block partition of [0, n).  Errors as skel_map. */
 int skel_map_index(skel_ctx_t ctx, const char *src, size_t n, skel_vec_t out, const skel_arg *args, int nargs);
+/* map_lanes: Map (eq. (1)) in which each element is processed by
+ * `lanes` consecutive threads of one warp (lanes = 1, 2, 4, 8, 16 or 32).  The
+ * user function has the form  R f(T x, int lane, int lanes, args...)  and is
+ * called once per (element, lane); it may combine values across the lanes of
+ * its element with the prelude's skel_group_sum(v, lanes) (every lane must
+ * call it).  out[i] = lane 0's result; out = NULL for a void f.  For elements
+ * that are long sequential jobs (an LM OSEM line of response) on
+ * parts too small to fill the GPU with one thread per element.  Distribution,
+ * ownership and errors as skel_map; lanes outside the set -> SKEL_ERR_ARG. */
+int skel_map_lanes(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, int lanes,
+                   const skel_arg *args, int nargs);
 int skel_zip(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_vec_t out,
              const skel_arg *args, int nargs);
 /* Fused form of Listing 4's tail:

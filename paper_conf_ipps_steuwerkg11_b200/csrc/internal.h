@@ -28,7 +28,7 @@ struct Error {
 // ---------------------------------------------------------------------------
 // JIT modules (NVRTC injection + kernel cache)
 // ---------------------------------------------------------------------------
-enum class Kind { Map = 0, Zip = 1, Red = 2, Idx = 3 };
+enum class Kind { Map = 0, Zip = 1, Red = 2, Idx = 3, Lanes = 4 };
 
 struct Module {
     Kind kind;

@@ -144,6 +144,7 @@ static const char *kind_name(Kind k) {
         case Kind::Map: return "map";
         case Kind::Zip: return "zip";
         case Kind::Idx: return "idx";
+        case Kind::Lanes: return "lanes";
         default: return "red";
     }
 }
@@ -190,6 +191,8 @@ static int assemble(Kind kind, const std::string &user, int block, bool fmad, st
     if (kind == Kind::Map) defs = "#define SKEL_NIN 1\n#define SKEL_BLOCK " + std::to_string(block) + "\n";
     if (kind == Kind::Zip) defs = "#define SKEL_NIN 2\n#define SKEL_BLOCK " + std::to_string(block) + "\n";
     if (kind == Kind::Idx) defs = "#define SKEL_NIN 0\n#define SKEL_BLOCK " + std::to_string(block) + "\n";
+    if (kind == Kind::Lanes)
+        defs = "#define SKEL_NIN 1\n#define SKEL_LANES 1\n#define SKEL_BLOCK " + std::to_string(block) + "\n";
     text->clear();
     text->reserve(user.size() + 65536);
     *text += "#line 1 \"skel_prelude.cuh\"\n";

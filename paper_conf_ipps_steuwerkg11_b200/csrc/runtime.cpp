@@ -1840,6 +1840,52 @@ int skel_map_index(skel_ctx_t ctx, const char *src, size_t n, skel_vec_t out, co
     return SKEL_OK;
 }
 
+// lanes Map: `lanes` threads per element (see map.cuh, SKEL_LANES)
+int skel_map_lanes(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, int lanes, const skel_arg *args,
+                   int nargs) {
+    if (!ctx || !src || !in || in->ctx != ctx || (out && out->ctx != ctx) || (nargs && !args) || nargs < 0)
+        return fail(ctx, SKEL_ERR_ARG, "bad map_lanes arguments");
+    if (lanes < 1 || lanes > 32 || (lanes & (lanes - 1)))
+        return fail(ctx, SKEL_ERR_ARG, "lanes must be a power of two in [1, 32]");
+    Module *m = nullptr;
+    TRY(get_module(ctx, Kind::Lanes, src, &m));
+    const uint64_t rsz = m->sig[3];
+    if (m->sig[4] != in->es)
+        return fail(ctx, SKEL_ERR_TYPE, "element size " + std::to_string(in->es) + " != sizeof(parameter 0) = " +
+                                            std::to_string(m->sig[4]));
+    if (rsz != 0 && !out) return fail(ctx, SKEL_ERR_ARG, "non-void function needs an output vector");
+    if (rsz != 0 && out->es != rsz)
+        return fail(ctx, SKEL_ERR_TYPE, "output element size " + std::to_string(out->es) + " != sizeof(result) = " +
+                                            std::to_string(rsz));
+    TRY(check_args(ctx, m, args, nargs));
+    TRY(ensure_device(in));
+    if (rsz != 0) TRY(prepare_output(out, in->n, in->dist, out == in));
+    const int block = (int)m->sig[9];
+    std::vector<unsigned char> abuf;
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        uint64_t cnt = in->bufs[li].count;
+        if (!cnt) continue;
+        const void *pa = in->bufs[li].ptr(in->es);
+        const void *pb = nullptr;
+        void *po = (rsz != 0) ? out->bufs[li].ptr(out->es) : nullptr;
+        pack_args(m, args, nargs, li, abuf);
+        // one thread per (element, lane): whole warps, up to the grid cap
+        const uint64_t threads = (cnt + 32 / lanes - 1) / (32 / lanes) * 32;
+        const int grid = ew_grid(s, (size_t)threads, block, 1);
+        int ln = lanes;
+        void *params[] = {&pa, &pb, &po, &cnt, &ln, abuf.data()};
+        DevGuard g(s.dev);
+        CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+        ctx->stats.kernel_launches++;
+    }
+    if (rsz != 0) {
+        out->dev_valid = true;
+        device_wrote(out);
+    }
+    return SKEL_OK;
+}
+
 int skel_zip(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_vec_t out, const skel_arg *args,
              int nargs) {
     if (!ctx || !src || !a || !b || !out || a->ctx != ctx || b->ctx != ctx || out->ctx != ctx || (nargs && !args) ||
@@ -2191,7 +2237,8 @@ int skel_prepare(skel_ctx_t ctx, const char *kind, const char *src) {
     else if (!strcmp(kind, "zip")) k = Kind::Zip;
     else if (!strcmp(kind, "reduce") || !strcmp(kind, "scan")) k = Kind::Red;
     else if (!strcmp(kind, "index")) k = Kind::Idx;
-    else return fail(ctx, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan|index");
+    else if (!strcmp(kind, "lanes")) k = Kind::Lanes;
+    else return fail(ctx, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan|index|lanes");
     Module *m = nullptr;
     return get_module(ctx, k, src, &m);
 }
@@ -2297,7 +2344,8 @@ int skel_compile_check(const char *kind, const char *src, int fmad, char *log, s
     else if (!strcmp(kind, "zip")) k = Kind::Zip;
     else if (!strcmp(kind, "reduce") || !strcmp(kind, "scan")) k = Kind::Red;
     else if (!strcmp(kind, "index")) k = Kind::Idx;
-    else return fail(nullptr, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan|index");
+    else if (!strcmp(kind, "lanes")) k = Kind::Lanes;
+    else return fail(nullptr, SKEL_ERR_ARG, "kind must be map|zip|reduce|scan|index|lanes");
     std::string l;
     std::vector<char> cubin;
     const int st = compile_only(k, src, 256, fmad != 0, &l, &cubin);

@@ -28,7 +28,11 @@
 
 using skel_F = decltype(&SKEL_FN);
 using skel_FT = skel::fn<skel_F>;
-constexpr int SKEL_NPOS = SKEL_NIN == 0 ? 1 : SKEL_NIN;  // positional (element / index) parameters
+#ifndef SKEL_LANES
+#define SKEL_LANES 0
+#endif
+// positional (element / index [/ lane, lanes]) parameters
+constexpr int SKEL_NPOS = SKEL_NIN == 0 ? 1 : (SKEL_LANES ? SKEL_NIN + 2 : SKEL_NIN);
 static_assert(skel_FT::arity >= SKEL_NPOS, "user function has too few parameters for this skeleton");
 using skel_A = typename skel_FT::template param<0>;
 #if SKEL_NIN == 2
@@ -188,7 +192,48 @@ __device__ __forceinline__ void skel_one(const skel_A *a, const skel_B *b, skel_
     }
 }
 
-#if SKEL_NIN == 0
+#if SKEL_LANES
+// ---------------------------------------------------------------------------
+// lanes Map (skel_map_lanes): element i is processed by `lanes` consecutive
+// threads of one warp (lanes = 1, 2, 4, ..., 32), which call
+// SKEL_FN(a[i], lane, lanes, args...) with lane = 0..lanes-1 and may combine
+// values across the group (skel_group_sum).  Lane 0's result is stored.  A
+// warp takes 32/lanes consecutive elements per trip of a warp-uniform
+// grid-stride loop, so the lanes of an element are always present together.
+// Used where one element is a long sequential job and a launch over the
+// elements alone would not fill the GPU (the LM OSEM error-image Map over one
+// GPU's part of a subset).
+// ---------------------------------------------------------------------------
+static_assert(SKEL_NIN == 1, "lanes Map: one input vector");
+static_assert(skel::same<skel::decay_t<typename skel_FT::template param<1>>, int>::value &&
+                  skel::same<skel::decay_t<typename skel_FT::template param<2>>, int>::value,
+              "a lanes Map's user function takes (element, int lane, int lanes, args...)");
+template <bool V = skel_void, class Tup>
+__device__ __forceinline__ void skel_lanes_one(const skel_A *a, skel_O *out, skel_u64 i, int sub, int lanes, Tup &t) {
+    if constexpr (V) {
+        skel::caller<skel_Seq>::call(&SKEL_FN, t, a[i], sub, lanes);
+    } else {
+        const skel_O r = skel::caller<skel_Seq>::call(&SKEL_FN, t, a[i], sub, lanes);
+        if (sub == 0) out[i] = r;
+    }
+}
+extern "C" __global__ void SKEL_EW_BOUNDS
+    skel_ew_kernel(const skel_A *__restrict__ a, const skel_B *__restrict__ b, skel_O *__restrict__ out, skel_u64 n,
+                   int lanes, const skel_Buf args) {
+    (void)b;
+    auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    const int lane = (int)(threadIdx.x & 31u);
+    const int sub = lane & (lanes - 1);
+    const skel_u64 per_warp = (skel_u64)(32 / lanes);
+    const skel_u64 gw = ((skel_u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const skel_u64 wstride = ((skel_u64)gridDim.x * blockDim.x) >> 5;
+#pragma unroll 1
+    for (skel_u64 base = gw * per_warp; base < n; base += wstride * per_warp) {  // warp-uniform
+        const skel_u64 i = base + (skel_u64)(lane / lanes);
+        if (i < n) skel_lanes_one(a, out, i, sub, lanes, t);
+    }
+}
+#elif SKEL_NIN == 0
 static_assert(skel::is_arith<skel::decay_t<skel_A>>::value, "an index Map's first parameter must be an integer index");
 // index Map: element c*E + e of this part is index base + c*E + e; outputs are
 // staged per chunk and stored with one 128-bit store, like Map.  (The bodies are

@@ -280,3 +280,20 @@ template <class T> __device__ __forceinline__ T ld_value(const T *p) {
 }
 
 }  // namespace skel
+
+// ---- lanes Map (skel_map_lanes): the `lanes` consecutive threads that share
+// one element.  A user function of a lanes Map receives (element, lane, lanes,
+// args...) and may combine values across the element's lanes with these
+// (every lane of the group must call them: they are warp shuffles restricted
+// to the group's lanes; lanes is a power of two <= 32).
+__device__ __forceinline__ unsigned skel_group_mask(int lanes) {
+    const unsigned lane = threadIdx.x & 31u;
+    return lanes >= 32 ? 0xffffffffu : (((1u << lanes) - 1u) << (lane & ~(unsigned)(lanes - 1)));
+}
+// sum over the group (butterfly: every lane gets the same value, since each
+// step adds the same two operands in every lane and + is commutative)
+template <class T> __device__ __forceinline__ T skel_group_sum(T v, int lanes) {
+    const unsigned m = skel_group_mask(lanes);
+    for (int o = 1; o < lanes; o <<= 1) v += __shfl_xor_sync(m, v, o, lanes);
+    return v;
+}

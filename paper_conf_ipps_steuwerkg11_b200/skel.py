@@ -87,6 +87,7 @@ def lib() -> ctypes.CDLL:
             "skel_vector_device_ptr": [P, I, PP, ctypes.POINTER(S)],
             "skel_map": [P, ctypes.c_char_p, P, P, P, I], "skel_zip": [P, ctypes.c_char_p, P, P, P, P, I],
             "skel_map_index": [P, ctypes.c_char_p, S, P, P, I],
+            "skel_map_lanes": [P, ctypes.c_char_p, P, P, I, P, I],
             "skel_reduce": [P, ctypes.c_char_p, P, P, P, I],
             "skel_zip_combine": [P, ctypes.c_char_p, P, P, I, P, P, I], "skel_reduce_to": [P, ctypes.c_char_p, P, P, P, I],
             "skel_scan": [P, ctypes.c_char_p, P, P, P, P, I], "skel_prepare": [P, ctypes.c_char_p, ctypes.c_char_p],
@@ -276,6 +277,13 @@ class Context:
         a, keep = self._args(args)
         _check(lib().skel_map_index(self._h, src.encode(), n, vout._h if vout is not None else None, a, len(args)),
                self._h)
+        return vout
+
+    def map_lanes(self, src: str, vin: "Vector", vout: "Vector | None" = None, lanes: int = 1, args=()):
+        """Map with `lanes` threads per element: f(x, lane, lanes, args...)."""
+        a, keep = self._args(args)
+        _check(lib().skel_map_lanes(self._h, src.encode(), vin._h, vout._h if vout is not None else None, lanes,
+                                    a, len(args)), self._h)
         return vout
 
     def zip(self, src: str, va: "Vector", vb: "Vector", vout: "Vector", args=()):

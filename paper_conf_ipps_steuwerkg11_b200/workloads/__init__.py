@@ -19,6 +19,10 @@ LMOSEM_ERROR = source("lmosem_error")
 # Map is bound by L1TEX requests: 16-byte gathers per 4-float group in the
 # forward projection too; in the given order they are slower
 LMOSEM_ERROR_PREPARED = "#define LMOSEM_VEC_FWD 1\n" + LMOSEM_ERROR
+# the same Listing 3 body on a lanes Map: `lanes` threads per event, each
+# walking an alpha piece of the line of response (small per-GPU parts, §4.2)
+LMOSEM_LANES = LMOSEM_ERROR + source("lmosem_lanes")
+LMOSEM_LANES_PREPARED = "#define LMOSEM_VEC_FWD 1\n" + LMOSEM_LANES
 LMOSEM_UPDATE = source("lmosem_update")
 # voxel visits of one event's path (measurement only: the LM OSEM roofline
 # counts one scattered request per visit in each of the two walks)

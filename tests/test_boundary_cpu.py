@@ -42,6 +42,22 @@ def test_nvrtc_injection_compiles_for_sm100a(kind, src):
     assert nbytes > 1000
 
 
+def test_lanes_map_compiles_for_sm100a():
+    from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_LANES, LMOSEM_LANES_PREPARED
+    for src in (LMOSEM_LANES, LMOSEM_LANES_PREPARED):
+        st, log, nbytes = skel.compile_check("lanes", src)
+        assert st == 0, log
+    # a lanes function needs (element, int lane, int lanes, ...)
+    st, log, _ = skel.compile_check("lanes", "float f(float x) { return x; }")
+    assert st != 0
+
+
+def _unused(kind, src):
+    st, log, nbytes = skel.compile_check(kind, src)
+    assert st == 0, log
+    assert nbytes > 1000
+
+
 def test_listing2_as_printed_is_rejected():
     st, log, _ = skel.compile_check("map", "float f(float input, float number) { return input * number }")
     assert st == 4 and 'expected a ";"' in log

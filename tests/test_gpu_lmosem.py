@@ -160,3 +160,50 @@ def test_events_prepare_option(D):
         f = rec.image()
     want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
     assert rel_l2(f, want) <= 1e-4
+
+
+@pytest.mark.parametrize("lanes", [1, 2, 4, 8, 32])
+def test_lanes_map_error_image_matches_oracle(lanes):
+    """The error image on a lanes Map (skel_map_lanes: `lanes` threads per
+    event, each walking an alpha piece of the line of response, the partial
+    forward projections summed over the group): the oracle's image (relL2 1e-4
+    bar; here 1e-5 on a random tiny grid with ties and at the paper's volume)."""
+    from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_LANES
+    g = np.random.default_rng(3)
+    dims = (4, 3, 5)
+    n = 600
+    e = np.zeros(n, si.EVENT_DTYPE)
+    for k in ("x1", "y1", "z1", "x2", "y2", "z2"):
+        e[k] = g.integers(-8, 28, n) / 4.0
+    f = g.uniform(0.5, 2.0, int(np.prod(dims))).astype(np.float32)
+    events = si.lmosem_events(50_003, subset=7)
+    with skel.Context(1) as ctx:
+        for evs, ff, dd in ((e, f, dims), (events, np.ones(150 * 150 * 280, np.float32), (150, 150, 280))):
+            fv = ctx.vector(ff)
+            c = ctx.vector(n=int(np.prod(dd)), dtype=np.float32)
+            ctx.map_lanes(LMOSEM_LANES, ctx.vector(evs), None, lanes, args=[fv, c, *[np.int32(d) for d in dd]])
+            c.mark_device_modified()
+            got = c.download()
+            want, _ = oracle.lmosem_error_image(evs, ff.astype(np.float64), dd)
+            assert np.array_equal(got > 0, want > 0)
+            assert rel_l2(got, want) <= 1e-5
+
+
+def test_lanes_map_generic_group_sum():
+    """skel_map_lanes semantics on a plain function: lane l of element x
+    contributes x * (l + 1); the group sum is x * lanes (lanes + 1) / 2 in every
+    lane, lane 0's result is stored (eq. (1) with a cooperative element)."""
+    src = """
+    float tri(float x, int lane, int lanes) {
+        return skel_group_sum(x * (float)(lane + 1), lanes);
+    }"""
+    x = np.arange(1, 10_001, dtype=np.float32)
+    with skel.Context(1) as ctx:
+        vx = ctx.vector(x)
+        out = ctx.vector(n=x.size, dtype=np.float32)
+        for lanes in (1, 2, 4, 8, 16, 32):
+            ctx.map_lanes(src, vx, out, lanes)
+            assert np.array_equal(out.download(), x * np.float32(lanes * (lanes + 1) // 2))
+        with pytest.raises(skel.SkelError) as e:
+            ctx.map_lanes(src, vx, out, 3)
+        assert e.value.name == "SKEL_ERR_ARG"
