@@ -861,9 +861,13 @@ def lm_subsets(nev, nsub, lo, hi):
 
 
 def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
-    """configs[3]/[4]: one subset of 10^6 events into 150x150x280, events block-distributed."""
+    """configs[3]/[4]: one subset of 10^6 events into 150x150x280, events
+    block-distributed; the error-image Map in the form lmosem.LMOSEM.plan picks
+    for 10^6/N events per GPU (a lanes Map with 4 threads per event in the
+    given order).  `device_order`: the same subset with every GPU's events
+    reordered by path length ON THE DEVICE first (counting Map + Scan +
+    scattering Map, included in the time)."""
     import torch
-    import skel_inputs as si
     from paper_conf_ipps_steuwerkg11_b200.lmosem import LMOSEM
     nev = 1_000_000
     ev = lm_subsets(nev, 1, 0, nev)[0]
@@ -891,24 +895,6 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         return max_over_ranks(e0.elapsed_time(e1) / reps)
 
     ms = timed(lambda: rec.subset(evv))
-    # the same subset with its events ordered longest path first (host
-    # preprocessing per subset, lmosem.order_by_path; each rank orders its part)
-    from paper_conf_ipps_steuwerkg11_b200.lmosem import prepare_part
-    t0 = time.perf_counter()
-    ev_ord, ord_block = prepare_part(ev[lo:hi])
-    order_host_s = time.perf_counter() - t0
-    rec.map_block = ord_block
-    from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_ERROR, LMOSEM_ERROR_PREPARED
-    rec.error_src = LMOSEM_ERROR_PREPARED
-    evo = ctx.vector(n=nev, dtype=ev.dtype)
-    if world > 1:
-        evo.set_distribution(skel.BLOCK)
-    evo.upload_part(lo, ev_ord)
-    for _ in range(TUNE):
-        rec.subset(evo)
-    ms_ord = timed(lambda: rec.subset(evo))
-    rec.map_block = 0
-    rec.error_src = LMOSEM_ERROR
     for _ in range(TUNE):
         rec.subset(evv, fused=True)
     ms_fused = timed(lambda: rec.subset(evv, fused=True))
@@ -920,6 +906,13 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         g.destroy()
     except skel.SkelError:  # a collective backend that cannot be captured
         ms_graph = ms
+    # the same subset with the events ordered on the device (sort inside the time)
+    recd = LMOSEM(ctx, order="device")
+    recd.prepare()
+    for _ in range(TUNE):
+        recd.subset(evv)
+    ms_dev = timed(lambda: recd.subset(evv))
+    ms_sort = timed(lambda: recd.order_on_device(evv))
     coll = None
     if world > 1:  # the exchange steps alone, bus GB/s vs NVLink
         S = rec.nvox * 4
@@ -941,27 +934,23 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
                 "all_gather_busbw_GBps": S * busf / (ms_ag * 1e-3) / 1e9,
                 "peak_GBps": 770.0, "peak_source": "B200_PROFILING.md measured peer copy per direction "
                                                   "(900 nominal)"}
-    roof = lmosem_roofline(ctx, skel, rec, evv, timed, world, evo, ord_block)
-    evo.destroy()
+    roof = lmosem_roofline(ctx, skel, rec, recd, evv, timed, world)
     evv.destroy()
     # configs[4]: the full reconstruction -- 10 subsets of 10^6 events (10^7,
     # P:L603-605), each subset a different synthetic draw, all events staged on
     # the devices beforehand (240 MB); one pass over the subsets from f0 = 1
     nsub = 10
     full = {}
-    for mode in ("given", "ordered"):
-        subs = []
-        for evl in lm_subsets(nev, nsub, lo, hi):
-            if mode == "ordered":
-                evl, _ = prepare_part(evl)
-            v = ctx.vector(n=nev, dtype=evl.dtype)
-            if world > 1:
-                v.set_distribution(skel.BLOCK)
-            v.upload_part(lo, evl)
-            subs.append(v)
-        rec2 = LMOSEM(ctx)
-        rec2.map_block = ord_block if mode == "ordered" else 0
-        rec2.error_src = LMOSEM_ERROR_PREPARED if mode == "ordered" else LMOSEM_ERROR
+    subs = []
+    for evl in lm_subsets(nev, nsub, lo, hi):
+        v = ctx.vector(n=nev, dtype=evl.dtype)
+        if world > 1:
+            v.set_distribution(skel.BLOCK)
+        v.upload_part(lo, evl)
+        subs.append(v)
+    for mode in ("given", "device"):
+        rec2 = LMOSEM(ctx, order=mode)
+        rec2.prepare()
         for v in subs:  # stage every subset (lazy H2D) and warm up
             rec2.subset(v)
         ctx.sync()
@@ -975,38 +964,51 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         e1.record(stream)
         ctx.sync()
         full[mode] = max_over_ranks(e0.elapsed_time(e1))
-        for v in subs:
-            v.destroy()
-    ms_full = full["given"]
+    for v in subs:
+        v.destroy()
+    src, lanes = rec.plan(-(-nev // world))
     return {"config": "configs[3]/[4]: one subset, 10^6 events, 150x150x280, events block over GPUs",
             "subset_s": ms * 1e-3, "subset_s_graph": ms_graph * 1e-3, "subset_s_fused": ms_fused * 1e-3,
+            "map_form": {"lanes": lanes, "cta_threads": 128},
             "roofline": roof, "exchange": coll,
-            "events_per_s": nev / (min(ms_graph, ms_fused) * 1e-3),
-            "full_recon_s": ms_full * 1e-3, "full_recon": "10 subsets x 10^6 events (configs[4]), f0 = 1, "
-                                                          "events resident on the devices",
-            "ordered": {"subset_s": ms_ord * 1e-3, "full_recon_s": full["ordered"] * 1e-3,
-                        "order_host_s_per_subset": order_host_s, "map_cta_threads": ord_block or 256,
-                        "note": "events of each device's part ordered on the host before upload (lmosem.prepare_part: "
-                                "longest path first, or below 1.5e5 events per device warp groups dealt over "
-                                "128-thread CTAs; list-mode events carry no order, same image up to float rounding)"},
+            "events_per_s": nev / (min(ms, ms_graph, ms_fused) * 1e-3),
+            "full_recon_s": full["given"] * 1e-3, "full_recon": "10 subsets x 10^6 events (configs[4]), f0 = 1, "
+                                                                "events resident on the devices",
+            "device_order": {"subset_s": ms_dev * 1e-3, "order_s": ms_sort * 1e-3,
+                             "full_recon_s": full["device"] * 1e-3,
+                             "map_lanes": recd.plan(-(-nev // world))[1],
+                             "note": "every GPU's events reordered by path length on the device (lmosem_order.cu: "
+                                     "counting Map + Scan + scattering Map, inside the timed subset) before the "
+                                     "error-image Map; same image up to float rounding (R10(x))"},
             "note": "includes f all-gather, c zero-fill, Siddon Map, c reduce-scatter and update Zip; "
                     "subset_s = eager calls, subset_s_graph = the same subset replayed as a CUDA graph, "
                     "subset_s_fused = the tail as one peer-memory kernel (skel_zip_combine, NEXT-1)"}
 
 
-def lmosem_roofline(ctx, skel, rec, evv, timed, nd, evo=None, evo_block=0):
+def lmosem_l1_hit():
+    """L1 hit rate of the forward-projection gathers of the error-image Map,
+    from the committed ncu capture (profiles/lmosem_l1.json), or None."""
+    try:
+        with open(os.path.join(ROOT, "profiles", "lmosem_l1.json")) as fh:
+            return json.load(fh)
+    except Exception:
+        return None
+
+
+def lmosem_roofline(ctx, skel, rec, recd, evv, timed, nd):
     """Roofline of the error-image Map.  Every voxel visit of a
     path is one scattered 4-byte request in each walk (a gather of f forward,
     a red.add into c backward) and the lanes of a warp are on different rays,
     so the Map is bound by how fast the SMs' L1TEX units can issue scattered
     requests to L2.  The peaks are measured in the same run by probe Maps
-    (workloads/probe_*.cu) issuing random scattered gathers / scalar and
-    vector reductions; the Map's ideal time is V/peak_gather + R/peak_red_v4
-    for V voxel visits and R vector reductions (4-float groups entered),
-    both counted by Maps over the same events."""
-    from paper_conf_ipps_steuwerkg11_b200.workloads import (LMOSEM_ERROR, LMOSEM_GROUPS, LMOSEM_VISITS,
-                                                            PROBE_GATHER, PROBE_K, PROBE_SCATTER_RED,
-                                                            PROBE_SCATTER_RED4, SUM_I32)
+    (workloads/probe_*.cu) issuing random scattered gathers / vector
+    reductions; a gather costs h/peak_resident + (1-h)/peak_image with h the
+    Map's measured L1 hit rate (profiles/lmosem_l1.json, ncu); the Map's ideal
+    time is V x that + R/peak_red_v4 for V voxel visits and R vector
+    reductions (4-float groups entered), both counted by Maps over the same
+    events."""
+    from paper_conf_ipps_steuwerkg11_b200.workloads import (LMOSEM_GROUPS, LMOSEM_VISITS, PROBE_GATHER, PROBE_K,
+                                                            PROBE_SCATTER_RED, PROBE_SCATTER_RED4, SUM_I32)
     dims = rec.dims_args
     nvis = ctx.vector(n=evv.n, dtype=np.int32)
     if evv.distribution == skel.BLOCK:
@@ -1019,17 +1021,17 @@ def lmosem_roofline(ctx, skel, rec, evv, timed, nd, evo=None, evo_block=0):
     f, c = rec.f, rec.c
     f.set_distribution(skel.COPY)
     c.fill_dist(skel.COPY, np.float32(0))
-    ctx.map(LMOSEM_ERROR, evv, None, args=[f, c, *dims])
-    ms_map = timed(lambda: ctx.map(LMOSEM_ERROR, evv, None, args=[f, c, *dims]))
-    ms_map_ord = None
-    if evo is not None:  # the prepared part, its CTA size and function (lmosem.prepare_part)
-        from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_ERROR_PREPARED
-        ctx.set_block_size(evo_block)
-        for _ in range(TUNE):
-            ctx.map(LMOSEM_ERROR_PREPARED, evo, None, args=[f, c, *dims])
-        ms_map_ord = timed(lambda: ctx.map(LMOSEM_ERROR_PREPARED, evo, None, args=[f, c, *dims]))
-        ctx.set_block_size(0)
+    for _ in range(TUNE):
+        rec.error_map(evv)
+    ms_map = timed(lambda: rec.error_map(evv))
+    recd.f.set_distribution(skel.COPY)
+    recd.c.fill_dist(skel.COPY, np.float32(0))
+    evo = recd.order_on_device(evv)
+    for _ in range(TUNE):
+        recd.error_map(evo)
+    ms_map_ord = timed(lambda: recd.error_map(evo))
     c.mark_device_modified()
+    recd.c.mark_device_modified()
     # probes: 2^20 elements x PROBE_K scattered requests each (per GPU), into (a) an
     # image-sized 25 MB buffer (random lines: L2 hit/miss and far-partition traffic
     # included) and (b) a small buffer (64 KB gathers: L1-resident; 1 MB reductions:
@@ -1054,32 +1056,40 @@ def lmosem_roofline(ctx, skel, rec, evv, timed, nd, evo=None, evo_block=0):
         probes[tag] = tuple(npr * PROBE_K / (t * 1e-3) / 1e9 for t in (ms_g, ms_r, ms_r4))
     for v in (idx, img, acc, gout):
         v.destroy()
-    peak_g = max(p[0] for p in probes.values())  # G requests/s per GPU
-    peak_r = max(p[1] for p in probes.values())
     peak_r4 = max(p[2] for p in probes.values())
+    l1 = lmosem_l1_hit()
+    h = float(l1["given"]["l1_hit_rate"]) if l1 else None
+    hd = float(l1["device"]["l1_hit_rate"]) if l1 and "device" in l1 else h
+    g_res, g_img = probes["resident"][0], probes["image"][0]
+
+    def gather_rate(hit):  # G gathers/s at L1 hit rate `hit` (None: the resident probe, an upper bound)
+        if hit is None:
+            return g_res
+        return 1.0 / (hit / g_res + (1.0 - hit) / g_img)
+    pg, pgd = gather_rate(h), gather_rate(hd)
     # requests of the Map: one gather per visit (forward), one vector reduction per
     # 4-float group entered (back projection); ideal = each at its measured peak
     reqs = (visits + groups) / nd
-    ideal_ms = (visits / nd) / (peak_g * 1e9) * 1e3 + (groups / nd) / (peak_r4 * 1e9) * 1e3
-    achieved = reqs / (ms_map * 1e-3) / 1e9
-    ideal_ord_ms = (groups / nd) / (peak_g * 1e9) * 1e3 + (groups / nd) / (peak_r4 * 1e9) * 1e3
-    peak = reqs / (ideal_ms * 1e-3) / 1e9
-    return {"kernel": "LM OSEM error-image Map (skel_ew_kernel + lmosem_error)", "bound": "l1tex",
-            "achieved": achieved, "peak": peak, "unit": "G scattered requests/s per GPU",
+    ideal_ms = (visits / nd) / (pg * 1e9) * 1e3 + (groups / nd) / (peak_r4 * 1e9) * 1e3
+    # device order: the forward projection gathers 16 bytes per 4-float group
+    ideal_ord_ms = (groups / nd) / (pgd * 1e9) * 1e3 + (groups / nd) / (peak_r4 * 1e9) * 1e3
+    return {"kernel": "LM OSEM error-image Map (skel_ew_kernel, lanes Map + lmosem_lanes)", "bound": "l1tex",
+            "achieved": reqs / (ms_map * 1e-3) / 1e9, "peak": reqs / (ideal_ms * 1e-3) / 1e9,
+            "unit": "G scattered requests/s per GPU",
             "frac": ideal_ms / ms_map, "map_ms": ms_map, "ideal_ms": ideal_ms, "visits_per_subset": visits,
-            "ordered": None if ms_map_ord is None else {
-                "map_ms": ms_map_ord, "frac": ideal_ord_ms / ms_map_ord, "ideal_ms": ideal_ord_ms,
-                "achieved": 2 * groups / nd / (ms_map_ord * 1e-3) / 1e9,
-                "note": "the prepared subset (lmosem.prepare_part) and function (LMOSEM_ERROR_PREPARED: one 16-byte "
-                        "gather per 4-float group forward, one red.v4 per group backward), so the requests are "
-                        "2 x groups; ideal = groups/peak_gather + groups/peak_red_v4 (the 16-byte gather taken at "
-                        "the 4-byte probe rate)"},
-            "vector_reductions_per_subset": groups, "peak_gather": peak_g, "peak_red_v4": peak_r4,
-            "peak_red": peak_r,
+            "l1_hit_rate": h, "gather_rate_G_per_s": pg,
+            "device_order": {"map_ms": ms_map_ord, "frac": ideal_ord_ms / ms_map_ord, "ideal_ms": ideal_ord_ms,
+                             "l1_hit_rate": hd,
+                             "note": "the Map over the device-ordered events with the prepared function (one 16-byte "
+                                     "gather per 4-float group forward, one red.v4 per group backward): 2 x groups "
+                                     "requests"},
+            "vector_reductions_per_subset": groups, "peak_red_v4": peak_r4, "peak_red": max(p[1] for p in probes.values()),
             "probes_Greq_per_s": {k: {"gather": v[0], "red": v[1], "red_v4": v[2]} for k, v in probes.items()},
             "peak_source": "measured in this run: probe Maps workloads/probe_gather.cu, probe_scatter.cu, "
                            "probe_scatter4.cu (random 4-byte gathers / red.add.f32 / red.add.v4.f32, 32 lanes on "
-                           "32 lines; best of a 25 MB image-sized buffer and an L1/L2-resident one)"}
+                           "32 lines) into a 25 MB image-sized buffer and an L1/L2-resident one; the gather rate "
+                           "is the two probes' rates weighted by the Map's ncu L1 hit rate (profiles/lmosem_l1.json; "
+                           "absent: the resident probe, an upper bound)"}
 
 
 if __name__ == "__main__":

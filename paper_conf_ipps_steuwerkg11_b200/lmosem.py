@@ -6,82 +6,47 @@ updated by a Zip on the blocks.
 Reading R10(i): c is reset to 0 at the start of every subset (Listing 3/4 do
 not show it, but without it the combine would re-add the previous subset's
 error image D times).
+
+The error-image Map (Listing 3 lines 4-13 inside Listing 4's Map) runs in one
+of two forms, picked per subset from the events each device holds
+(`LMOSEM.plan`):
+
+* a Map with one thread per event (workloads/lmosem_error.cu), or
+* a lanes Map (skel_map_lanes) with `lanes` threads per event, each walking an
+  alpha piece of the line of response (workloads/lmosem_lanes.cu) -- the form
+  that fills the GPU when one device's part of a subset is small (10^6/8
+  events at 8 GPUs).
+
+`order="device"` first reorders every device's events by path length on the
+device with the library's own skeletons (a counting Map, a Scan of the
+bucket counts and a scattering Map; workloads/lmosem_order.cu): list-mode
+events carry no order and the error image is a sum over events (R10(x)), so
+the image is the same up to float rounding, and rays of similar length then
+share a warp.
 """
 from __future__ import annotations
 
 import numpy as np
 
 from . import skel
-from .workloads import LMOSEM_ERROR, LMOSEM_ERROR_PREPARED, LMOSEM_UPDATE
+from .workloads import (LMOSEM_ERROR, LMOSEM_ERROR_PREPARED, LMOSEM_LANES, LMOSEM_LANES_PREPARED,
+                        LMOSEM_ORDER_BUCKETS, LMOSEM_ORDER_HIST, LMOSEM_ORDER_SCATTER, LMOSEM_UPDATE, SUM_I32)
 
 DIMS = (150, 150, 280)  # P:L604
 
-
-def order_by_path(ev: np.ndarray, dims=DIMS) -> np.ndarray:
-    """The events of a subset reordered longest path first (host preprocessing,
-    like reading the subset from file).  List-mode events carry no
-    order, and the error image is a sum over them, so any order gives the same
-    image up to float rounding (R10(x)).  With similar path lengths next to each
-    other, the 32 rays of a warp finish together (thread efficiency) and the
-    longest rays start first (shorter launch tail): DESIGN.md §4.2.
-    Key: the L1 length |dx|+|dy|+|dz| of the segment clipped to the volume
-    (slab clipping, float64) -- proportional to the voxel steps of the walk."""
-    p = np.stack([ev["x1"], ev["y1"], ev["z1"]]).astype(np.float64)
-    d = np.stack([ev["x2"], ev["y2"], ev["z2"]]).astype(np.float64) - p
-    amin = np.zeros(len(ev))
-    amax = np.ones(len(ev))
-    for a, n in enumerate(dims):
-        nz = d[a] != 0
-        with np.errstate(divide="ignore", invalid="ignore"):
-            a0 = np.where(nz, (0.0 - p[a]) / d[a], -np.inf)
-            a1 = np.where(nz, (float(n) - p[a]) / d[a], np.inf)
-        inside = (p[a] >= 0) & (p[a] < n)
-        amin = np.maximum(amin, np.where(nz, np.minimum(a0, a1), np.where(inside, -np.inf, np.inf)))
-        amax = np.minimum(amax, np.where(nz, np.maximum(a0, a1), np.inf))
-    key = np.where(amax > amin, (amax - amin) * np.abs(d).sum(axis=0), 0.0)
-    return ev[np.argsort(-key, kind="stable")]
-
-
-def deal_warps(ev: np.ndarray, block: int = 256, warp: int = 32) -> np.ndarray:
-    """Events ordered longest path first (order_by_path), then their groups of
-    `warp` consecutive events dealt round-robin to the `block`-thread CTAs of a
-    one-event-per-thread launch (snake order): a warp keeps rays of similar
-    length, and every CTA gets one group from each length range, so the CTAs
-    (and the SMs that host them) carry equal work."""
-    o = order_by_path(ev)
-    n = len(o)
-    ng = -(-n // warp)
-    per_cta = block // warp
-    ncta = -(-ng // per_cta)
-    # group g (in length order) goes to slot g // ncta of a CTA dealt in snake
-    # order (0..ncta-1, then ncta-1..0, ...), which evens out the CTAs' sums
-    gid = np.arange(ng)
-    rnd, pos = gid // ncta, gid % ncta
-    cta = np.where(rnd % 2 == 0, pos, ncta - 1 - pos)
-    dest = cta * per_cta + rnd
-    order = np.argsort(dest, kind="stable")
-    idx = (order[:, None] * warp + np.arange(warp)[None, :]).ravel()
-    return o[idx[idx < n]]
-
-
-# events per device below which a launch is well under one wave of the GPU
-# (148 SMs x 2048 threads); there 128-thread CTAs and warp-dealt order balance
-# the SMs better (DESIGN.md §4.2; measured: better at 1.25e5 events per GPU,
-# worse at 2.5e5)
-SMALL_PART = 150_000
-
-
-def prepare_part(ev: np.ndarray, dims=DIMS) -> tuple[np.ndarray, int]:
-    """(events, CTA size for the error-image Map) for one device's part of a
-    subset: longest path first at the default CTA size, or -- for parts below
-    SMALL_PART events -- warp groups dealt over 128-thread CTAs."""
-    if len(ev) <= SMALL_PART:
-        return deal_warps(ev, block=128), 128
-    return order_by_path(ev, dims), 0
+# CTA size of every error-image Map (measured at 10^6/D events, D = 1..8,
+# tools/lm_lanes_probe.py: 128 is as fast or faster than 256 everywhere)
+MAP_BLOCK = 128
+# events per device from which the one-thread-per-event Map beats the lanes
+# Map on length-ordered events (measured crossover between 1.25e5 and 2.5e5)
+ORDERED_LANES_BELOW = 200_000
 
 
 class LMOSEM:
-    def __init__(self, ctx: skel.Context, dims=DIMS, f0: float = 1.0):
+    def __init__(self, ctx: skel.Context, dims=DIMS, f0: float = 1.0, order: str = "given",
+                 lanes: int | None = None):
+        if order not in ("given", "device"):
+            raise ValueError("order must be 'given' or 'device'")
         self.ctx = ctx
         self.dims = tuple(int(d) for d in dims)
         self.nvox = int(np.prod(self.dims))
@@ -89,36 +54,88 @@ class LMOSEM:
         self.c = ctx.vector(n=self.nvox, dtype=np.float32)
         self.f.fill_dist(skel.BLOCK, np.float32(f0))  # f0 = 1 everywhere (reading R10(ii))
         self.dims_args = [np.int32(d) for d in self.dims]
-        self.map_block = 0  # CTA size of the error-image Map (0 = the context's default)
-        self.error_src = LMOSEM_ERROR  # LMOSEM_ERROR_PREPARED for prepared event order
+        self.order = order
+        self.lanes = lanes  # None: LMOSEM.plan decides per subset
+        self._hist = self._cursor = self._sorted = None
+
+    # ---- policy ------------------------------------------------------------
+    def plan(self, per_device: int) -> tuple[str, int]:
+        """(error-image function source, lanes) for parts of `per_device`
+        events.  Given order: 4 lanes per event at every measured part size
+        (10^6/D events, D = 1..8: 1.29 / 0.655 / 0.337 / 0.179 ms against
+        1.37 / 0.727 / 0.394 / 0.211 ms with one thread per event).
+        Length-ordered events: one thread per event down to ORDERED_LANES_BELOW,
+        4 lanes below it (D = 1: 1.14 vs 1.26 ms; D = 8: 0.169 vs 0.175 ms)."""
+        ordered = self.order == "device"
+        lanes = self.lanes
+        if lanes is None:
+            lanes = 4 if (not ordered or per_device < ORDERED_LANES_BELOW) else 1
+        if lanes == 1:
+            return (LMOSEM_ERROR_PREPARED if ordered else LMOSEM_ERROR), 1
+        return (LMOSEM_LANES_PREPARED if ordered else LMOSEM_LANES), lanes
 
     def prepare(self):
-        if self.map_block:
-            self.ctx.set_block_size(self.map_block)
-        self.ctx.prepare("map", self.error_src)
-        if self.map_block:
-            self.ctx.set_block_size(0)
-        self.ctx.prepare("zip", LMOSEM_UPDATE)
+        """Compile every function a subset may use (before timing or capturing)."""
+        ctx = self.ctx
+        ctx.set_block_size(MAP_BLOCK)
+        for src in (LMOSEM_ERROR, LMOSEM_ERROR_PREPARED):
+            ctx.prepare("map", src)
+        for src in (LMOSEM_LANES, LMOSEM_LANES_PREPARED):
+            ctx.prepare("lanes", src)
+        ctx.set_block_size(0)
+        ctx.prepare("zip", LMOSEM_UPDATE)
+        if self.order == "device":
+            ctx.prepare("map", LMOSEM_ORDER_HIST)
+            ctx.prepare("map", LMOSEM_ORDER_SCATTER)
+            ctx.prepare("scan", SUM_I32)
 
-    def events(self, ev: np.ndarray, prepare: bool = False) -> skel.Vector:
+    # ---- data ----------------------------------------------------------------
+    def events(self, ev: np.ndarray) -> skel.Vector:
         """Vector<Event> of one subset, block-distributed (Listing 4).
-        prepare=True: each device's part [k*ceil(n/D), ...) reordered by
-        prepare_part (the error-image Map then uses the CTA size it picks).
         In rank mode pass the whole subset on every rank, as for a plain upload."""
-        if prepare and len(ev):
-            D = self.ctx.D
-            ps = -(-len(ev) // D)
-            parts = []
-            for k in range(D):
-                part, blk = prepare_part(ev[k * ps:(k + 1) * ps], self.dims)
-                parts.append(part)
-                if k == 0:
-                    self.map_block = blk
-            self.error_src = LMOSEM_ERROR_PREPARED
-            ev = np.concatenate(parts)
         v = self.ctx.vector(ev)
         v.set_distribution(skel.BLOCK)
         return v
+
+    def order_on_device(self, events: skel.Vector) -> skel.Vector:
+        """Every device's events reordered longest path first, on the device:
+        bucket counts (void Map, one atomic per bucket and warp), exclusive Scan
+        of the counts, and a void Map that moves each event to its bucket's next
+        slot.  Returns a vector with the same distribution and part sizes."""
+        ctx, nb = self.ctx, LMOSEM_ORDER_BUCKETS
+        if self._hist is None:
+            self._hist = ctx.vector(n=nb, dtype=np.int32)
+            self._cursor = ctx.vector(n=nb, dtype=np.int32)
+        if self._sorted is None or self._sorted.n != events.n or \
+                self._sorted.distribution != events.distribution:
+            if self._sorted is not None:
+                self._sorted.destroy()
+            self._sorted = ctx.vector(n=events.n, dtype=events.dtype)
+            self._sorted.fill_dist(events.distribution, np.zeros(1, events.dtype)[0])
+        hist, cursor, out = self._hist, self._cursor, self._sorted
+        hist.fill_dist(skel.COPY, np.int32(0))   # one histogram per device
+        ctx.map(LMOSEM_ORDER_HIST, events, None, args=[hist, *self.dims_args, np.int32(nb)])
+        hist.mark_device_modified()              # per-device counts (diverged copies)
+        ctx.scan(SUM_I32, hist, cursor, np.int32(0))  # each device scans its own counts
+        ctx.map(LMOSEM_ORDER_SCATTER, events, None, args=[cursor, out, *self.dims_args, np.int32(nb)])
+        cursor.mark_device_modified()
+        out.mark_device_modified()
+        return out
+
+    # ---- Listing 4's loop body -------------------------------------------------
+    def error_map(self, events: skel.Vector):
+        """The error-image Map c += ... over the (already ordered) events."""
+        ctx, f, c = self.ctx, self.f, self.c
+        per_device = -(-events.n // ctx.D) if events.distribution == skel.BLOCK else events.n
+        src, lanes = self.plan(per_device)
+        ctx.set_block_size(MAP_BLOCK)
+        try:
+            if lanes == 1:
+                ctx.map(src, events, None, args=[f, c, *self.dims_args])
+            else:
+                ctx.map_lanes(src, events, None, lanes, args=[f, c, *self.dims_args])
+        finally:
+            ctx.set_block_size(0)
 
     def subset(self, events: skel.Vector, fused: bool = False):
         """One iteration of Listing 4's loop body.  fused=True runs the tail
@@ -126,11 +143,8 @@ class LMOSEM:
         ctx, f, c = self.ctx, self.f, self.c
         f.set_distribution(skel.COPY)                     # block -> copy: all-gather (no-op after a fused tail)
         c.fill_dist(skel.COPY, np.float32(0))             # fresh zero copy on every device
-        if self.map_block:
-            ctx.set_block_size(self.map_block)
-        ctx.map(self.error_src, events, None, args=[f, c, *self.dims_args])
-        if self.map_block:
-            ctx.set_block_size(0)
+        ev = self.order_on_device(events) if self.order == "device" else events
+        self.error_map(ev)
         c.mark_device_modified()                          # dataOnDevicesModified()
         if fused:
             ctx.zip_combine(LMOSEM_UPDATE, f, c, skel.COMBINE_ADD, f)

@@ -24,6 +24,29 @@ LMOSEM_ERROR_PREPARED = "#define LMOSEM_VEC_FWD 1\n" + LMOSEM_ERROR
 LMOSEM_LANES = LMOSEM_ERROR + source("lmosem_lanes")
 LMOSEM_LANES_PREPARED = "#define LMOSEM_VEC_FWD 1\n" + LMOSEM_LANES
 LMOSEM_UPDATE = source("lmosem_update")
+# on-device ordering of a subset's events by path length (Map + Scan + Map):
+# bucket counts, then the scatter into bucket order (lmosem_order.cu)
+_ORDER = LMOSEM_ERROR + source("lmosem_order")
+LMOSEM_ORDER_HIST = _ORDER + """
+void lm_order_hist(Event e, int *hist, int nx, int ny, int nz, int nb) {
+    const int b = lm_bucket(e, nx, ny, nz, nb);
+    // lanes of a warp with the same bucket add once (one atomic per bucket per warp)
+    const unsigned peers = __match_any_sync(__activemask(), b);
+    if ((int)(threadIdx.x & 31u) == __ffs(peers) - 1) atomicAdd(&hist[b], __popc(peers));
+}
+"""
+LMOSEM_ORDER_SCATTER = _ORDER + """
+void lm_order_scatter(Event e, int *cursor, Event *out, int nx, int ny, int nz, int nb) {
+    const int b = lm_bucket(e, nx, ny, nz, nb);
+    const unsigned peers = __match_any_sync(__activemask(), b);
+    const int lane = (int)(threadIdx.x & 31u), leader = __ffs(peers) - 1;
+    int base = 0;
+    if (lane == leader) base = atomicAdd(&cursor[b], __popc(peers));
+    base = __shfl_sync(peers, base, leader);
+    out[base + __popc(peers & ((1u << lane) - 1u))] = e;
+}
+"""
+LMOSEM_ORDER_BUCKETS = 64
 # voxel visits of one event's path (measurement only: the LM OSEM roofline
 # counts one scattered request per visit in each of the two walks)
 LMOSEM_VISITS = LMOSEM_ERROR + """

@@ -108,21 +108,16 @@ def test_full_size_subset_matches_oracle():
     assert abs(float(f[c > 0].astype(np.float64).sum()) - nv) <= 1e-4 * nv
 
 
-@pytest.mark.parametrize("n,D,prepared_fn", [(1_000_000, 1, False), (1_000_000, 1, True), (40_000, 4, True)])
-def test_path_ordered_events_match_oracle_in_given_order(n, D, prepared_fn):
-    """The events reordered longest path first (lmosem.order_by_path, host
-    preprocessing) -- with the plain error function or the one
-    for prepared order (16-byte forward gathers) -- give the oracle's image for
-    the events in their given order: the error image is a sum over events
-    (R10(x))."""
-    from paper_conf_ipps_steuwerkg11_b200.lmosem import order_by_path
-    from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_ERROR_PREPARED
+@pytest.mark.parametrize("n,D", [(1_000_000, 1), (60_000, 4), (20_001, 8)])
+def test_device_ordered_events_match_oracle_in_given_order(n, D):
+    """order="device": each device's events reordered longest path first on the
+    device (counting Map, Scan, scattering Map; workloads/lmosem_order.cu) --
+    the oracle's image for the events in their given order (the error image is
+    a sum over events, R10(x)), with both Map forms the policy picks."""
     events = si.lmosem_events(n, subset=3)
     with skel.Context(D) as ctx:
-        rec = LMOSEM(ctx)
-        if prepared_fn:
-            rec.error_src = LMOSEM_ERROR_PREPARED
-        rec.subset(rec.events(order_by_path(events)))
+        rec = LMOSEM(ctx, order="device")
+        rec.subset(rec.events(events))
         f = rec.image()
     want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
     assert rel_l2(f, want) <= 1e-4
@@ -130,36 +125,31 @@ def test_path_ordered_events_match_oracle_in_given_order(n, D, prepared_fn):
 
 
 @pytest.mark.parametrize("D", [1, 3])
-def test_dealt_parts_on_128_thread_ctas_match_oracle(D):
-    """lmosem.prepare_part for a small part (warp groups of similar length dealt
-    over 128-thread CTAs, the error-image Map compiled for that CTA size): the
-    same image as the oracle's for the events in their given order."""
-    from paper_conf_ipps_steuwerkg11_b200.lmosem import prepare_part
-    events = si.lmosem_events(30_000, subset=6)
-    prepared, block = prepare_part(events)
-    assert block == 128 and len(prepared) == len(events)
+def test_device_order_is_a_per_device_permutation_by_bucket(D):
+    """The reordered vector holds, on every device, a permutation of that
+    device's own events, and their length buckets never increase along it
+    (bucket of an event recomputed on the host from the oracle's exact path:
+    longer paths first, up to bucket-boundary rounding)."""
+    from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_ORDER_BUCKETS
+    n = 30_011
+    events = si.lmosem_events(n, subset=9)
     with skel.Context(D) as ctx:
-        rec = LMOSEM(ctx)
-        rec.map_block = block
-        rec.subset(rec.events(prepared))
-        f = rec.image()
-    want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
-    assert rel_l2(f, want) <= 1e-4
-    assert abs(float(f[c > 0].astype(np.float64).sum()) - nv) <= 1e-4 * nv
-
-
-@pytest.mark.parametrize("D", [1, 4])
-def test_events_prepare_option(D):
-    """LMOSEM.events(ev, prepare=True): each device's part reordered (and the
-    Map's CTA size picked) by prepare_part; the image is the oracle's."""
-    events = si.lmosem_events(24_000, subset=8)
-    with skel.Context(D) as ctx:
-        rec = LMOSEM(ctx)
-        rec.subset(rec.events(events, prepare=True))
-        assert rec.map_block == 128
-        f = rec.image()
-    want, c, nv = oracle.lmosem_subset(events, np.ones(150 * 150 * 280))
-    assert rel_l2(f, want) <= 1e-4
+        rec = LMOSEM(ctx, order="device")
+        ev = rec.events(events)
+        out = rec.order_on_device(ev).download()
+        parts = [ev.part(k) for k in range(D)]
+    rows = lambda a: sorted(map(bytes, a.view(np.uint8).reshape(len(a), -1)))  # noqa: E731
+    nb = LMOSEM_ORDER_BUCKETS
+    for lo, hi in parts:
+        assert rows(out[lo:hi]) == rows(events[lo:hi])
+        seg = out[lo:hi]
+        nvox = np.array([len(oracle.compute_path((e["x1"], e["y1"], e["z1"]), (e["x2"], e["y2"], e["z2"]))[0])
+                         for e in seg[:: max(1, len(seg) // 2000)]])
+        # the oracle's voxel count per path decreases along the order
+        from scipy.stats import spearmanr
+        r = spearmanr(np.arange(len(nvox)), nvox).statistic
+        assert r < -0.95, r
+    assert nb >= 16
 
 
 @pytest.mark.parametrize("lanes", [1, 2, 4, 8, 32])

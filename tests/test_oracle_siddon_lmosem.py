@@ -199,39 +199,3 @@ def test_events_on_detector_cylinder():
     for a, b in (("x1", "y1"), ("x2", "y2")):
         r = np.hypot(ev[a].astype(np.float64) - 75, ev[b].astype(np.float64) - 75)
         assert np.allclose(r, 110.0, atol=1e-4)
-
-
-def test_order_by_path_is_a_permutation_longest_first():
-    """lmosem.order_by_path (host preprocessing of a subset):
-    a permutation of the events whose order follows the exact path lengths of
-    the oracle's compute_path (Siddon, float64) -- longest first."""
-    import skel_inputs as si
-    from paper_conf_ipps_steuwerkg11_b200.lmosem import order_by_path
-    ev = si.lmosem_events(3000, subset=5)
-    o = order_by_path(ev)
-    rows = lambda a: sorted(map(bytes, a.view(np.uint8).reshape(len(a), -1)))  # noqa: E731
-    assert rows(o) == rows(ev)
-    nvox = np.array([len(oracle.compute_path((e["x1"], e["y1"], e["z1"]), (e["x2"], e["y2"], e["z2"]))[0])
-                     for e in o])
-    # rank correlation of position with the voxel count: strongly decreasing
-    r = np.corrcoef(np.argsort(np.argsort(nvox)), np.arange(len(o)))[0, 1]
-    assert r < -0.97, r
-    assert nvox[: len(o) // 10].mean() > 1.5 * nvox[-len(o) // 10:].mean()
-
-
-def test_deal_warps_balances_ctas():
-    """lmosem.deal_warps: a permutation; every 128-thread CTA receives one warp
-    group from each length range, so the CTAs' summed path lengths (the oracle's
-    exact voxel counts) are nearly equal while a warp's lengths stay close."""
-    import skel_inputs as si
-    from paper_conf_ipps_steuwerkg11_b200.lmosem import deal_warps
-    ev = si.lmosem_events(4096, subset=7)
-    d = deal_warps(ev, block=128)
-    rows = lambda a: sorted(map(bytes, a.view(np.uint8).reshape(len(a), -1)))  # noqa: E731
-    assert rows(d) == rows(ev)
-    nvox = np.array([len(oracle.compute_path((e["x1"], e["y1"], e["z1"]), (e["x2"], e["y2"], e["z2"]))[0])
-                     for e in d], dtype=np.float64)
-    per_cta = nvox.reshape(-1, 128).sum(axis=1)
-    assert per_cta.std() / per_cta.mean() < 0.03
-    per_warp_spread = (nvox.reshape(-1, 32).max(axis=1) - nvox.reshape(-1, 32).min(axis=1)).mean()
-    assert per_warp_spread < 0.25 * nvox.mean()

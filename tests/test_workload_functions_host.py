@@ -170,3 +170,52 @@ def test_blocked_mandelbrot_equals_the_plain_iteration(mandel_blocked, golden_di
         with open(os.path.join(golden_dir, "mandelbrot.json")) as fh:
             case = [c for c in json.load(fh)["cases"] if (c["width"], c["height"], c["cap"]) == (1024, 768, 256)][0]
         assert zlib.crc32(got.tobytes()) == int(case["crc32"], 16)
+
+
+ORDER_SHIM = r'''
+#include <cmath>
+#include <algorithm>
+using std::min; using std::max; using std::fmin; using std::fmax; using std::fabs;
+#define __forceinline__ inline
+template <class T> static T __ldg(const T* p) { return *p; }
+struct float4 { float x, y, z, w; };
+static inline float4 make_float4(float a, float b, float c, float d) { return float4{a, b, c, d}; }
+#include "ERR"
+#include "ORD"
+extern "C" void buckets(const float* ev, int n, int nx, int ny, int nz, int nb, int* out) {
+    for (int i = 0; i < n; ++i) {
+        Event e{ev[6*i], ev[6*i+1], ev[6*i+2], ev[6*i+3], ev[6*i+4], ev[6*i+5]};
+        out[i] = lm_bucket(e, nx, ny, nz, nb);
+    }
+}
+'''
+
+
+def test_device_order_key_follows_the_exact_path_length(tmp_path):
+    """lm_bucket (workloads/lmosem_order.cu, the key of the on-device event
+    ordering): bucket 0 = longest clipped path; checked against the oracle's
+    exact Siddon path lengths (rank correlation), range [0, nb), and a ray that
+    misses the volume goes last."""
+    wl = ROOT / "paper_conf_ipps_steuwerkg11_b200" / "workloads"
+    src = tmp_path / "order.cpp"
+    src.write_text(ORDER_SHIM.replace("ERR", str(wl / "lmosem_error.cu")).replace("ORD", str(wl / "lmosem_order.cu")))
+    so = tmp_path / "order.so"
+    subprocess.run(["g++", "-O2", "-std=c++17", "-ffp-contract=off", "-shared", "-fPIC", str(src), "-o", str(so)],
+                   check=True)
+    lib = ctypes.CDLL(str(so))
+    lib.buckets.argtypes = [ctypes.c_void_p, ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_int,
+                            ctypes.c_void_p]
+    ev = si.lmosem_events(3000, subset=5)
+    miss = np.zeros(1, si.EVENT_DTYPE)
+    miss["x1"], miss["y1"], miss["z1"], miss["x2"], miss["y2"], miss["z2"] = -5, -5, -5, -9, -1, -7
+    ev = np.concatenate([ev, miss])
+    nb = 64
+    b = np.zeros(ev.size, np.int32)
+    lib.buckets(ev.ctypes.data, ev.size, 150, 150, 280, nb, b.ctypes.data)
+    assert b.min() >= 0 and b.max() <= nb - 1 and b[-1] == nb - 1
+    # the walk's work is its voxel count: the oracle's number of path segments
+    nvox = np.array([len(oracle.compute_path((e["x1"], e["y1"], e["z1"]), (e["x2"], e["y2"], e["z2"]))[0])
+                     for e in ev[:-1]])
+    from scipy.stats import spearmanr
+    r = spearmanr(b[:-1], -nvox).statistic  # ties (a bucket holds many events) ranked by their mean
+    assert r > 0.95, r

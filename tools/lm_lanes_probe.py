@@ -13,7 +13,7 @@ import torch
 
 import skel_inputs as si
 from paper_conf_ipps_steuwerkg11_b200 import skel
-from paper_conf_ipps_steuwerkg11_b200.lmosem import order_by_path
+from paper_conf_ipps_steuwerkg11_b200.lmosem import LMOSEM
 from paper_conf_ipps_steuwerkg11_b200.workloads import (LMOSEM_ERROR, LMOSEM_ERROR_PREPARED, LMOSEM_LANES,
                                                         LMOSEM_LANES_PREPARED)
 
@@ -45,7 +45,9 @@ with skel.Context(1) as ctx:
     for D in Ds:
         part = ev[: 1_000_000 // D]
         for order in ("given", "length"):
-            e = ctx.vector(part if order == "given" else order_by_path(part))
+            e = ctx.vector(part)
+            if order == "length":  # ordered on the device (lmosem.LMOSEM.order_on_device)
+                e = LMOSEM(ctx, order="device").order_on_device(e)
             for blk in BLOCKS:
                 ctx.set_block_size(blk)
                 res = {"D": D, "events": len(part), "order": order, "block": blk}

@@ -1,6 +1,19 @@
-"""Per-GPU work of LM OSEM at D GPUs, measured on one GPU: the error-image
-Map over 10^6/D events (what each GPU runs per subset at D GPUs), plus the
-other per-subset kernels.  Prints ms per Map for D = 1, 2, 4, 8."""
+"""LM OSEM subset time at D GPUs projected from pieces measured on ONE GPU
+(only one GPU is available to this build).  For D = 1, 2, 4, 8 it times what
+each GPU runs per subset at D GPUs (Listing 4's loop body, PAPER.md
+P:L518-549), with the library's own policy (lmosem.LMOSEM.plan):
+
+  fill   c <- 0 on the device's whole copy (25.2 MB)
+  order  the device's 10^6/D events reordered by path length (order="device")
+  map    the error-image Map over the 10^6/D events (given / device order)
+  zip    the update Zip over the device's 6.3M/D voxels
+
+and adds the exchange, which one GPU cannot run: copy->block+add
+(reduce-scatter) and block->copy (all-gather) of the 25.2 MB image move
+(D-1)/D x 25.2 MB into and out of each GPU, at the measured 770 GB/s peer
+copy per direction (B200_PROFILING.md; NVLS in-switch reduction would move
+1/D of it).  Prints one JSON line per D and a summary with T1/TD."""
+import json
 import os
 import sys
 
@@ -10,33 +23,56 @@ import torch
 
 import skel_inputs as si
 from paper_conf_ipps_steuwerkg11_b200 import skel
-from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_ERROR
+from paper_conf_ipps_steuwerkg11_b200.lmosem import LMOSEM
+from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_UPDATE
 
-if os.environ.get("LM_SRC"):  # A/B: an alternative error-image function text
-    LMOSEM_ERROR = open(os.environ["LM_SRC"]).read()
-
+NVLINK_GBPS = 770.0
+S = 150 * 150 * 280 * 4
 ev = si.lmosem_events(1_000_000, subset=0)
+rows = []
 with skel.Context(1) as ctx:
     stream = torch.cuda.ExternalStream(ctx.stream(0))
-    f = ctx.vector(n=150 * 150 * 280, dtype=np.float32).fill(np.float32(1))
-    c = ctx.vector(n=150 * 150 * 280, dtype=np.float32)
-    dims = [np.int32(150), np.int32(150), np.int32(280)]
-    for D in (1, 2, 4, 8):
-        part = ev[: 1_000_000 // D]
-        if os.environ.get("LM_ORDER") == "dealt":  # longest first, warp groups dealt to the CTAs
-            from paper_conf_ipps_steuwerkg11_b200.lmosem import deal_warps
-            part = deal_warps(part, block=int(os.environ.get("SKEL_BLOCK_SIZE", "256")))
-        elif os.environ.get("LM_ORDER"):  # each GPU orders its part longest path first
-            from paper_conf_ipps_steuwerkg11_b200.lmosem import order_by_path
-            part = order_by_path(part)
-        e = ctx.vector(part)
+
+    def timed(fn, reps=20):
         for _ in range(3):
-            ctx.map(LMOSEM_ERROR, e, None, args=[f, c, *dims])
+            fn()
         ctx.sync()
         e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         e0.record(stream)
-        for _ in range(10):
-            ctx.map(LMOSEM_ERROR, e, None, args=[f, c, *dims])
+        for _ in range(reps):
+            fn()
         e1.record(stream)
         ctx.sync()
-        print(f"D={D} events={1_000_000 // D} map_ms={e0.elapsed_time(e1) / 10:.4f}", flush=True)
+        return e0.elapsed_time(e1) / reps
+
+    for D in (1, 2, 4, 8):
+        part = ev[: 1_000_000 // D]
+        r = {"D": D, "events_per_gpu": len(part)}
+        for order in ("given", "device"):
+            rec = LMOSEM(ctx, order=order)
+            rec.prepare()
+            e = ctx.vector(part)
+            rec.f.set_distribution(skel.COPY)
+            rec.c.fill_dist(skel.COPY, np.float32(0))
+            r[f"{order}_map_ms"] = timed(lambda: rec.error_map(e))
+            if order == "device":
+                r["order_ms"] = timed(lambda: rec.order_on_device(e))
+                ordered = rec.order_on_device(e)
+                r["device_map_ms"] = timed(lambda: rec.error_map(ordered))
+            r["fill_ms"] = timed(lambda: rec.c.fill_dist(skel.COPY, np.float32(0)))
+            e.destroy()
+        nv = -(-150 * 150 * 280 // D)
+        fp, cp = ctx.vector(n=nv, dtype=np.float32).fill(np.float32(1)), ctx.vector(n=nv, dtype=np.float32)
+        cp.fill(np.float32(0.5))
+        r["zip_ms"] = timed(lambda: ctx.zip(LMOSEM_UPDATE, fp, cp, fp))
+        r["exchange_ms_model"] = 2 * S * (D - 1) / D / (NVLINK_GBPS * 1e9) * 1e3
+        for order in ("given", "device"):
+            extra = r["order_ms"] if order == "device" else 0.0
+            r[f"{order}_subset_ms"] = r["fill_ms"] + extra + r[f"{order}_map_ms"] + r["zip_ms"] + r["exchange_ms_model"]
+        rows.append(r)
+        print(json.dumps({k: (round(v, 4) if isinstance(v, float) else v) for k, v in r.items()}), flush=True)
+summary = {}
+for order in ("given", "device"):
+    t1 = rows[0][f"{order}_subset_ms"]
+    summary[order] = {f"T1/T{r['D']}": round(t1 / r[f"{order}_subset_ms"], 2) for r in rows}
+print(json.dumps({"projection": summary, "exchange": f"RS + AG of {S / 1e6:.1f} MB at {NVLINK_GBPS} GB/s per direction"}))

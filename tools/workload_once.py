@@ -16,10 +16,10 @@ with skel.Context(1) as ctx:
         for _ in range(3):
             ctx.map(MANDELBROT, vin, out, args=[np.int32(256)])
         ctx.sync()
-    if which in ("both", "lmosem", "lmosem_prepared"):
+    if which in ("both", "lmosem", "lmosem_device"):
         ev = si.lmosem_events(1_000_000, subset=0)
-        rec = LMOSEM(ctx)
-        evv = rec.events(ev, prepare=which == "lmosem_prepared")
+        rec = LMOSEM(ctx, order="device" if which == "lmosem_device" else "given")
+        evv = rec.events(ev)
         for _ in range(3):
             rec.subset(evv)
         ctx.sync()
