@@ -30,7 +30,8 @@ import numpy as np
 
 from . import skel
 from .workloads import (LMOSEM_ERROR, LMOSEM_ERROR_PREPARED, LMOSEM_LANES, LMOSEM_LANES_PREPARED,
-                        LMOSEM_ORDER_BUCKETS, LMOSEM_ORDER_HIST, LMOSEM_ORDER_SCATTER, LMOSEM_UPDATE, SUM_I32)
+                        LMOSEM_ORDER_BUCKETS, LMOSEM_ORDER_HIST, LMOSEM_ORDER_SCATTER, LMOSEM_ORDER_SLOTS,
+                        LMOSEM_UPDATE, SUM_I32)
 
 DIMS = (150, 150, 280)
 
@@ -103,9 +104,9 @@ class LMOSEM:
         of the counts, and a void Map that moves each event to its bucket's next
         slot.  Returns a vector with the same distribution and part sizes."""
         ctx, nb = self.ctx, LMOSEM_ORDER_BUCKETS
-        if self._hist is None:
-            self._hist = ctx.vector(n=nb, dtype=np.int32)
-            self._cursor = ctx.vector(n=nb, dtype=np.int32)
+        if self._hist is None:  # bucket-major counter slots (lmosem_order.cu: lm_slot)
+            self._hist = ctx.vector(n=LMOSEM_ORDER_SLOTS, dtype=np.int32)
+            self._cursor = ctx.vector(n=LMOSEM_ORDER_SLOTS, dtype=np.int32)
         if self._sorted is None or self._sorted.n != events.n or \
                 self._sorted.distribution != events.distribution:
             if self._sorted is not None:

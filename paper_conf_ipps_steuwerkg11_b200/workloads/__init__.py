@@ -29,24 +29,26 @@ LMOSEM_UPDATE = source("lmosem_update")
 _ORDER = LMOSEM_ERROR + source("lmosem_order")
 LMOSEM_ORDER_HIST = _ORDER + """
 void lm_order_hist(Event e, int *hist, int nx, int ny, int nz, int nb) {
-    const int b = lm_bucket(e, nx, ny, nz, nb);
-    // lanes of a warp with the same bucket add once (one atomic per bucket per warp)
-    const unsigned peers = __match_any_sync(__activemask(), b);
-    if ((int)(threadIdx.x & 31u) == __ffs(peers) - 1) atomicAdd(&hist[b], __popc(peers));
+    const int k = lm_slot(e, nx, ny, nz, nb);
+    // lanes of a warp with the same counter add once
+    const unsigned peers = __match_any_sync(__activemask(), k);
+    if ((int)(threadIdx.x & 31u) == __ffs(peers) - 1) atomicAdd(&hist[k], __popc(peers));
 }
 """
 LMOSEM_ORDER_SCATTER = _ORDER + """
 void lm_order_scatter(Event e, int *cursor, Event *out, int nx, int ny, int nz, int nb) {
-    const int b = lm_bucket(e, nx, ny, nz, nb);
-    const unsigned peers = __match_any_sync(__activemask(), b);
+    const int k = lm_slot(e, nx, ny, nz, nb);
+    const unsigned peers = __match_any_sync(__activemask(), k);
     const int lane = (int)(threadIdx.x & 31u), leader = __ffs(peers) - 1;
     int base = 0;
-    if (lane == leader) base = atomicAdd(&cursor[b], __popc(peers));
+    if (lane == leader) base = atomicAdd(&cursor[k], __popc(peers));
     base = __shfl_sync(peers, base, leader);
     out[base + __popc(peers & ((1u << lane) - 1u))] = e;
 }
 """
 LMOSEM_ORDER_BUCKETS = 64
+LMOSEM_ORDER_REPLICAS = 128  # counters per bucket (lmosem_order.cu: lm_slot)
+LMOSEM_ORDER_SLOTS = LMOSEM_ORDER_BUCKETS * LMOSEM_ORDER_REPLICAS
 # voxel visits of one event's path (measurement only: the LM OSEM roofline
 # counts one scattered request per visit in each of the two walks)
 LMOSEM_VISITS = LMOSEM_ERROR + """

@@ -18,3 +18,18 @@ static __forceinline__ int lm_bucket(const Event &e, int nx, int ny, int nz, int
     const int k = (int)(l1 * (double)nb / (double)(nx + ny + nz));
     return nb - 1 - min(max(k, 0), nb - 1);
 }
+
+// Counter slot of an event: bucket-major, LM_ORDER_R replica counters per
+// bucket picked by a hash of the event's bits.  With one counter per bucket
+// the few busiest buckets serialise ~10^4 atomics each on one L2 address (the
+// ordering measured 133 us for 10^6 events); the replicas spread them.  The
+// slot depends only on the event, so the counting and the scattering Map
+// agree on it, and the scan over the slots in index order still puts the
+// buckets in order.
+#define LM_ORDER_R 128
+static __forceinline__ int lm_slot(const Event &e, int nx, int ny, int nz, int nb) {
+    unsigned h = __float_as_uint(e.x1) * 0x9E3779B1u ^ __float_as_uint(e.y2) * 0x85EBCA77u ^
+                 __float_as_uint(e.z1) * 0xC2B2AE3Du;
+    h ^= h >> 15;
+    return lm_bucket(e, nx, ny, nz, nb) * LM_ORDER_R + (int)(h & (LM_ORDER_R - 1));
+}

@@ -180,6 +180,8 @@ using std::min; using std::max; using std::fmin; using std::fmax; using std::fab
 template <class T> static T __ldg(const T* p) { return *p; }
 struct float4 { float x, y, z, w; };
 static inline float4 make_float4(float a, float b, float c, float d) { return float4{a, b, c, d}; }
+#include <cstring>
+static inline unsigned __float_as_uint(float f) { unsigned u; std::memcpy(&u, &f, 4); return u; }
 #include "ERR"
 #include "ORD"
 extern "C" void buckets(const float* ev, int n, int nx, int ny, int nz, int nb, int* out) {

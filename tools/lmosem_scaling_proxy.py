@@ -65,14 +65,22 @@ with skel.Context(1) as ctx:
         fp, cp = ctx.vector(n=nv, dtype=np.float32).fill(np.float32(1)), ctx.vector(n=nv, dtype=np.float32)
         cp.fill(np.float32(0.5))
         r["zip_ms"] = timed(lambda: ctx.zip(LMOSEM_UPDATE, fp, cp, fp))
+        # RS then AG (NCCL, one after the other): (D-1)/D x S out of each GPU, then into it
         r["exchange_ms_model"] = 2 * S * (D - 1) / D / (NVLINK_GBPS * 1e9) * 1e3
+        # fused peer-memory tail (skel_zip_combine): the loads of the peers' copies
+        # (into the GPU) and the stores of the new f part (out of it) overlap on the
+        # full-duplex links: (D-1)/D x S per direction
+        r["exchange_fused_ms_model"] = S * (D - 1) / D / (NVLINK_GBPS * 1e9) * 1e3
         for order in ("given", "device"):
             extra = r["order_ms"] if order == "device" else 0.0
-            r[f"{order}_subset_ms"] = r["fill_ms"] + extra + r[f"{order}_map_ms"] + r["zip_ms"] + r["exchange_ms_model"]
+            base = r["fill_ms"] + extra + r[f"{order}_map_ms"] + r["zip_ms"]
+            r[f"{order}_subset_ms"] = base + r["exchange_ms_model"]
+            r[f"{order}_subset_fused_ms"] = base + r["exchange_fused_ms_model"]
         rows.append(r)
         print(json.dumps({k: (round(v, 4) if isinstance(v, float) else v) for k, v in r.items()}), flush=True)
 summary = {}
 for order in ("given", "device"):
-    t1 = rows[0][f"{order}_subset_ms"]
-    summary[order] = {f"T1/T{r['D']}": round(t1 / r[f"{order}_subset_ms"], 2) for r in rows}
+    for tail in ("", "_fused"):
+        t1 = rows[0][f"{order}_subset{tail}_ms"]
+        summary[order + tail] = {f"T1/T{r['D']}": round(t1 / r[f"{order}_subset{tail}_ms"], 2) for r in rows}
 print(json.dumps({"projection": summary, "exchange": f"RS + AG of {S / 1e6:.1f} MB at {NVLINK_GBPS} GB/s per direction"}))
