@@ -45,18 +45,11 @@ struct Module {
     cudaKernel_t k_zipcomb = nullptr;  // Zip modules: fused combine + zip + broadcast
     uint64_t sig[16 + 4 * 32] = {0};
     std::set<int> attr_set_on;  // devices on which smem attributes were set
-    // element-wise grid policy per size class (log2 of the chunk count), chosen
-    // by measurement: 0 = UNROLL chunks in flight per thread (bandwidth-bound
-    // user functions), 1 = one chunk per thread, 2 = one element per thread
-    // through the scalar path (compute-bound, divergent ones: finer work items
-    // even out the lanes of a warp)
-    static constexpr int kPolicies = 3, kRounds = 2;
-    struct EwTune {
-        int trial = 0;   // launches timed so far (policies in turn: 0,1,2,0,1,2)
-        int best = -1;   // decided policy, -1 while measuring
-        cudaEvent_t ev[2 * kPolicies * kRounds] = {};
-    };
-    std::map<int, EwTune> ew_tune;
+    // element-wise grid policy (runtime.cpp ew_decide): 0 = UNROLL chunks in
+    // flight per thread, 1 = one chunk per thread, 2 = one element per thread
+    // through the scalar path; -1 until decided on a sample at the first launch
+    static constexpr int kPolicies = 3;
+    int ew_policy = -1;
     int red_occ = 0;  // resident Reduce CTAs per SM (0 = not yet queried)
 };
 

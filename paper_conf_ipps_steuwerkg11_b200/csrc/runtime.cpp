@@ -824,51 +824,117 @@ int ew_grid(const Slot &s, size_t chunks, int block, int per_thread) {
     return (int)std::max<size_t>(g, 1);
 }
 
-// element-wise grid policy for a module and size class (log2 of the chunk
-// count), chosen by measurement among the policies in `mask` (bit p = policy
-// p; the lowest one is the default another must beat by 3%): the first
-// launches on the first device time each in turn, twice (events around the
-// launch, outside graph captures); later launches use the fastest
-struct EwChoice {
-    int policy = 0, tslot = -1;
-    Module::EwTune *tu = nullptr;
-};
-int ew_choose(skel_ctx_s *ctx, Module *m, Slot &s, size_t li, uint64_t chunks, unsigned mask, EwChoice &ch) {
+// Element-wise grid policy of a module (Module::ew_policy): 0 = UNROLL chunks
+// in flight per thread (bandwidth-bound functions), 1 = one chunk per thread,
+// 2 = one element per thread through the scalar path (compute-bound, divergent
+// functions: finer work items even out the lanes of a warp).  Decided ONCE per
+// module, at its first launch, by timing the policies in `mask` on a SAMPLE of
+// that launch's data copied to scratch memory -- never on the user's buffers,
+// so no user launch runs with a losing policy and nothing the user owns is
+// written twice.  The sample: 256 evenly spread blocks of the input(s), 2^21
+// elements in all (the whole vector if smaller); an index Map samples four
+// contiguous index ranges spread over [0, n).  Functions with pointer
+// (vector) arguments may have side effects and are not sampled: they take the
+// mask's lowest policy.  The lowest policy is also the default another must
+// beat by 3%.
+bool has_ptr_args(const Module *m) {
+    for (uint64_t i = 0; i < m->sig[6] && i < 32; ++i)
+        if (m->sig[18 + 4 * i]) return true;
+    return false;
+}
+
+int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, size_t esa, const void *pb, size_t esb,
+              size_t eso, uint64_t cnt, uint64_t base, std::vector<unsigned char> &abuf, unsigned mask, int *policy) {
     int pol[Module::kPolicies], P = 0;
     for (int p = 0; p < Module::kPolicies; ++p)
         if (mask & (1u << p)) pol[P++] = p;
-    ch.policy = pol[0];
-    Module::EwTune *tu = &m->ew_tune[64 - __builtin_clzll((unsigned long long)std::max<uint64_t>(chunks, 1))];
-    ch.tu = tu;
+    *policy = pol[0];
+    if (m->ew_policy >= 0) {
+        *policy = m->ew_policy;
+        return SKEL_OK;
+    }
     cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
     cudaStreamIsCapturing(s.stream, &cs);
-    const int NT = P * Module::kRounds;
-    if (tu->best < 0 && li == 0 && cs == cudaStreamCaptureStatusNone) {
-        if (tu->trial == NT) {  // all samples recorded: decide (one wait, once per class)
-            CK(ctx, cudaEventSynchronize(tu->ev[2 * NT - 1]));
-            float best_t[Module::kPolicies];
-            for (int p = 0; p < P; ++p) best_t[p] = 3.0e38f;
-            for (int k = 0; k < NT; ++k) {
-                float t = 0;
-                CK(ctx, cudaEventElapsedTime(&t, tu->ev[2 * k], tu->ev[2 * k + 1]));
-                best_t[k % P] = std::min(best_t[k % P], t);
-            }
-            int b = 0;
-            for (int p = 1; p < P; ++p)
-                if (best_t[p] < 0.97f * best_t[0] && best_t[p] < best_t[b]) b = p;
-            tu->best = pol[b];
-            for (cudaEvent_t &e : tu->ev) {
-                if (e) cudaEventDestroy(e);
-                e = nullptr;
-            }
-        } else {
-            ch.tslot = tu->trial++;
-            ch.policy = pol[ch.tslot % P];
-            for (int k = 0; k < 2; ++k)
-                if (!tu->ev[2 * ch.tslot + k]) CK(ctx, cudaEventCreate(&tu->ev[2 * ch.tslot + k]));
-        }
+    if (cs != cudaStreamCaptureStatusNone || eso == 0 || has_ptr_args(m) || P < 2) {
+        if (cs == cudaStreamCaptureStatusNone) m->ew_policy = pol[0];
+        return SKEL_OK;
     }
-    if (tu->best >= 0) ch.policy = tu->best;
+    const uint64_t E = m->sig[8];
+    const int block = (int)m->sig[9];
+    const int unroll = std::max<int>(1, (int)m->sig[10]);
+    constexpr uint64_t kSample = 1ull << 21, kBlocks = 256;
+    uint64_t ns = std::min<uint64_t>(cnt, kSample) / E * E;
+    if (ns == 0) return SKEL_OK;  // decide at a larger launch
+    const size_t oa = 0, ob = align_up(ns * esa, 256), oo = ob + align_up(pb ? ns * esb : 0, 256);
+    TRY(scratch(ctx, s, oo + align_up(ns * eso, 256)));
+    char *sa = s.scratch + oa, *sb = s.scratch + ob, *so = s.scratch + oo;
+    DevGuard g(s.dev);
+    std::vector<std::pair<uint64_t, uint64_t>> ranges;  // index Map: (base, count) per launch
+    if (kind == Kind::Idx) {
+        const uint64_t part = ns / 4 / E * E;
+        for (int r = 0; r < 4 && part; ++r) {
+            const uint64_t lo = std::min<uint64_t>(cnt - part, (cnt / 4) * r + cnt / 8 - std::min(cnt / 8, part / 2));
+            ranges.push_back({base + lo, part});
+        }
+        if (ranges.empty()) ranges.push_back({base, ns});
+    } else if (cnt <= kSample) {
+        CK(ctx, cudaMemcpyAsync(sa, pa, ns * esa, cudaMemcpyDeviceToDevice, s.stream));
+        if (pb) CK(ctx, cudaMemcpyAsync(sb, pb, ns * esb, cudaMemcpyDeviceToDevice, s.stream));
+        ranges.push_back({0, ns});
+    } else {
+        const uint64_t blk = std::max<uint64_t>(E, ns / kBlocks / E * E), nblk = ns / blk;
+        const uint64_t stride = cnt / nblk;  // >= blk
+        CK(ctx, cudaMemcpy2DAsync(sa, blk * esa, pa, stride * esa, blk * esa, nblk, cudaMemcpyDeviceToDevice,
+                                  s.stream));
+        if (pb)
+            CK(ctx, cudaMemcpy2DAsync(sb, blk * esb, pb, stride * esb, blk * esb, nblk, cudaMemcpyDeviceToDevice,
+                                      s.stream));
+        ns = blk * nblk;
+        ranges.push_back({0, ns});
+    }
+    cudaEvent_t ev[2 * Module::kPolicies * 2] = {};
+    for (auto &e : ev) CK(ctx, cudaEventCreate(&e));
+    auto launch = [&](int policy) -> int {
+        for (auto &rg : ranges) {
+            uint64_t n = rg.second, b0 = rg.first;
+            const size_t chunks = std::max<uint64_t>(n / E, 1);
+            int vk = policy == 2 ? 0 : 1;
+            const void *qa = sa, *qb = pb ? (const void *)sb : nullptr;
+            void *qo = so;
+            int grid;
+            if (kind == Kind::Idx) {
+                grid = ew_grid(s, policy == 2 ? n : chunks, block, 1);
+                void *params[] = {&qo, &n, &b0, &vk, abuf.data()};
+                CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+            } else {
+                grid = policy == 2 ? ew_grid(s, n, block, 1) : ew_grid(s, chunks, block, policy == 0 ? unroll : 1);
+                void *params[] = {&qa, &qb, &qo, &n, &vk, abuf.data()};
+                CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+            }
+        }
+        return SKEL_OK;
+    };
+    TRY(launch(pol[0]));  // warm (first touch of the module on this device)
+    for (int k = 0; k < 2 * P; ++k) {
+        CK(ctx, cudaEventRecord(ev[2 * k], s.stream));
+        TRY(launch(pol[k % P]));
+        CK(ctx, cudaEventRecord(ev[2 * k + 1], s.stream));
+    }
+    CK(ctx, cudaEventSynchronize(ev[4 * P - 1]));
+    float best_t[Module::kPolicies];
+    for (int p = 0; p < P; ++p) best_t[p] = 3.0e38f;
+    for (int k = 0; k < 2 * P; ++k) {
+        float t = 0;
+        CK(ctx, cudaEventElapsedTime(&t, ev[2 * k], ev[2 * k + 1]));
+        best_t[k % P] = std::min(best_t[k % P], t);
+    }
+    for (auto &e : ev) cudaEventDestroy(e);
+    int b = 0;
+    for (int p = 1; p < P; ++p)
+        if (best_t[p] < 0.97f * best_t[0] && best_t[p] < best_t[b]) b = p;
+    m->ew_policy = pol[b];
+    ctx->stats.kernel_launches += (uint64_t)(2 * P + 1) * ranges.size();
+    *policy = m->ew_policy;
     return SKEL_OK;
 }
 
@@ -909,19 +975,16 @@ int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_
         const size_t chunks = vec_ok ? std::max<uint64_t>(cnt / E, 1) : cnt;
         const int unroll = std::max<int>(1, (int)m->sig[10]);
         DevGuard g(s.dev);
-        // grid policy (Module::EwTune): measured among policies 0/1/2
-        EwChoice ch;
-        if (vec_ok && E > 1 && unroll > 1) TRY(ew_choose(ctx, m, s, li, chunks, 0x7u, ch));
-        const int policy = ch.policy, tslot = ch.tslot;
-        Module::EwTune *tu = ch.tu;
+        // grid policy (Module::ew_policy): decided on a sample at the module's first launch
+        int policy = 0;
+        if (vec_ok && E > 1 && unroll > 1)
+            TRY(ew_decide(ctx, m, s, kind, pa, a->es, pb, b ? b->es : 0, rsz, cnt, 0, abuf, 0x7u, &policy));
         // policy 2: the scalar path, one element per thread
         int vk = policy == 2 ? 0 : vec_ok;
         const int grid = policy == 2 ? ew_grid(s, cnt, block, 1)
                                      : ew_grid(s, chunks, block, policy == 0 && vec_ok && E > 1 ? unroll : 1);
         void *params[] = {&pa, &pb, &po, &cnt, &vk, abuf.data()};
-        if (tslot >= 0) CK(ctx, cudaEventRecord(tu->ev[2 * tslot], s.stream));
         CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
-        if (tslot >= 0) CK(ctx, cudaEventRecord(tu->ev[2 * tslot + 1], s.stream));
         ctx->stats.kernel_launches++;
     }
     if (rsz != 0) {
@@ -1414,9 +1477,6 @@ int skel_finalize(skel_ctx_t ctx) {
     for (auto *v : vs) skel_vector_destroy(v);
     for (auto &kv : ctx->modules) {
         if (kv.second->lib) cudaLibraryUnload(kv.second->lib);
-        for (auto &t : kv.second->ew_tune)
-            for (cudaEvent_t e : t.second.ev)
-                if (e) cudaEventDestroy(e);
     }
     if (ctx->comm) ncclCommDestroy(ctx->comm);
     for (auto &s : ctx->slots) {
@@ -1474,9 +1534,6 @@ int skel_clear_kernel_cache(skel_ctx_t ctx) {
     TRY(sync_all(ctx));
     for (auto &kv : ctx->modules) {
         if (kv.second->lib) cudaLibraryUnload(kv.second->lib);
-        for (auto &t : kv.second->ew_tune)
-            for (cudaEvent_t e : t.second.ev)
-                if (e) cudaEventDestroy(e);
     }
     ctx->modules.clear();
     ctx->fast_modules.clear();
@@ -1822,15 +1879,13 @@ int skel_map_index(skel_ctx_t ctx, const char *src, size_t n, skel_vec_t out, co
         // measured choice between one chunk of E outputs per thread (policy 1) and
         // one element per thread through the scalar path (policy 2): a divergent,
         // compute-bound function (Mandelbrot) balances better with the second
-        EwChoice ch;
-        ch.policy = 1;
-        if (vec_ok && rsz != 0 && E > 1) TRY(ew_choose(ctx, m, s, li, chunks, 0x6u, ch));
-        int vk = ch.policy == 2 ? 0 : vec_ok;
-        const int grid = ew_grid(s, ch.policy == 2 ? cnt : chunks, block, 1);
+        int policy = 1;
+        if (vec_ok && rsz != 0 && E > 1)
+            TRY(ew_decide(ctx, m, s, Kind::Idx, nullptr, 0, nullptr, 0, rsz, cnt, base, abuf, 0x6u, &policy));
+        int vk = policy == 2 ? 0 : vec_ok;
+        const int grid = ew_grid(s, policy == 2 ? cnt : chunks, block, 1);
         void *params[] = {&po, &cnt, &base, &vk, abuf.data()};
-        if (ch.tslot >= 0) CK(ctx, cudaEventRecord(ch.tu->ev[2 * ch.tslot], s.stream));
         CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
-        if (ch.tslot >= 0) CK(ctx, cudaEventRecord(ch.tu->ev[2 * ch.tslot + 1], s.stream));
         ctx->stats.kernel_launches++;
     }
     if (rsz != 0) {

@@ -14,6 +14,8 @@ def source(name: str) -> str:
 MANDELBROT = source("mandelbrot")
 MANDELBROT_INDEX = source("mandelbrot_index")  # index Map variant (NEXT-4)
 MANDELBROT_BLOCKED = source("mandelbrot_blocked")  # loop control per block of updates (NEXT-4)
+# pairs of neighbouring pixels per element, packed FP32x2 arithmetic (NEXT-4)
+MANDELBROT_PAIRS = source("mandelbrot_pairs")
 LMOSEM_ERROR = source("lmosem_error")
 # the same function for prepared (longest-path-first) event order, where the
 # Map is bound by L1TEX requests: 16-byte gathers per 4-float group in the

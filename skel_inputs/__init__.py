@@ -24,6 +24,10 @@ SEED_BASE = 20110516
 
 # Vector<{float re, im}> element of the Mandelbrot Map (8 bytes, AoS).
 POS_DTYPE = np.dtype([("re", np.float32), ("im", np.float32)])
+# Vector<{Pos, Pos}>: two neighbouring pixels per element (the same bytes as a
+# Vector<Pos> of twice the length; workloads/mandelbrot_pairs.cu)
+POS2_DTYPE = np.dtype([("re0", np.float32), ("im0", np.float32), ("re1", np.float32), ("im1", np.float32)])
+CNT2_DTYPE = np.dtype([("n0", np.int32), ("n1", np.int32)])
 # Vector<Event> element of LM OSEM: {float x1,y1,z1,x2,y2,z2} (24 bytes, AoS),
 # DESIGN.md reading R8 (PAPER.md P:L520 leaves the fields unspecified).
 EVENT_DTYPE = np.dtype([("x1", np.float32), ("y1", np.float32), ("z1", np.float32),

@@ -89,3 +89,27 @@ def test_blocked_variant_bit_exact(golden_dir, w, h, cap, D):
         assert zlib.crc32(got.tobytes()) == int(case[0]["crc32"], 16)
     if w * h <= 1 << 20:
         assert np.array_equal(got, oracle.mandelbrot(pos, cap))
+
+
+@pytest.mark.parametrize("w,h,cap,D", [(1024, 768, 256, 1), (4096, 3072, 256, 1), (1024, 768, 4096, 1),
+                                       (1024, 768, 256, 4), (1024, 768, 7, 1), (1024, 768, 1500, 1)])
+def test_pairs_variant_bit_exact(golden_dir, w, h, cap, D):
+    """mandelbrot_pairs.cu (two neighbouring pixels per element, packed FFMA2 /
+    FADD2 arithmetic with the multiplies kept unfused): the same counts as eq.
+    (5) as written -- golden CRCs and the oracle, on one and on four devices."""
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_PAIRS
+    pos = si.mandelbrot_positions(w, h)
+    pairs = pos.view(si.POS2_DTYPE)
+    with skel.Context(D) as ctx:
+        vin = ctx.vector(pairs)
+        if D > 1:
+            vin.set_distribution(skel.BLOCK)
+        out = ctx.vector(n=pairs.size, dtype=si.CNT2_DTYPE)
+        ctx.map(MANDELBROT_PAIRS, vin, out, args=[np.int32(cap)])
+        got = out.download().view(np.int32)
+    with open(os.path.join(golden_dir, "mandelbrot.json")) as fh:
+        cases = [c for c in json.load(fh)["cases"] if (c["width"], c["height"], c["cap"]) == (w, h, cap)]
+    if cases:
+        assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)
+    if w * h <= 1 << 20:
+        assert np.array_equal(got, oracle.mandelbrot(pos, cap))

@@ -221,3 +221,43 @@ def test_device_order_key_follows_the_exact_path_length(tmp_path):
     from scipy.stats import spearmanr
     r = spearmanr(b[:-1], -nvox).statistic  # ties (a bucket holds many events) ranked by their mean
     assert r > 0.95, r
+
+
+PAIRS_SHIM = r'''
+#define __forceinline__ inline
+#include "SRC"
+extern "C" void run(const float* pos, long npairs, int cap, int* out) {
+    for (long i = 0; i < npairs; ++i) {
+        Cnt2 r = mandelbrot_pairs(Pos2{pos[4*i], pos[4*i+1], pos[4*i+2], pos[4*i+3]}, cap);
+        out[2*i] = r.n0;
+        out[2*i+1] = r.n1;
+    }
+}
+'''
+
+
+@pytest.mark.parametrize("cap", [1, 5, 8, 9, 17, 256, 1500])
+def test_pairs_mandelbrot_equals_the_plain_iteration(tmp_path, golden_dir, cap):
+    """mandelbrot_pairs.cu (two neighbouring pixels per element, packed updates
+    emulated one float at a time on the host): bit-identical to eq. (5) as
+    written (the oracle) on the whole 1024x768 image, caps below/at/above the
+    prefix and block lengths, and to the golden CRC at cap 256."""
+    import json
+    import os
+    import zlib
+    src = tmp_path / "pairs.cpp"
+    src.write_text(PAIRS_SHIM.replace(
+        "SRC", str(ROOT / "paper_conf_ipps_steuwerkg11_b200" / "workloads" / "mandelbrot_pairs.cu")))
+    so = tmp_path / "pairs.so"
+    subprocess.run(["g++", "-O2", "-std=c++17", "-ffp-contract=off", "-shared", "-fPIC", str(src), "-o", str(so)],
+                   check=True)
+    lib = ctypes.CDLL(str(so))
+    lib.run.argtypes = [ctypes.c_void_p, ctypes.c_long, ctypes.c_int, ctypes.c_void_p]
+    pos = np.ascontiguousarray(si.mandelbrot_positions(1024, 768))
+    got = np.zeros(pos.size, np.int32)
+    lib.run(pos.ctypes.data, pos.size // 2, cap, got.ctypes.data)
+    assert np.array_equal(got, oracle.mandelbrot(pos, cap))
+    if cap == 256:
+        with open(os.path.join(golden_dir, "mandelbrot.json")) as fh:
+            case = [c for c in json.load(fh)["cases"] if (c["width"], c["height"], c["cap"]) == (1024, 768, 256)][0]
+        assert zlib.crc32(got.tobytes()) == int(case["crc32"], 16)
