@@ -16,6 +16,10 @@ MANDELBROT_INDEX = source("mandelbrot_index")  # index Map variant (NEXT-4)
 MANDELBROT_BLOCKED = source("mandelbrot_blocked")  # loop control per block of updates (NEXT-4)
 # pairs of neighbouring pixels per element, packed FP32x2 arithmetic (NEXT-4)
 MANDELBROT_PAIRS = source("mandelbrot_pairs")
+# cyclic rows: index Map over a permuted row order (device k: rows k, k+D, ...),
+# then an index Map that restores row-major order (NEXT-4; mandelbrot.py)
+MANDELBROT_CYCLIC = MANDELBROT_PAIRS + source("mandelbrot_cyclic")
+MANDELBROT_UNPERMUTE = source("mandelbrot_unpermute")
 LMOSEM_ERROR = source("lmosem_error")
 # the same function for prepared (longest-path-first) event order, where the
 # Map is bound by L1TEX requests: 16-byte gathers per 4-float group in the

@@ -113,3 +113,25 @@ def test_pairs_variant_bit_exact(golden_dir, w, h, cap, D):
         assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)
     if w * h <= 1 << 20:
         assert np.array_equal(got, oracle.mandelbrot(pos, cap))
+
+
+@pytest.mark.parametrize("w,h,cap,D", [(1024, 768, 256, 1), (1024, 768, 256, 2), (1024, 768, 256, 3),
+                                       (1024, 768, 256, 4), (1024, 768, 256, 8), (4096, 3072, 256, 8),
+                                       (1024, 768, 4096, 4), (258, 7, 50, 3)])
+def test_cyclic_rows_bit_exact(golden_dir, w, h, cap, D):
+    """NEXT-4 cyclic rows (mandelbrot.CyclicMandelbrot): device k computes rows
+    k, k+D, ... into a permuted, block-distributed image; gathered and
+    un-permuted on device 0 it is the golden image (and the oracle's), also
+    when the rows do not divide evenly (258x7 at D = 3: padding slots)."""
+    from paper_conf_ipps_steuwerkg11_b200.mandelbrot import CyclicMandelbrot
+    with skel.Context(D) as ctx:
+        cm = CyclicMandelbrot(ctx, w, h)
+        got = cm.counts(cap)
+        again = cm.counts(cap)  # buffers reused
+    assert np.array_equal(got, again)
+    cases = [c for c in json.load(open(os.path.join(golden_dir, "mandelbrot.json")))["cases"]
+             if (c["width"], c["height"], c["cap"]) == (w, h, cap)]
+    if cases:
+        assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)
+    if w * h <= 1 << 20:
+        assert np.array_equal(got, oracle.mandelbrot(si.mandelbrot_positions(w, h), cap))

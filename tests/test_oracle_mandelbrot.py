@@ -123,3 +123,23 @@ def test_golden_generator_reproduces_the_small_pin(golden_dir):
     with open(os.path.join(golden_dir, "mandelbrot.json")) as fh:
         want = json.load(fh)["cases"][0]
     assert mk.pins(want["width"], want["height"], want["cap"]) == want
+
+
+def test_cyclic_rows_balance_the_devices():
+    """NEXT-4: work per device (the oracle's iteration counts summed over the
+    rows each device computes) for the paper's image (4096x3072, cap 256).
+    Block rows: the busiest device carries 1.997 / 2.115 / 3.112x
+    the mean at D = 2 / 4 / 8 (SURVEY §8d config 3's ideal-speedup ceiling).
+    Cyclic rows (device k: rows k, k+D, ...): every device within 5% of the
+    busiest (mean/max >= 0.95)."""
+    W, H = 4096, 3072
+    rows = oracle.mandelbrot(mandelbrot_positions(W, H), 256).astype(np.int64).reshape(H, W).sum(axis=1)
+    total = rows.sum()
+    for D, ceiling in ((2, 1.997), (3, None), (4, 2.115), (8, 3.112)):
+        R = -(-H // D)
+        block = np.array([rows[k * R:(k + 1) * R].sum() for k in range(D)])
+        if ceiling is not None:
+            assert abs(total / block.max() - ceiling) < 0.002, (D, total / block.max())
+        cyc = np.array([rows[k::D].sum() for k in range(D)])
+        assert cyc.sum() == total
+        assert cyc.mean() / cyc.max() >= 0.95, (D, cyc.mean() / cyc.max())
