@@ -14,6 +14,8 @@ def source(name: str) -> str:
 MANDELBROT = source("mandelbrot")
 MANDELBROT_INDEX = source("mandelbrot_index")  # index Map variant (NEXT-4)
 MANDELBROT_BLOCKED = source("mandelbrot_blocked")  # loop control per block of updates (NEXT-4)
+# 8 x 4 pixel tiles per warp: a void index Map writing the row-major image (NEXT-4)
+MANDELBROT_TILES = MANDELBROT_BLOCKED + source("mandelbrot_tiles")
 # pairs of neighbouring pixels per element, packed FP32x2 arithmetic (NEXT-4)
 MANDELBROT_PAIRS = source("mandelbrot_pairs")
 # cyclic rows: index Map over a permuted row order (device k: rows k, k+D, ...),

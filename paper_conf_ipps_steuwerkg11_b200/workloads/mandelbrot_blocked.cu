@@ -17,9 +17,26 @@
 #define MANDEL_B 8
 #endif
 struct Pos { float re, im; };
+// MANDEL_PRE: updates done by the plain loop before the blocks start -- most
+// pixels outside the set escape within a few updates (93.5% within 8 on the
+// paper image), and for them a first block would be computed, rolled back and
+// replayed
+#ifndef MANDEL_PRE
+#define MANDEL_PRE 0
+#endif
 template <int B> static int mandel_blocked(Pos c, int cap) {
     float x = 0.0f, y = 0.0f;
     int n = 0;
+    if (MANDEL_PRE > 0) {
+        const int p = cap < MANDEL_PRE ? cap : MANDEL_PRE;
+        while (n < p && x * x + y * y <= 4.0f) {
+            float xt = (x * x - y * y) + c.re;
+            y = (2.0f * x) * y + c.im;
+            x = xt;
+            ++n;
+        }
+        if (n < p) return n;  // escaped in the prefix
+    }
     while (n + B <= cap) {
         const float x0 = x, y0 = y;
         bool out = false;

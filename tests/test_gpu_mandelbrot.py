@@ -135,3 +135,22 @@ def test_cyclic_rows_bit_exact(golden_dir, w, h, cap, D):
         assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)
     if w * h <= 1 << 20:
         assert np.array_equal(got, oracle.mandelbrot(si.mandelbrot_positions(w, h), cap))
+
+
+@pytest.mark.parametrize("w,h,cap,D", [(1024, 768, 256, 1), (4096, 3072, 256, 1), (1024, 768, 4096, 1),
+                                       (1024, 768, 256, 3)])
+def test_tiles_variant_bit_exact(golden_dir, w, h, cap, D):
+    """NEXT-4: 8 x 4 pixel tiles per warp (void index Map writing the row-major
+    image through a vector argument): the golden image."""
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_TILES
+    with skel.Context(D) as ctx:
+        img = ctx.vector(n=w * h, dtype=np.int32)
+        img.fill_dist(skel.COPY if D > 1 else skel.SINGLE, np.int32(-1))
+        ctx.map_index(MANDELBROT_TILES, w * h, None, args=[img, np.int32(w), np.int32(h), np.int32(cap)])
+        img.mark_device_modified()
+        if D > 1:  # each device wrote its own tiles into its copy: combine (max over -1 fill)
+            img.set_distribution(skel.SINGLE, skel.COMBINE_MAX)
+        got = img.download()
+    cases = [c for c in json.load(open(os.path.join(golden_dir, "mandelbrot.json")))["cases"]
+             if (c["width"], c["height"], c["cap"]) == (w, h, cap)]
+    assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)

@@ -5,7 +5,7 @@ import numpy as np
 import torch
 import skel_inputs as si
 from paper_conf_ipps_steuwerkg11_b200 import skel
-from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT, MANDELBROT_BLOCKED, MANDELBROT_PAIRS
+from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT, MANDELBROT_BLOCKED, MANDELBROT_PAIRS, MANDELBROT_TILES
 
 pos = si.mandelbrot_positions(4096, 3072)
 with skel.Context(1) as ctx:
@@ -29,7 +29,21 @@ with skel.Context(1) as ctx:
             ctx.sync()
             res[f"{name}_{cap}_ms"] = round(e0.elapsed_time(e1) / 10, 4)
             outs[name] = out.download().view(np.int32)
-        res[f"same_{cap}"] = bool(np.array_equal(outs["paper"], outs["blocked"])) and \
-            bool(np.array_equal(outs["paper"], outs["pairs"]))
+        # 8 x 4 tiles per warp: void index Map over W*H indices writing the image
+        img = ctx.vector(n=pos.size, dtype=np.int32)
+        targs = [img, np.int32(4096), np.int32(3072), np.int32(cap)]
+        for _ in range(2):
+            ctx.map_index(MANDELBROT_TILES, pos.size, None, args=targs)
+        ctx.sync()
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        e0.record(st)
+        for _ in range(10):
+            ctx.map_index(MANDELBROT_TILES, pos.size, None, args=targs)
+        e1.record(st)
+        ctx.sync()
+        res[f"tiles_{cap}_ms"] = round(e0.elapsed_time(e1) / 10, 4)
+        img.mark_device_modified()
+        outs["tiles"] = img.download()
+        res[f"same_{cap}"] = all(bool(np.array_equal(outs["paper"], outs[k])) for k in ("blocked", "pairs", "tiles"))
         res[f"iters_{cap}"] = int(outs["paper"].astype(np.int64).sum())
     print(json.dumps(res))
