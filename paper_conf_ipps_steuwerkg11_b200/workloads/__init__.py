@@ -14,6 +14,9 @@ def source(name: str) -> str:
 MANDELBROT = source("mandelbrot")
 MANDELBROT_INDEX = source("mandelbrot_index")  # index Map variant (NEXT-4)
 MANDELBROT_BLOCKED = source("mandelbrot_blocked")  # loop control per block of updates (NEXT-4)
+# the blocked function with exact periodicity checking (a member is recognised
+# when its float32 orbit repeats bit for bit; NEXT-4)
+MANDELBROT_PERIODIC = "#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n" + MANDELBROT_BLOCKED
 # 8 x 4 pixel tiles per warp: a void index Map writing the row-major image (NEXT-4)
 MANDELBROT_TILES = MANDELBROT_BLOCKED + source("mandelbrot_tiles")
 # pairs of neighbouring pixels per element, packed FP32x2 arithmetic (NEXT-4)

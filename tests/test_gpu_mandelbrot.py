@@ -154,3 +154,21 @@ def test_tiles_variant_bit_exact(golden_dir, w, h, cap, D):
     cases = [c for c in json.load(open(os.path.join(golden_dir, "mandelbrot.json")))["cases"]
              if (c["width"], c["height"], c["cap"]) == (w, h, cap)]
     assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)
+
+
+@pytest.mark.parametrize("w,h,cap,D", [(1024, 768, 256, 1), (4096, 3072, 256, 1), (1024, 768, 4096, 1),
+                                       (1024, 768, 256, 4), (257, 3, 9, 1)])
+def test_periodic_variant_bit_exact(golden_dir, w, h, cap, D):
+    """NEXT-4: the blocked function with exact periodicity checking (a member
+    recognised when its float32 orbit repeats bit for bit): the counts of eq.
+    (5) as written -- golden CRCs and the oracle."""
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_PERIODIC
+    pos = si.mandelbrot_positions(w, h)
+    with skel.Context(D) as ctx:
+        got = run(ctx, pos, cap, skel.BLOCK if D > 1 else None, fn=MANDELBROT_PERIODIC)
+    cases = [c for c in json.load(open(os.path.join(golden_dir, "mandelbrot.json")))["cases"]
+             if (c["width"], c["height"], c["cap"]) == (w, h, cap)]
+    if cases:
+        assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)
+    if w * h <= 1 << 20:
+        assert np.array_equal(got, oracle.mandelbrot(pos, cap))

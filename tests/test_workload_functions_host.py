@@ -154,6 +154,33 @@ def mandel_blocked(tmp_path_factory):
     return run
 
 
+@pytest.mark.parametrize("cap", [1, 7, 8, 9, 17, 256, 1024, 1500])
+def test_periodic_mandelbrot_equals_the_plain_iteration(tmp_path, golden_dir, cap):
+    """mandelbrot_blocked.cu with MANDEL_PERIODIC (exact periodicity checking,
+    Brent's save schedule at block ends) and an 8-update plain prefix: the
+    counts of eq. (5) as written on the whole 1024x768 image, and the golden CRC
+    at cap 256."""
+    import json
+    import os
+    import zlib
+    src = tmp_path / "periodic.cpp"
+    src.write_text("#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n" + MANDEL_SHIM.replace(
+        "SRC", str(ROOT / "paper_conf_ipps_steuwerkg11_b200" / "workloads" / "mandelbrot_blocked.cu")))
+    so = tmp_path / "periodic.so"
+    subprocess.run(["g++", "-O2", "-std=c++17", "-ffp-contract=off", "-shared", "-fPIC", str(src), "-o", str(so)],
+                   check=True)
+    lib = ctypes.CDLL(str(so))
+    lib.run.argtypes = [ctypes.c_void_p, ctypes.c_long, ctypes.c_int, ctypes.c_void_p]
+    pos = np.ascontiguousarray(si.mandelbrot_positions(1024, 768))
+    got = np.zeros(pos.size, np.int32)
+    lib.run(pos.ctypes.data, pos.size, cap, got.ctypes.data)
+    assert np.array_equal(got, oracle.mandelbrot(pos, cap))
+    if cap == 256:
+        with open(os.path.join(golden_dir, "mandelbrot.json")) as fh:
+            case = [c for c in json.load(fh)["cases"] if (c["width"], c["height"], c["cap"]) == (1024, 768, 256)][0]
+        assert zlib.crc32(got.tobytes()) == int(case["crc32"], 16)
+
+
 @pytest.mark.parametrize("cap", [1, 7, 8, 9, 256, 1024, 1500])
 def test_blocked_mandelbrot_equals_the_plain_iteration(mandel_blocked, golden_dir, cap):
     """mandelbrot_blocked.cu (loop control per block of 8 updates, roll back on
