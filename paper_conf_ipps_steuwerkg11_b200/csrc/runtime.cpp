@@ -22,9 +22,35 @@
 #include <cstring>
 #include <mutex>
 
+#include <nvtx3/nvToolsExt.h>
+
 #include "internal.h"
 
 using namespace skelrt;
+
+// NVTX ranges: every skeleton call and every planner operation
+// is a named range in the "skel" domain, so Nsight timelines show the paper's
+// operations (Map/Zip/Reduce/Scan, distribution changes, transfers) around the
+// kernels and collectives they launch.  Header-only NVTX3: free unless a tool
+// is attached.
+namespace {
+nvtxDomainHandle_t nvtx_domain() {
+    static nvtxDomainHandle_t d = nvtxDomainCreateA("skel");
+    return d;
+}
+struct NvtxRange {
+    explicit NvtxRange(const char *name) {
+        nvtxEventAttributes_t a = {};
+        a.version = NVTX_VERSION;
+        a.size = NVTX_EVENT_ATTRIB_STRUCT_SIZE;
+        a.messageType = NVTX_MESSAGE_TYPE_ASCII;
+        a.message.ascii = name;
+        nvtxDomainRangePushEx(nvtx_domain(), &a);
+    }
+    ~NvtxRange() { nvtxDomainRangePop(nvtx_domain()); }
+};
+}  // namespace
+#define SKEL_RANGE(name) NvtxRange skel_nvtx_range_(name)
 
 namespace {
 
@@ -1541,6 +1567,7 @@ int skel_clear_kernel_cache(skel_ctx_t ctx) {
 }
 
 int skel_sync(skel_ctx_t ctx) {
+    SKEL_RANGE("skel_sync");
     if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
     return sync_all(ctx);
 }
@@ -1617,6 +1644,7 @@ int skel_vector_size(skel_vec_t v, size_t *n, size_t *es) {
 }
 
 int skel_vector_upload(skel_vec_t v, const void *src, size_t n) {
+    SKEL_RANGE("skel_vector_upload");
     if (!v || (!src && n)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad upload arguments");
     if (n != v->n) return fail(v->ctx, SKEL_ERR_SIZE, "upload length != vector length");
     TRY(host_mirror(v));  // (replaces a rank-local part mirror)
@@ -1630,6 +1658,7 @@ int skel_vector_upload(skel_vec_t v, const void *src, size_t n) {
 }
 
 int skel_vector_upload_part(skel_vec_t v, size_t lo, const void *src, size_t count) {
+    SKEL_RANGE("skel_vector_upload_part");
     if (!v || (!src && count)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad upload_part arguments");
     skel_ctx_s *ctx = v->ctx;
     if (lo > v->n || count > v->n - lo) return fail(ctx, SKEL_ERR_SIZE, "range outside the vector");
@@ -1665,6 +1694,7 @@ int skel_vector_upload_part(skel_vec_t v, size_t lo, const void *src, size_t cou
 }
 
 int skel_vector_download(skel_vec_t v, void *dst, size_t n) {
+    SKEL_RANGE("skel_vector_download");
     if (!v || (!dst && n)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad download arguments");
     if (n != v->n) return fail(v->ctx, SKEL_ERR_SIZE, "download length != vector length");
     if (partial_mirror(v)) {
@@ -1680,6 +1710,7 @@ int skel_vector_download(skel_vec_t v, void *dst, size_t n) {
 }
 
 int skel_vector_download_part(skel_vec_t v, size_t lo, void *dst, size_t count) {
+    SKEL_RANGE("skel_vector_download_part");
     if (!v || (!dst && count)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad download_part arguments");
     skel_ctx_s *ctx = v->ctx;
     if (lo > v->n || count > v->n - lo) return fail(ctx, SKEL_ERR_SIZE, "range outside the vector");
@@ -1737,6 +1768,7 @@ int skel_vector_download_part(skel_vec_t v, size_t lo, void *dst, size_t count) 
 }
 
 int skel_vector_host_ptr(skel_vec_t v, void **host) {
+    SKEL_RANGE("skel_vector_host_ptr");
     if (!v || !host) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad arguments");
     TRY(ensure_host(v));
     *host = v->host;
@@ -1758,6 +1790,7 @@ int skel_vector_fill(skel_vec_t v, const void *value) {
 }
 
 int skel_vector_fill_dist(skel_vec_t v, skel_dist dist, const void *value) {
+    SKEL_RANGE("skel_vector_fill_dist");
     if (!v || !value || (int)dist < 0 || (int)dist > 2)
         return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad fill arguments");
     skel_ctx_s *ctx = v->ctx;
@@ -1779,6 +1812,7 @@ int skel_vector_fill_dist(skel_vec_t v, skel_dist dist, const void *value) {
 }
 
 int skel_vector_set_distribution(skel_vec_t v, skel_dist dist, skel_combine combine) {
+    SKEL_RANGE("skel_vector_set_distribution");
     if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
     if ((int)dist < 0 || (int)dist > 2 || (int)combine < 0 || (int)combine > 4)
         return fail(v->ctx, SKEL_ERR_ARG, "bad distribution or combine");
@@ -1786,6 +1820,7 @@ int skel_vector_set_distribution(skel_vec_t v, skel_dist dist, skel_combine comb
 }
 
 int skel_vector_set_distribution_fn(skel_vec_t v, skel_dist dist, const char *combine_src) {
+    SKEL_RANGE("skel_vector_set_distribution_fn");
     if (!v || !combine_src) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad arguments");
     if ((int)dist < 0 || (int)dist > 2) return fail(v->ctx, SKEL_ERR_ARG, "bad distribution");
     return set_distribution_fn(v, dist, combine_src);
@@ -1798,6 +1833,7 @@ int skel_vector_get_distribution(skel_vec_t v, skel_dist *dist) {
 }
 
 int skel_vector_mark_device_modified(skel_vec_t v) {
+    SKEL_RANGE("skel_vector_mark_device_modified");
     if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
     TRY(ensure_device(v));
     device_wrote(v);
@@ -1828,6 +1864,7 @@ int skel_vector_device_ptr(skel_vec_t v, int li, void **ptr, size_t *count) {
 
 // ---- skeletons -------------------------------------------------------------------
 int skel_map(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, const skel_arg *args, int nargs) {
+    SKEL_RANGE("skel_map");
     if (!ctx || !src || !in || in->ctx != ctx || (out && out->ctx != ctx) || (nargs && !args) || nargs < 0)
         return fail(ctx, SKEL_ERR_ARG, "bad map arguments");
     return run_ew(ctx, Kind::Map, src, in, nullptr, out, args, nargs);
@@ -1837,6 +1874,7 @@ int skel_map(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, con
 // input vector; each device computes the indices of its part of out (block: its
 // part, copy: all, single: device 0); a void f runs over a block partition of [0, n)
 int skel_map_index(skel_ctx_t ctx, const char *src, size_t n, skel_vec_t out, const skel_arg *args, int nargs) {
+    SKEL_RANGE("skel_map_index");
     if (!ctx || !src || (out && out->ctx != ctx) || (nargs && !args) || nargs < 0)
         return fail(ctx, SKEL_ERR_ARG, "bad map_index arguments");
     Module *m = nullptr;
@@ -1898,6 +1936,7 @@ int skel_map_index(skel_ctx_t ctx, const char *src, size_t n, skel_vec_t out, co
 // lanes Map: `lanes` threads per element (see map.cuh, SKEL_LANES)
 int skel_map_lanes(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, int lanes, const skel_arg *args,
                    int nargs) {
+    SKEL_RANGE("skel_map_lanes");
     if (!ctx || !src || !in || in->ctx != ctx || (out && out->ctx != ctx) || (nargs && !args) || nargs < 0)
         return fail(ctx, SKEL_ERR_ARG, "bad map_lanes arguments");
     if (lanes < 1 || lanes > 32 || (lanes & (lanes - 1)))
@@ -1943,6 +1982,7 @@ int skel_map_lanes(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t ou
 
 int skel_zip(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_vec_t out, const skel_arg *args,
              int nargs) {
+    SKEL_RANGE("skel_zip");
     if (!ctx || !src || !a || !b || !out || a->ctx != ctx || b->ctx != ctx || out->ctx != ctx || (nargs && !args) ||
         nargs < 0)
         return fail(ctx, SKEL_ERR_ARG, "bad zip arguments");
@@ -1952,6 +1992,7 @@ int skel_zip(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_v
 
 int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b, skel_combine combine,
                      skel_vec_t out, const skel_arg *args, int nargs) {
+    SKEL_RANGE("skel_zip_combine");
     if (!ctx || !src || !a || !b || !out || a->ctx != ctx || b->ctx != ctx || out->ctx != ctx || (nargs && !args) ||
         nargs < 0 || (int)combine < 1 || (int)combine > 4 || out == b)
         return fail(ctx, SKEL_ERR_ARG, "bad zip_combine arguments");
@@ -2067,6 +2108,7 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
 
 int skel_reduce_to(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t result, const skel_arg *args,
                    int nargs) {
+    SKEL_RANGE("skel_reduce_to");
     if (!ctx || !src || !in || !result || in->ctx != ctx || result->ctx != ctx || (nargs && !args) || nargs < 0)
         return fail(ctx, SKEL_ERR_ARG, "bad reduce arguments");
     if (in->n == 0) return fail(ctx, SKEL_ERR_SIZE, "reduce of an empty vector (eq. 3 has no identity)");
@@ -2107,6 +2149,7 @@ int skel_reduce_to(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t re
 }
 
 int skel_reduce(skel_ctx_t ctx, const char *src, skel_vec_t in, void *result_host, const skel_arg *args, int nargs) {
+    SKEL_RANGE("skel_reduce");
     if (!ctx || !src || !in || !result_host || in->ctx != ctx || (nargs && !args) || nargs < 0)
         return fail(ctx, SKEL_ERR_ARG, "bad reduce arguments");
     if (in->n == 0) return fail(ctx, SKEL_ERR_SIZE, "reduce of an empty vector (eq. 3 has no identity)");
@@ -2129,6 +2172,7 @@ int skel_reduce(skel_ctx_t ctx, const char *src, skel_vec_t in, void *result_hos
 
 int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, const void *identity,
               const skel_arg *args, int nargs) {
+    SKEL_RANGE("skel_scan");
     if (!ctx || !src || !in || !out || !identity || in->ctx != ctx || out->ctx != ctx || (nargs && !args) ||
         nargs < 0)
         return fail(ctx, SKEL_ERR_ARG, "bad scan arguments");
@@ -2346,6 +2390,7 @@ int skel_capture_end(skel_ctx_t ctx, skel_graph_t *out) {
 }
 
 int skel_graph_launch(skel_graph_t g) {
+    SKEL_RANGE("skel_graph_launch");
     if (!g) return fail(nullptr, SKEL_ERR_ARG, "graph is NULL");
     skel_ctx_s *ctx = g->ctx;
     Slot &s0 = ctx->slots[0];

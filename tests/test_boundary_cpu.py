@@ -157,3 +157,14 @@ def test_scan_window_probe_variants_compile(monkeypatch, defines):
     st, log, nb = skel.compile_check("scan", SUM_F32)
     assert st == 0, log
     assert nb > 1000 and nb != base[2]
+
+
+def test_nvtx_ranges_are_compiled_in():
+    """skeleton calls and planner operations are NVTX ranges in the
+    'skel' domain (header-only NVTX3: the injection hook and the range names are
+    in the library)."""
+    data = open(skel.LIB_PATH if hasattr(skel, "LIB_PATH") else
+                __import__("os").path.join(__import__("os").path.dirname(skel.__file__), "libskel.so"), "rb").read()
+    assert b"NVTX_INJECTION64_PATH" in data
+    for name in (b"skel_map", b"skel_scan", b"skel_vector_set_distribution", b"skel_zip_combine"):
+        assert name + b"\x00" in data
