@@ -98,6 +98,9 @@ typedef struct {
     double disk_load_ms; /* total time loading cubins from the disk cache */
     uint64_t scan_coop_fallbacks; /* persistent Scans that could not be made co-resident
                                      (cooperative launch refused) and ran as two launches */
+    uint64_t vmm_allocs;          /* vector buffers allocated through VMM (cuMemCreate)     */
+    uint64_t mc_binds;            /* multicast objects bound to a vector's device buffers   */
+    uint64_t multimem_launches;   /* fused tails run through NVSwitch multicast (multimem)  */
 } skel_stats;
 
 /* ---- context ------------------------------------------------------------

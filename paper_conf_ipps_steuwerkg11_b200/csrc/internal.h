@@ -42,7 +42,8 @@ struct Module {
     cudaKernel_t k_scan_small = nullptr;  // small-vector Scan: seeded tile scans
     cudaKernel_t k_fold_aggs = nullptr;   // small-vector Reduce: ordered fold of the tile aggregates
     cudaKernel_t k_red_agg2 = nullptr;    // small-vector Reduce: aggregates of double-size tiles
-    cudaKernel_t k_zipcomb = nullptr;  // Zip modules: fused combine + zip + broadcast
+    cudaKernel_t k_zipcomb = nullptr;  // Zip modules: fused combine + zip + broadcast (peer memory)
+    cudaKernel_t k_zipcomb_mm = nullptr;  // ... the same through NVSwitch multicast (multimem)
     uint64_t sig[16 + 4 * 32] = {0};
     std::set<int> attr_set_on;  // devices on which smem attributes were set
     // element-wise grid policy (runtime.cpp ew_decide): 0 = UNROLL chunks in
@@ -83,6 +84,21 @@ struct Slot {
     size_t scratch_cap = 0;
 };
 
+struct VmmRec {  // a VMM (cuMemCreate) allocation backing a vector buffer
+    unsigned long long handle = 0;
+    size_t size = 0;
+    int dev = 0;
+};
+
+// a multicast object (NVSwitch NVLS) bound to every device's buffer of a vector
+struct McRec {
+    unsigned long long handle = 0;  // CUmemGenericAllocationHandle of the multicast object
+    unsigned long long va = 0;      // its mapping (one address reaches all bound buffers)
+    size_t size = 0;
+    std::vector<char *> bases;      // the buffers it is bound to (one per local slot)
+    std::vector<int> devs;
+};
+
 struct Buf {  // one logical device's storage of a vector
     char *base = nullptr;
     size_t cap = 0;    // bytes allocated at base
@@ -111,6 +127,13 @@ struct skel_ctx_s {
     // every pair of distinct physical devices has peer access enabled (in-process
     // mode); the fused peer-memory paths need it, else they take the unfused one
     bool peer_all = true;
+    // vector buffers of at least vmm_min bytes are VMM allocations (cuMemCreate,
+    // exportable), so one allocation can be bound to a multicast object; rank
+    // mode keeps cudaMalloc (its fused tail opens peers through CUDA IPC)
+    bool vmm_on = true;
+    size_t vmm_min = 2u << 20;
+    std::unordered_map<char *, skelrt::VmmRec> vmm;
+    int mc_ok = -1;  // every local device supports multicast (-1: not yet queried)
     skel_stats stats{};
     std::string last_error;
     std::map<std::string, std::unique_ptr<skelrt::Module>> modules;
@@ -141,6 +164,7 @@ struct skel_vec_s {
     bool diverged = false;  // copy distribution after mark_device_modified
     std::vector<skelrt::Buf> bufs;  // indexed like ctx->slots
     uint64_t serial = 0;            // unique per context (graphs refer to vectors by it)
+    skelrt::McRec mc;               // multicast binding of bufs (fused NVLS tail), if any
 };
 
 namespace skelrt {

@@ -113,7 +113,120 @@ struct DevGuard {
     explicit DevGuard(int dev) { cudaSetDevice(dev); }
 };
 
+// ---- CUDA driver entry points (VMM, multicast), resolved through the runtime ----
+struct Drv {
+    PFN_cuMemCreate_v10020 create = nullptr;
+    PFN_cuMemRelease_v10020 release = nullptr;
+    PFN_cuMemAddressReserve_v10020 reserve = nullptr;
+    PFN_cuMemAddressFree_v10020 addr_free = nullptr;
+    PFN_cuMemMap_v10020 map = nullptr;
+    PFN_cuMemUnmap_v10020 unmap = nullptr;
+    PFN_cuMemSetAccess_v10020 set_access = nullptr;
+    PFN_cuMemGetAllocationGranularity_v10020 granularity = nullptr;
+    PFN_cuMulticastCreate_v12010 mc_create = nullptr;
+    PFN_cuMulticastAddDevice_v12010 mc_add = nullptr;
+    PFN_cuMulticastBindMem_v12010 mc_bind = nullptr;
+    PFN_cuMulticastUnbind_v12010 mc_unbind = nullptr;
+    PFN_cuMulticastGetGranularity_v12010 mc_granularity = nullptr;
+    PFN_cuDeviceGetAttribute_v2000 attr = nullptr;
+    bool vmm = false, mc = false;
+};
+const Drv &drv() {
+    static Drv d;
+    static std::once_flag once;
+    std::call_once(once, [] {
+        auto get = [](const char *name, int ver, void **fn) {
+            cudaDriverEntryPointQueryResult q;
+            if (cudaGetDriverEntryPointByVersion(name, fn, ver, cudaEnableDefault, &q) != cudaSuccess ||
+                q != cudaDriverEntryPointSuccess) {
+                cudaGetLastError();
+                *fn = nullptr;
+            }
+        };
+        get("cuMemCreate", 10020, (void **)&d.create);
+        get("cuMemRelease", 10020, (void **)&d.release);
+        get("cuMemAddressReserve", 10020, (void **)&d.reserve);
+        get("cuMemAddressFree", 10020, (void **)&d.addr_free);
+        get("cuMemMap", 10020, (void **)&d.map);
+        get("cuMemUnmap", 10020, (void **)&d.unmap);
+        get("cuMemSetAccess", 10020, (void **)&d.set_access);
+        get("cuMemGetAllocationGranularity", 10020, (void **)&d.granularity);
+        get("cuMulticastCreate", 12010, (void **)&d.mc_create);
+        get("cuMulticastAddDevice", 12010, (void **)&d.mc_add);
+        get("cuMulticastBindMem", 12010, (void **)&d.mc_bind);
+        get("cuMulticastUnbind", 12010, (void **)&d.mc_unbind);
+        get("cuMulticastGetGranularity", 12010, (void **)&d.mc_granularity);
+        get("cuDeviceGetAttribute", 2000, (void **)&d.attr);
+        d.vmm = d.create && d.release && d.reserve && d.addr_free && d.map && d.unmap && d.set_access &&
+                d.granularity;
+        d.mc = d.vmm && d.mc_create && d.mc_add && d.mc_bind && d.mc_unbind && d.mc_granularity && d.attr;
+    });
+    return d;
+}
+
+// distinct physical devices of the context's local slots
+std::vector<int> local_devices(const skel_ctx_s *ctx) {
+    std::vector<int> devs;
+    for (const auto &s : ctx->slots)
+        if (std::find(devs.begin(), devs.end(), s.dev) == devs.end()) devs.push_back(s.dev);
+    return devs;
+}
+
 // ---- device memory -----------------------------------------------------------
+// VMM allocation (cuMemCreate + cuMemMap) on slot s's device, readable and
+// writable from every local device (in-process peers need cuMemSetAccess, not
+// cudaDeviceEnablePeerAccess, for VMM memory).  The physical memory is
+// exportable as a POSIX file descriptor where the driver allows it.  Size:
+// rounded up to the allocation granularity (2 MB), which is also the minimum
+// multicast granularity, so the buffer can be bound to a multicast object.
+// *out = nullptr (and SKEL_OK) when VMM is unavailable: the caller falls back.
+int vmm_alloc(skel_ctx_s *ctx, Slot &s, size_t bytes, char **out) {
+    *out = nullptr;
+    const Drv &d = drv();
+    if (!d.vmm) return SKEL_OK;
+    DevGuard g(s.dev);
+    CUmemAllocationProp prop = {};
+    prop.type = CU_MEM_ALLOCATION_TYPE_PINNED;
+    prop.location.type = CU_MEM_LOCATION_TYPE_DEVICE;
+    prop.location.id = s.dev;
+    prop.requestedHandleTypes = CU_MEM_HANDLE_TYPE_POSIX_FILE_DESCRIPTOR;
+    size_t gran = 0;
+    if (d.granularity(&gran, &prop, CU_MEM_ALLOC_GRANULARITY_RECOMMENDED) != CUDA_SUCCESS || !gran) return SKEL_OK;
+    const size_t size = align_up(std::max<size_t>(bytes, 1), gran);
+    CUmemGenericAllocationHandle h = 0;
+    CUresult r = d.create(&h, size, &prop, 0);
+    if (r != CUDA_SUCCESS) {  // not exportable here: a plain VMM allocation
+        prop.requestedHandleTypes = CU_MEM_HANDLE_TYPE_NONE;
+        r = d.create(&h, size, &prop, 0);
+    }
+    if (r == CUDA_ERROR_OUT_OF_MEMORY) return fail(ctx, SKEL_ERR_OOM, "cuMemCreate(" + std::to_string(size) + ")");
+    if (r != CUDA_SUCCESS) return SKEL_OK;
+    CUdeviceptr va = 0;
+    if (d.reserve(&va, size, gran, 0, 0) != CUDA_SUCCESS) {
+        d.release(h);
+        return SKEL_OK;
+    }
+    std::vector<CUmemAccessDesc> acc;
+    for (int dev : local_devices(ctx)) {
+        CUmemAccessDesc a = {};
+        a.location.type = CU_MEM_LOCATION_TYPE_DEVICE;
+        a.location.id = dev;
+        a.flags = CU_MEM_ACCESS_FLAGS_PROT_READWRITE;
+        acc.push_back(a);
+    }
+    if (d.map(va, size, 0, h, 0) != CUDA_SUCCESS || d.set_access(va, size, acc.data(), acc.size()) != CUDA_SUCCESS) {
+        d.unmap(va, size);
+        d.addr_free(va, size);
+        d.release(h);
+        return SKEL_OK;
+    }
+    char *p = reinterpret_cast<char *>(va);
+    ctx->vmm[p] = VmmRec{(unsigned long long)h, size, s.dev};
+    ctx->stats.vmm_allocs++;
+    *out = p;
+    return SKEL_OK;
+}
+
 int dev_alloc(skel_ctx_s *ctx, Slot &s, size_t bytes, char **out) {
     DevGuard g(s.dev);
     void *p = nullptr;
@@ -133,8 +246,138 @@ int dev_free(skel_ctx_s *ctx, Slot &s, char *p) {
                                          "eagerly before capturing it");
     DevGuard g(s.dev);
     CK(ctx, cudaStreamSynchronize(s.stream));
+    auto it = ctx->vmm.find(p);
+    if (it != ctx->vmm.end()) {
+        const Drv &d = drv();
+        for (auto &o : ctx->slots)  // peers may still read it (exchanges): drain every local stream
+            if (&o != &s) {
+                DevGuard go(o.dev);
+                cudaStreamSynchronize(o.stream);
+            }
+        const CUdeviceptr va = reinterpret_cast<CUdeviceptr>(p);
+        d.unmap(va, it->second.size);
+        d.addr_free(va, it->second.size);
+        d.release((CUmemGenericAllocationHandle)it->second.handle);
+        ctx->vmm.erase(it);
+        return SKEL_OK;
+    }
     CK(ctx, cudaFree(p));
     return SKEL_OK;
+}
+
+// storage of a vector buffer: VMM when large enough (in-process contexts)
+int vec_alloc(skel_ctx_s *ctx, Slot &s, size_t bytes, char **out) {
+    if (!ctx->rank_mode && ctx->vmm_on && bytes >= ctx->vmm_min) {
+        TRY(vmm_alloc(ctx, s, bytes, out));
+        if (*out) return SKEL_OK;
+    }
+    return dev_alloc(ctx, s, bytes, out);
+}
+
+// ---- multicast (NVLS) binding of a vector's device buffers -----------------------
+void mc_release(skel_vec_s *v) {
+    McRec &m = v->mc;
+    if (!m.handle) return;
+    const Drv &d = drv();
+    skel_ctx_s *ctx = v->ctx;
+    for (auto &s : ctx->slots) {
+        DevGuard g(s.dev);
+        cudaStreamSynchronize(s.stream);
+    }
+    d.unmap((CUdeviceptr)m.va, m.size);
+    d.addr_free((CUdeviceptr)m.va, m.size);
+    for (int dev : m.devs) d.mc_unbind((CUmemGenericAllocationHandle)m.handle, (CUdevice)dev, 0, m.size);
+    d.release((CUmemGenericAllocationHandle)m.handle);
+    m = McRec{};
+}
+// release the multicast binding of any vector bound to buffer p (before p is freed)
+void mc_release_base(skel_ctx_s *ctx, const char *p) {
+    for (skel_vec_s *v : ctx->vecs)
+        if (v->mc.handle && std::find(v->mc.bases.begin(), v->mc.bases.end(), p) != v->mc.bases.end())
+            mc_release(v);
+}
+
+// every local device supports multicast (queried once)
+bool mc_supported(skel_ctx_s *ctx) {
+    if (ctx->mc_ok >= 0) return ctx->mc_ok == 1;
+    const Drv &d = drv();
+    bool ok = d.mc && !ctx->rank_mode;
+    if (const char *e = getenv("SKEL_MULTIMEM")) ok = ok && atoi(e) != 0;
+    for (int dev : local_devices(ctx)) {
+        int v = 0;
+        if (!ok || d.attr(&v, CU_DEVICE_ATTRIBUTE_MULTICAST_SUPPORTED, (CUdevice)dev) != CUDA_SUCCESS || !v) ok = false;
+    }
+    ctx->mc_ok = ok ? 1 : 0;
+    return ok;
+}
+
+// one multicast object bound to the first `bytes` of every local slot's buffer
+// of v (each slot a distinct device, every buffer a VMM allocation large
+// enough); false (no error) if that is not possible
+bool mc_bind(skel_vec_s *v, size_t bytes) {
+    skel_ctx_s *ctx = v->ctx;
+    std::vector<char *> bases;
+    for (auto &b : v->bufs) bases.push_back(b.base);
+    if (v->mc.handle && v->mc.bases == bases && v->mc.size >= bytes) return true;
+    mc_release(v);
+    if (!mc_supported(ctx) || local_devices(ctx).size() != ctx->slots.size()) return false;
+    const Drv &d = drv();
+    CUmulticastObjectProp prop = {};
+    prop.numDevices = (unsigned)ctx->slots.size();
+    prop.handleTypes = CU_MEM_HANDLE_TYPE_NONE;
+    prop.size = std::max<size_t>(bytes, 1);
+    size_t gran = 0;
+    if (d.mc_granularity(&gran, &prop, CU_MULTICAST_GRANULARITY_MINIMUM) != CUDA_SUCCESS || !gran) return false;
+    prop.size = align_up(prop.size, gran);
+    for (auto &b : v->bufs) {
+        auto it = ctx->vmm.find(b.base);
+        if (it == ctx->vmm.end() || it->second.size < prop.size) return false;
+    }
+    CUmemGenericAllocationHandle mc = 0;
+    if (d.mc_create(&mc, &prop) != CUDA_SUCCESS) {
+        cudaGetLastError();
+        return false;
+    }
+    McRec m;
+    m.handle = (unsigned long long)mc;
+    m.size = prop.size;
+    bool ok = true;
+    for (auto &s : ctx->slots) ok = ok && d.mc_add(mc, (CUdevice)s.dev) == CUDA_SUCCESS;
+    for (size_t li = 0; ok && li < ctx->slots.size(); ++li) {
+        DevGuard g(ctx->slots[li].dev);
+        const VmmRec &r = ctx->vmm[v->bufs[li].base];
+        ok = d.mc_bind(mc, 0, (CUmemGenericAllocationHandle)r.handle, 0, prop.size, 0) == CUDA_SUCCESS;
+        if (ok) m.devs.push_back(ctx->slots[li].dev);
+    }
+    CUdeviceptr va = 0;
+    if (ok) ok = d.reserve(&va, prop.size, gran, 0, 0) == CUDA_SUCCESS;
+    if (ok) {
+        ok = d.map(va, prop.size, 0, mc, 0) == CUDA_SUCCESS;
+        std::vector<CUmemAccessDesc> acc;
+        for (auto &s : ctx->slots) {
+            CUmemAccessDesc a = {};
+            a.location.type = CU_MEM_LOCATION_TYPE_DEVICE;
+            a.location.id = s.dev;
+            a.flags = CU_MEM_ACCESS_FLAGS_PROT_READWRITE;
+            acc.push_back(a);
+        }
+        if (ok) ok = d.set_access(va, prop.size, acc.data(), acc.size()) == CUDA_SUCCESS;
+        if (!ok) {
+            d.unmap(va, prop.size);
+            d.addr_free(va, prop.size);
+        }
+    }
+    if (!ok) {
+        cudaGetLastError();
+        for (int dev : m.devs) d.mc_unbind(mc, (CUdevice)dev, 0, prop.size);
+        d.release(mc);
+        return false;
+    }
+    m.va = (unsigned long long)va;
+    m.bases = bases;
+    v->mc = m;
+    ctx->stats.mc_binds++;
+    return true;
 }
 // make b hold at least `bytes`; the first `keep` bytes at element offset
 // b.off move to byte offset new_off_bytes of the new allocation
@@ -151,10 +394,11 @@ int buf_grow(skel_ctx_s *ctx, Slot &s, Buf &b, size_t bytes, size_t es, size_t k
         return SKEL_OK;
     }
     char *nb = nullptr;
-    TRY(dev_alloc(ctx, s, bytes, &nb));
+    TRY(vec_alloc(ctx, s, bytes, &nb));
     DevGuard g(s.dev);
     if (keep) CK(ctx, cudaMemcpyAsync(nb + new_off_elems * es, b.base + b.off * es, keep, cudaMemcpyDeviceToDevice,
                                       s.stream));
+    if (b.base) mc_release_base(ctx, b.base);
     TRY(dev_free(ctx, s, b.base));
     b.base = nb;
     b.cap = bytes;
@@ -1405,6 +1649,8 @@ static int init_slot(skel_ctx_s *ctx, int d, int dev) {
 static void ctx_defaults(skel_ctx_s *ctx) {
     const char *f = getenv("SKEL_FMAD");
     ctx->fmad = f && atoi(f) != 0;
+    if (const char *e = getenv("SKEL_VMM")) ctx->vmm_on = atoi(e) != 0;  // 0: cudaMalloc only
+    if (const char *e = getenv("SKEL_VMM_MIN")) ctx->vmm_min = (size_t)strtoull(e, nullptr, 10);
     const char *b = getenv("SKEL_BLOCK_SIZE");
     if (b) ctx->block_size = atoi(b);
 }
@@ -1619,6 +1865,7 @@ int skel_vector_create(skel_ctx_t ctx, size_t n, size_t es, skel_vec_t *out) {
 int skel_vector_destroy(skel_vec_t v) {
     if (!v) return fail(nullptr, SKEL_ERR_ARG, "vector is NULL");
     skel_ctx_s *ctx = v->ctx;
+    mc_release(v);
     for (auto &b : v->bufs) close_peers(b);
     for (size_t li = 0; li < v->bufs.size(); ++li) dev_free(ctx, ctx->slots[li], v->bufs[li].base);
     if (v->host) cudaFreeHost(v->host);
@@ -2004,8 +2251,14 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
     // in-process mode loads and stores through the other devices' buffers: only
     // with peer access between every pair of distinct GPUs (else the unfused
     // reduce-scatter + Zip + all-gather, which moves data with copies)
-    const bool fused = D > 1 && D <= 16 && (a->dist == SKEL_COPY || a->dist == SKEL_BLOCK) &&
-                       (out != a || a->dist == SKEL_COPY) && !ctx->capturing && (ctx->rank_mode || ctx->peer_all);
+    // SKEL_FORCE_MULTIMEM=1 (test hook): a one-device context takes the fused
+    // multicast path too (a multicast object of one device), so the NVLS
+    // kernel and the binding can be exercised on a single GPU
+    static const bool force_mm = getenv("SKEL_FORCE_MULTIMEM") && atoi(getenv("SKEL_FORCE_MULTIMEM")) != 0;
+    const bool fused = ((D > 1 && D <= 16) || (force_mm && D == 1 && !ctx->rank_mode)) &&
+                       (a->dist == SKEL_COPY || a->dist == SKEL_BLOCK || D == 1) &&
+                       (out != a || a->dist == SKEL_COPY || D == 1) && !ctx->capturing &&
+                       (ctx->rank_mode || ctx->peer_all);
     if (!fused) {  // the same result as the unfused sequence
         if (D > 1) TRY(set_distribution(b, SKEL_BLOCK, combine));
         if (a->dist != b->dist) TRY(set_distribution(a, b->dist, SKEL_COMBINE_NONE));
@@ -2054,7 +2307,40 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
         ctx->stats.d2d_bytes += (uint64_t)(D - 1) * cnt * (esb + eso);
         return SKEL_OK;
     };
-    if (!ctx->rank_mode) {
+    // NVSwitch multicast form (skel_zipcomb_mm_kernel): float32 '+' combine and
+    // 4-byte elements, every local slot on its own multicast-capable device,
+    // b's and out's buffers VMM allocations bound to one multicast object each
+    bool mm = !ctx->rank_mode && m->k_zipcomb_mm && b->dt == SKEL_DT_F32 && combine == SKEL_COMBINE_ADD &&
+              esa == 4 && eso == 4 && E == 4;
+    if (mm) {
+        TRY(join(ctx));
+        mm = mc_bind(b, full_bytes(b)) && mc_bind(out, full_bytes(out));
+    }
+    if (mm) {
+        for (size_t li = 0; li < ctx->slots.size(); ++li) {
+            Slot &s = ctx->slots[li];
+            const int k = s.d;
+            uint64_t cnt = want_count(a, SKEL_BLOCK, k);
+            const size_t lo = part_lo(a, k);
+            if (!cnt) continue;
+            const void *pa = a->dist == SKEL_COPY ? a->bufs[li].base + lo * esa : a->bufs[li].ptr(esa);
+            const float *mcb = reinterpret_cast<const float *>(b->mc.va) + lo;
+            void *bown = b->bufs[li].base + lo * esb;
+            float *mco = reinterpret_cast<float *>(out->mc.va) + lo;
+            int vec_ok = al16(pa) && al16(mcb) && al16(bown) && al16(mco);
+            pack_args(m, args, nargs, li, abuf);
+            const uint64_t work = vec_ok ? cnt / 4 : cnt;
+            const int grid = ew_grid(s, std::max<uint64_t>(work, 1), block);
+            uint64_t ncall = cnt;
+            void *params[] = {&pa, &mcb, &bown, &mco, &ncall, &vec_ok, abuf.data()};
+            DevGuard g(s.dev);
+            CK(ctx, cudaLaunchKernel((const void *)m->k_zipcomb_mm, dim3(grid), dim3(block), params, 0, s.stream));
+            ctx->stats.kernel_launches++;
+            ctx->stats.multimem_launches++;
+            ctx->stats.d2d_bytes += (uint64_t)cnt * (esb + eso);
+        }
+        TRY(join(ctx));
+    } else if (!ctx->rank_mode) {
         TRY(join(ctx));
         for (size_t li = 0; li < ctx->slots.size(); ++li) {
             Slot &s = ctx->slots[li];

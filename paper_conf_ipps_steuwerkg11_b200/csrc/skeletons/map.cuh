@@ -413,4 +413,69 @@ extern "C" __global__ void SKEL_EW_BOUNDS
 #pragma unroll 1
     for (skel_u64 i = done + tid; i < n; i += stride) skel_zipcomb_elem(a[i], bsrc, nsrc, bown, odst, ndst, i, op, t);
 }
+
+// ---------------------------------------------------------------------------
+// The same fused tail through NVSwitch multicast (NVLS; SURVEY.md §8f NEXT-1 in
+// its specified form).  b's D copies and out's D copies are each bound to a
+// multicast object, so ONE address reaches the same element on every device:
+//   multimem.ld_reduce.add  -- the switch reads the element from all D copies
+//                              and returns their sum (the copy->block combine),
+//   multimem.st             -- the switch writes the result into all D copies
+//                              of out (the block->copy all-gather).
+// Device k's kernel walks its part [lo, hi): per 16-byte chunk one
+// ld_reduce.v4.f32 of b, the combined chunk kept in its own part of b, the
+// Zip function applied, one st.v4 of the result.  Each device moves S/D bytes
+// of b in and S/D bytes of out out over NVLink (the switch does the fan-in and
+// fan-out), against (D-1)/D x S each way for peer loads/stores.  float32 `+`
+// combine and 4-byte outputs only; other types use skel_zipcomb_kernel.
+// ---------------------------------------------------------------------------
+template <class Tup>
+__device__ __forceinline__ void skel_mm_chunk(const skel_A *a, const float *mcb, skel_B *bown, float *mco, skel_u64 c,
+                                              Tup &t) {
+    if constexpr (skel::same<skel::decay_t<skel_B>, float>::value && sizeof(skel_O) == 4 && SKEL_E == 4 &&
+                  !skel_void) {
+        float4 v;
+        asm volatile("multimem.ld_reduce.relaxed.sys.global.add.v4.f32 {%0, %1, %2, %3}, [%4];"
+                     : "=f"(v.x), "=f"(v.y), "=f"(v.z), "=f"(v.w)
+                     : "l"(mcb + 4 * c)
+                     : "memory");
+        skel::arr<skel_B, 4> acc;
+        acc.v[0] = v.x;
+        acc.v[1] = v.y;
+        acc.v[2] = v.z;
+        acc.v[3] = v.w;
+        skel_st<16>(reinterpret_cast<char *>(bown) + c * 16, skel::bit_cast<skel::chunk<16>>(acc));
+        const auto xa = skel::bit_cast<skel::arr<skel_A, 4>>(skel_ld<skel_CA>(reinterpret_cast<const char *>(a) + c * skel_CA));
+        skel::arr<skel_O, 4> yo;
+        skel_apply_chunk(xa.v, acc.v, yo.v, t);
+        const auto r = skel::bit_cast<float4>(yo);
+        asm volatile("multimem.st.relaxed.sys.global.v4.f32 [%0], {%1, %2, %3, %4};" ::"l"(mco + 4 * c), "f"(r.x),
+                     "f"(r.y), "f"(r.z), "f"(r.w)
+                     : "memory");
+    }
+}
+template <class Tup>
+__device__ __forceinline__ void skel_mm_one(const skel_A *a, const float *mcb, skel_B *bown, float *mco, skel_u64 i,
+                                            Tup &t) {
+    if constexpr (skel::same<skel::decay_t<skel_B>, float>::value && sizeof(skel_O) == 4 && !skel_void) {
+        float v;
+        asm volatile("multimem.ld_reduce.relaxed.sys.global.add.f32 %0, [%1];" : "=f"(v) : "l"(mcb + i) : "memory");
+        bown[i] = v;
+        const skel_O r = skel::caller<skel_Seq>::call(&SKEL_FN, t, a[i], v);
+        asm volatile("multimem.st.relaxed.sys.global.f32 [%0], %1;" ::"l"(mco + i), "f"(skel::bit_cast<float>(r))
+                     : "memory");
+    }
+}
+extern "C" __global__ void SKEL_EW_BOUNDS
+    skel_zipcomb_mm_kernel(const skel_A *__restrict__ a, const float *mcb, skel_B *bown, float *mco, skel_u64 n,
+                           int vec_ok, const skel_Buf args) {
+    auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
+    const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;
+    const skel_u64 nch = (SKEL_E == 4 && vec_ok) ? n / 4 : 0;  // 16-byte chunks (all pointers aligned)
+#pragma unroll 1
+    for (skel_u64 c = tid; c < nch; c += stride) skel_mm_chunk(a, mcb, bown, mco, c, t);
+#pragma unroll 1
+    for (skel_u64 i = nch * 4 + tid; i < n; i += stride) skel_mm_one(a, mcb, bown, mco, i, t);
+}
 #endif

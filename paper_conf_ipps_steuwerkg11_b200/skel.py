@@ -47,7 +47,8 @@ class Stats(ctypes.Structure):
                 ("kernel_launches", ctypes.c_uint64), ("compile_mem_hits", ctypes.c_uint64),
                 ("compile_disk_hits", ctypes.c_uint64), ("compile_misses", ctypes.c_uint64),
                 ("compile_ms", ctypes.c_double), ("disk_load_ms", ctypes.c_double),
-                ("scan_coop_fallbacks", ctypes.c_uint64)]
+                ("scan_coop_fallbacks", ctypes.c_uint64), ("vmm_allocs", ctypes.c_uint64),
+                ("mc_binds", ctypes.c_uint64), ("multimem_launches", ctypes.c_uint64)]
 
     def asdict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}

@@ -90,3 +90,59 @@ def test_lmosem_fused_subsets_match_oracle(D):
         img = rec.image()
     want = oracle.lmosem_reconstruct(subsets)
     assert np.linalg.norm(img - want) <= 1e-4 * np.linalg.norm(want)
+
+
+MM_BODY = r'''
+import sys
+sys.path.insert(0, ROOT)
+import numpy as np
+import oracle
+import skel_inputs as si
+from paper_conf_ipps_steuwerkg11_b200 import skel
+from paper_conf_ipps_steuwerkg11_b200.lmosem import LMOSEM
+from paper_conf_ipps_steuwerkg11_b200.workloads import LMOSEM_UPDATE
+with skel.Context(1) as ctx:
+    # n not a multiple of 4: chunked multimem loads/stores plus the scalar tail
+    n = 2_000_003
+    f0 = si.uniform_f32(n, 3)
+    c0 = si.uniform_f32(n, 4) - np.float32(0.25)
+    f = ctx.vector(f0); c = ctx.vector(c0)
+    ctx.zip_combine(LMOSEM_UPDATE, f, c, skel.COMBINE_ADD, f)
+    st = ctx.stats()
+    got_f, got_c = f.download(), c.download()
+    want = oracle.skel_zip(LMOSEM_UPDATE, f0, c0, np.float32)
+    assert np.array_equal(got_c, c0)
+    assert np.array_equal(got_f, want)
+    # LM OSEM subset with the fused tail through multicast: the oracle's image
+    ev = si.lmosem_events(20_000, subset=2)
+    rec = LMOSEM(ctx)
+    rec.subset(rec.events(ev), fused=True)
+    img = rec.image()
+    ref, cc, nv = oracle.lmosem_subset(ev, np.ones(150 * 150 * 280))
+    rel = float(np.linalg.norm(img.astype(np.float64) - ref) / np.linalg.norm(ref))
+    assert rel <= 1e-4, rel
+    print("STATS", ctx.stats()["multimem_launches"], ctx.stats()["mc_binds"], st["vmm_allocs"])
+'''
+
+
+def test_fused_tail_through_multicast_on_one_gpu():
+    """NEXT-1 in its NVLS form (skel_zipcomb_mm_kernel: multimem.ld_reduce.add +
+    multimem.st through a multicast object bound to VMM buffers), exercised on
+    one GPU with a one-device multicast object (SKEL_FORCE_MULTIMEM=1): the
+    update Zip's result and the combined c are exact, and an LM OSEM subset
+    with this tail is the oracle's image.  Skipped where the device reports no
+    multicast support."""
+    import os
+    import subprocess
+    import sys
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    env = dict(os.environ, SKEL_FORCE_MULTIMEM="1")
+    r = subprocess.run([sys.executable, "-c", f"ROOT = {root!r}\n" + MM_BODY], env=env, cwd=root,
+                       capture_output=True, text=True, timeout=600)
+    assert r.returncode == 0, r.stdout[-2000:] + r.stderr[-3000:]
+    line = [x for x in r.stdout.splitlines() if x.startswith("STATS")][0].split()
+    launches, binds, vmm = int(line[1]), int(line[2]), int(line[3])
+    assert vmm > 0  # the 8 MB vectors are VMM allocations
+    if binds == 0:
+        pytest.skip("device reports no multicast support: the peer-memory tail ran (results checked)")
+    assert launches >= 2
