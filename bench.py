@@ -37,10 +37,10 @@ METRIC = "skeleton step GB/s (Map+Zip+Reduce+Scan, float32, 2^30 elements per GP
 SEED = 20110516
 
 
-# untimed launches before any timing of an element-wise skeleton: the first
-# 6 launches of a module and size class time its three grid policies
-# (K1/K2), the 7th uses the decided one
-TUNE = 7
+# untimed launches of a skeleton before it is timed: its first launch compiles
+# (or loads) the module and decides the element-wise grid policy on a sample
+# (runtime.cpp ew_decide; no trial policies on user launches)
+TUNE = 1
 
 
 def bench_config(nloc: int, world: int) -> dict:
@@ -726,100 +726,94 @@ def bench_overhead_small(ctx, hw, stream):
     return out
 
 
+FP32_PEAK_OPS = 148 * 128 * 1.965e9  # nominal: 148 SMs x 128 FP32 lanes x 1.965 GHz (no measured FP32 peak)
+
+
 def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
-    """configs[2]: 4096x3072, cap 256, rows block-distributed over the GPUs."""
+    """configs[2]: 4096x3072, cap 256, rows block-distributed over the GPUs --
+    the paper's Map over positions and the NEXT-4 variants (all bit-identical
+    to eq. (5) as written, tests/test_gpu_mandelbrot.py): index Map, blocked
+    loop control, pixel pairs with packed FP32x2, exact periodicity checking,
+    cyclic rows; the cap-4096 heavy variant; configs[0] 1024x768 on one GPU.
+    FP32 fraction = 8 FP32 operations per iteration AS WRITTEN x sum of the
+    counts / time / nominal FP32 lane peak (the periodicity variant executes
+    fewer iterations than that sum: its figure is an algorithmic-equivalent
+    rate, not pipe utilisation)."""
     import torch
     import skel_inputs as si
-    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT
+    from paper_conf_ipps_steuwerkg11_b200.mandelbrot import CyclicMandelbrot
+    from paper_conf_ipps_steuwerkg11_b200.workloads import (MANDELBROT, MANDELBROT_BLOCKED, MANDELBROT_INDEX,
+                                                            MANDELBROT_PAIRS, MANDELBROT_PERIODIC)
     W, H, cap = 4096, 3072, 256
-    pos = si.mandelbrot_positions(W, H)
-    vin = ctx.vector(n=pos.size, dtype=pos.dtype)
-    if world > 1:
-        vin.set_distribution(skel.BLOCK)
-    lo, hi = vin.part(rank) if world > 1 else (0, pos.size)
-    vin.upload_part(lo, pos[lo:hi])
-    out = ctx.vector(n=pos.size, dtype=np.int32)
-    capv = np.int32(cap)
-    ctx.map(MANDELBROT, vin, out, args=[capv])
-    ctx.sync()
-    for _ in range(TUNE):
-        ctx.map(MANDELBROT, vin, out, args=[capv])
-    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     reps = max(args.steps, 10)
-    barrier()
-    torch.cuda.synchronize()
-    e0.record(stream)
-    for _ in range(reps):
-        ctx.map(MANDELBROT, vin, out, args=[capv])
-    e1.record(stream)
-    ctx.sync()
-    ms = max_over_ranks(e0.elapsed_time(e1) / reps)
-    res = {"config": "configs[2]: 4096x3072, cap 256, block rows", "ms": ms,
-           "Mpix_per_s": W * H / (ms * 1e-3) / 1e6}
-    # NEXT-4: the same image from an index Map (c computed in-kernel, no position vector)
-    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_INDEX
-    oi = ctx.vector(n=pos.size, dtype=np.int32)
-    if world > 1:
-        oi.set_distribution(skel.BLOCK)
-    iargs = [np.int32(W), np.int32(H), capv]
-    for _ in range(TUNE):
-        ctx.map_index(MANDELBROT_INDEX, W * H, oi, args=iargs)
-    barrier()
-    torch.cuda.synchronize()
-    e0.record(stream)
-    for _ in range(reps):
-        ctx.map_index(MANDELBROT_INDEX, W * H, oi, args=iargs)
-    e1.record(stream)
-    ctx.sync()
-    res["index_map_ms"] = max_over_ranks(e0.elapsed_time(e1) / reps)
-    oi.destroy()
-    # NEXT-4: the blocked user function (same counts, loop control per 8 updates)
-    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_BLOCKED
-    ob = ctx.vector(n=pos.size, dtype=np.int32)
-    for _ in range(TUNE):
-        ctx.map(MANDELBROT_BLOCKED, vin, ob, args=[capv])
-    barrier()
-    torch.cuda.synchronize()
-    e0.record(stream)
-    for _ in range(reps):
-        ctx.map(MANDELBROT_BLOCKED, vin, ob, args=[capv])
-    e1.record(stream)
-    ctx.sync()
-    ms_blk = max_over_ranks(e0.elapsed_time(e1) / reps)
-    res["blocked_ms"] = ms_blk
-    same = ob.download()
-    counts = out.download()  # collective in rank mode: every rank takes part
-    # heavy variant (SURVEY §8d config 1/3: "also report the cap-4096 variant")
-    heavy = {}
-    for name, fn in (("paper", MANDELBROT), ("blocked", MANDELBROT_BLOCKED)):
-        c4 = np.int32(4096)
-        ctx.map(fn, vin, ob, args=[c4])
+
+    def timed(fn, n=reps):
+        for _ in range(3):
+            fn()
+        ctx.sync()
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         barrier()
         torch.cuda.synchronize()
         e0.record(stream)
-        for _ in range(3):
-            ctx.map(fn, vin, ob, args=[c4])
+        for _ in range(n):
+            fn()
         e1.record(stream)
         ctx.sync()
-        heavy[name] = max_over_ranks(e0.elapsed_time(e1) / 3)
-    it4096 = int(ob.download().astype(np.int64).sum())
-    ob.destroy()
-    if rank == 0:
-        res["blocked_bit_identical"] = bool(np.array_equal(same, counts))
-    if rank == 0:
-        iters = int(counts.astype(np.int64).sum())
-        res["sum_iter"] = iters
-        res["Giter_per_s"] = iters / (ms * 1e-3) / 1e9
-        # FP32 pipe roofline: 8 FP32 ops per iteration as written (3 FMUL, 4 FADD/FSUB, 1 scale)
-        # vs 148 SM x 128 lanes x 1.965 GHz = 37.2 T FP32 instr/s
-        peak_ops = 148 * 128 * 1.965e9
-        res["fp32_frac"] = 8 * iters / (ms * 1e-3) / peak_ops
-        res["blocked_fp32_frac"] = 8 * iters / (ms_blk * 1e-3) / peak_ops
-        res["cap4096"] = {"sum_iter": it4096, "ms": heavy["paper"], "blocked_ms": heavy["blocked"],
-                          "fp32_frac": 8 * it4096 / (heavy["paper"] * 1e-3) / peak_ops,
-                          "blocked_fp32_frac": 8 * it4096 / (heavy["blocked"] * 1e-3) / peak_ops}
-    vin.destroy()
-    out.destroy()
+        return max_over_ranks(e0.elapsed_time(e1) / n)
+
+    pos = si.mandelbrot_positions(W, H)
+    vin = ctx.vector(n=pos.size, dtype=pos.dtype)
+    pairs = pos.view(si.POS2_DTYPE)
+    vin2 = ctx.vector(n=pairs.size, dtype=pairs.dtype)
+    if world > 1:
+        vin.set_distribution(skel.BLOCK)
+        vin2.set_distribution(skel.BLOCK)
+    lo, hi = vin.part(rank) if world > 1 else (0, pos.size)
+    vin.upload_part(lo, pos[lo:hi])
+    lo2, hi2 = vin2.part(rank) if world > 1 else (0, pairs.size)
+    vin2.upload_part(lo2, pairs[lo2:hi2])
+    out = ctx.vector(n=pos.size, dtype=np.int32)
+    out2 = ctx.vector(n=pairs.size, dtype=si.CNT2_DTYPE)
+    oi = ctx.vector(n=pos.size, dtype=np.int32)
+    if world > 1:
+        oi.set_distribution(skel.BLOCK)
+    capv = np.int32(cap)
+    ms = {}
+    ms["paper"] = timed(lambda: ctx.map(MANDELBROT, vin, out, args=[capv]))
+    counts = out.download()  # collective in rank mode: every rank takes part
+    ms["index_map"] = timed(lambda: ctx.map_index(MANDELBROT_INDEX, W * H, oi, args=[np.int32(W), np.int32(H), capv]))
+    ms["blocked"] = timed(lambda: ctx.map(MANDELBROT_BLOCKED, vin, out, args=[capv]))
+    same = np.array_equal(out.download(), counts)
+    ms["pairs"] = timed(lambda: ctx.map(MANDELBROT_PAIRS, vin2, out2, args=[capv]))
+    same &= np.array_equal(out2.download().view(np.int32), counts)
+    ms["periodic"] = timed(lambda: ctx.map(MANDELBROT_PERIODIC, vin, out, args=[capv]))
+    same &= np.array_equal(out.download(), counts)
+    # cyclic rows (device k: rows k, k+D, ...): the compute step alone and the
+    # whole image on device 0 (gather + un-permute)
+    cm = CyclicMandelbrot(ctx, W, H)
+    ms["cyclic_compute"] = timed(lambda: cm.compute(cap))
+    ms["cyclic_image"] = timed(lambda: cm.image(cap))
+    same &= np.array_equal(cm.counts(cap), counts)
+    iters = int(counts.astype(np.int64).sum())
+    res = {"config": "configs[2]: 4096x3072, cap 256, block rows", "ms": ms["paper"],
+           "Mpix_per_s": W * H / (ms["paper"] * 1e-3) / 1e6, "variants_ms": ms,
+           "all_bit_identical": bool(same), "sum_iter": iters,
+           "Giter_per_s": iters / (ms["paper"] * 1e-3) / 1e9,
+           "fp32_peak": {"value": FP32_PEAK_OPS, "unit": "FP32 ops/s", "source": "nominal (148 SMs x 128 lanes x "
+                         "1.965 GHz); MEASURED_PEAKS.json has no FP32 entry"},
+           "fp32_frac": {k: 8 * iters / (v * 1e-3) / FP32_PEAK_OPS for k, v in ms.items()
+                         if not k.startswith("cyclic_image")}}
+    # heavy variant (SURVEY §8d config 1/3: "also report the cap-4096 variant")
+    c4 = np.int32(4096)
+    heavy = {}
+    for name, fn, vi, vo in (("paper", MANDELBROT, vin, out), ("blocked", MANDELBROT_BLOCKED, vin, out),
+                             ("periodic", MANDELBROT_PERIODIC, vin, out)):
+        heavy[name] = timed(lambda: ctx.map(fn, vi, vo, args=[c4]), n=3)
+    it4096 = int(out.download().astype(np.int64).sum())
+    res["cap4096"] = {"sum_iter": it4096, "ms": heavy,
+                      "fp32_frac": {k: 8 * it4096 / (v * 1e-3) / FP32_PEAK_OPS for k, v in heavy.items()}}
+    for v in (vin, vin2, out, out2, oi):
+        v.destroy()
     # configs[0]: 1024x768, cap 256, single distribution (device 0 / rank 0)
     ps = si.mandelbrot_positions(1024, 768)
     vs = ctx.vector(n=ps.size, dtype=ps.dtype)
@@ -827,22 +821,21 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
     vs.upload(ps)
     os_ = ctx.vector(n=ps.size, dtype=np.int32)
     os_.set_distribution(skel.SINGLE)
-    for _ in range(TUNE):
-        ctx.map(MANDELBROT, vs, os_, args=[capv])
-    barrier()
-    torch.cuda.synchronize()
-    e0.record(stream)
-    for _ in range(reps):
-        ctx.map(MANDELBROT, vs, os_, args=[capv])
-    e1.record(stream)
-    ctx.sync()
-    ms_s = max_over_ranks(e0.elapsed_time(e1) / reps)
-    res["configs0_1024x768"] = {"ms": ms_s, "Mpix_per_s": ps.size / (ms_s * 1e-3) / 1e6,
-                                "sum_iter": 28347768,
-                                "fp32_frac": 8 * 28347768 / (ms_s * 1e-3) / (148 * 128 * 1.965e9),
+    ps2 = ps.view(si.POS2_DTYPE)
+    vs2 = ctx.vector(n=ps2.size, dtype=ps2.dtype)
+    vs2.set_distribution(skel.SINGLE)
+    vs2.upload(ps2)
+    os2 = ctx.vector(n=ps2.size, dtype=si.CNT2_DTYPE)
+    os2.set_distribution(skel.SINGLE)
+    ms0 = {"paper": timed(lambda: ctx.map(MANDELBROT, vs, os_, args=[capv])),
+           "pairs": timed(lambda: ctx.map(MANDELBROT_PAIRS, vs2, os2, args=[capv])),
+           "periodic": timed(lambda: ctx.map(MANDELBROT_PERIODIC, vs, os_, args=[capv]))}
+    res["configs0_1024x768"] = {"ms": ms0["paper"], "variants_ms": ms0,
+                                "Mpix_per_s": ps.size / (ms0["paper"] * 1e-3) / 1e6, "sum_iter": 28347768,
+                                "fp32_frac": {k: 8 * 28347768 / (v * 1e-3) / FP32_PEAK_OPS for k, v in ms0.items()},
                                 "note": "single distribution: one GPU computes, 2.6 waves (latency-sized)"}
-    vs.destroy()
-    os_.destroy()
+    for v in (vs, os_, vs2, os2):
+        v.destroy()
     return res
 
 

@@ -305,7 +305,11 @@ bool mc_supported(skel_ctx_s *ctx) {
     if (const char *e = getenv("SKEL_MULTIMEM")) ok = ok && atoi(e) != 0;
     for (int dev : local_devices(ctx)) {
         int v = 0;
-        if (!ok || d.attr(&v, CU_DEVICE_ATTRIBUTE_MULTICAST_SUPPORTED, (CUdevice)dev) != CUDA_SUCCESS || !v) ok = false;
+        CUresult r = ok ? d.attr(&v, CU_DEVICE_ATTRIBUTE_MULTICAST_SUPPORTED, (CUdevice)dev) : CUDA_SUCCESS;
+        if (getenv("SKEL_LOG"))
+            fprintf(stderr, "[skel] multicast: driver entry points %d, device %d attribute %d (query %d)\n", (int)d.mc,
+                    dev, v, (int)r);
+        if (!ok || r != CUDA_SUCCESS || !v) ok = false;
     }
     ctx->mc_ok = ok ? 1 : 0;
     return ok;
@@ -334,7 +338,9 @@ bool mc_bind(skel_vec_s *v, size_t bytes) {
         if (it == ctx->vmm.end() || it->second.size < prop.size) return false;
     }
     CUmemGenericAllocationHandle mc = 0;
-    if (d.mc_create(&mc, &prop) != CUDA_SUCCESS) {
+    const CUresult cr = d.mc_create(&mc, &prop);
+    if (cr != CUDA_SUCCESS) {
+        if (getenv("SKEL_LOG")) fprintf(stderr, "[skel] cuMulticastCreate: %d\n", (int)cr);
         cudaGetLastError();
         return false;
     }
@@ -368,6 +374,7 @@ bool mc_bind(skel_vec_s *v, size_t bytes) {
         }
     }
     if (!ok) {
+        if (getenv("SKEL_LOG")) fprintf(stderr, "[skel] multicast bind/map failed\n");
         cudaGetLastError();
         for (int dev : m.devs) d.mc_unbind(mc, (CUdevice)dev, 0, prop.size);
         d.release(mc);

@@ -429,24 +429,25 @@ extern "C" __global__ void SKEL_EW_BOUNDS
 // fan-out), against (D-1)/D x S each way for peer loads/stores.  float32 `+`
 // combine and 4-byte outputs only; other types use skel_zipcomb_kernel.
 // ---------------------------------------------------------------------------
-template <class Tup>
-__device__ __forceinline__ void skel_mm_chunk(const skel_A *a, const float *mcb, skel_B *bown, float *mco, skel_u64 c,
+// (templates on the element types B, O so that nothing is checked for the
+// element types the host never launches this kernel with)
+template <class B, class O, class Tup>
+__device__ __forceinline__ void skel_mm_chunk(const skel_A *a, const float *mcb, B *bown, float *mco, skel_u64 c,
                                               Tup &t) {
-    if constexpr (skel::same<skel::decay_t<skel_B>, float>::value && sizeof(skel_O) == 4 && SKEL_E == 4 &&
-                  !skel_void) {
+    if constexpr (skel::same<skel::decay_t<B>, float>::value && sizeof(O) == 4 && SKEL_E == 4 && !skel_void) {
         float4 v;
         asm volatile("multimem.ld_reduce.relaxed.sys.global.add.v4.f32 {%0, %1, %2, %3}, [%4];"
                      : "=f"(v.x), "=f"(v.y), "=f"(v.z), "=f"(v.w)
                      : "l"(mcb + 4 * c)
                      : "memory");
-        skel::arr<skel_B, 4> acc;
+        skel::arr<B, 4> acc;
         acc.v[0] = v.x;
         acc.v[1] = v.y;
         acc.v[2] = v.z;
         acc.v[3] = v.w;
         skel_st<16>(reinterpret_cast<char *>(bown) + c * 16, skel::bit_cast<skel::chunk<16>>(acc));
         const auto xa = skel::bit_cast<skel::arr<skel_A, 4>>(skel_ld<skel_CA>(reinterpret_cast<const char *>(a) + c * skel_CA));
-        skel::arr<skel_O, 4> yo;
+        skel::arr<O, 4> yo;
         skel_apply_chunk(xa.v, acc.v, yo.v, t);
         const auto r = skel::bit_cast<float4>(yo);
         asm volatile("multimem.st.relaxed.sys.global.v4.f32 [%0], {%1, %2, %3, %4};" ::"l"(mco + 4 * c), "f"(r.x),
@@ -454,14 +455,14 @@ __device__ __forceinline__ void skel_mm_chunk(const skel_A *a, const float *mcb,
                      : "memory");
     }
 }
-template <class Tup>
-__device__ __forceinline__ void skel_mm_one(const skel_A *a, const float *mcb, skel_B *bown, float *mco, skel_u64 i,
+template <class B, class O, class Tup>
+__device__ __forceinline__ void skel_mm_one(const skel_A *a, const float *mcb, B *bown, float *mco, skel_u64 i,
                                             Tup &t) {
-    if constexpr (skel::same<skel::decay_t<skel_B>, float>::value && sizeof(skel_O) == 4 && !skel_void) {
+    if constexpr (skel::same<skel::decay_t<B>, float>::value && sizeof(O) == 4 && !skel_void) {
         float v;
         asm volatile("multimem.ld_reduce.relaxed.sys.global.add.f32 %0, [%1];" : "=f"(v) : "l"(mcb + i) : "memory");
         bown[i] = v;
-        const skel_O r = skel::caller<skel_Seq>::call(&SKEL_FN, t, a[i], v);
+        const O r = skel::caller<skel_Seq>::call(&SKEL_FN, t, a[i], v);
         asm volatile("multimem.st.relaxed.sys.global.f32 [%0], %1;" ::"l"(mco + i), "f"(skel::bit_cast<float>(r))
                      : "memory");
     }
@@ -472,10 +473,13 @@ extern "C" __global__ void SKEL_EW_BOUNDS
     auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
     const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;
-    const skel_u64 nch = (SKEL_E == 4 && vec_ok) ? n / 4 : 0;  // 16-byte chunks (all pointers aligned)
+    skel_u64 nch = 0;  // 16-byte chunks (all pointers aligned)
+    if constexpr (SKEL_E == 4) {
+        nch = vec_ok ? n / 4 : 0;
 #pragma unroll 1
-    for (skel_u64 c = tid; c < nch; c += stride) skel_mm_chunk(a, mcb, bown, mco, c, t);
+        for (skel_u64 c = tid; c < nch; c += stride) skel_mm_chunk<skel_B, skel_O>(a, mcb, bown, mco, c, t);
+    }
 #pragma unroll 1
-    for (skel_u64 i = nch * 4 + tid; i < n; i += stride) skel_mm_one(a, mcb, bown, mco, i, t);
+    for (skel_u64 i = nch * 4 + tid; i < n; i += stride) skel_mm_one<skel_B, skel_O>(a, mcb, bown, mco, i, t);
 }
 #endif
