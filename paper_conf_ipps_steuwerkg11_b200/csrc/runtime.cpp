@@ -338,9 +338,19 @@ bool mc_bind(skel_vec_s *v, size_t bytes) {
         if (it == ctx->vmm.end() || it->second.size < prop.size) return false;
     }
     CUmemGenericAllocationHandle mc = 0;
-    const CUresult cr = d.mc_create(&mc, &prop);
+    // the handle type of the multicast object: exportable kinds first (what the
+    // driver accepts depends on the platform), then none
+    CUresult cr = CUDA_ERROR_INVALID_VALUE;
+    for (CUmemAllocationHandleType ht : {CU_MEM_HANDLE_TYPE_POSIX_FILE_DESCRIPTOR, CU_MEM_HANDLE_TYPE_FABRIC,
+                                         CU_MEM_HANDLE_TYPE_NONE}) {
+        prop.handleTypes = ht;
+        cr = d.mc_create(&mc, &prop);
+        if (getenv("SKEL_LOG"))
+            fprintf(stderr, "[skel] cuMulticastCreate(handle type %d, size %zu, devices %u): %d\n", (int)ht,
+                    (size_t)prop.size, prop.numDevices, (int)cr);
+        if (cr == CUDA_SUCCESS) break;
+    }
     if (cr != CUDA_SUCCESS) {
-        if (getenv("SKEL_LOG")) fprintf(stderr, "[skel] cuMulticastCreate: %d\n", (int)cr);
         cudaGetLastError();
         return false;
     }

@@ -124,3 +124,59 @@ def test_bench_reference_arm_under_torchrun():
     d = json.loads(lines[0])
     assert d["impl"] == "reference" and d["n_gpus"] == 2 and d["value"] > 0
     assert d["e2e"]["h2d_bytes_per_step"] == 0 and d["cpu_baseline"]["kind"] == "oracle"
+
+
+def _cyclic_worker(rank, world, port, q):
+    """Cyclic Mandelbrot rows at world 2 (mandelbrot.CyclicMandelbrot's layout):
+    the permuted image is block-distributed with R = ceil(H/D) row slots per
+    rank, slot t of rank k holding row k + t*D.  Each rank computes its slots
+    with the oracle; gathered on rank 0 in block order and un-permuted (row r at
+    slot (r mod D)*R + r div D) they must be the whole image, and the ranks'
+    work (sum of counts) must be balanced."""
+    sys.path.insert(0, ROOT)
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import oracle
+        import skel_inputs as si
+        from paper_conf_ipps_steuwerkg11_b200 import skel
+        W, H, cap = 256, 190, 64   # H not a multiple of D: padding slots
+        R = -(-H // world)
+        n_perm = world * R * W
+        lo, hi = skel.plan_part(n_perm, world, rank)
+        assert (lo, hi) == (rank * R * W, (rank + 1) * R * W)
+        pos = si.mandelbrot_positions(W, H).reshape(H, W)
+        mine = np.zeros((R, W), np.int32)
+        for t in range(R):
+            row = rank + t * world
+            if row < H:
+                mine[t] = oracle.mandelbrot(np.ascontiguousarray(pos[row]), cap)
+        parts = [torch.zeros(R * W, dtype=torch.int32) for _ in range(world)]
+        dist.all_gather(parts, torch.from_numpy(mine.reshape(-1)))
+        perm = torch.cat(parts).numpy().reshape(world * R, W)
+        img = np.stack([perm[(r % world) * R + r // world] for r in range(H)])
+        want = oracle.mandelbrot(np.ascontiguousarray(pos.reshape(-1)), cap).reshape(H, W)
+        work = torch.tensor([float(mine.astype(np.int64).sum())], dtype=torch.float64)
+        works = [torch.zeros(1, dtype=torch.float64) for _ in range(world)]
+        dist.all_gather(works, work)
+        w = np.array([float(x) for x in works])
+        q.put((rank, {"image": bool(np.array_equal(img, want)), "balance": float(w.mean() / w.max())}))
+    finally:
+        dist.destroy_process_group()
+
+
+def test_cyclic_rows_layout_world2():
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = free_port()
+    procs = [ctx.Process(target=_cyclic_worker, args=(r, 2, port, q)) for r in range(2)]
+    for p in procs:
+        p.start()
+    out = dict(q.get(timeout=180) for _ in procs)
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    for r in range(2):
+        assert out[r]["image"]
+        assert out[r]["balance"] >= 0.95, out[r]
