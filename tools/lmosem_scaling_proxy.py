@@ -65,22 +65,28 @@ with skel.Context(1) as ctx:
         fp, cp = ctx.vector(n=nv, dtype=np.float32).fill(np.float32(1)), ctx.vector(n=nv, dtype=np.float32)
         cp.fill(np.float32(0.5))
         r["zip_ms"] = timed(lambda: ctx.zip(LMOSEM_UPDATE, fp, cp, fp))
-        # RS then AG (NCCL, one after the other): (D-1)/D x S out of each GPU, then into it
+        # Bytes per GPU and direction (full-duplex links, S = 25.2 MB):
+        # RS + AG (NCCL ring): (D-1)/D S each way for the RS, then again for the AG
         r["exchange_ms_model"] = 2 * S * (D - 1) / D / (NVLINK_GBPS * 1e9) * 1e3
-        # fused peer-memory tail (skel_zip_combine): the loads of the peers' copies
-        # (into the GPU) and the stores of the new f part (out of it) overlap on the
-        # full-duplex links: (D-1)/D x S per direction
-        r["exchange_fused_ms_model"] = S * (D - 1) / D / (NVLINK_GBPS * 1e9) * 1e3
+        # fused peer-memory tail (skel_zip_combine): a GPU loads its part of the
+        # D-1 other copies and stores its result part into D-1 copies, and serves
+        # the same to every peer: 2 (D-1)/D S each way, in ONE kernel
+        r["exchange_fused_ms_model"] = 2 * S * (D - 1) / D / (NVLINK_GBPS * 1e9) * 1e3
+        # NVLS tail (multimem.ld_reduce + multimem.st): in, S/D reduced + (D-1)/D S of
+        # the others' results; out, (D-1)/D S of its copy to the switch + S/D of its
+        # result: S each way
+        r["exchange_nvls_ms_model"] = S / (NVLINK_GBPS * 1e9) * 1e3 if D > 1 else 0.0
         for order in ("given", "device"):
             extra = r["order_ms"] if order == "device" else 0.0
             base = r["fill_ms"] + extra + r[f"{order}_map_ms"] + r["zip_ms"]
             r[f"{order}_subset_ms"] = base + r["exchange_ms_model"]
             r[f"{order}_subset_fused_ms"] = base + r["exchange_fused_ms_model"]
+            r[f"{order}_subset_nvls_ms"] = base + r["exchange_nvls_ms_model"]
         rows.append(r)
         print(json.dumps({k: (round(v, 4) if isinstance(v, float) else v) for k, v in r.items()}), flush=True)
 summary = {}
 for order in ("given", "device"):
-    for tail in ("", "_fused"):
+    for tail in ("", "_fused", "_nvls"):
         t1 = rows[0][f"{order}_subset{tail}_ms"]
         summary[order + tail] = {f"T1/T{r['D']}": round(t1 / r[f"{order}_subset{tail}_ms"], 2) for r in rows}
 print(json.dumps({"projection": summary, "exchange": f"RS + AG of {S / 1e6:.1f} MB at {NVLINK_GBPS} GB/s per direction"}))
