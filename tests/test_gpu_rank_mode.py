@@ -64,7 +64,7 @@ def test_bench_rank_path(fake_nccl):
     assert d["n_gpus"] == 2 and d["value"] > 0 and d["config"]["distribution"] == "block"
     assert d["e2e"]["h2d_bytes_per_step"] == 2 * (1 << 22) * 4  # this rank's parts of x and y
     assert d["mandelbrot"]["sum_iter"] == 453197644
-    assert d["mandelbrot"]["blocked_bit_identical"] and d["mandelbrot"]["cap4096"]["sum_iter"] > 453197644
+    assert d["mandelbrot"]["all_bit_identical"] and d["mandelbrot"]["cap4096"]["sum_iter"] > 453197644
     ex = d["lmosem"]["exchange"]  # reduce-scatter / all-gather of the 25.2 MB image alone
     assert ex["bytes"] == 150 * 150 * 280 * 4 and ex["reduce_scatter_busbw_GBps"] > 0 and ex["all_gather_busbw_GBps"] > 0
     assert d["lmosem"]["full_recon_s"] > 0
