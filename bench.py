@@ -906,6 +906,17 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         recd.subset(evv)
     ms_dev = timed(lambda: recd.subset(evv))
     ms_sort = timed(lambda: recd.order_on_device(evv))
+    try:  # the same as CUDA graphs: GPU time without the per-call host overhead
+        if os.environ.get("SKEL_BENCH_NO_GRAPH"):
+            raise skel.SkelError(8, "graphs disabled")
+        g = ctx.capture(lambda: recd.subset(evv))
+        ms_dev_graph = timed(g.launch)
+        g.destroy()
+        g = ctx.capture(lambda: recd.order_on_device(evv))
+        ms_sort_graph = timed(g.launch)
+        g.destroy()
+    except skel.SkelError:
+        ms_dev_graph, ms_sort_graph = ms_dev, ms_sort
     coll = None
     if world > 1:  # the exchange steps alone, bus GB/s vs NVLink
         S = rec.nvox * 4
@@ -968,6 +979,7 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
             "full_recon_s": full["given"] * 1e-3, "full_recon": "10 subsets x 10^6 events (configs[4]), f0 = 1, "
                                                                 "events resident on the devices",
             "device_order": {"subset_s": ms_dev * 1e-3, "order_s": ms_sort * 1e-3,
+                             "subset_s_graph": ms_dev_graph * 1e-3, "order_s_graph": ms_sort_graph * 1e-3,
                              "full_recon_s": full["device"] * 1e-3,
                              "map_lanes": recd.plan(-(-nev // world))[1],
                              "note": "every GPU's events reordered by path length on the device (lmosem_order.cu: "

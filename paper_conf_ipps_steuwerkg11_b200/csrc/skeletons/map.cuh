@@ -177,8 +177,10 @@ __device__ __forceinline__ void skel_chunk_op(const skel::chunk<skel_CA> &ca, co
 }
 // Map over elements no 16-byte chunk covers (E == 1), sizes multiple of 4 up
 // to 64 bytes: staged through shared memory (see skel_ew_kernel)
+// (power-of-two sizes keep the direct loads: measured slower staged for the
+// 16-byte pixel pairs of mandelbrot_pairs, a compute-bound Map)
 constexpr bool skel_stage = SKEL_NIN == 1 && SKEL_E == 1 && !SKEL_LANES && sizeof(skel_A) >= 8 &&
-                            sizeof(skel_A) % 4 == 0 && sizeof(skel_A) <= 64;
+                            sizeof(skel_A) % 4 == 0 && sizeof(skel_A) <= 64 && !skel::pow2(sizeof(skel_A));
 template <bool V = skel_void, class Tup>
 __device__ __forceinline__ void skel_one_val(const skel_A &x, skel_O *out, skel_u64 i, Tup &t) {
     if constexpr (V) {
@@ -348,8 +350,8 @@ extern "C" __global__ void SKEL_EW_BOUNDS
                 if (c + u * stride < nch) skel_chunk_op(ca[u], cb[u], po + (c + u * stride) * skel_CO, t);
         }
     }
-    // Elements that no 16-byte access covers one per thread (a 24-byte LM OSEM
-    // event, a 16-byte pixel pair): staged through shared memory.  The CTA
+    // Elements of a size no single load covers (a 24-byte LM OSEM event): staged
+    // through shared memory.  The CTA
     // copies its tile of blockDim elements with coalesced 16-byte loads, then
     // each thread reads its element from shared memory -- instead of every
     // thread issuing sizeof(A)/4 strided 4-byte loads (measured: a Map over

@@ -34,15 +34,21 @@ with skel.Context(1) as ctx:
     stream = torch.cuda.ExternalStream(ctx.stream(0))
 
     def timed(fn, reps=20):
+        """GPU time per call (captured once as a CUDA graph, the graph replayed:
+        eager Python calls would add their launch overhead to short pieces)."""
         for _ in range(3):
             fn()
+        ctx.sync()
+        g = ctx.capture(fn)
+        g.launch()
         ctx.sync()
         e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         e0.record(stream)
         for _ in range(reps):
-            fn()
+            g.launch()
         e1.record(stream)
         ctx.sync()
+        g.destroy()
         return e0.elapsed_time(e1) / reps
 
     for D in (1, 2, 4, 8):

@@ -31,15 +31,21 @@ with skel.Context(1) as ctx:
     dims = [np.int32(150), np.int32(150), np.int32(280), np.int32(64)]
 
     def timed(fn, reps=20):
+        """GPU time per call: the calls are captured once as a CUDA graph and the
+        graph replayed (eager timing would measure the Python/ctypes launch rate)."""
         for _ in range(3):
             fn()
+        ctx.sync()
+        g = ctx.capture(fn)
+        g.launch()
         ctx.sync()
         e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         e0.record(st)
         for _ in range(reps):
-            fn()
+            g.launch()
         e1.record(st)
         ctx.sync()
+        g.destroy()
         return round(e0.elapsed_time(e1) / reps * 1e3, 2)
     res = {}
     for blk in (256, 128):
@@ -52,5 +58,9 @@ with skel.Context(1) as ctx:
         hist.fill(np.int32(0))
         res[f"scatter_us_{blk}"] = timed(lambda: (hist.fill(np.int32(0)),
                                                   ctx.map(LMOSEM_ORDER_SCATTER, e, None, args=[hist, out, *dims])))
+        from paper_conf_ipps_steuwerkg11_b200.lmosem import LMOSEM
+        rec = LMOSEM(ctx, order="device")
+        rec.prepare()
+        res[f"order_on_device_us_{blk}"] = timed(lambda: rec.order_on_device(e))
     ctx.set_block_size(0)
     print(json.dumps(res))
