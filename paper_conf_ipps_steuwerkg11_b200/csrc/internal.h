@@ -99,6 +99,15 @@ struct McRec {
     std::vector<int> devs;
 };
 
+// rank mode: an NCCL symmetric window over a vector buffer (ncclMemAlloc +
+// ncclCommWindowRegister(NCCL_WIN_COLL_SYMMETRIC)) and the pointers it gives
+struct WinRec {
+    ncclWindow_t win = nullptr;
+    size_t size = 0;
+    std::vector<char *> peers;  // every rank's buffer, load/store-accessible from here
+    char *mc = nullptr;         // its multicast address (NVLS), if the device communicator has one
+};
+
 struct Buf {  // one logical device's storage of a vector
     char *base = nullptr;
     size_t cap = 0;    // bytes allocated at base
@@ -134,6 +143,14 @@ struct skel_ctx_s {
     size_t vmm_min = 2u << 20;
     std::unordered_map<char *, skelrt::VmmRec> vmm;
     int mc_ok = -1;  // every local device supports multicast (-1: not yet queried)
+    // rank mode, SKEL_NCCL_WINDOWS=1: the fused tail's vectors live in NCCL
+    // symmetric windows (peer pointers and the NVLS multicast address come from
+    // NCCL instead of CUDA IPC)
+    bool nccl_windows = false;
+    std::set<char *> nccl_mem;                        // buffers from ncclMemAlloc
+    std::unordered_map<char *, skelrt::WinRec> wins;  // registered windows by buffer
+    int devcomm_state = -1;                           // -1 not tried, 0 failed, 1 created
+    void *devcomm = nullptr;                          // ncclDevComm (nccl_device/impl/comm__types.h)
     skel_stats stats{};
     std::string last_error;
     std::map<std::string, std::unique_ptr<skelrt::Module>> modules;

@@ -22,6 +22,7 @@
 #include <cstring>
 #include <mutex>
 
+#include <nccl_device/impl/comm__types.h>  // host views of ncclDevComm / ncclWindow_vidmem
 #include <nvtx3/nvToolsExt.h>
 
 #include "internal.h"
@@ -246,6 +247,16 @@ int dev_free(skel_ctx_s *ctx, Slot &s, char *p) {
                                          "eagerly before capturing it");
     DevGuard g(s.dev);
     CK(ctx, cudaStreamSynchronize(s.stream));
+    if (ctx->nccl_mem.count(p)) {  // rank mode: an NCCL symmetric window's buffer
+        auto w = ctx->wins.find(p);
+        if (w != ctx->wins.end()) {
+            ncclCommWindowDeregister(ctx->comm, w->second.win);  // collective, like the registration
+            ctx->wins.erase(w);
+        }
+        ncclMemFree(p);
+        ctx->nccl_mem.erase(p);
+        return SKEL_OK;
+    }
     auto it = ctx->vmm.find(p);
     if (it != ctx->vmm.end()) {
         const Drv &d = drv();
@@ -1328,6 +1339,96 @@ int ipc_peers(skel_ctx_s *ctx, Slot &s, Buf &b) {
     return SKEL_OK;
 }
 
+// rank mode: do all ranks report ok?  (a one-word MIN all-reduce, then a sync)
+int rank_agree(skel_ctx_s *ctx, Slot &s, int ok, int *all_ok) {
+    DevGuard g(s.dev);
+    int v = ok ? 1 : 0;
+    CK(ctx, cudaMemcpyAsync(s.counters + 9, &v, sizeof v, cudaMemcpyHostToDevice, s.stream));
+    NK(ctx, ncclAllReduce(s.counters + 9, s.counters + 9, 1, ncclInt32, ncclMin, ctx->comm, s.stream));
+    CK(ctx, cudaMemcpyAsync(&v, s.counters + 9, sizeof v, cudaMemcpyDeviceToHost, s.stream));
+    CK(ctx, cudaStreamSynchronize(s.stream));
+    *all_ok = v;
+    return SKEL_OK;
+}
+
+// rank mode, SKEL_NCCL_WINDOWS=1: move vector v's buffer into an
+// NCCL symmetric window -- ncclMemAlloc (VMM memory NCCL can map on every
+// rank), the data copied over, ncclCommWindowRegister(NCCL_WIN_COLL_SYMMETRIC)
+// -- and read from the window every rank's load/store address (the LSA flat
+// mapping) and, with a device communicator that has multimem, the buffer's
+// multicast address.  Collective: every rank calls it for the same vector.
+// *ok = false (and SKEL_OK) on any failure, agreed by all ranks before the
+// collective registration; the caller then opens the peers with CUDA IPC.
+int win_setup(skel_ctx_s *ctx, Slot &s, skel_vec_s *v, bool *ok) {
+    *ok = false;
+    Buf &b = v->bufs[0];
+    if (ctx->wins.count(b.base)) {
+        *ok = true;
+        return SKEL_OK;
+    }
+    const size_t es = v->es;
+    const size_t size = align_up(std::max<size_t>(full_bytes(v), 1), NCCL_WIN_REQUIRED_ALIGNMENT);
+    DevGuard g(s.dev);
+    TRY(sync_all(ctx));
+    void *p = nullptr;
+    const bool alloc_ok = ncclMemAlloc(&p, size) == ncclSuccess && p;
+    int all = 0;
+    TRY(rank_agree(ctx, s, alloc_ok, &all));
+    if (!all) {
+        if (alloc_ok) ncclMemFree(p);
+        return SKEL_OK;
+    }
+    char *nb = static_cast<char *>(p);
+    if (b.count) CK(ctx, cudaMemcpyAsync(nb + b.off * es, b.base + b.off * es, b.count * es, cudaMemcpyDeviceToDevice,
+                                         s.stream));
+    CK(ctx, cudaStreamSynchronize(s.stream));
+    close_peers(b);
+    TRY(dev_free(ctx, s, b.base));
+    b.base = nb;
+    b.cap = size;
+    ctx->nccl_mem.insert(nb);
+    ncclWindow_t win = nullptr;
+    const bool reg_ok = ncclCommWindowRegister(ctx->comm, nb, size, &win, NCCL_WIN_COLL_SYMMETRIC) == ncclSuccess;
+    TRY(rank_agree(ctx, s, reg_ok, &all));
+    if (!all) {
+        if (reg_ok) ncclCommWindowDeregister(ctx->comm, win);
+        return SKEL_OK;  // the buffer stays an ncclMemAlloc one; peers through IPC will fail -> unfused
+    }
+    ncclWindow_vidmem wv;
+    CK(ctx, cudaMemcpy(&wv, win, sizeof wv, cudaMemcpyDefault));
+    WinRec rec;
+    rec.win = win;
+    rec.size = size;
+    const size_t four_g = (size_t)1 << 32;
+    for (int r = 0; r < ctx->D; ++r) rec.peers.push_back(wv.lsaFlatBase + (size_t)r * wv.stride4G * four_g);
+    if (ctx->devcomm_state < 0) {  // one device communicator per context, multimem if the fabric has it
+        auto *dc = new ncclDevComm();
+        ncclDevCommRequirements req = {};
+        req.lsaMultimem = true;
+        ncclResult_t r = ncclDevCommCreate(ctx->comm, &req, dc);
+        if (r != ncclSuccess) {
+            req.lsaMultimem = false;
+            r = ncclDevCommCreate(ctx->comm, &req, dc);
+        }
+        ctx->devcomm_state = r == ncclSuccess ? 1 : 0;
+        if (ctx->devcomm_state) ctx->devcomm = dc;
+        else delete dc;
+    }
+    if (ctx->devcomm_state == 1) {
+        const auto *dc = static_cast<const ncclDevComm *>(ctx->devcomm);
+        if (dc->lsaMultimem.mcBasePtr)
+            rec.mc = static_cast<char *>(dc->lsaMultimem.mcBasePtr) + (size_t)wv.mcOffset4K * 4096;
+    }
+    // the window's own slot must be this rank's buffer
+    if (wv.lsaRank != ctx->rank || rec.peers[ctx->rank] != nb) {
+        ncclCommWindowDeregister(ctx->comm, win);
+        return SKEL_OK;
+    }
+    ctx->wins[nb] = rec;
+    *ok = true;
+    return SKEL_OK;
+}
+
 // ---- Reduce / Scan -------------------------------------------------------------
 using PFN_encode = CUresult (*)(CUtensorMap *, CUtensorMapDataType, cuuint32_t, void *, const cuuint64_t *,
                                 const cuuint64_t *, const cuuint32_t *, const cuuint32_t *, CUtensorMapInterleave,
@@ -1667,6 +1768,7 @@ static void ctx_defaults(skel_ctx_s *ctx) {
     const char *f = getenv("SKEL_FMAD");
     ctx->fmad = f && atoi(f) != 0;
     if (const char *e = getenv("SKEL_VMM")) ctx->vmm_on = atoi(e) != 0;  // 0: cudaMalloc only
+    if (const char *e = getenv("SKEL_NCCL_WINDOWS")) ctx->nccl_windows = atoi(e) != 0;
     if (const char *e = getenv("SKEL_VMM_MIN")) ctx->vmm_min = (size_t)strtoull(e, nullptr, 10);
     const char *b = getenv("SKEL_BLOCK_SIZE");
     if (b) ctx->block_size = atoi(b);
@@ -1766,6 +1868,11 @@ int skel_finalize(skel_ctx_t ctx) {
     for (auto *v : vs) skel_vector_destroy(v);
     for (auto &kv : ctx->modules) {
         if (kv.second->lib) cudaLibraryUnload(kv.second->lib);
+    }
+    if (ctx->devcomm) {
+        ncclDevCommDestroy(ctx->comm, static_cast<const ncclDevComm *>(ctx->devcomm));
+        delete static_cast<ncclDevComm *>(ctx->devcomm);
+        ctx->devcomm = nullptr;
     }
     if (ctx->comm) ncclCommDestroy(ctx->comm);
     for (auto &s : ctx->slots) {
@@ -2376,17 +2483,44 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
     } else {
         Slot &s = ctx->slots[0];
         const int k = ctx->rank;
-        TRY(ipc_peers(ctx, s, b->bufs[0]));
-        TRY(ipc_peers(ctx, s, out->bufs[0]));
+        // peers: NCCL symmetric windows (SKEL_NCCL_WINDOWS=1), else CUDA IPC
+        bool win = false;
+        if (ctx->nccl_windows) {
+            bool wb = false, wo = false;
+            TRY(win_setup(ctx, s, b, &wb));
+            if (wb) TRY(win_setup(ctx, s, out, &wo));
+            win = wb && wo;
+        }
+        const WinRec *wrb = win ? &ctx->wins[b->bufs[0].base] : nullptr;
+        const WinRec *wro = win ? &ctx->wins[out->bufs[0].base] : nullptr;
+        if (!win) {
+            TRY(ipc_peers(ctx, s, b->bufs[0]));
+            TRY(ipc_peers(ctx, s, out->bufs[0]));
+        }
         TRY(rank_barrier(ctx, s));  // every rank's copy of b is complete
         const size_t lo = part_lo(a, k), cnt = want_count(a, SKEL_BLOCK, k);
-        if (cnt) {
+        const void *pa = a->dist == SKEL_COPY ? a->bufs[0].base + lo * esa : a->bufs[0].ptr(esa);
+        const bool mm_rank = win && wrb->mc && wro->mc && m->k_zipcomb_mm && b->dt == SKEL_DT_F32 &&
+                             combine == SKEL_COMBINE_ADD && esa == 4 && eso == 4 && E == 4;
+        if (cnt && mm_rank) {  // NVLS through the windows' multicast addresses
+            const float *mcb = reinterpret_cast<const float *>(wrb->mc) + lo;
+            float *mco = reinterpret_cast<float *>(wro->mc) + lo;
+            void *bown = b->bufs[0].base + lo * esb;
+            int vec_ok = al16(pa) && al16(mcb) && al16(bown) && al16(mco);
+            pack_args(m, args, nargs, 0, abuf);
+            const int grid = ew_grid(s, std::max<uint64_t>(vec_ok ? cnt / 4 : cnt, 1), block);
+            uint64_t ncall = cnt;
+            void *params[] = {&pa, &mcb, &bown, &mco, &ncall, &vec_ok, abuf.data()};
+            DevGuard g(s.dev);
+            CK(ctx, cudaLaunchKernel((const void *)m->k_zipcomb_mm, dim3(grid), dim3(block), params, 0, s.stream));
+            ctx->stats.kernel_launches++;
+            ctx->stats.multimem_launches++;
+        } else if (cnt) {
             Ptrs bs{}, os{};
             for (int j = 0; j < D; ++j) {
-                bs.p[j] = b->bufs[0].peers[j] + lo * esb;
-                os.p[j] = out->bufs[0].peers[j] + lo * eso;
+                bs.p[j] = (win ? wrb->peers[j] : b->bufs[0].peers[j]) + lo * esb;
+                os.p[j] = (win ? wro->peers[j] : out->bufs[0].peers[j]) + lo * eso;
             }
-            const void *pa = a->dist == SKEL_COPY ? a->bufs[0].base + lo * esa : a->bufs[0].ptr(esa);
             TRY(launch(s, 0, bs, b->bufs[0].base + lo * esb, os, pa, cnt));
         }
         TRY(rank_barrier(ctx, s));  // every rank's part of out has landed everywhere

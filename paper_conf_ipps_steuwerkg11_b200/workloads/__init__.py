@@ -59,7 +59,7 @@ void lm_order_scatter(Event e, int *cursor, Event *out, int nx, int ny, int nz, 
 """
 LMOSEM_ORDER_BUCKETS = 64
 LMOSEM_ORDER_REPLICAS = 128  # counters per bucket (lmosem_order.cu: lm_slot)
-LMOSEM_ORDER_SLOTS = LMOSEM_ORDER_BUCKETS * LMOSEM_ORDER_REPLICAS
+LMOSEM_ORDER_SLOTS = LMOSEM_ORDER_BUCKETS * LMOSEM_ORDER_REPLICAS * 8  # one counter per 32-byte sector
 # voxel visits of one event's path (measurement only: the LM OSEM roofline
 # counts one scattered request per visit in each of the two walks)
 LMOSEM_VISITS = LMOSEM_ERROR + """

@@ -26,10 +26,15 @@ static __forceinline__ int lm_bucket(const Event &e, int nx, int ny, int nz, int
 // slot depends only on the event, so the counting and the scattering Map
 // agree on it, and the scan over the slots in index order still puts the
 // buckets in order.
+// Each counter sits alone in a 32-byte sector (LM_ORDER_PAD ints apart; the
+// zeros between them do not change the scan): atomics on one L2 line are
+// serialised, and with consecutive counters the replicas of a busy bucket
+// shared four lines.
 #define LM_ORDER_R 128
+#define LM_ORDER_PAD 8
 static __forceinline__ int lm_slot(const Event &e, int nx, int ny, int nz, int nb) {
     unsigned h = __float_as_uint(e.x1) * 0x9E3779B1u ^ __float_as_uint(e.y2) * 0x85EBCA77u ^
                  __float_as_uint(e.z1) * 0xC2B2AE3Du;
     h ^= h >> 15;
-    return lm_bucket(e, nx, ny, nz, nb) * LM_ORDER_R + (int)(h & (LM_ORDER_R - 1));
+    return (lm_bucket(e, nx, ny, nz, nb) * LM_ORDER_R + (int)(h & (LM_ORDER_R - 1))) * LM_ORDER_PAD;
 }

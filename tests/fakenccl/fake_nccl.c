@@ -216,3 +216,24 @@ ncclResult_t ncclAllReduce(const void *s, void *r, size_t n, ncclDataType_t t, n
                            cudaStream_t st) {
     return coll(AR, s, r, n, t, op, 0, c, st);
 }
+
+/* Symmetric-window API (SKEL_NCCL_WINDOWS=1): not available in this stand-in,
+ * so libskel takes its CUDA-IPC path -- the tests check that fallback. */
+ncclResult_t ncclMemAlloc(void **ptr, size_t size) {
+    (void)size;
+    if (ptr) *ptr = NULL;
+    return ncclInvalidUsage;
+}
+ncclResult_t ncclMemFree(void *ptr) {
+    (void)ptr;
+    return ncclSuccess;
+}
+ncclResult_t ncclCommWindowRegister(ncclComm_t comm, void *buff, size_t size, ncclWindow_t *win, int flags) {
+    (void)comm; (void)buff; (void)size; (void)flags;
+    if (win) *win = NULL;
+    return ncclInvalidUsage;
+}
+ncclResult_t ncclCommWindowDeregister(ncclComm_t comm, ncclWindow_t win) {
+    (void)comm; (void)win;
+    return ncclSuccess;
+}

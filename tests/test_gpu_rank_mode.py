@@ -68,3 +68,15 @@ def test_bench_rank_path(fake_nccl):
     ex = d["lmosem"]["exchange"]  # reduce-scatter / all-gather of the 25.2 MB image alone
     assert ex["bytes"] == 150 * 150 * 280 * 4 and ex["reduce_scatter_busbw_GBps"] > 0 and ex["all_gather_busbw_GBps"] > 0
     assert d["lmosem"]["full_recon_s"] > 0
+
+
+def test_rank_mode_nccl_windows_fall_back(fake_nccl):
+    """SKEL_NCCL_WINDOWS=1: the fused LM OSEM tail asks NCCL for symmetric
+    windows (ncclMemAlloc + ncclCommWindowRegister).  The
+    host-staged stand-in has no such memory, so every rank must agree to fall
+    back to CUDA IPC -- the self-test (incl. the fused tail against the oracle)
+    still passes at 2 ranks."""
+    r = torchrun(2, ["tools/rank_selftest.py"], fake_nccl, extra_env={"SKEL_NCCL_WINDOWS": "1"})
+    oks = [ln for ln in r.stdout.splitlines() if ln.startswith("rank ")]
+    assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-3000:]
+    assert len(oks) == 2 and all(": OK" in ln for ln in oks), oks
