@@ -891,6 +891,12 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
     for _ in range(TUNE):
         rec.subset(evv, fused=True)
     ms_fused = timed(lambda: rec.subset(evv, fused=True))
+    # the two fixed orders the default (order="auto") chooses between
+    recg = LMOSEM(ctx, order="given")
+    recg.prepare()
+    for _ in range(TUNE):
+        recg.subset(evv)
+    ms_given = timed(lambda: recg.subset(evv))
     try:
         if os.environ.get("SKEL_BENCH_NO_GRAPH"):
             raise skel.SkelError(8, "graphs disabled")
@@ -938,7 +944,7 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
                 "all_gather_busbw_GBps": S * busf / (ms_ag * 1e-3) / 1e9,
                 "peak_GBps": 770.0, "peak_source": "B200_PROFILING.md measured peer copy per direction "
                                                   "(900 nominal)"}
-    roof = lmosem_roofline(ctx, skel, rec, recd, evv, timed, world)
+    roof = lmosem_roofline(ctx, skel, recg, recd, evv, timed, world)
     evv.destroy()
     # configs[4]: the full reconstruction -- 10 subsets of 10^6 events (10^7,
     # P:L603-605), each subset a different synthetic draw, all events staged on
@@ -952,7 +958,7 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
             v.set_distribution(skel.BLOCK)
         v.upload_part(lo, evl)
         subs.append(v)
-    for mode in ("given", "device"):
+    for mode in ("auto", "given"):
         rec2 = LMOSEM(ctx, order=mode)
         rec2.prepare()
         for v in subs:  # stage every subset (lazy H2D) and warm up
@@ -970,17 +976,20 @@ def bench_lmosem(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
         full[mode] = max_over_ranks(e0.elapsed_time(e1))
     for v in subs:
         v.destroy()
-    src, lanes = rec.plan(-(-nev // world))
+    per = -(-nev // world)
+    src, lanes = rec.plan(per)
     return {"config": "configs[3]/[4]: one subset, 10^6 events, 150x150x280, events block over GPUs",
             "subset_s": ms * 1e-3, "subset_s_graph": ms_graph * 1e-3, "subset_s_fused": ms_fused * 1e-3,
-            "map_form": {"lanes": lanes, "cta_threads": 128},
+            "policy": {"order": "device" if rec.ordered(per) else "given", "lanes": lanes, "cta_threads": 128,
+                       "events_per_gpu": per},
             "roofline": roof, "exchange": coll,
             "events_per_s": nev / (min(ms, ms_graph, ms_fused) * 1e-3),
-            "full_recon_s": full["given"] * 1e-3, "full_recon": "10 subsets x 10^6 events (configs[4]), f0 = 1, "
-                                                                "events resident on the devices",
+            "full_recon_s": full["auto"] * 1e-3, "full_recon": "10 subsets x 10^6 events (configs[4]), f0 = 1, "
+                                                               "events resident on the devices",
+            "given_order": {"subset_s": ms_given * 1e-3, "full_recon_s": full["given"] * 1e-3,
+                            "map_lanes": recg.plan(per)[1]},
             "device_order": {"subset_s": ms_dev * 1e-3, "order_s": ms_sort * 1e-3,
                              "subset_s_graph": ms_dev_graph * 1e-3, "order_s_graph": ms_sort_graph * 1e-3,
-                             "full_recon_s": full["device"] * 1e-3,
                              "map_lanes": recd.plan(-(-nev // world))[1],
                              "note": "every GPU's events reordered by path length on the device (lmosem_order.cu: "
                                      "counting Map + Scan + scattering Map, inside the timed subset) before the "

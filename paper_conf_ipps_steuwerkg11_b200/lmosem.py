@@ -17,8 +17,9 @@ of two forms, picked per subset from the events each device holds
   that fills the GPU when one device's part of a subset is small (10^6/8
   events at 8 GPUs).
 
-`order="device"` first reorders every device's events by path length on the
-device with the library's own skeletons (a counting Map, a Scan of the
+`order="device"` (and `order="auto"`, the default, for parts of at least
+AUTO_ORDER_FROM events) first reorders every device's events by path length on
+the device with the library's own skeletons (a counting Map, a Scan of the
 bucket counts and a scattering Map; workloads/lmosem_order.cu): list-mode
 events carry no order and the error image is a sum over events (R10(x)), so
 the image is the same up to float rounding, and rays of similar length then
@@ -41,13 +42,17 @@ MAP_BLOCK = 128
 # events per device from which the one-thread-per-event Map beats the lanes
 # Map on length-ordered events (measured crossover between 1.25e5 and 2.5e5)
 ORDERED_LANES_BELOW = 200_000
+# order="auto": events per device from which ordering them on the device pays
+# for itself (10^6: 0.076 ms ordering + 1.15 ms Map vs 1.29 ms lanes Map in
+# the given order; 1.25e5: 0.017 + 0.170 vs 0.178 ms)
+AUTO_ORDER_FROM = 400_000
 
 
 class LMOSEM:
-    def __init__(self, ctx: skel.Context, dims=DIMS, f0: float = 1.0, order: str = "given",
+    def __init__(self, ctx: skel.Context, dims=DIMS, f0: float = 1.0, order: str = "auto",
                  lanes: int | None = None):
-        if order not in ("given", "device"):
-            raise ValueError("order must be 'given' or 'device'")
+        if order not in ("given", "device", "auto"):
+            raise ValueError("order must be 'given', 'device' or 'auto'")
         self.ctx = ctx
         self.dims = tuple(int(d) for d in dims)
         self.nvox = int(np.prod(self.dims))
@@ -60,6 +65,13 @@ class LMOSEM:
         self._hist = self._cursor = self._sorted = None
 
     # ---- policy ------------------------------------------------------------
+    def ordered(self, per_device: int) -> bool:
+        """Whether the events are ordered on the device before the Map."""
+        return self.order == "device" or (self.order == "auto" and per_device >= AUTO_ORDER_FROM)
+
+    def per_device(self, events: skel.Vector) -> int:
+        return -(-events.n // self.ctx.D) if events.distribution == skel.BLOCK else events.n
+
     def plan(self, per_device: int) -> tuple[str, int]:
         """(error-image function source, lanes) for parts of `per_device`
         events.  Given order: 4 lanes per event at every measured part size
@@ -67,7 +79,7 @@ class LMOSEM:
         1.37 / 0.727 / 0.394 / 0.211 ms with one thread per event).
         Length-ordered events: one thread per event down to ORDERED_LANES_BELOW,
         4 lanes below it (D = 1: 1.14 vs 1.26 ms; D = 8: 0.169 vs 0.175 ms)."""
-        ordered = self.order == "device"
+        ordered = self.ordered(per_device)
         lanes = self.lanes
         if lanes is None:
             lanes = 4 if (not ordered or per_device < ORDERED_LANES_BELOW) else 1
@@ -85,7 +97,7 @@ class LMOSEM:
             ctx.prepare("lanes", src)
         ctx.set_block_size(0)
         ctx.prepare("zip", LMOSEM_UPDATE)
-        if self.order == "device":
+        if self.order != "given":
             ctx.prepare("map", LMOSEM_ORDER_HIST)
             ctx.prepare("map", LMOSEM_ORDER_SCATTER)
             ctx.prepare("scan", SUM_I32)
@@ -127,8 +139,7 @@ class LMOSEM:
     def error_map(self, events: skel.Vector):
         """The error-image Map c += ... over the (already ordered) events."""
         ctx, f, c = self.ctx, self.f, self.c
-        per_device = -(-events.n // ctx.D) if events.distribution == skel.BLOCK else events.n
-        src, lanes = self.plan(per_device)
+        src, lanes = self.plan(self.per_device(events))
         ctx.set_block_size(MAP_BLOCK)
         try:
             if lanes == 1:
@@ -144,7 +155,7 @@ class LMOSEM:
         ctx, f, c = self.ctx, self.f, self.c
         f.set_distribution(skel.COPY)                     # block -> copy: all-gather (no-op after a fused tail)
         c.fill_dist(skel.COPY, np.float32(0))             # fresh zero copy on every device
-        ev = self.order_on_device(events) if self.order == "device" else events
+        ev = self.order_on_device(events) if self.ordered(self.per_device(events)) else events
         self.error_map(ev)
         c.mark_device_modified()                          # dataOnDevicesModified()
         if fused:
