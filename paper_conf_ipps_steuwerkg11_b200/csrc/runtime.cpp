@@ -1129,9 +1129,10 @@ int ew_grid(const Slot &s, size_t chunks, int block, int per_thread) {
 // module, at its first launch, by timing the policies in `mask` on a SAMPLE of
 // that launch's data copied to scratch memory -- never on the user's buffers,
 // so no user launch runs with a losing policy and nothing the user owns is
-// written twice.  The sample: 256 evenly spread blocks of the input(s), 2^21
-// elements in all (the whole vector if smaller); an index Map samples four
-// contiguous index ranges spread over [0, n).  Functions with pointer
+// written twice.  The sample: 256 evenly spread blocks of the input(s), up to
+// 256 MB of operands in all (the whole vector if smaller), each policy timed
+// three times (best of three); an index Map samples four contiguous index
+// ranges spread over [0, n).  Functions with pointer
 // (vector) arguments may have side effects and are not sampled: they take the
 // mask's lowest policy.  The lowest policy is also the default another must
 // beat by 3%.
@@ -1160,7 +1161,11 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     const uint64_t E = m->sig[8];
     const int block = (int)m->sig[9];
     const int unroll = std::max<int>(1, (int)m->sig[10]);
-    constexpr uint64_t kSample = 1ull << 21, kBlocks = 256;
+    // sample: up to 256 MB of operands -- more than the 126 MB L2, so the trials
+    // see the memory system the full launch sees (an L2-resident sample once
+    // made the scalar path look as fast as the vector path for a Zip)
+    constexpr uint64_t kSampleBytes = 256ull << 20, kBlocks = 256;
+    const uint64_t kSample = std::max<uint64_t>(kSampleBytes / std::max<size_t>(esa + esb + eso, 1), 4096);
     uint64_t ns = std::min<uint64_t>(cnt, kSample) / E * E;
     if (ns == 0) return SKEL_OK;  // decide at a larger launch
     const size_t oa = 0, ob = align_up(ns * esa, 256), oo = ob + align_up(pb ? ns * esb : 0, 256);
@@ -1190,7 +1195,8 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
         ns = blk * nblk;
         ranges.push_back({0, ns});
     }
-    cudaEvent_t ev[2 * Module::kPolicies * 2] = {};
+    constexpr int kRounds = 3;
+    cudaEvent_t ev[2 * Module::kPolicies * kRounds] = {};
     for (auto &e : ev) CK(ctx, cudaEventCreate(&e));
     auto launch = [&](int policy) -> int {
         for (auto &rg : ranges) {
@@ -1213,15 +1219,15 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
         return SKEL_OK;
     };
     TRY(launch(pol[0]));  // warm (first touch of the module on this device)
-    for (int k = 0; k < 2 * P; ++k) {
+    for (int k = 0; k < kRounds * P; ++k) {
         CK(ctx, cudaEventRecord(ev[2 * k], s.stream));
         TRY(launch(pol[k % P]));
         CK(ctx, cudaEventRecord(ev[2 * k + 1], s.stream));
     }
-    CK(ctx, cudaEventSynchronize(ev[4 * P - 1]));
+    CK(ctx, cudaEventSynchronize(ev[2 * kRounds * P - 1]));
     float best_t[Module::kPolicies];
     for (int p = 0; p < P; ++p) best_t[p] = 3.0e38f;
-    for (int k = 0; k < 2 * P; ++k) {
+    for (int k = 0; k < kRounds * P; ++k) {
         float t = 0;
         CK(ctx, cudaEventElapsedTime(&t, ev[2 * k], ev[2 * k + 1]));
         best_t[k % P] = std::min(best_t[k % P], t);
@@ -1231,7 +1237,7 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     for (int p = 1; p < P; ++p)
         if (best_t[p] < 0.97f * best_t[0] && best_t[p] < best_t[b]) b = p;
     m->ew_policy = pol[b];
-    ctx->stats.kernel_launches += (uint64_t)(2 * P + 1) * ranges.size();
+    ctx->stats.kernel_launches += (uint64_t)(kRounds * P + 1) * ranges.size();
     *policy = m->ew_policy;
     return SKEL_OK;
 }

@@ -73,6 +73,27 @@ with skel.Context(1) as ctx:
     rec.subset(rec.events(ev))
     img = rec.image()
     check(np.isfinite(img).all() and int((img != 1.0).sum()) > 1000, "lmosem subset")
+    # round 2: lanes Map (LM OSEM pieces), on-device ordering + shared-memory staged
+    # 24-byte Map, persistent Scan (cooperative) at a size above the small path
+    recd = LMOSEM(ctx, order="device", lanes=4)
+    recd.subset(recd.events(ev))
+    img2 = recd.image()
+    check(float(np.abs(img2 - img).max()) < 1e-3, "lmosem lanes + device order")
+    from paper_conf_ipps_steuwerkg11_b200.workloads import (MANDELBROT_PAIRS, MANDELBROT_PERIODIC,  # noqa: E402
+                                                            MANDELBROT_TILES)
+    pos2 = pos.view(si.POS2_DTYPE)
+    mp = ctx.vector(n=pos2.size, dtype=si.CNT2_DTYPE)
+    ctx.map(MANDELBROT_PAIRS, ctx.vector(pos2), mp, args=[np.int32(64)])
+    check(np.array_equal(mp.download().view(np.int32), mo.download()), "mandelbrot pairs")
+    ctx.map(MANDELBROT_PERIODIC, ctx.vector(pos), mo, args=[np.int32(64)])
+    img_t = ctx.vector(n=pos.size, dtype=np.int32)
+    ctx.map_index(MANDELBROT_TILES, pos.size, None, args=[img_t, np.int32(256), np.int32(192), np.int32(64)])
+    img_t.mark_device_modified()
+    check(np.array_equal(img_t.download(), mo.download()), "mandelbrot periodic + tiles")
+    big = si.uniform_int01(1 << 22, 5)
+    bo = ctx.vector(n=big.size, dtype=np.int32)
+    ctx.scan(SUM_I32, ctx.vector(big), bo, np.int32(0))
+    check(int(bo.download()[-1]) == int(big[:-1].sum()), "persistent scan (cooperative)")
 
 with skel.Context(3) as ctx:  # virtual devices: exchanges, unaligned views, fused zip_combine
     x = si.uniform_int01(N, 3)
@@ -93,4 +114,7 @@ with skel.Context(3) as ctx:  # virtual devices: exchanges, unaligned views, fus
     rec.subset(rec.events(ev), fused=True)
     img = rec.image()
     check(np.isfinite(img).all() and int((img != 1.0).sum()) > 1000, "fused zip_combine")
+    from paper_conf_ipps_steuwerkg11_b200.mandelbrot import CyclicMandelbrot  # noqa: E402
+    cyc = CyclicMandelbrot(ctx, 256, 190).counts(64)
+    check(int(cyc.max()) == 64 and cyc.size == 256 * 190, "cyclic rows (gather + un-permute)")
 print("sanitize_run: all ok")
