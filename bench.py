@@ -456,7 +456,8 @@ def main():
     # ---- end to end through the C-ABI: pinned host inputs -> every result on the host
     e2e = None
     if args.e2e_steps > 0:
-        hbuf = torch.empty(nloc, dtype=torch.float32, pin_memory=True).numpy()  # the user's result buffer
+        # the user's result buffers (pinned host memory)
+        hbufs = [torch.empty(nloc, dtype=torch.float32, pin_memory=True).numpy() for _ in range(3)]
         ctx.sync()
         barrier()
         st0 = ctx.stats()
@@ -469,18 +470,21 @@ def main():
             ctx.zip(SAXPY_F32, x, y, z, args=[a])
             ctx.scan(SUM_F32, x, s, np.float32(0))
             ctx.reduce(SUM_F32, x)  # blocking: the scalar on the host
-            for v in (m, z, s):     # this rank's block of every output vector on the host
-                v.download_part(lo, hbuf)
-        ctx.sync()
+            # this rank's block of every output vector to the host, asynchronously:
+            # the copies overlap the next step's uploads (opposite PCIe direction)
+            for v, hb in zip((m, z, s), hbufs):
+                v.download_part_async(lo, hb)
+        ctx.sync()  # every download has landed
         dt = max_over_ranks(time.perf_counter() - t0) / args.e2e_steps
         st1 = ctx.stats()
         e2e = {"value": STEP_BYTES * N / dt / 1e9, "unit": "GB/s", "ms_per_step": dt * 1e3,
                "h2d_bytes_per_step": (st1["h2d_bytes"] - st0["h2d_bytes"]) // args.e2e_steps,
                "d2h_bytes_per_step": (st1["d2h_bytes"] - st0["d2h_bytes"]) // args.e2e_steps,
                "path": "skel_vector_mark_host_modified on pinned host mirrors of x, y, then map/zip/scan/reduce "
-                       "(lazy H2D inside), skel_reduce's blocking D2H of the scalar, and skel_vector_download_part "
-                       "of the Map, Zip and Scan outputs into a pinned host buffer"}
-        del hbuf
+                       "(lazy H2D inside), skel_reduce's blocking D2H of the scalar, and "
+                       "skel_vector_download_part_async of the Map, Zip and Scan outputs into pinned host buffers "
+                       "(overlapping the next step's uploads); skel_sync after the last step"}
+        del hbufs
 
     # free the big vectors before the side measurements
     for v in (x, y, m, z, s):

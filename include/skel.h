@@ -130,7 +130,7 @@ int skel_set_block_size(skel_ctx_t ctx, int threads);
 int skel_set_cache_dir(skel_ctx_t ctx, const char *dir);
 /* Clear the in-memory kernel cache (the disk cache is kept). */
 int skel_clear_kernel_cache(skel_ctx_t ctx);
-int skel_sync(skel_ctx_t ctx);
+int skel_sync(skel_ctx_t ctx); /* waits for the main streams and every asynchronous download */
 int skel_get_stats(skel_ctx_t ctx, skel_stats *out);
 int skel_reset_stats(skel_ctx_t ctx);
 const char *skel_last_error(skel_ctx_t ctx);
@@ -174,6 +174,14 @@ int skel_vector_download(skel_vec_t v, void *dst, size_t n);
  * and not diverged, or single on rank 0), else SKEL_ERR_STATE.  Blocks.
  * SKEL_ERR_SIZE if the range is outside the vector. */
 int skel_vector_download_part(skel_vec_t v, size_t lo, void *dst, size_t count);
+/* The same without waiting: the device-to-host copies are enqueued on a
+ * per-device download stream (after everything already enqueued for v) and
+ * the call returns, so they overlap later uploads and kernels.  dst must be
+ * pinned host memory (pageable memory makes the copy synchronous) and stay
+ * valid and untouched until skel_sync; operations that write v wait for the
+ * copy on the device.  Ranges served from a valid host mirror are copied
+ * before the call returns. */
+int skel_vector_download_part_async(skel_vec_t v, size_t lo, void *dst, size_t count);
 int skel_vector_host_ptr(skel_vec_t v, void **host);
 int skel_vector_mark_host_modified(skel_vec_t v);
 int skel_vector_fill(skel_vec_t v, const void *value);

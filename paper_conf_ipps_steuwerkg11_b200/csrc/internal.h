@@ -69,6 +69,10 @@ struct Slot {
     cudaStream_t stream = nullptr;
     cudaEvent_t ev = nullptr;  // join event
     cudaEvent_t ev_scan = nullptr;  // after this slot's persistent Scan (chains slots sharing a GPU)
+    // asynchronous downloads (skel_vector_download_part_async) run on their own
+    // stream, so a D2H overlaps the next uploads and kernels of the main stream
+    cudaStream_t dl_stream = nullptr;
+    cudaEvent_t dl_ready = nullptr;  // main-stream point a download waits for
     bool ev_scan_live = false;      // ev_scan has been recorded at least once
     // grow-only workspace for reduce/scan partials, look-back status, seeds
     char *ws = nullptr;
@@ -114,6 +118,9 @@ struct Buf {  // one logical device's storage of a vector
     size_t off = 0;    // element offset of the live data inside base
     size_t count = 0;  // live elements
     char *ptr(size_t es) const { return base ? base + off * es : nullptr; }
+    // an asynchronous download still reading this buffer: writers wait for it
+    cudaEvent_t dl_done = nullptr;
+    bool dl_pending = false;
     // rank mode: every rank's `base` of this vector, opened through CUDA IPC
     std::vector<char *> peers;
     char *peers_of = nullptr;  // the local base the peer table was built for

@@ -114,6 +114,9 @@ struct DevGuard {
     explicit DevGuard(int dev) { cudaSetDevice(dev); }
 };
 
+int wait_dl(skel_vec_s *v);
+int sync_downloads(skel_ctx_s *ctx);
+
 // ---- CUDA driver entry points (VMM, multicast), resolved through the runtime ----
 struct Drv {
     PFN_cuMemCreate_v10020 create = nullptr;
@@ -247,6 +250,7 @@ int dev_free(skel_ctx_s *ctx, Slot &s, char *p) {
                                          "eagerly before capturing it");
     DevGuard g(s.dev);
     CK(ctx, cudaStreamSynchronize(s.stream));
+    if (s.dl_stream) CK(ctx, cudaStreamSynchronize(s.dl_stream));  // a download may still read it
     if (ctx->nccl_mem.count(p)) {  // rank mode: an NCCL symmetric window's buffer
         auto w = ctx->wins.find(p);
         if (w != ctx->wins.end()) {
@@ -511,6 +515,7 @@ int ensure_device(skel_vec_s *v) {
     if (v->dev_valid) return SKEL_OK;
     skel_ctx_s *ctx = v->ctx;
     if (!v->host_valid || !v->host) return fail(ctx, SKEL_ERR_STATE, "vector has no valid copy");
+    TRY(wait_dl(v));
     TRY(place(v, v->dist));
     for (size_t li = 0; li < ctx->slots.size(); ++li) {
         Slot &s = ctx->slots[li];
@@ -540,6 +545,30 @@ int sync_all(skel_ctx_s *ctx) {
         ncclResult_t ae = ncclSuccess;
         NK(ctx, ncclCommGetAsyncError(ctx->comm, &ae));
         if (ae != ncclSuccess) return fail(ctx, SKEL_ERR_NCCL, std::string("NCCL async: ") + ncclGetErrorString(ae));
+    }
+    return SKEL_OK;
+}
+
+// every asynchronous download has finished
+int sync_downloads(skel_ctx_s *ctx) {
+    for (auto &s : ctx->slots) {
+        DevGuard g(s.dev);
+        CK(ctx, cudaStreamSynchronize(s.dl_stream));
+    }
+    return SKEL_OK;
+}
+
+// v is about to be written on the main streams: wait (on the device) for any
+// asynchronous download still reading its buffers
+int wait_dl(skel_vec_s *v) {
+    skel_ctx_s *ctx = v->ctx;
+    for (size_t li = 0; li < v->bufs.size(); ++li) {
+        Buf &b = v->bufs[li];
+        if (!b.dl_pending) continue;
+        Slot &s = ctx->slots[li];
+        DevGuard g(s.dev);
+        CK(ctx, cudaStreamWaitEvent(s.stream, b.dl_done, 0));
+        b.dl_pending = false;
     }
     return SKEL_OK;
 }
@@ -876,6 +905,7 @@ int xchg_rank(skel_vec_s *v, int x, skel_combine combine) {
 
 int set_distribution(skel_vec_s *v, skel_dist dist, skel_combine combine) {
     skel_ctx_s *ctx = v->ctx;
+    TRY(wait_dl(v));  // exchanges rewrite the buffers
     const int x = plan_exchange(v->dist, dist, combine);
     if (x < 0) return fail(ctx, SKEL_ERR_STATE, "a combine merges per-device copies: the vector must be SKEL_COPY");
     if (combine != SKEL_COMBINE_NONE && v->dt == SKEL_DT_OPAQUE)
@@ -940,6 +970,7 @@ int fold_raw(skel_ctx_s *ctx, Module *m, Slot &s, const std::vector<const char *
 
 int set_distribution_fn(skel_vec_s *v, skel_dist dist, const char *src) {
     skel_ctx_s *ctx = v->ctx;
+    TRY(wait_dl(v));
     if (v->dist != SKEL_COPY) return fail(ctx, SKEL_ERR_STATE, "a combine merges per-device copies: the vector must be SKEL_COPY");
     Module *m = nullptr;
     TRY(get_module(ctx, Kind::Zip, src, &m));
@@ -1061,7 +1092,10 @@ int check_args(skel_ctx_s *ctx, const Module *m, const skel_arg *args, int nargs
         }
     }
     for (int i = 0; i < nargs; ++i)
-        if (args[i].kind == SKEL_ARG_VECTOR) TRY(ensure_device(args[i].vec));
+        if (args[i].kind == SKEL_ARG_VECTOR) {
+            TRY(ensure_device(args[i].vec));
+            TRY(wait_dl(args[i].vec));  // a side-effect Map may write it
+        }
     return SKEL_OK;
 }
 void pack_args(const Module *m, const skel_arg *args, int nargs, size_t li, std::vector<unsigned char> &buf) {
@@ -1079,6 +1113,7 @@ void pack_args(const Module *m, const skel_arg *args, int nargs, size_t li, std:
 }
 
 int prepare_output(skel_vec_s *out, size_t n, skel_dist dist, bool same_as_input) {
+    TRY(wait_dl(out));
     if (!same_as_input) {
         if (out->n != n) {  // resize: the output gets the input's length
             out->n = n;
@@ -1759,6 +1794,8 @@ static int init_slot(skel_ctx_s *ctx, int d, int dev) {
     CK(ctx, cudaStreamCreateWithFlags(&s.stream, cudaStreamNonBlocking));
     CK(ctx, cudaEventCreateWithFlags(&s.ev, cudaEventDisableTiming));
     CK(ctx, cudaEventCreateWithFlags(&s.ev_scan, cudaEventDisableTiming));
+    CK(ctx, cudaStreamCreateWithFlags(&s.dl_stream, cudaStreamNonBlocking));
+    CK(ctx, cudaEventCreateWithFlags(&s.dl_ready, cudaEventDisableTiming));
     void *p = nullptr;
     CK(ctx, cudaMalloc(&p, 256));
     CK(ctx, cudaMemsetAsync(p, 0, 256, s.stream));  // ordered with the epoch write below
@@ -1870,6 +1907,7 @@ int skel_vector_destroy(skel_vec_t v);
 int skel_finalize(skel_ctx_t ctx) {
     if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
     sync_all(ctx);
+    sync_downloads(ctx);
     std::vector<skel_vec_s *> vs(ctx->vecs.begin(), ctx->vecs.end());
     for (auto *v : vs) skel_vector_destroy(v);
     for (auto &kv : ctx->modules) {
@@ -1890,6 +1928,8 @@ int skel_finalize(skel_ctx_t ctx) {
         cudaFree(s.fl32);
         cudaEventDestroy(s.ev);
         cudaEventDestroy(s.ev_scan);
+        cudaEventDestroy(s.dl_ready);
+        cudaStreamDestroy(s.dl_stream);
         cudaStreamDestroy(s.stream);
     }
     delete ctx;
@@ -1945,7 +1985,8 @@ int skel_clear_kernel_cache(skel_ctx_t ctx) {
 int skel_sync(skel_ctx_t ctx) {
     SKEL_RANGE("skel_sync");
     if (!ctx) return fail(nullptr, SKEL_ERR_ARG, "ctx is NULL");
-    return sync_all(ctx);
+    TRY(sync_all(ctx));
+    return sync_downloads(ctx);
 }
 
 int skel_get_stats(skel_ctx_t ctx, skel_stats *out) {
@@ -1998,6 +2039,11 @@ int skel_vector_destroy(skel_vec_t v) {
     mc_release(v);
     for (auto &b : v->bufs) close_peers(b);
     for (size_t li = 0; li < v->bufs.size(); ++li) dev_free(ctx, ctx->slots[li], v->bufs[li].base);
+    for (size_t li = 0; li < v->bufs.size(); ++li)
+        if (v->bufs[li].dl_done) {
+            DevGuard g(ctx->slots[li].dev);
+            cudaEventDestroy(v->bufs[li].dl_done);
+        }
     if (v->host) cudaFreeHost(v->host);
     ctx->vecs.erase(v);
     delete v;
@@ -2086,8 +2132,19 @@ int skel_vector_download(skel_vec_t v, void *dst, size_t n) {
     return SKEL_OK;
 }
 
+namespace {
+int download_range(skel_vec_s *v, size_t lo, void *dst, size_t count, bool async);
+}
 int skel_vector_download_part(skel_vec_t v, size_t lo, void *dst, size_t count) {
     SKEL_RANGE("skel_vector_download_part");
+    return download_range(v, lo, dst, count, false);
+}
+int skel_vector_download_part_async(skel_vec_t v, size_t lo, void *dst, size_t count) {
+    SKEL_RANGE("skel_vector_download_part_async");
+    return download_range(v, lo, dst, count, true);
+}
+namespace {
+int download_range(skel_vec_s *v, size_t lo, void *dst, size_t count, bool async) {
     if (!v || (!dst && count)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad download_part arguments");
     skel_ctx_s *ctx = v->ctx;
     if (lo > v->n || count > v->n - lo) return fail(ctx, SKEL_ERR_SIZE, "range outside the vector");
@@ -2134,15 +2191,26 @@ int skel_vector_download_part(skel_vec_t v, size_t lo, void *dst, size_t count) 
     }
     for (const Piece &p : pieces) {
         Slot &s = ctx->slots[p.li];
-        const Buf &b = v->bufs[p.li];
+        Buf &b = v->bufs[p.li];
         DevGuard g(s.dev);
-        CK(ctx, cudaMemcpyAsync(static_cast<char *>(dst) + (p.lo - lo) * es, b.ptr(es) + p.src_off * es, p.cnt * es,
-                                cudaMemcpyDeviceToHost, s.stream));
+        char *to = static_cast<char *>(dst) + (p.lo - lo) * es;
+        const char *from = b.ptr(es) + p.src_off * es;
+        if (async) {  // on the download stream, after everything enqueued on the main stream so far
+            CK(ctx, cudaEventRecord(s.dl_ready, s.stream));
+            CK(ctx, cudaStreamWaitEvent(s.dl_stream, s.dl_ready, 0));
+            CK(ctx, cudaMemcpyAsync(to, from, p.cnt * es, cudaMemcpyDeviceToHost, s.dl_stream));
+            if (!b.dl_done) CK(ctx, cudaEventCreateWithFlags(&b.dl_done, cudaEventDisableTiming));
+            CK(ctx, cudaEventRecord(b.dl_done, s.dl_stream));
+            b.dl_pending = true;
+        } else {
+            CK(ctx, cudaMemcpyAsync(to, from, p.cnt * es, cudaMemcpyDeviceToHost, s.stream));
+        }
         ctx->stats.d2h_bytes += p.cnt * es;
         ctx->stats.d2h_copies++;
     }
-    return sync_all(ctx);
+    return async ? SKEL_OK : sync_all(ctx);
 }
+}  // namespace
 
 int skel_vector_host_ptr(skel_vec_t v, void **host) {
     SKEL_RANGE("skel_vector_host_ptr");
@@ -2171,6 +2239,7 @@ int skel_vector_fill_dist(skel_vec_t v, skel_dist dist, const void *value) {
     if (!v || !value || (int)dist < 0 || (int)dist > 2)
         return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad fill arguments");
     skel_ctx_s *ctx = v->ctx;
+    TRY(wait_dl(v));
     v->dist = dist;  // old contents are discarded: no exchange needed
     if (v->es > 64) return fail(ctx, SKEL_ERR_TYPE, "fill supports elements up to 64 bytes");
     TRY(place(v, v->dist));
@@ -2404,6 +2473,8 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
     TRY(check_args(ctx, m, args, nargs));
     TRY(ensure_device(a));
     TRY(ensure_device(b));
+    TRY(wait_dl(b));  // both are rewritten
+    TRY(wait_dl(out));
     const size_t n = a->n, esa = a->es, esb = b->es, eso = out->es;
     if (out != a) {
         if (out->n != n) {
@@ -2569,6 +2640,7 @@ int skel_reduce_to(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t re
             result->host = nullptr;
         }
     }
+    TRY(wait_dl(result));
     result->dist = SKEL_COPY;
     TRY(place(result, SKEL_COPY));
     std::vector<RedLayout> Ls;

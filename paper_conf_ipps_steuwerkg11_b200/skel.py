@@ -79,7 +79,7 @@ def lib() -> ctypes.CDLL:
             "skel_reset_stats": [P],
             "skel_vector_create": [P, S, S, PP], "skel_vector_destroy": [P], "skel_vector_set_dtype": [P, I],
             "skel_vector_size": [P, ctypes.POINTER(S), ctypes.POINTER(S)], "skel_vector_upload": [P, P, S],
-            "skel_vector_download": [P, P, S], "skel_vector_download_part": [P, S, P, S], "skel_vector_upload_part": [P, S, P, S], "skel_vector_host_ptr": [P, PP],
+            "skel_vector_download": [P, P, S], "skel_vector_download_part": [P, S, P, S], "skel_vector_download_part_async": [P, S, P, S], "skel_vector_upload_part": [P, S, P, S], "skel_vector_host_ptr": [P, PP],
             "skel_vector_mark_host_modified": [P], "skel_vector_fill": [P, P], "skel_vector_fill_dist": [P, I, P],
             "skel_vector_set_distribution": [P, I, I], "skel_vector_get_distribution": [P, ctypes.POINTER(I)],
             "skel_vector_set_distribution_fn": [P, I, ctypes.c_char_p],
@@ -392,6 +392,13 @@ class Vector:
         holding them; pass pinned memory for full-rate copies)."""
         assert out.dtype == self.dtype and out.flags["C_CONTIGUOUS"]
         _check(lib().skel_vector_download_part(self._h, lo, out.ctypes.data, out.size), self.ctx._h)
+        return out
+
+    def download_part_async(self, lo: int, out: np.ndarray) -> np.ndarray:
+        """As download_part, without waiting: `out` (pinned memory) is filled by the
+        time of the next ctx.sync()."""
+        assert out.dtype == self.dtype and out.flags["C_CONTIGUOUS"]
+        _check(lib().skel_vector_download_part_async(self._h, lo, out.ctypes.data, out.size), self.ctx._h)
         return out
 
     def host_view(self) -> np.ndarray:

@@ -134,3 +134,32 @@ def test_download_part_reads_the_range_from_the_devices(D, dist):
         with pytest.raises(skel.SkelError) as e:
             out.download_part(n - 2, np.empty(3, np.float32))
         assert e.value.name == "SKEL_ERR_SIZE"
+
+
+def test_download_part_async_overlaps_and_orders_writes():
+    """skel_vector_download_part_async: the copy is enqueued on the download
+    stream after everything already enqueued for the vector; a later skeleton
+    that rewrites the vector waits for it on the device (write-after-read), so
+    the host buffer holds the values as of the call; skel_sync completes it."""
+    import torch
+    n = (1 << 22) + 3
+    x = si.uniform_f32(n, 12)
+    with skel.Context(1) as ctx:
+        v = ctx.vector(x)
+        out = ctx.vector(n=n, dtype=np.float32)
+        ctx.map(MAP_F32, v, out)
+        host = torch.empty(n, dtype=torch.float32, pin_memory=True).numpy()
+        out.download_part_async(0, host)
+        for _ in range(5):  # rewrite out in place right away: must not race the copy
+            ctx.map(MAP_F32, out, out)
+        ctx.sync()
+        want = oracle.skel_map(MAP_F32, x, np.float32)
+        assert np.array_equal(host, want)
+        w = want
+        for _ in range(5):
+            w = oracle.skel_map(MAP_F32, w, np.float32)
+        assert np.array_equal(out.download(), w)
+        part = torch.empty(1000, dtype=torch.float32, pin_memory=True).numpy()
+        out.download_part_async(n - 1000, part)
+        ctx.sync()
+        assert np.array_equal(part, w[-1000:])
