@@ -329,7 +329,7 @@ def main():
     ap.add_argument("--warmup", type=int, default=5)
     ap.add_argument("--impl", default="skel", choices=["skel", "reference"])
     ap.add_argument("--log2n", type=int, default=30, help="elements per GPU (log2)")
-    ap.add_argument("--e2e-steps", type=int, default=3)
+    ap.add_argument("--e2e-steps", type=int, default=5)
     ap.add_argument("--no-extras", action="store_true", help="skip Mandelbrot / LM OSEM side measurements")
     ap.add_argument("--no-cpu", action="store_true", help="skip the cpu_baseline oracle timing")
     args = ap.parse_args()
