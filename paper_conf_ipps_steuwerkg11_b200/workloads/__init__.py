@@ -19,6 +19,8 @@ MANDELBROT_BLOCKED = source("mandelbrot_blocked")  # loop control per block of u
 MANDELBROT_PERIODIC = "#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n" + MANDELBROT_BLOCKED
 # 8 x 4 pixel tiles per warp: a void index Map writing the row-major image (NEXT-4)
 MANDELBROT_TILES = MANDELBROT_BLOCKED + source("mandelbrot_tiles")
+# the tiles with periodicity checking (coherent warps stop together: deep caps)
+MANDELBROT_TILES_PERIODIC = "#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n" + MANDELBROT_TILES
 # pairs of neighbouring pixels per element, packed FP32x2 arithmetic (NEXT-4)
 MANDELBROT_PAIRS = source("mandelbrot_pairs")
 # cyclic rows: index Map over a permuted row order (device k: rows k, k+D, ...),

@@ -172,3 +172,16 @@ def test_periodic_variant_bit_exact(golden_dir, w, h, cap, D):
         assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)
     if w * h <= 1 << 20:
         assert np.array_equal(got, oracle.mandelbrot(pos, cap))
+
+
+@pytest.mark.parametrize("w,h,cap", [(1024, 768, 256), (1024, 768, 4096), (4096, 3072, 256)])
+def test_tiles_periodic_variant_bit_exact(golden_dir, w, h, cap):
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_TILES_PERIODIC
+    with skel.Context(1) as ctx:
+        img = ctx.vector(n=w * h, dtype=np.int32)
+        ctx.map_index(MANDELBROT_TILES_PERIODIC, w * h, None, args=[img, np.int32(w), np.int32(h), np.int32(cap)])
+        img.mark_device_modified()
+        got = img.download()
+    cases = [c for c in json.load(open(os.path.join(golden_dir, "mandelbrot.json")))["cases"]
+             if (c["width"], c["height"], c["cap"]) == (w, h, cap)]
+    assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)
