@@ -48,9 +48,10 @@ struct Module {
     std::set<int> attr_set_on;  // devices on which smem attributes were set
     // element-wise grid policy (runtime.cpp ew_decide): 0 = UNROLL chunks in
     // flight per thread, 1 = one chunk per thread, 2 = one element per thread
-    // through the scalar path; -1 until decided on a sample at the first launch
+    // through the scalar path; decided on a sample at the first launch of each
+    // size class
     static constexpr int kPolicies = 3;
-    int ew_policy = -1;
+    std::map<int, int> ew_policy;  // size class (log2 of the chunk count) -> decided policy
     int red_occ = 0;  // resident Reduce CTAs per SM (0 = not yet queried)
 };
 

@@ -1160,9 +1160,10 @@ int ew_grid(const Slot &s, size_t chunks, int block, int per_thread) {
 // Element-wise grid policy of a module (Module::ew_policy): 0 = UNROLL chunks
 // in flight per thread (bandwidth-bound functions), 1 = one chunk per thread,
 // 2 = one element per thread through the scalar path (compute-bound, divergent
-// functions: finer work items even out the lanes of a warp).  Decided ONCE per
-// module, at its first launch, by timing the policies in `mask` on a SAMPLE of
-// that launch's data copied to scratch memory -- never on the user's buffers,
+// functions: finer work items even out the lanes of a warp).  Decided once per
+// module and size class (log2 of the chunk count), at the first launch of that
+// class, by timing the policies in `mask` on a SAMPLE of that launch's data
+// copied to scratch memory -- never on the user's buffers,
 // so no user launch runs with a losing policy and nothing the user owns is
 // written twice.  The sample: 256 evenly spread blocks of the input(s), up to
 // 256 MB of operands in all (the whole vector if smaller), each policy timed
@@ -1183,14 +1184,17 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     for (int p = 0; p < Module::kPolicies; ++p)
         if (mask & (1u << p)) pol[P++] = p;
     *policy = pol[0];
-    if (m->ew_policy >= 0) {
-        *policy = m->ew_policy;
+    const uint64_t E0 = std::max<uint64_t>(m->sig[8], 1);
+    const int cls = 64 - __builtin_clzll((unsigned long long)std::max<uint64_t>(cnt / E0, 1));
+    auto known = m->ew_policy.find(cls);
+    if (known != m->ew_policy.end()) {
+        *policy = known->second;
         return SKEL_OK;
     }
     cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
     cudaStreamIsCapturing(s.stream, &cs);
     if (cs != cudaStreamCaptureStatusNone || eso == 0 || has_ptr_args(m) || P < 2) {
-        if (cs == cudaStreamCaptureStatusNone) m->ew_policy = pol[0];
+        if (cs == cudaStreamCaptureStatusNone) m->ew_policy[cls] = pol[0];
         return SKEL_OK;
     }
     const uint64_t E = m->sig[8];
@@ -1271,9 +1275,9 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     int b = 0;
     for (int p = 1; p < P; ++p)
         if (best_t[p] < 0.97f * best_t[0] && best_t[p] < best_t[b]) b = p;
-    m->ew_policy = pol[b];
+    m->ew_policy[cls] = pol[b];
     ctx->stats.kernel_launches += (uint64_t)(kRounds * P + 1) * ranges.size();
-    *policy = m->ew_policy;
+    *policy = pol[b];
     return SKEL_OK;
 }
 
