@@ -21,10 +21,6 @@ MANDELBROT_PERIODIC = "#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n" + MAND
 MANDELBROT_TILES = MANDELBROT_BLOCKED + source("mandelbrot_tiles")
 # the tiles with periodicity checking (coherent warps stop together: deep caps)
 MANDELBROT_TILES_PERIODIC = "#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n" + MANDELBROT_TILES
-# persistent warps that refill finished lanes with new pixels (a void index Map
-# over one resident wave of threads, a work counter as argument; NEXT-4)
-MANDELBROT_REFILL = MANDELBROT_BLOCKED + source("mandelbrot_refill")
-MANDELBROT_REFILL_PERIODIC = "#define MANDEL_PERIODIC 1\n" + MANDELBROT_REFILL
 # pairs of neighbouring pixels per element, packed FP32x2 arithmetic (NEXT-4)
 MANDELBROT_PAIRS = source("mandelbrot_pairs")
 # cyclic rows: index Map over a permuted row order (device k: rows k, k+D, ...),

@@ -185,28 +185,3 @@ def test_tiles_periodic_variant_bit_exact(golden_dir, w, h, cap):
     cases = [c for c in json.load(open(os.path.join(golden_dir, "mandelbrot.json")))["cases"]
              if (c["width"], c["height"], c["cap"]) == (w, h, cap)]
     assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)
-
-
-@pytest.mark.parametrize("w,h,cap", [(1024, 768, 256), (4096, 3072, 256), (1024, 768, 4096), (258, 7, 50)])
-@pytest.mark.parametrize("periodic", [False, True])
-def test_refill_variant_bit_exact(golden_dir, w, h, cap, periodic):
-    """NEXT-4: persistent warps that give a finished lane the next pixel (a void
-    index Map over ~one wave of threads, a work counter vector): every pixel
-    computed once, with the counts of eq. (5) as written."""
-    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_REFILL, MANDELBROT_REFILL_PERIODIC
-    src = MANDELBROT_REFILL_PERIODIC if periodic else MANDELBROT_REFILL
-    with skel.Context(1) as ctx:
-        img = ctx.vector(n=w * h, dtype=np.int32)
-        img.fill(np.int32(-1))
-        ctr = ctx.vector(n=1, dtype=np.int32)
-        for _ in range(2):  # the counter is reset before every launch
-            ctr.fill(np.int32(0))
-            ctx.map_index(src, 148 * 1024, None, args=[img, ctr, np.int32(w), np.int32(h), np.int32(cap)])
-        img.mark_device_modified()
-        got = img.download()
-    cases = [c for c in json.load(open(os.path.join(golden_dir, "mandelbrot.json")))["cases"]
-             if (c["width"], c["height"], c["cap"]) == (w, h, cap)]
-    if cases:
-        assert zlib.crc32(got.tobytes()) == int(cases[0]["crc32"], 16)
-    if w * h <= 1 << 20:
-        assert np.array_equal(got, oracle.mandelbrot(si.mandelbrot_positions(w, h), cap))

@@ -5,7 +5,7 @@ import numpy as np
 import torch
 import skel_inputs as si
 from paper_conf_ipps_steuwerkg11_b200 import skel
-from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT, MANDELBROT_BLOCKED, MANDELBROT_PAIRS, MANDELBROT_PERIODIC, MANDELBROT_REFILL, MANDELBROT_REFILL_PERIODIC, MANDELBROT_TILES
+from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT, MANDELBROT_BLOCKED, MANDELBROT_PAIRS, MANDELBROT_PERIODIC, MANDELBROT_TILES
 
 pos = si.mandelbrot_positions(4096, 3072)
 with skel.Context(1) as ctx:
@@ -45,24 +45,6 @@ with skel.Context(1) as ctx:
         res[f"tiles_{cap}_ms"] = round(e0.elapsed_time(e1) / 10, 4)
         img.mark_device_modified()
         outs["tiles"] = img.download()
-        # persistent warps with pixel refill (plain and periodic), n threads = SMs x 1024
-        ctr = ctx.vector(n=1, dtype=np.int32)
-        nthreads = int(os.environ.get("MANDEL_THREADS", 148 * 1024))
-        for name, fn in (("refill", MANDELBROT_REFILL), ("refill_periodic", MANDELBROT_REFILL_PERIODIC)):
-            def run():
-                ctr.fill(np.int32(0))
-                ctx.map_index(fn, nthreads, None, args=[img, ctr, np.int32(4096), np.int32(3072), np.int32(cap)])
-            for _ in range(2):
-                run()
-            ctx.sync()
-            e0.record(st)
-            for _ in range(10):
-                run()
-            e1.record(st)
-            ctx.sync()
-            res[f"{name}_{cap}_ms"] = round(e0.elapsed_time(e1) / 10, 4)
-            img.mark_device_modified()
-            outs[name] = img.download()
-        res[f"same_{cap}"] = all(bool(np.array_equal(outs["paper"], outs[k])) for k in ("blocked", "pairs", "tiles", "periodic", "refill", "refill_periodic"))
+        res[f"same_{cap}"] = all(bool(np.array_equal(outs["paper"], outs[k])) for k in ("blocked", "pairs", "tiles", "periodic"))
         res[f"iters_{cap}"] = int(outs["paper"].astype(np.int64).sum())
     print(json.dumps(res))
