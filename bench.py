@@ -329,7 +329,7 @@ def main():
     ap.add_argument("--warmup", type=int, default=5)
     ap.add_argument("--impl", default="skel", choices=["skel", "reference"])
     ap.add_argument("--log2n", type=int, default=30, help="elements per GPU (log2)")
-    ap.add_argument("--e2e-steps", type=int, default=5)
+    ap.add_argument("--e2e-steps", type=int, default=8)
     ap.add_argument("--no-extras", action="store_true", help="skip Mandelbrot / LM OSEM side measurements")
     ap.add_argument("--no-cpu", action="store_true", help="skip the cpu_baseline oracle timing")
     args = ap.parse_args()
@@ -752,17 +752,31 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
     reps = max(args.steps, 10)
 
     def timed(fn, n=reps):
+        """GPU time per call: the call captured once as a CUDA graph and replayed
+        n times (a 25 us launch timed eagerly would measure the Python/ctypes call
+        rate); eager calls where graphs are unavailable."""
         for _ in range(3):
             fn()
         ctx.sync()
+        run, g = fn, None
+        if not os.environ.get("SKEL_BENCH_NO_GRAPH"):
+            try:
+                g = ctx.capture(fn)
+                g.launch()
+                ctx.sync()
+                run = g.launch
+            except skel.SkelError:
+                g, run = None, fn
         e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         barrier()
         torch.cuda.synchronize()
         e0.record(stream)
         for _ in range(n):
-            fn()
+            run()
         e1.record(stream)
         ctx.sync()
+        if g is not None:
+            g.destroy()
         return max_over_ranks(e0.elapsed_time(e1) / n)
 
     pos = si.mandelbrot_positions(W, H)
