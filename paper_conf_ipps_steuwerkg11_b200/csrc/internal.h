@@ -35,6 +35,7 @@ struct Module {
     std::string key;
     cudaLibrary_t lib = nullptr;
     cudaKernel_t k_main = nullptr;  // skel_ew_kernel | skel_reduce_kernel
+    cudaKernel_t k_main_u1 = nullptr;  // Map/Zip: one chunk in flight per thread (fewer registers)
     cudaKernel_t k_scan = nullptr;
     cudaKernel_t k_fold = nullptr;
     cudaKernel_t k_seed = nullptr;
@@ -48,9 +49,10 @@ struct Module {
     std::set<int> attr_set_on;  // devices on which smem attributes were set
     // element-wise grid policy (runtime.cpp ew_decide): 0 = UNROLL chunks in
     // flight per thread, 1 = one chunk per thread, 2 = one element per thread
-    // through the scalar path; decided on a sample at the first launch of each
-    // size class
-    static constexpr int kPolicies = 3;
+    // through the scalar path, 3 = one chunk per thread with the low-register
+    // kernel (k_main_u1); decided on a sample at the first launch of each size
+    // class
+    static constexpr int kPolicies = 4;
     std::map<int, int> ew_policy;  // size class (log2 of the chunk count) -> decided policy
     int red_occ = 0;  // resident Reduce CTAs per SM (0 = not yet queried)
 };

@@ -360,6 +360,7 @@ int get_module_slow(skel_ctx_s *ctx, Kind kind, const char *src, Module **out) {
             return SKEL_ERR_CUDA;
     } else {
         if (!getk("skel_ew_kernel", &m->k_main)) return SKEL_ERR_CUDA;
+        if ((kind == Kind::Map || kind == Kind::Zip) && !getk("skel_ew_kernel_u1", &m->k_main_u1)) return SKEL_ERR_CUDA;
         if (kind == Kind::Zip && !getk("skel_zipcomb_kernel", &m->k_zipcomb)) return SKEL_ERR_CUDA;
         if (kind == Kind::Zip && !getk("skel_zipcomb_mm_kernel", &m->k_zipcomb_mm)) return SKEL_ERR_CUDA;
     }

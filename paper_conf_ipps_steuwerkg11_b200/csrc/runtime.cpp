@@ -1160,7 +1160,9 @@ int ew_grid(const Slot &s, size_t chunks, int block, int per_thread) {
 // Element-wise grid policy of a module (Module::ew_policy): 0 = UNROLL chunks
 // in flight per thread (bandwidth-bound functions), 1 = one chunk per thread,
 // 2 = one element per thread through the scalar path (compute-bound, divergent
-// functions: finer work items even out the lanes of a warp).  Decided once per
+// functions: finer work items even out the lanes of a warp), 3 = one chunk per
+// thread with the low-register kernel (small vectors: twice the CTAs per SM,
+// so a single-wave launch).  Decided once per
 // module and size class (log2 of the chunk count), at the first launch of that
 // class, by timing the policies in `mask` on a SAMPLE of that launch's data
 // copied to scratch memory -- never on the user's buffers,
@@ -1252,7 +1254,8 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
             } else {
                 grid = policy == 2 ? ew_grid(s, n, block, 1) : ew_grid(s, chunks, block, policy == 0 ? unroll : 1);
                 void *params[] = {&qa, &qb, &qo, &n, &vk, abuf.data()};
-                CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+                const void *kf = policy == 3 ? (const void *)m->k_main_u1 : (const void *)m->k_main;
+                CK(ctx, cudaLaunchKernel(kf, dim3(grid), dim3(block), params, 0, s.stream));
             }
         }
         return SKEL_OK;
@@ -1321,13 +1324,15 @@ int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_
         // grid policy (Module::ew_policy): decided on a sample at the module's first launch
         int policy = 0;
         if (vec_ok && E > 1 && unroll > 1)
-            TRY(ew_decide(ctx, m, s, kind, pa, a->es, pb, b ? b->es : 0, rsz, cnt, 0, abuf, 0x7u, &policy));
-        // policy 2: the scalar path, one element per thread
+            TRY(ew_decide(ctx, m, s, kind, pa, a->es, pb, b ? b->es : 0, rsz, cnt, 0, abuf,
+                          m->k_main_u1 ? 0xFu : 0x7u, &policy));
+        // policy 2: the scalar path, one element per thread; 3: the low-register kernel
         int vk = policy == 2 ? 0 : vec_ok;
         const int grid = policy == 2 ? ew_grid(s, cnt, block, 1)
                                      : ew_grid(s, chunks, block, policy == 0 && vec_ok && E > 1 ? unroll : 1);
         void *params[] = {&pa, &pb, &po, &cnt, &vk, abuf.data()};
-        CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+        const void *kf = policy == 3 ? (const void *)m->k_main_u1 : (const void *)m->k_main;
+        CK(ctx, cudaLaunchKernel(kf, dim3(grid), dim3(block), params, 0, s.stream));
         ctx->stats.kernel_launches++;
     }
     if (rsz != 0) {

@@ -179,7 +179,13 @@ __device__ __forceinline__ void skel_chunk_op(const skel::chunk<skel_CA> &ca, co
 // to 64 bytes: staged through shared memory (see skel_ew_kernel)
 // (power-of-two sizes keep the direct loads: measured slower staged for the
 // 16-byte pixel pairs of mandelbrot_pairs, a compute-bound Map)
-constexpr bool skel_stage = SKEL_NIN == 1 && SKEL_E == 1 && !SKEL_LANES && sizeof(skel_A) >= 8 &&
+// A user function may turn the staging off (`#define SKEL_STAGE_ELEMS 0`): the
+// LM OSEM error-image Map, whose event load is negligible next to its walk and
+// which would pay the staging's registers in occupancy.
+#ifndef SKEL_STAGE_ELEMS
+#define SKEL_STAGE_ELEMS 1
+#endif
+constexpr bool skel_stage = SKEL_STAGE_ELEMS && SKEL_NIN == 1 && SKEL_E == 1 && !SKEL_LANES && sizeof(skel_A) >= 8 &&
                             sizeof(skel_A) % 4 == 0 && sizeof(skel_A) <= 64 && !skel::pow2(sizeof(skel_A));
 template <bool V = skel_void, class Tup>
 __device__ __forceinline__ void skel_one_val(const skel_A &x, skel_O *out, skel_u64 i, Tup &t) {
@@ -289,9 +295,13 @@ extern "C" __global__ void SKEL_EW_BOUNDS
     for (skel_u64 i = done + tid; i < n; i += stride) skel_idx_one(out, i, base, t);
 }
 #else
-extern "C" __global__ void SKEL_EW_BOUNDS
-    skel_ew_kernel(const skel_A *__restrict__ a, const skel_B *__restrict__ b, skel_O *__restrict__ out, skel_u64 n,
-                   int vec_ok, const skel_Buf args) {
+// the element-wise body with U chunks in flight per thread (U = U for
+// the main kernel; U = 1 for skel_ew_kernel_u1, which needs fewer registers and
+// so fits twice the CTAs per SM: the better grid for small vectors, whose
+// launch is a single wave -- the grid policy decides, runtime.cpp ew_decide)
+template <int U>
+__device__ __forceinline__ void skel_ew_body(const skel_A *__restrict__ a, const skel_B *__restrict__ b,
+                                             skel_O *__restrict__ out, skel_u64 n, int vec_ok, const skel_Buf &args) {
     auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
     const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;
@@ -317,38 +327,48 @@ extern "C" __global__ void SKEL_EW_BOUNDS
 #define SKEL_MAIN_UNROLL _Pragma("unroll 1")
 #endif
 #endif
+        if constexpr (U == 1) {  // one chunk in flight: the low-register kernel
+#pragma unroll 1
+            for (; c < nch; c += stride) {
+                const skel::chunk<skel_CA> ca = skel_ld<skel_CA>(pa + c * skel_CA);
+                skel::chunk<skel_CB> cb{};
+                if constexpr (SKEL_NIN == 2) cb = skel_ld<skel_CB>(pb + c * skel_CB);
+                skel_chunk_op(ca, cb, po + c * skel_CO, t);
+            }
+        } else {
         SKEL_MAIN_UNROLL
-        for (; c + (SKEL_UNROLL - 1) * stride < nch; c += SKEL_UNROLL * stride) {
-            skel::chunk<skel_CA> ca[SKEL_UNROLL];
-            skel::chunk<skel_CB> cb[SKEL_UNROLL];
+        for (; c + (U - 1) * stride < nch; c += U * stride) {
+            skel::chunk<skel_CA> ca[U];
+            skel::chunk<skel_CB> cb[U];
 #pragma unroll
-            for (int u = 0; u < SKEL_UNROLL; ++u) {
+            for (int u = 0; u < U; ++u) {
                 ca[u] = skel_ld<skel_CA>(pa + (c + u * stride) * skel_CA);
                 if constexpr (SKEL_NIN == 2) cb[u] = skel_ld<skel_CB>(pb + (c + u * stride) * skel_CB);
             }
 #pragma unroll
-            for (int u = 0; u < SKEL_UNROLL; ++u) {
+            for (int u = 0; u < U; ++u) {
                 skel_chunk_op(ca[u], cb[u], po + (c + u * stride) * skel_CO, t);
             }
         }
-        // the < SKEL_UNROLL chunks left to this thread: one predicated round, so
+        // the < U chunks left to this thread: one predicated round, so
         // their loads are in flight together (a loop would pay one memory round
         // trip per chunk -- what bounded vectors of 2^21..2^23 elements, where a
         // thread holds 2-4 chunks)
         if (c < nch) {
-            skel::chunk<skel_CA> ca[SKEL_UNROLL];
-            skel::chunk<skel_CB> cb[SKEL_UNROLL];
+            skel::chunk<skel_CA> ca[U];
+            skel::chunk<skel_CB> cb[U];
 #pragma unroll
-            for (int u = 0; u < SKEL_UNROLL; ++u) {
+            for (int u = 0; u < U; ++u) {
                 if (c + u * stride < nch) {
                     ca[u] = skel_ld<skel_CA>(pa + (c + u * stride) * skel_CA);
                     if constexpr (SKEL_NIN == 2) cb[u] = skel_ld<skel_CB>(pb + (c + u * stride) * skel_CB);
                 }
             }
 #pragma unroll
-            for (int u = 0; u < SKEL_UNROLL; ++u)
+            for (int u = 0; u < U; ++u)
                 if (c + u * stride < nch) skel_chunk_op(ca[u], cb[u], po + (c + u * stride) * skel_CO, t);
         }
+        }  // U > 1
     }
     // Elements of a size no single load covers (a 24-byte LM OSEM event): staged
     // through shared memory.  The CTA
@@ -385,6 +405,16 @@ extern "C" __global__ void SKEL_EW_BOUNDS
     // scalar path: the tail, or everything for non-vectorisable element types
 #pragma unroll 1
     for (skel_u64 i = done + tid; i < n; i += stride) skel_one(a, b, out, i, t);
+}
+extern "C" __global__ void SKEL_EW_BOUNDS
+    skel_ew_kernel(const skel_A *__restrict__ a, const skel_B *__restrict__ b, skel_O *__restrict__ out, skel_u64 n,
+                   int vec_ok, const skel_Buf args) {
+    skel_ew_body<SKEL_UNROLL>(a, b, out, n, vec_ok, args);
+}
+extern "C" __global__ void SKEL_EW_BOUNDS
+    skel_ew_kernel_u1(const skel_A *__restrict__ a, const skel_B *__restrict__ b, skel_O *__restrict__ out, skel_u64 n,
+                      int vec_ok, const skel_Buf args) {
+    skel_ew_body<1>(a, b, out, n, vec_ok, args);
 }
 #endif  // SKEL_NIN == 0
 

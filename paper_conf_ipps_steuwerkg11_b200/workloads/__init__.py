@@ -27,7 +27,8 @@ MANDELBROT_PAIRS = source("mandelbrot_pairs")
 # then an index Map that restores row-major order (NEXT-4; mandelbrot.py)
 MANDELBROT_CYCLIC = MANDELBROT_PAIRS + source("mandelbrot_cyclic")
 MANDELBROT_UNPERMUTE = source("mandelbrot_unpermute")
-LMOSEM_ERROR = source("lmosem_error")
+# (the error-image Maps keep their direct event loads: SKEL_STAGE_ELEMS 0)
+LMOSEM_ERROR = "#define SKEL_STAGE_ELEMS 0\n" + source("lmosem_error")
 # the same function for prepared (longest-path-first) event order, where the
 # Map is bound by L1TEX requests: 16-byte gathers per 4-float group in the
 # forward projection too; in the given order they are slower
@@ -39,7 +40,7 @@ LMOSEM_LANES_PREPARED = "#define LMOSEM_VEC_FWD 1\n" + LMOSEM_LANES
 LMOSEM_UPDATE = source("lmosem_update")
 # on-device ordering of a subset's events by path length (Map + Scan + Map):
 # bucket counts, then the scatter into bucket order (lmosem_order.cu)
-_ORDER = LMOSEM_ERROR + source("lmosem_order")
+_ORDER = source("lmosem_error") + source("lmosem_order")  # staged 24-byte event loads
 LMOSEM_ORDER_HIST = _ORDER + """
 void lm_order_hist(Event e, int *hist, int nx, int ny, int nz, int nb) {
     const int k = lm_slot(e, nx, ny, nz, nb);
