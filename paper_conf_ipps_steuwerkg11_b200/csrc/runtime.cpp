@@ -1207,6 +1207,15 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     // made the scalar path look as fast as the vector path for a Zip)
     constexpr uint64_t kSampleBytes = 256ull << 20, kBlocks = 256;
     const uint64_t kSample = std::max<uint64_t>(kSampleBytes / std::max<size_t>(esa + esb + eso, 1), 4096);
+    if (cnt > kSample && (mask & 8u)) {
+        // the low-register kernel is a small-vector policy: judged only where the
+        // sample IS the launch (at 2^30 a sample once preferred it by noise, 1.7%
+        // slower at full size)
+        mask &= ~8u;
+        P = 0;
+        for (int p = 0; p < Module::kPolicies; ++p)
+            if (mask & (1u << p)) pol[P++] = p;
+    }
     uint64_t ns = std::min<uint64_t>(cnt, kSample) / E * E;
     if (ns == 0) return SKEL_OK;  // decide at a larger launch
     const size_t oa = 0, ob = align_up(ns * esa, 256), oo = ob + align_up(pb ? ns * esb : 0, 256);
