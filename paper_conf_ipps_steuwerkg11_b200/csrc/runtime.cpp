@@ -1263,7 +1263,7 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
             } else {
                 grid = policy == 2 ? ew_grid(s, n, block, 1) : ew_grid(s, chunks, block, policy == 0 ? unroll : 1);
                 void *params[] = {&qa, &qb, &qo, &n, &vk, abuf.data()};
-                const void *kf = policy == 3 ? (const void *)m->k_main_u1 : (const void *)m->k_main;
+                const void *kf = (policy >= 2 && m->k_main_u1) ? (const void *)m->k_main_u1 : (const void *)m->k_main;
                 CK(ctx, cudaLaunchKernel(kf, dim3(grid), dim3(block), params, 0, s.stream));
             }
         }
@@ -1335,12 +1335,14 @@ int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_
         if (vec_ok && E > 1 && unroll > 1)
             TRY(ew_decide(ctx, m, s, kind, pa, a->es, pb, b ? b->es : 0, rsz, cnt, 0, abuf,
                           m->k_main_u1 ? 0xFu : 0x7u, &policy));
-        // policy 2: the scalar path, one element per thread; 3: the low-register kernel
+        // policy 2: the scalar path, one element per thread; 3: one chunk per thread;
+        // both through the low-register kernel (the scalar path never needs the
+        // main kernel's registers for chunks in flight)
         int vk = policy == 2 ? 0 : vec_ok;
         const int grid = policy == 2 ? ew_grid(s, cnt, block, 1)
                                      : ew_grid(s, chunks, block, policy == 0 && vec_ok && E > 1 ? unroll : 1);
         void *params[] = {&pa, &pb, &po, &cnt, &vk, abuf.data()};
-        const void *kf = policy == 3 ? (const void *)m->k_main_u1 : (const void *)m->k_main;
+        const void *kf = (policy >= 2 && m->k_main_u1) ? (const void *)m->k_main_u1 : (const void *)m->k_main;
         CK(ctx, cudaLaunchKernel(kf, dim3(grid), dim3(block), params, 0, s.stream));
         ctx->stats.kernel_launches++;
     }
