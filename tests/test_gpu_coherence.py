@@ -163,3 +163,27 @@ def test_download_part_async_overlaps_and_orders_writes():
         out.download_part_async(n - 1000, part)
         ctx.sync()
         assert np.array_equal(part, w[-1000:])
+
+
+@pytest.mark.parametrize("D", [3, 4])
+def test_download_part_async_block_parts_on_virtual_devices(D):
+    """download_part_async of a range spanning several devices' block parts:
+    one D2H per overlapping part on each device's download stream."""
+    import torch
+    n = 1_000_003
+    x = si.uniform_f32(n, 14)
+    with skel.Context(D) as ctx:
+        v = ctx.vector(x)
+        v.set_distribution(skel.BLOCK)
+        out = ctx.vector(n=n, dtype=np.float32)
+        ctx.map(MAP_F32, v, out)
+        lo, cnt = n // 7, n // 2
+        host = torch.empty(cnt, dtype=torch.float32, pin_memory=True).numpy()
+        ctx.reset_stats()
+        out.download_part_async(lo, host)
+        ctx.map(MAP_F32, out, out)  # waits for the copies on every device
+        ctx.sync()
+        assert ctx.stats()["d2h_bytes"] == 4 * cnt
+        want = oracle.skel_map(MAP_F32, x, np.float32)
+        assert np.array_equal(host, want[lo:lo + cnt])
+        assert np.array_equal(out.download(), oracle.skel_map(MAP_F32, want, np.float32))
