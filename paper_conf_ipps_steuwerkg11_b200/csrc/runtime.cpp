@@ -2166,6 +2166,8 @@ int skel_vector_download_part_async(skel_vec_t v, size_t lo, void *dst, size_t c
 namespace {
 int download_range(skel_vec_s *v, size_t lo, void *dst, size_t count, bool async) {
     if (!v || (!dst && count)) return fail(v ? v->ctx : nullptr, SKEL_ERR_ARG, "bad download_part arguments");
+    if (v->ctx->capturing)
+        return fail(v->ctx, SKEL_ERR_STATE, "downloads cannot be captured into a graph (skel_capture_begin)");
     skel_ctx_s *ctx = v->ctx;
     if (lo > v->n || count > v->n - lo) return fail(ctx, SKEL_ERR_SIZE, "range outside the vector");
     if (!count) return SKEL_OK;
