@@ -806,6 +806,9 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
     same &= np.array_equal(out2.download().view(np.int32), counts)
     ms["periodic"] = timed(lambda: ctx.map(MANDELBROT_PERIODIC, vin, out, args=[capv]))
     same &= np.array_equal(out.download(), counts)
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_PAIRS_PERIODIC
+    ms["pairs_periodic"] = timed(lambda: ctx.map(MANDELBROT_PAIRS_PERIODIC, vin2, out2, args=[capv]))
+    same &= np.array_equal(out2.download().view(np.int32), counts)
     # cyclic rows (device k: rows k, k+D, ...): the compute step alone and the
     # whole image on device 0 (gather + un-permute)
     cm = CyclicMandelbrot(ctx, W, H)

@@ -23,6 +23,7 @@ MANDELBROT_TILES = MANDELBROT_BLOCKED + source("mandelbrot_tiles")
 MANDELBROT_TILES_PERIODIC = "#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n" + MANDELBROT_TILES
 # pairs of neighbouring pixels per element, packed FP32x2 arithmetic (NEXT-4)
 MANDELBROT_PAIRS = source("mandelbrot_pairs")
+MANDELBROT_PAIRS_PERIODIC = "#define MANDEL_PERIODIC 1\n" + MANDELBROT_PAIRS  # + exact periodicity checking
 # cyclic rows: index Map over a permuted row order (device k: rows k, k+D, ...),
 # then an index Map that restores row-major order (NEXT-4; mandelbrot.py)
 MANDELBROT_CYCLIC = MANDELBROT_PAIRS + source("mandelbrot_cyclic")

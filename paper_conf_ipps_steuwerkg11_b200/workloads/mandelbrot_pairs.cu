@@ -60,6 +60,7 @@ static __forceinline__ mandel_f2 sub2(mandel_f2 a, mandel_f2 b) {
     return d;
 }
 static __forceinline__ mandel_f2 load_negzero2() { return *(volatile mandel_f2 *)&mandel_negzero2; }
+static __forceinline__ bool same2(mandel_f2 a, mandel_f2 b) { return a == b; }  // bit for bit
 #else
 // host build of this function (tests/test_workload_functions_host.py): the same
 // arithmetic one float at a time (compiled with -ffp-contract=off)
@@ -73,6 +74,15 @@ static inline mandel_f2 mul2z(mandel_f2 a, mandel_f2 b, mandel_f2 nz) {
 static inline mandel_f2 add2(mandel_f2 a, mandel_f2 b) { return mandel_f2{a.lo + b.lo, a.hi + b.hi}; }
 static inline mandel_f2 sub2(mandel_f2 a, mandel_f2 b) { return mandel_f2{a.lo - b.lo, a.hi - b.hi}; }
 static inline mandel_f2 load_negzero2() { return mandel_f2{-0.0f, -0.0f}; }
+#include <cstring>
+static inline bool same2(mandel_f2 a, mandel_f2 b) { return std::memcmp(&a, &b, sizeof a) == 0; }
+#endif
+// MANDEL_PERIODIC: exact periodicity checking for the pair (as in
+// mandelbrot_blocked.cu): after each packed block both pixels' states are
+// compared bit for bit with the states saved at block 1, 2, 4, ... (Brent's
+// schedule); if BOTH repeat, neither ever escapes and both counts are the cap
+#ifndef MANDEL_PERIODIC
+#define MANDEL_PERIODIC 0
 #endif
 
 // plain loop (eq. (5) as written) for at most `lim` updates from (x, y, n)
@@ -119,6 +129,10 @@ Cnt2 mandelbrot_pairs(Pos2 c, int cap) {
         const mandel_f2 cr = mk2(c.re0, c.re1), ci = mk2(c.im0, c.im1);
         mandel_f2 X = mk2(x0, x1), Y = mk2(y0, y1);
         int n = p;
+#if MANDEL_PERIODIC
+        mandel_f2 SX = X, SY = Y;
+        int blk = 0, next_save = 1;
+#endif
         while (n + MANDEL_PB <= cap) {
             const mandel_f2 Xs = X, Ys = Y;
             bool out0 = false, out1 = false;
@@ -138,6 +152,19 @@ Cnt2 mandelbrot_pairs(Pos2 c, int cap) {
                 break;
             }
             n += MANDEL_PB;
+#if MANDEL_PERIODIC
+            if (same2(X, SX) && same2(Y, SY)) {  // both orbits repeat exactly: members
+                Cnt2 m;
+                m.n0 = cap;
+                m.n1 = cap;
+                return m;
+            }
+            if (++blk == next_save) {
+                SX = X;
+                SY = Y;
+                next_save <<= 1;
+            }
+#endif
         }
         x0 = lo2(X);
         y0 = lo2(Y);

@@ -97,9 +97,14 @@ def test_pairs_variant_bit_exact(golden_dir, w, h, cap, D):
     """mandelbrot_pairs.cu (two neighbouring pixels per element, packed FFMA2 /
     FADD2 arithmetic with the multiplies kept unfused): the same counts as eq.
     (5) as written -- golden CRCs and the oracle, on one and on four devices."""
-    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_PAIRS
+    from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT_PAIRS, MANDELBROT_PAIRS_PERIODIC
     pos = si.mandelbrot_positions(w, h)
     pairs = pos.view(si.POS2_DTYPE)
+    for fn in (MANDELBROT_PAIRS, MANDELBROT_PAIRS_PERIODIC):
+        _pairs_check(golden_dir, w, h, cap, D, pos, pairs, fn)
+
+
+def _pairs_check(golden_dir, w, h, cap, D, pos, pairs, MANDELBROT_PAIRS):
     with skel.Context(D) as ctx:
         vin = ctx.vector(pairs)
         if D > 1:

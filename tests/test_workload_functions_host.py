@@ -263,8 +263,9 @@ extern "C" void run(const float* pos, long npairs, int cap, int* out) {
 '''
 
 
+@pytest.mark.parametrize("periodic", [False, True])
 @pytest.mark.parametrize("cap", [1, 5, 8, 9, 17, 256, 1500])
-def test_pairs_mandelbrot_equals_the_plain_iteration(tmp_path, golden_dir, cap):
+def test_pairs_mandelbrot_equals_the_plain_iteration(tmp_path, golden_dir, cap, periodic):
     """mandelbrot_pairs.cu (two neighbouring pixels per element, packed updates
     emulated one float at a time on the host): bit-identical to eq. (5) as
     written (the oracle) on the whole 1024x768 image, caps below/at/above the
@@ -273,7 +274,7 @@ def test_pairs_mandelbrot_equals_the_plain_iteration(tmp_path, golden_dir, cap):
     import os
     import zlib
     src = tmp_path / "pairs.cpp"
-    src.write_text(PAIRS_SHIM.replace(
+    src.write_text(("#define MANDEL_PERIODIC 1\n" if periodic else "") + PAIRS_SHIM.replace(
         "SRC", str(ROOT / "paper_conf_ipps_steuwerkg11_b200" / "workloads" / "mandelbrot_pairs.cu")))
     so = tmp_path / "pairs.so"
     subprocess.run(["g++", "-O2", "-std=c++17", "-ffp-contract=off", "-shared", "-fPIC", str(src), "-o", str(so)],

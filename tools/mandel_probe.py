@@ -5,7 +5,7 @@ import numpy as np
 import torch
 import skel_inputs as si
 from paper_conf_ipps_steuwerkg11_b200 import skel
-from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT, MANDELBROT_BLOCKED, MANDELBROT_PAIRS, MANDELBROT_PERIODIC, MANDELBROT_TILES
+from paper_conf_ipps_steuwerkg11_b200.workloads import MANDELBROT, MANDELBROT_BLOCKED, MANDELBROT_PAIRS, MANDELBROT_PAIRS_PERIODIC, MANDELBROT_PERIODIC, MANDELBROT_TILES
 
 pos = si.mandelbrot_positions(4096, 3072)
 with skel.Context(1) as ctx:
@@ -16,9 +16,9 @@ with skel.Context(1) as ctx:
     for cap in (256, 4096):
         outs = {}
         for name, fn in (("paper", MANDELBROT), ("blocked", MANDELBROT_BLOCKED), ("pairs", MANDELBROT_PAIRS),
-                         ("periodic", MANDELBROT_PERIODIC)):
-            v = vin2 if name == "pairs" else vin
-            out = ctx.vector(n=v.n, dtype=si.CNT2_DTYPE if name == "pairs" else np.int32)
+                         ("periodic", MANDELBROT_PERIODIC), ("pairs_periodic", MANDELBROT_PAIRS_PERIODIC)):
+            v = vin2 if name.startswith("pairs") else vin
+            out = ctx.vector(n=v.n, dtype=si.CNT2_DTYPE if name.startswith("pairs") else np.int32)
             for _ in range(2):  # first launch decides the grid policy on a sample
                 ctx.map(fn, v, out, args=[np.int32(cap)])
             ctx.sync()
@@ -45,6 +45,6 @@ with skel.Context(1) as ctx:
         res[f"tiles_{cap}_ms"] = round(e0.elapsed_time(e1) / 10, 4)
         img.mark_device_modified()
         outs["tiles"] = img.download()
-        res[f"same_{cap}"] = all(bool(np.array_equal(outs["paper"], outs[k])) for k in ("blocked", "pairs", "tiles", "periodic"))
+        res[f"same_{cap}"] = all(bool(np.array_equal(outs["paper"], outs[k])) for k in ("blocked", "pairs", "tiles", "periodic", "pairs_periodic"))
         res[f"iters_{cap}"] = int(outs["paper"].astype(np.int64).sum())
     print(json.dumps(res))
