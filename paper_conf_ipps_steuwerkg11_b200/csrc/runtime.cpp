@@ -1269,10 +1269,19 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
         }
         return SKEL_OK;
     };
-    TRY(launch(pol[0]));  // warm (first touch of the module on this device)
+    // warm every policy once (first touch of the module on this device) and time
+    // that pass, so that short launches are measured in repetitions of about
+    // 200 us (a lone 25 us launch is at the mercy of launch gaps)
+    CK(ctx, cudaEventRecord(ev[0], s.stream));
+    for (int p = 0; p < P; ++p) TRY(launch(pol[p]));
+    CK(ctx, cudaEventRecord(ev[1], s.stream));
+    CK(ctx, cudaEventSynchronize(ev[1]));
+    float warm = 0;
+    CK(ctx, cudaEventElapsedTime(&warm, ev[0], ev[1]));
+    const int reps = std::max(1, std::min(16, (int)(0.2f / std::max(warm / P, 1e-3f))));
     for (int k = 0; k < kRounds * P; ++k) {
         CK(ctx, cudaEventRecord(ev[2 * k], s.stream));
-        TRY(launch(pol[k % P]));
+        for (int r = 0; r < reps; ++r) TRY(launch(pol[k % P]));
         CK(ctx, cudaEventRecord(ev[2 * k + 1], s.stream));
     }
     CK(ctx, cudaEventSynchronize(ev[2 * kRounds * P - 1]));
@@ -1288,7 +1297,7 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     for (int p = 1; p < P; ++p)
         if (best_t[p] < 0.97f * best_t[0] && best_t[p] < best_t[b]) b = p;
     m->ew_policy[cls] = pol[b];
-    ctx->stats.kernel_launches += (uint64_t)(kRounds * P + 1) * ranges.size();
+    ctx->stats.kernel_launches += (uint64_t)(kRounds * P * reps + P) * ranges.size();
     *policy = pol[b];
     return SKEL_OK;
 }
