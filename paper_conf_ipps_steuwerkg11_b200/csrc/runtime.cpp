@@ -1219,7 +1219,12 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     uint64_t ns = std::min<uint64_t>(cnt, kSample) / E * E;
     if (ns == 0) return SKEL_OK;  // decide at a larger launch
     const size_t oa = 0, ob = align_up(ns * esa, 256), oo = ob + align_up(pb ? ns * esb : 0, 256);
-    TRY(scratch(ctx, s, oo + align_up(ns * eso, 256)));
+    const size_t per_copy = oo + align_up(ns * eso, 256);
+    // a sample smaller than L2 is replicated so that consecutive trial launches
+    // touch different copies and stream from HBM, as a user's launches on
+    // distinct vectors would (an L2-resident sample hides the memory behaviour)
+    const int copies = per_copy < (128ull << 20) ? (int)std::min<uint64_t>(16, (256ull << 20) / per_copy) : 1;
+    TRY(scratch(ctx, s, per_copy * copies));
     char *sa = s.scratch + oa, *sb = s.scratch + ob, *so = s.scratch + oo;
     DevGuard g(s.dev);
     std::vector<std::pair<uint64_t, uint64_t>> ranges;  // index Map: (base, count) per launch
@@ -1245,16 +1250,22 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
         ns = blk * nblk;
         ranges.push_back({0, ns});
     }
+    for (int k = 1; k < copies && kind != Kind::Idx; ++k) {  // the replicas of the inputs
+        CK(ctx, cudaMemcpyAsync(sa + k * per_copy, sa, ns * esa, cudaMemcpyDeviceToDevice, s.stream));
+        if (pb) CK(ctx, cudaMemcpyAsync(sb + k * per_copy, sb, ns * esb, cudaMemcpyDeviceToDevice, s.stream));
+    }
+    int rot = 0;  // the copy the next trial launch uses
     constexpr int kRounds = 3;
     cudaEvent_t ev[2 * Module::kPolicies * kRounds] = {};
     for (auto &e : ev) CK(ctx, cudaEventCreate(&e));
     auto launch = [&](int policy) -> int {
+        const size_t off = (size_t)(rot++ % copies) * per_copy;
         for (auto &rg : ranges) {
             uint64_t n = rg.second, b0 = rg.first;
             const size_t chunks = std::max<uint64_t>(n / E, 1);
             int vk = policy == 2 ? 0 : 1;
-            const void *qa = sa, *qb = pb ? (const void *)sb : nullptr;
-            void *qo = so;
+            const void *qa = sa + off, *qb = pb ? (const void *)(sb + off) : nullptr;
+            void *qo = so + off;
             int grid;
             if (kind == Kind::Idx) {
                 grid = ew_grid(s, policy == 2 ? n : chunks, block, 1);
