@@ -50,10 +50,11 @@ struct Module {
     // element-wise grid policy (runtime.cpp ew_decide): 0 = UNROLL chunks in
     // flight per thread, 1 = one chunk per thread, 2 = one element per thread
     // through the scalar path, 3 = one chunk per thread with the low-register
-    // kernel (k_main_u1); decided on a sample at the first launch of each size
-    // class
-    static constexpr int kPolicies = 4;
-    std::map<int, int> ew_policy;  // size class (log2 of the chunk count) -> decided policy
+    // kernel (k_main_u1), 4 = the scalar path through k_main_u1; decided on a
+    // sample at the first launch of each size class
+    static constexpr int kPolicies = 5;
+    // (size class = log2 of the chunk count, hash of the scalar arguments) -> decided policy
+    std::map<std::pair<int, uint64_t>, int> ew_policy;
     int red_occ = 0;  // resident Reduce CTAs per SM (0 = not yet queried)
 };
 

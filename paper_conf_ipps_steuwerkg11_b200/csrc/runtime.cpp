@@ -1162,9 +1162,9 @@ int ew_grid(const Slot &s, size_t chunks, int block, int per_thread) {
 // 2 = one element per thread through the scalar path (compute-bound, divergent
 // functions: finer work items even out the lanes of a warp), 3 = one chunk per
 // thread with the low-register kernel (small vectors: twice the CTAs per SM,
-// so a single-wave launch).  Decided once per
-// module and size class (log2 of the chunk count), at the first launch of that
-// class, by timing the policies in `mask` on a SAMPLE of that launch's data
+// so a single-wave launch), 4 = the scalar path through the low-register kernel.  Decided once per
+// module, size class (log2 of the chunk count) and set of scalar arguments (up
+// to four per class), at the first launch of that class and set, by timing the policies in `mask` on a SAMPLE of that launch's data
 // copied to scratch memory -- never on the user's buffers,
 // so no user launch runs with a losing policy and nothing the user owns is
 // written twice.  The sample: 256 evenly spread blocks of the input(s), up to
@@ -1188,15 +1188,35 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     *policy = pol[0];
     const uint64_t E0 = std::max<uint64_t>(m->sig[8], 1);
     const int cls = 64 - __builtin_clzll((unsigned long long)std::max<uint64_t>(cnt / E0, 1));
-    auto known = m->ew_policy.find(cls);
+    // the scalar arguments can change a function's cost profile (Mandelbrot's
+    // iteration cap: at 4096 the periodicity check makes the work far more
+    // uneven than at 256), so they are part of the key -- up to kArgKeys
+    // argument sets per size class; later sets reuse a decided one (no trials
+    // for a function whose argument changes at every launch)
+    constexpr int kArgKeys = 4;
+    uint64_t ah = 1469598103934665603ull;  // FNV-1a of the packed scalar arguments
+    for (unsigned char c : abuf) ah = (ah ^ c) * 1099511628211ull;
+    const auto key = std::make_pair(cls, ah);
+    auto known = m->ew_policy.find(key);
     if (known != m->ew_policy.end()) {
         *policy = known->second;
         return SKEL_OK;
     }
+    {
+        auto it = m->ew_policy.lower_bound(std::make_pair(cls, (uint64_t)0));
+        int seen = 0;
+        int first = -1;
+        for (; it != m->ew_policy.end() && it->first.first == cls; ++it, ++seen)
+            if (first < 0) first = it->second;
+        if (seen >= kArgKeys) {
+            *policy = first;
+            return SKEL_OK;
+        }
+    }
     cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
     cudaStreamIsCapturing(s.stream, &cs);
     if (cs != cudaStreamCaptureStatusNone || eso == 0 || has_ptr_args(m) || P < 2) {
-        if (cs == cudaStreamCaptureStatusNone) m->ew_policy[cls] = pol[0];
+        if (cs == cudaStreamCaptureStatusNone) m->ew_policy[key] = pol[0];
         return SKEL_OK;
     }
     const uint64_t E = m->sig[8];
@@ -1207,11 +1227,11 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     // made the scalar path look as fast as the vector path for a Zip)
     constexpr uint64_t kSampleBytes = 256ull << 20, kBlocks = 256;
     const uint64_t kSample = std::max<uint64_t>(kSampleBytes / std::max<size_t>(esa + esb + eso, 1), 4096);
-    if (cnt > kSample && (mask & 8u)) {
+    if (cnt > kSample && (mask & 24u)) {
         // the low-register kernel is a small-vector policy: judged only where the
         // sample IS the launch (at 2^30 a sample once preferred it by noise, 1.7%
         // slower at full size)
-        mask &= ~8u;
+        mask &= ~24u;
         P = 0;
         for (int p = 0; p < Module::kPolicies; ++p)
             if (mask & (1u << p)) pol[P++] = p;
@@ -1228,7 +1248,11 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     char *sa = s.scratch + oa, *sb = s.scratch + ob, *so = s.scratch + oo;
     DevGuard g(s.dev);
     std::vector<std::pair<uint64_t, uint64_t>> ranges;  // index Map: (base, count) per launch
-    if (kind == Kind::Idx) {
+    if (kind == Kind::Idx && cnt <= kSample) {
+        ranges.push_back({base, cnt});  // the trial launch is the user's launch
+    } else if (kind == Kind::Idx) {
+        // four pieces spread over the index range (a divergent function's cost
+        // varies along it, e.g. the rows of a Mandelbrot image)
         const uint64_t part = ns / 4 / E * E;
         for (int r = 0; r < 4 && part; ++r) {
             const uint64_t lo = std::min<uint64_t>(cnt - part, (cnt / 4) * r + cnt / 8 - std::min(cnt / 8, part / 2));
@@ -1263,18 +1287,19 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
         for (auto &rg : ranges) {
             uint64_t n = rg.second, b0 = rg.first;
             const size_t chunks = std::max<uint64_t>(n / E, 1);
-            int vk = policy == 2 ? 0 : 1;
+            const bool scalar = policy == 2 || policy == 4;
+            int vk = scalar ? 0 : 1;
             const void *qa = sa + off, *qb = pb ? (const void *)(sb + off) : nullptr;
             void *qo = so + off;
             int grid;
             if (kind == Kind::Idx) {
-                grid = ew_grid(s, policy == 2 ? n : chunks, block, 1);
+                grid = ew_grid(s, scalar ? n : chunks, block, 1);
                 void *params[] = {&qo, &n, &b0, &vk, abuf.data()};
                 CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
             } else {
-                grid = policy == 2 ? ew_grid(s, n, block, 1) : ew_grid(s, chunks, block, policy == 0 ? unroll : 1);
+                grid = scalar ? ew_grid(s, n, block, 1) : ew_grid(s, chunks, block, policy == 0 ? unroll : 1);
                 void *params[] = {&qa, &qb, &qo, &n, &vk, abuf.data()};
-                const void *kf = (policy >= 2 && m->k_main_u1) ? (const void *)m->k_main_u1 : (const void *)m->k_main;
+                const void *kf = policy >= 3 ? (const void *)m->k_main_u1 : (const void *)m->k_main;
                 CK(ctx, cudaLaunchKernel(kf, dim3(grid), dim3(block), params, 0, s.stream));
             }
         }
@@ -1307,7 +1332,12 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     int b = 0;
     for (int p = 1; p < P; ++p)
         if (best_t[p] < 0.97f * best_t[0] && best_t[p] < best_t[b]) b = p;
-    m->ew_policy[cls] = pol[b];
+    m->ew_policy[key] = pol[b];
+    if (getenv("SKEL_LOG")) {
+        fprintf(stderr, "[skel] grid policy, size class %d, %d x %d reps:", cls, (int)ranges.size(), reps);
+        for (int p = 0; p < P; ++p) fprintf(stderr, " p%d %.4f ms", pol[p], best_t[p] / reps);
+        fprintf(stderr, " -> p%d\n", pol[b]);
+    }
     ctx->stats.kernel_launches += (uint64_t)(kRounds * P * reps + P) * ranges.size();
     *policy = pol[b];
     return SKEL_OK;
@@ -1354,15 +1384,15 @@ int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_
         int policy = 0;
         if (vec_ok && E > 1 && unroll > 1)
             TRY(ew_decide(ctx, m, s, kind, pa, a->es, pb, b ? b->es : 0, rsz, cnt, 0, abuf,
-                          m->k_main_u1 ? 0xFu : 0x7u, &policy));
-        // policy 2: the scalar path, one element per thread; 3: one chunk per thread;
-        // both through the low-register kernel (the scalar path never needs the
-        // main kernel's registers for chunks in flight)
-        int vk = policy == 2 ? 0 : vec_ok;
-        const int grid = policy == 2 ? ew_grid(s, cnt, block, 1)
-                                     : ew_grid(s, chunks, block, policy == 0 && vec_ok && E > 1 ? unroll : 1);
+                          m->k_main_u1 ? 0x1Fu : 0x7u, &policy));
+        // policy 2: the scalar path, one element per thread; 3: one chunk per thread
+        // through the low-register kernel; 4: the scalar path through it
+        const bool scalar = policy == 2 || policy == 4;
+        int vk = scalar ? 0 : vec_ok;
+        const int grid = scalar ? ew_grid(s, cnt, block, 1)
+                                : ew_grid(s, chunks, block, policy == 0 && vec_ok && E > 1 ? unroll : 1);
         void *params[] = {&pa, &pb, &po, &cnt, &vk, abuf.data()};
-        const void *kf = (policy >= 2 && m->k_main_u1) ? (const void *)m->k_main_u1 : (const void *)m->k_main;
+        const void *kf = policy >= 3 ? (const void *)m->k_main_u1 : (const void *)m->k_main;
         CK(ctx, cudaLaunchKernel(kf, dim3(grid), dim3(block), params, 0, s.stream));
         ctx->stats.kernel_launches++;
     }
