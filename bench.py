@@ -424,10 +424,12 @@ def main():
     torch.cuda.synchronize()
     sampler.start()
     time.sleep(0.3)
+    torch.cuda.nvtx.range_push("timed")  # ncu --nvtx --nvtx-include timed/ selects the timed launches
     t_start.record(stream)
     for k in range(args.steps):
         step(evs[k])
     t_stop.record(stream)
+    torch.cuda.nvtx.range_pop()
     ctx.sync()
     torch.cuda.synchronize()
     barrier()

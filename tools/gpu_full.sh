@@ -10,8 +10,8 @@ timeout 1200 python bench.py > gpurun_out/${T}_bench.json 2> gpurun_out/${T}_ben
 timeout 600 python bench.py --impl reference --steps 3 --warmup 3 > gpurun_out/${T}_bench_ref.json 2> gpurun_out/${T}_bench_ref.err
 timeout 1200 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/${T}_launches.csv \
     python bench.py --steps 2 --warmup 3 --e2e-steps 0 --no-cpu > gpurun_out/${T}_launches_bench.json 2> gpurun_out/${T}_launches.err
-timeout 900 ncu --set full --clock-control none --import-source on -k regex:skel_ew_kernel -s 20 -c 2 \
+timeout 900 ncu --set full --clock-control none --import-source on --nvtx --nvtx-include timed/ -k regex:skel_ew_kernel -c 2 \
     -o gpurun_out/${T}_prof_ew -f python bench.py --steps 1 --warmup 3 --e2e-steps 0 --no-cpu --no-extras > gpurun_out/${T}_prof_ew.log 2>&1
-timeout 900 ncu --set full --clock-control none --import-source on -k 'regex:skel_(reduce|scan)_kernel' -s 3 -c 2 \
+timeout 900 ncu --set full --clock-control none --import-source on --nvtx --nvtx-include timed/ -k 'regex:skel_(reduce|scan)_kernel' -c 2 \
     -o gpurun_out/${T}_prof_rs -f python bench.py --steps 1 --warmup 3 --e2e-steps 0 --no-cpu --no-extras > gpurun_out/${T}_prof_rs.log 2>&1
 tail -3 gpurun_out/${T}_pytest.log; tail -2 gpurun_out/${T}_smoke.log; cut -c1-400 gpurun_out/${T}_bench.json; tail -2 gpurun_out/${T}_bench.err
