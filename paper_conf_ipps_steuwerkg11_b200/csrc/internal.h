@@ -55,6 +55,12 @@ struct Module {
     static constexpr int kPolicies = 5;
     // (size class = log2 of the chunk count, hash of the scalar arguments) -> decided policy
     std::map<std::pair<int, uint64_t>, int> ew_policy;
+    // decisions persist next to the cached cubin (<key>.policy, one line per
+    // decision: device tag, size class, argument hash, policy), so a later
+    // process -- or one under a profiler, where trial timings are meaningless --
+    // launches what an earlier one measured; empty: no disk cache
+    std::string policy_path;
+    bool policy_loaded = false;
     int red_occ = 0;  // resident Reduce CTAs per SM (0 = not yet queried)
 };
 
@@ -70,6 +76,7 @@ struct Slot {
     int d = 0;      // logical device index (0..D-1)
     int dev = 0;    // CUDA device ordinal
     int sms = 148;  // multiprocessor count
+    int cc = 100;   // compute capability, major * 10 + minor
     cudaStream_t stream = nullptr;
     cudaEvent_t ev = nullptr;  // join event
     cudaEvent_t ev_scan = nullptr;  // after this slot's persistent Scan (chains slots sharing a GPU)

@@ -334,6 +334,8 @@ int get_module_slow(skel_ctx_s *ctx, Kind kind, const char *src, Module **out) {
     auto m = std::make_unique<Module>();
     m->kind = kind;
     m->key = key;
+    if (!path.empty() && !(getenv("SKEL_POLICY_CACHE") && atoi(getenv("SKEL_POLICY_CACHE")) == 0))
+        m->policy_path = dir + "/" + key + ".policy";
     if (ctx->slots.empty()) {
         ctx->last_error = "context has no devices";
         return SKEL_ERR_STATE;

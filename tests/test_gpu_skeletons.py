@@ -391,12 +391,13 @@ def test_double_reduce_scan(ctx, n):
 
 
 @pytest.mark.parametrize("n", [(1 << 22) + 5, 1 << 24])
-def test_map_zip_grid_policy_trials_bit_identical(n):
+def test_map_zip_grid_policy_trials_bit_identical(n, tmp_path):
     """The element-wise grid policy is chosen per module and size class by timing
     the three candidates on the first launches (K1/K2): every
     launch -- trials of each policy (incl. the scalar one-element-per-thread
     path) and the decided one -- must give the same bits."""
     with skel.Context(1) as c:
+        c.set_cache_dir(str(tmp_path))  # no decisions persisted by earlier processes: trials run
         x, y = si.uniform_f32(n, 11), si.uniform_f32(n, 12)
         vx, vy = c.vector(x), c.vector(y)
         want_m = oracle.skel_map(MAP_F32, x, np.float32)
@@ -410,6 +411,48 @@ def test_map_zip_grid_policy_trials_bit_identical(n):
             assert np.array_equal(vz.download(), want_z)
             vm.destroy()
             vz.destroy()
+
+
+_POLICY_CHILD = r"""
+import sys, numpy as np
+sys.path.insert(0, {root!r})
+import skel_inputs as si
+from paper_conf_ipps_steuwerkg11_b200 import skel
+from paper_conf_ipps_steuwerkg11_b200.workloads import MAP_F32
+with skel.Context(1) as c:
+    c.set_cache_dir({cache!r})
+    x = si.uniform_f32(1 << 22, 3)
+    vx, vm = c.vector(x), c.vector(n=x.size, dtype=np.float32)
+    c.map(MAP_F32, vx, vm)
+    c.sync()
+    print("LAUNCHES", c.stats()["kernel_launches"])
+"""
+
+
+def test_grid_policy_decisions_persist_across_processes(tmp_path):
+    """A decided grid policy is written next to the cached cubin (<key>.policy)
+    and a later process takes it without trials (one launch instead of the
+    trial launches); SKEL_POLICY_CACHE=0 turns the file off."""
+    import os, re, subprocess, sys
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    code = _POLICY_CHILD.format(root=root, cache=str(tmp_path))
+
+    def run(env_extra):
+        env = dict(os.environ, SKEL_LOG="1", **env_extra)
+        r = subprocess.run([sys.executable, "-c", code], capture_output=True, text=True, env=env, timeout=300)
+        assert r.returncode == 0, r.stderr
+        return int(re.search(r"LAUNCHES (\d+)", r.stdout).group(1)), r.stderr.count("grid policy")
+
+    n1, t1 = run({})
+    assert t1 == 1 and n1 > 1  # trials, then the launch
+    files = [f for f in os.listdir(tmp_path) if f.endswith(".policy")]
+    assert len(files) == 1
+    tag, cls, _h, pol = open(tmp_path / files[0]).read().split()
+    assert tag.startswith("cc") and int(pol) in range(5) and int(cls) >= 18
+    n2, t2 = run({})
+    assert (n2, t2) == (1, 0)  # decision from the file, no trials
+    n3, t3 = run({"SKEL_POLICY_CACHE": "0"})
+    assert t3 == 1 and n3 > 1
 
 
 IDX_I64 = "long long poly(long long i, long long k){ return i * i - k * i + 7; }"
