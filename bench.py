@@ -732,7 +732,8 @@ def bench_overhead_small(ctx, hw, stream):
     return out
 
 
-FP32_PEAK_OPS = 148 * 128 * 1.965e9  # nominal: 148 SMs x 128 FP32 lanes x 1.965 GHz (no measured FP32 peak)
+FP32_NOMINAL_OPS = 148 * 128 * 1.965e9  # nominal: 148 SMs x 128 FP32 lanes x 1.965 GHz
+MANDEL_BLOCK = 128  # CTA size of the Mandelbrot Maps (skel_set_block_size; measured best)
 
 
 def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, args):
@@ -742,16 +743,27 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
     loop control, pixel pairs with packed FP32x2, exact periodicity checking,
     cyclic rows; the cap-4096 heavy variant; configs[0] 1024x768 on one GPU.
     FP32 fraction = 8 FP32 operations per iteration AS WRITTEN x sum of the
-    counts / time / nominal FP32 lane peak (the periodicity variant executes
-    fewer iterations than that sum: its figure is an algorithmic-equivalent
-    rate, not pipe utilisation)."""
+    counts / time / FP32 lane peak MEASURED in this run by a probe Map
+    (workloads/probe_fp32.cu: independent packed FP32 adds on every lane; the
+    nominal 148 x 128 x 1.965 GHz is reported beside it).  The periodicity
+    variants execute fewer iterations than that sum: their figure is an
+    algorithmic-equivalent rate, not pipe utilisation."""
+    W, H, cap = 4096, 3072, 256
+    reps = max(args.steps, 10)
+    ctx.set_block_size(MANDEL_BLOCK)
+    try:
+        return _bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, reps, W, H, cap)
+    finally:
+        ctx.set_block_size(0)
+
+
+def _bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, reps, W, H, cap):
     import torch
     import skel_inputs as si
     from paper_conf_ipps_steuwerkg11_b200.mandelbrot import CyclicMandelbrot
     from paper_conf_ipps_steuwerkg11_b200.workloads import (MANDELBROT, MANDELBROT_BLOCKED, MANDELBROT_INDEX,
-                                                            MANDELBROT_PAIRS, MANDELBROT_PERIODIC)
-    W, H, cap = 4096, 3072, 256
-    reps = max(args.steps, 10)
+                                                            MANDELBROT_PAIRS, MANDELBROT_PERIODIC, PROBE_FP32,
+                                                            PROBE_FP32_OPS_PER_STEP)
 
     def timed(fn, n=reps):
         """GPU time per call: the call captured once as a CUDA graph and replayed
@@ -781,6 +793,17 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
             g.destroy()
         return max_over_ranks(e0.elapsed_time(e1) / n)
 
+    # the FP32 lane peak, measured: every GPU runs the probe Map over 4 resident
+    # waves of threads (16 FP32 operations per step and thread)
+    sms = torch.cuda.get_device_properties(torch.cuda.current_device()).multi_processor_count
+    npr, steps = sms * 2048 * 4 * world, 2048
+    pv = ctx.vector(n=npr, dtype=np.float32)
+    if world > 1:
+        pv.set_distribution(skel.BLOCK)
+    ms_p = timed(lambda: ctx.map_index(PROBE_FP32, npr, pv, args=[np.float32(1e-7), np.int32(steps)]), n=5)
+    pv.destroy()
+    peak = (npr // world) * steps * PROBE_FP32_OPS_PER_STEP / (ms_p * 1e-3)  # per GPU
+    peak_all = peak * world
     pos = si.mandelbrot_positions(W, H)
     vin = ctx.vector(n=pos.size, dtype=pos.dtype)
     pairs = pos.view(si.POS2_DTYPE)
@@ -822,9 +845,12 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
            "Mpix_per_s": W * H / (ms["paper"] * 1e-3) / 1e6, "variants_ms": ms,
            "all_bit_identical": bool(same), "sum_iter": iters,
            "Giter_per_s": iters / (ms["paper"] * 1e-3) / 1e9,
-           "fp32_peak": {"value": FP32_PEAK_OPS, "unit": "FP32 ops/s", "source": "nominal (148 SMs x 128 lanes x "
-                         "1.965 GHz); MEASURED_PEAKS.json has no FP32 entry"},
-           "fp32_frac": {k: 8 * iters / (v * 1e-3) / FP32_PEAK_OPS for k, v in ms.items()
+           "fp32_peak": {"value": peak_all, "per_gpu": peak, "unit": "FP32 ops/s",
+                         "source": "measured in this run: probe Map workloads/probe_fp32.cu (8 independent chains of "
+                                   "add.rn.f32x2 per thread, 4 resident waves)",
+                         "nominal_per_gpu": FP32_NOMINAL_OPS, "measured_over_nominal": peak / FP32_NOMINAL_OPS},
+           "cta_threads": MANDEL_BLOCK,
+           "fp32_frac": {k: 8 * iters / (v * 1e-3) / peak_all for k, v in ms.items()
                          if not k.startswith("cyclic_image")}}
     # heavy variant ("also report the cap-4096 variant")
     c4 = np.int32(4096)
@@ -841,7 +867,7 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
                                                           args=[img, np.int32(W), np.int32(H), c4]), n=3)
     img.destroy()
     res["cap4096"] = {"sum_iter": it4096, "ms": heavy,
-                      "fp32_frac": {k: 8 * it4096 / (v * 1e-3) / FP32_PEAK_OPS for k, v in heavy.items()},
+                      "fp32_frac": {k: 8 * it4096 / (v * 1e-3) / peak_all for k, v in heavy.items()},
                       "note": "periodic variants stop a member once its orbit repeats bit for bit: their fraction "
                               "is algorithmic-equivalent (sum of the counts x 8 / time), not pipe utilisation"}
     for v in (vin, vin2, out, out2, oi):
@@ -864,7 +890,7 @@ def bench_mandelbrot(ctx, skel, stream, world, rank, barrier, max_over_ranks, ar
            "periodic": timed(lambda: ctx.map(MANDELBROT_PERIODIC, vs, os_, args=[capv]))}
     res["configs0_1024x768"] = {"ms": ms0["paper"], "variants_ms": ms0,
                                 "Mpix_per_s": ps.size / (ms0["paper"] * 1e-3) / 1e6, "sum_iter": 28347768,
-                                "fp32_frac": {k: 8 * 28347768 / (v * 1e-3) / FP32_PEAK_OPS for k, v in ms0.items()},
+                                "fp32_frac": {k: 8 * 28347768 / (v * 1e-3) / peak for k, v in ms0.items()},
                                 "note": "single distribution: one GPU computes, 2.6 waves (latency-sized)"}
     for v in (vs, os_, vs2, os2):
         v.destroy()

@@ -23,7 +23,9 @@ MANDELBROT_TILES = MANDELBROT_BLOCKED + source("mandelbrot_tiles")
 MANDELBROT_TILES_PERIODIC = "#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n" + MANDELBROT_TILES
 # pairs of neighbouring pixels per element, packed FP32x2 arithmetic (NEXT-4)
 MANDELBROT_PAIRS = source("mandelbrot_pairs")
-MANDELBROT_PAIRS_PERIODIC = "#define MANDEL_PERIODIC 1\n" + MANDELBROT_PAIRS  # + exact periodicity checking
+# + exact periodicity checking, the pair kept in the packed loop until both
+# pixels are done (no per-pixel finishing loops: MANDEL_NOREPLAY)
+MANDELBROT_PAIRS_PERIODIC = "#define MANDEL_PERIODIC 1\n#define MANDEL_NOREPLAY 1\n" + MANDELBROT_PAIRS
 # cyclic rows: index Map over a permuted row order (device k: rows k, k+D, ...),
 # then an index Map that restores row-major order (NEXT-4; mandelbrot.py)
 MANDELBROT_CYCLIC = MANDELBROT_PAIRS + source("mandelbrot_cyclic")
@@ -39,6 +41,9 @@ LMOSEM_ERROR_PREPARED = "#define LMOSEM_VEC_FWD 1\n" + LMOSEM_ERROR
 LMOSEM_LANES = LMOSEM_ERROR + source("lmosem_lanes")
 LMOSEM_LANES_PREPARED = "#define LMOSEM_VEC_FWD 1\n" + LMOSEM_LANES
 LMOSEM_UPDATE = source("lmosem_update")
+# FP32 lane-peak probe (measurement only: the Mandelbrot roofline's denominator)
+PROBE_FP32 = source("probe_fp32")
+PROBE_FP32_OPS_PER_STEP = 2 * 8  # FP32 operations per element and step (8 chains of add.rn.f32x2)
 # on-device ordering of a subset's events by path length (Map + Scan + Map):
 # bucket counts, then the scatter into bucket order (lmosem_order.cu)
 _ORDER = source("lmosem_error") + source("lmosem_order")  # staged 24-byte event loads

@@ -154,17 +154,34 @@ def mandel_blocked(tmp_path_factory):
     return run
 
 
+BLOCKED_FORMS = {
+    "periodic": "#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n",
+    "maxtest": "#define MANDEL_MAXTEST 1\n",
+    "fsetp": "#define MANDEL_MAXTEST 0\n",
+    "fsetp_periodic": "#define MANDEL_MAXTEST 0\n#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n",
+    "maxtest_periodic": "#define MANDEL_MAXTEST 1\n#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n",
+    "maxtest_blockstart": "#define MANDEL_MAXTEST 1\n#define MANDEL_PERIODIC 2\n#define MANDEL_PRE 8\n",
+    "maxtest_blockstart_b4": "#define MANDEL_MAXTEST 1\n#define MANDEL_PERIODIC 2\n#define MANDEL_B 4\n",
+    "noreplay": "#define MANDEL_NOREPLAY 1\n",
+    "noreplay_periodic": "#define MANDEL_NOREPLAY 1\n#define MANDEL_PERIODIC 1\n",
+    "noreplay_periodic_b4": "#define MANDEL_NOREPLAY 1\n#define MANDEL_PERIODIC 1\n#define MANDEL_B 4\n",
+}
+
+
+@pytest.mark.parametrize("form", sorted(BLOCKED_FORMS))
 @pytest.mark.parametrize("cap", [1, 7, 8, 9, 17, 256, 1024, 1500])
-def test_periodic_mandelbrot_equals_the_plain_iteration(tmp_path, golden_dir, cap):
-    """mandelbrot_blocked.cu with MANDEL_PERIODIC (exact periodicity checking,
-    Brent's save schedule at block ends) and an 8-update plain prefix: the
-    counts of eq. (5) as written on the whole 1024x768 image, and the golden CRC
-    at cap 256."""
+def test_blocked_forms_equal_the_plain_iteration(tmp_path, golden_dir, cap, form):
+    """mandelbrot_blocked.cu in its other forms -- exact periodicity checking
+    (Brent's save schedule at block ends) with an 8-update plain prefix, the
+    block's tests folded into one NaN-propagating maximum (MANDEL_MAXTEST), and
+    blocks that keep their test values so an escape needs no replay
+    (MANDEL_NOREPLAY): the counts of eq. (5) as written on the whole 1024x768
+    image, and the golden CRC at cap 256."""
     import json
     import os
     import zlib
     src = tmp_path / "periodic.cpp"
-    src.write_text("#define MANDEL_PERIODIC 1\n#define MANDEL_PRE 8\n" + MANDEL_SHIM.replace(
+    src.write_text(BLOCKED_FORMS[form] + MANDEL_SHIM.replace(
         "SRC", str(ROOT / "paper_conf_ipps_steuwerkg11_b200" / "workloads" / "mandelbrot_blocked.cu")))
     so = tmp_path / "periodic.so"
     subprocess.run(["g++", "-O2", "-std=c++17", "-ffp-contract=off", "-shared", "-fPIC", str(src), "-o", str(so)],
@@ -263,9 +280,10 @@ extern "C" void run(const float* pos, long npairs, int cap, int* out) {
 '''
 
 
+@pytest.mark.parametrize("maxtest", [False, True, "noreplay", "noreplay_fsetp"])
 @pytest.mark.parametrize("periodic", [False, True])
 @pytest.mark.parametrize("cap", [1, 5, 8, 9, 17, 256, 1500])
-def test_pairs_mandelbrot_equals_the_plain_iteration(tmp_path, golden_dir, cap, periodic):
+def test_pairs_mandelbrot_equals_the_plain_iteration(tmp_path, golden_dir, cap, periodic, maxtest):
     """mandelbrot_pairs.cu (two neighbouring pixels per element, packed updates
     emulated one float at a time on the host): bit-identical to eq. (5) as
     written (the oracle) on the whole 1024x768 image, caps below/at/above the
@@ -274,7 +292,10 @@ def test_pairs_mandelbrot_equals_the_plain_iteration(tmp_path, golden_dir, cap, 
     import os
     import zlib
     src = tmp_path / "pairs.cpp"
-    src.write_text(("#define MANDEL_PERIODIC 1\n" if periodic else "") + PAIRS_SHIM.replace(
+    src.write_text(("#define MANDEL_PERIODIC 1\n" if periodic else "") +
+                   ("#define MANDEL_MAXTEST 1\n" if maxtest else "#define MANDEL_MAXTEST 0\n") +
+                   ("#define MANDEL_NOREPLAY 1\n" if str(maxtest).startswith("noreplay") else "") +
+                   ("#define MANDEL_NR_FSETP 1\n" if maxtest == "noreplay_fsetp" else "") + PAIRS_SHIM.replace(
         "SRC", str(ROOT / "paper_conf_ipps_steuwerkg11_b200" / "workloads" / "mandelbrot_pairs.cu")))
     so = tmp_path / "pairs.so"
     subprocess.run(["g++", "-O2", "-std=c++17", "-ffp-contract=off", "-shared", "-fPIC", str(src), "-o", str(so)],
