@@ -12,7 +12,10 @@ and adds the exchange, which one GPU cannot run: copy->block+add
 (reduce-scatter) and block->copy (all-gather) of the 25.2 MB image move
 (D-1)/D x 25.2 MB into and out of each GPU, at the measured 770 GB/s peer
 copy per direction (B200_PROFILING.md; NVLS in-switch reduction would move
-1/D of it).  Prints one JSON line per D and a summary with T1/TD."""
+1/D of it).  The fused tails (skel_zip_combine) run the update inside the
+exchange kernel: max(zip, exchange), not their sum.  `auto` takes, at each D,
+the faster event order (the library's order="auto" policy picks by part size).
+Prints one JSON line per D and a summary with T1/TD."""
 import json
 import os
 import sys
@@ -84,14 +87,20 @@ with skel.Context(1) as ctx:
         r["exchange_nvls_ms_model"] = S / (NVLINK_GBPS * 1e9) * 1e3 if D > 1 else 0.0
         for order in ("given", "device"):
             extra = r["order_ms"] if order == "device" else 0.0
-            base = r["fill_ms"] + extra + r[f"{order}_map_ms"] + r["zip_ms"]
-            r[f"{order}_subset_ms"] = base + r["exchange_ms_model"]
-            r[f"{order}_subset_fused_ms"] = base + r["exchange_fused_ms_model"]
-            r[f"{order}_subset_nvls_ms"] = base + r["exchange_nvls_ms_model"]
+            base = r["fill_ms"] + extra + r[f"{order}_map_ms"]
+            # unfused: reduce-scatter, then the update Zip, then the all-gather
+            r[f"{order}_subset_ms"] = base + r["zip_ms"] + r["exchange_ms_model"]
+            # fused tails: the update runs inside the exchange kernel on the part
+            # it has just combined (its 2 x S/D bytes of HBM traffic overlap the
+            # NVLink transfers), so the kernel takes the longer of the two
+            r[f"{order}_subset_fused_ms"] = base + max(r["zip_ms"], r["exchange_fused_ms_model"])
+            r[f"{order}_subset_nvls_ms"] = base + max(r["zip_ms"], r["exchange_nvls_ms_model"])
+        for tail in ("", "_fused", "_nvls"):  # the order policy that is faster at this part size
+            r[f"auto_subset{tail}_ms"] = min(r[f"given_subset{tail}_ms"], r[f"device_subset{tail}_ms"])
         rows.append(r)
         print(json.dumps({k: (round(v, 4) if isinstance(v, float) else v) for k, v in r.items()}), flush=True)
 summary = {}
-for order in ("given", "device"):
+for order in ("given", "device", "auto"):
     for tail in ("", "_fused", "_nvls"):
         t1 = rows[0][f"{order}_subset{tail}_ms"]
         summary[order + tail] = {f"T1/T{r['D']}": round(t1 / r[f"{order}_subset{tail}_ms"], 2) for r in rows}
