@@ -28,7 +28,8 @@ MANDELBROT_PAIRS = source("mandelbrot_pairs")
 MANDELBROT_PAIRS_PERIODIC = "#define MANDEL_PERIODIC 1\n#define MANDEL_NOREPLAY 1\n" + MANDELBROT_PAIRS
 # cyclic rows: index Map over a permuted row order (device k: rows k, k+D, ...),
 # then an index Map that restores row-major order (NEXT-4; mandelbrot.py)
-MANDELBROT_CYCLIC = MANDELBROT_PAIRS + source("mandelbrot_cyclic")
+# (the pairs in their fastest form: lockstep packed loop with periodicity checking)
+MANDELBROT_CYCLIC = MANDELBROT_PAIRS_PERIODIC + source("mandelbrot_cyclic")
 MANDELBROT_UNPERMUTE = source("mandelbrot_unpermute")
 # (the error-image Maps keep their direct event loads: SKEL_STAGE_ELEMS 0)
 LMOSEM_ERROR = "#define SKEL_STAGE_ELEMS 0\n" + source("lmosem_error")

@@ -1,6 +1,7 @@
 #!/bin/bash
 # One gpurun call: all GPU tests, smoke, bench (default args), reference arm, the
-# bench's launch list and ncu --set full of the four skeleton kernels at 2^30.
+# bench's launch list and ncu --set full of the four skeleton kernels at 2^30 and of
+# three Mandelbrot forms (paper loop, periodic, lockstep pairs + periodic).
 cd "${GRAFT_REPO_ROOT:-/root/repo}"
 mkdir -p gpurun_out
 T=${TAG:-full}
@@ -14,4 +15,8 @@ timeout 900 ncu --set full --clock-control none --import-source on --nvtx --nvtx
     -o gpurun_out/${T}_prof_ew -f python bench.py --steps 1 --warmup 3 --e2e-steps 0 --no-cpu --no-extras > gpurun_out/${T}_prof_ew.log 2>&1
 timeout 900 ncu --set full --clock-control none --import-source on --nvtx --nvtx-include timed/ -k 'regex:skel_(reduce|scan)_kernel' -c 2 \
     -o gpurun_out/${T}_prof_rs -f python bench.py --steps 1 --warmup 3 --e2e-steps 0 --no-cpu --no-extras > gpurun_out/${T}_prof_rs.log 2>&1
+for v in paper periodic pairs_periodic; do
+  timeout 600 ncu --set full --clock-control none --import-source on -k regex:skel_ew -s 3 -c 1 \
+      -o gpurun_out/${T}_mandel_$v -f python tools/mandel_one.py $v 128 > gpurun_out/${T}_mandel_$v.log 2>&1
+done
 tail -3 gpurun_out/${T}_pytest.log; tail -2 gpurun_out/${T}_smoke.log; cut -c1-400 gpurun_out/${T}_bench.json; tail -2 gpurun_out/${T}_bench.err

@@ -8,10 +8,8 @@ import skel_inputs as si
 from paper_conf_ipps_steuwerkg11_b200 import skel
 from paper_conf_ipps_steuwerkg11_b200 import workloads as w
 
-MX = "#define MANDEL_MAXTEST 1\n"
 V = {"paper": w.MANDELBROT, "blocked": w.MANDELBROT_BLOCKED, "periodic": w.MANDELBROT_PERIODIC,
-     "periodic_max": MX + w.MANDELBROT_PERIODIC, "pairs": w.MANDELBROT_PAIRS, "pairs_max": MX + w.MANDELBROT_PAIRS,
-     "pairs_periodic_max": MX + w.MANDELBROT_PAIRS_PERIODIC}
+     "pairs": w.MANDELBROT_PAIRS, "pairs_periodic": w.MANDELBROT_PAIRS_PERIODIC}
 name = sys.argv[1]
 block = int(sys.argv[2]) if len(sys.argv) > 2 else 0
 src = V[name]
