@@ -101,6 +101,8 @@ typedef struct {
     uint64_t vmm_allocs;          /* vector buffers allocated through VMM (cuMemCreate)     */
     uint64_t mc_binds;            /* multicast objects bound to a vector's device buffers   */
     uint64_t multimem_launches;   /* fused tails run through NVSwitch multicast (multimem)  */
+    uint64_t xdev_reduces;        /* block-distributed Reduces folded across devices in the
+                                     Reduce kernels themselves (last arriver, one pass)      */
 } skel_stats;
 
 /* ---- context ------------------------------------------------------------

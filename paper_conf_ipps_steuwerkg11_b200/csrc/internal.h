@@ -154,6 +154,7 @@ struct skel_ctx_s {
     // every pair of distinct physical devices has peer access enabled (in-process
     // mode); the fused peer-memory paths need it, else they take the unfused one
     bool peer_all = true;
+    bool peer_atomics = true;  // every distinct pair has native P2P atomics (the cross-device Reduce ticket)
     // vector buffers of at least vmm_min bytes are VMM allocations (cuMemCreate,
     // exportable), so one allocation can be bound to a multicast object; rank
     // mode keeps cudaMalloc (its fused tail opens peers through CUDA IPC)

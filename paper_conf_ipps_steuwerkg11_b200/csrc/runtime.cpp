@@ -1513,6 +1513,7 @@ int win_setup(skel_ctx_s *ctx, Slot &s, skel_vec_s *v, bool *ok) {
     TRY(rank_agree(ctx, s, alloc_ok, &all));
     if (!all) {
         if (alloc_ok) ncclMemFree(p);
+        if (getenv("SKEL_LOG")) fprintf(stderr, "[skel] NCCL symmetric window: ncclMemAlloc refused on some rank\n");
         return SKEL_OK;
     }
     char *nb = static_cast<char *>(p);
@@ -1529,6 +1530,8 @@ int win_setup(skel_ctx_s *ctx, Slot &s, skel_vec_s *v, bool *ok) {
     TRY(rank_agree(ctx, s, reg_ok, &all));
     if (!all) {
         if (reg_ok) ncclCommWindowDeregister(ctx->comm, win);
+        if (getenv("SKEL_LOG"))
+            fprintf(stderr, "[skel] NCCL symmetric window: ncclCommWindowRegister refused on some rank\n");
         return SKEL_OK;  // the buffer stays an ncclMemAlloc one; peers through IPC will fail -> unfused
     }
     ncclWindow_vidmem wv;
@@ -1556,13 +1559,20 @@ int win_setup(skel_ctx_s *ctx, Slot &s, skel_vec_s *v, bool *ok) {
         if (dc->lsaMultimem.mcBasePtr)
             rec.mc = static_cast<char *>(dc->lsaMultimem.mcBasePtr) + (size_t)wv.mcOffset4K * 4096;
     }
-    // the window's own slot must be this rank's buffer
-    if (wv.lsaRank != ctx->rank || rec.peers[ctx->rank] != nb) {
+    // the window's own slot must be this rank's (the flat mapping gives every
+    // rank's buffer a second address, its own included); agreed by all ranks
+    TRY(rank_agree(ctx, s, wv.lsaRank == ctx->rank, &all));
+    if (!all) {
         ncclCommWindowDeregister(ctx->comm, win);
+        if (getenv("SKEL_LOG")) fprintf(stderr, "[skel] NCCL symmetric window: LSA rank mismatch on some rank\n");
         return SKEL_OK;
     }
     ctx->wins[nb] = rec;
     *ok = true;
+    if (getenv("SKEL_LOG"))
+        fprintf(stderr, "[skel] NCCL symmetric window: rank %d, %zu bytes (ncclMemAlloc + ncclCommWindowRegister), "
+                        "%d LSA peers, multicast %s\n",
+                ctx->rank, size, ctx->D, rec.mc ? "yes" : "no (device communicator without lsaMultimem)");
     return SKEL_OK;
 }
 
@@ -1732,8 +1742,20 @@ bool red_small(const Module *m, uint64_t cnt) {
 }
 
 // local reduce of the slot's data into dst
+// host mirror of red.cuh's skel_xdev (the cross-device single-pass Reduce);
+// K == 0: a device-local Reduce
+struct XDev {
+    void *slots = nullptr;
+    unsigned *ticket = nullptr;
+    void *dst[16] = {};
+    void *gat[16] = {};
+    int k = 0, K = 0, ndst = 0;
+};
+constexpr int kXdevMax = 16;
+constexpr int kXdevTicket = 48;  // word of Slot::counters (logical device 0) holding the arrivals
+
 int launch_reduce(skel_ctx_s *ctx, Module *m, Slot &s, const void *in, uint64_t cnt, const RedLayout &L,
-                  std::vector<unsigned char> &abuf, void *dst) {
+                  std::vector<unsigned char> &abuf, void *dst, const XDev &xd = XDev()) {
     if (red_small(m, cnt)) {
         const uint64_t ST = red_small_tile(m, cnt);
         uint64_t nt = (cnt + ST - 1) / ST;
@@ -1743,7 +1765,7 @@ int launch_reduce(skel_ctx_s *ctx, Module *m, Slot &s, const void *in, uint64_t 
         const void *kagg = red_small_big_tiles(m, cnt) ? (const void *)m->k_red_agg2 : (const void *)m->k_scan_agg;
         CK(ctx, cudaLaunchKernel(kagg, dim3((unsigned)nt), dim3((unsigned)m->sig[9]), pa, 0, s.stream));
         const void *caggs = aggs;
-        void *pf[] = {&caggs, &nt, &dst, abuf.data()};
+        void *pf[] = {&caggs, &nt, &dst, const_cast<XDev *>(&xd), abuf.data()};
         CK(ctx, cudaLaunchKernel((const void *)m->k_fold_aggs, dim3(1), dim3((unsigned)m->sig[9]), pf, 0, s.stream));
         ctx->stats.kernel_launches += 2;
         return SKEL_OK;
@@ -1758,7 +1780,8 @@ int launch_reduce(skel_ctx_s *ctx, Module *m, Slot &s, const void *in, uint64_t 
     char *ws = s.ws;
     void *partials = ws + L.o_part, *pvalid = ws + L.o_pvalid, *result = dst;
     unsigned *counter = s.counters + 2;
-    void *params[] = {&tin, &in, &cnt, &use_tma, &partials, &pvalid, &counter, &result, abuf.data()};
+    void *params[] = {&tin, &in, &cnt, &use_tma, &partials, &pvalid, &counter, &result, const_cast<XDev *>(&xd),
+                      abuf.data()};
     DevGuard g(s.dev);
     CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3((unsigned)G), dim3((unsigned)RB), params,
                              use_tma ? m->sig[11] : 0, s.stream));
@@ -1773,9 +1796,20 @@ int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args
                 std::vector<RedLayout> &Ls, void *direct = nullptr) {
     const int D = ctx->D;
     const bool cross = D > 1 && in->dist == SKEL_BLOCK;
+    const size_t es = m->sig[4];
+    const size_t ps = part_size(in->n, D);
+    const int K = cross ? (int)((in->n + ps - 1) / ps) : 1;  // devices holding data
+    // in-process devices that can all reach each other's memory: one pass, the
+    // device-order fold done by the last device to finish (red.cuh skel_xdev)
+    static const bool xdev_env = [] {
+        const char *e = getenv("SKEL_XDEV_REDUCE");  // 0: gather + fold launches instead
+        return !(e && atoi(e) == 0);
+    }();
+    const bool single = cross && !ctx->rank_mode && ctx->peer_all && ctx->peer_atomics && xdev_env && K <= kXdevMax &&
+                        ctx->slots.size() <= (size_t)kXdevMax;
     std::vector<unsigned char> abuf;
     Ls.resize(ctx->slots.size());
-    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {  // every workspace before any launch (XDev points across)
         Slot &s = ctx->slots[li];
         const uint64_t cnt = in->bufs[li].count;
         TRY(set_smem_attr(ctx, m, s));  // before the occupancy query in red_grid
@@ -1783,13 +1817,30 @@ int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args
         const size_t extra =
             red_small(m, cnt) ? (size_t)((cnt + red_small_tile(m, cnt) - 1) / red_small_tile(m, cnt)) * Ls[li].slot : 0;
         TRY(ensure_ws(ctx, s, Ls[li].total + extra));
+    }
+    XDev xd;
+    if (single) {
+        xd.slots = ctx->slots[0].ws + Ls[0].o_gather;  // room for D packed slots
+        xd.ticket = ctx->slots[0].counters + kXdevTicket;
+        xd.K = K;
+        xd.ndst = (int)ctx->slots.size();
+        for (size_t j = 0; j < ctx->slots.size(); ++j) {
+            xd.dst[j] = ctx->slots[j].ws + Ls[j].o_fold;
+            xd.gat[j] = ctx->slots[j].ws + Ls[j].o_gather;
+        }
+    }
+    for (size_t li = 0; li < ctx->slots.size(); ++li) {
+        Slot &s = ctx->slots[li];
+        const uint64_t cnt = in->bufs[li].count;
         pack_args(m, args, nargs, li, abuf);
         char *dst = cross ? s.ws + Ls[li].o_res : (direct && D == 1 ? static_cast<char *>(direct) : s.ws + Ls[li].o_fold);
-        if (cnt) TRY(launch_reduce(ctx, m, s, in->bufs[li].ptr(in->es), cnt, Ls[li], abuf, dst));
+        xd.k = s.d;
+        if (cnt) TRY(launch_reduce(ctx, m, s, in->bufs[li].ptr(in->es), cnt, Ls[li], abuf, dst, xd));
     }
-    const size_t es = m->sig[4];
-    const size_t ps = part_size(in->n, D);
-    const int K = cross ? (int)((in->n + ps - 1) / ps) : 1;  // devices holding data
+    if (single) {
+        ctx->stats.xdev_reduces++;
+        return join(ctx);  // every device after the last arriver's stores
+    }
     if (cross && !ctx->rank_mode) {
         TRY(join(ctx));
         std::vector<const void *> src0(K);
@@ -1948,6 +1999,12 @@ int skel_init(int num_devices, skel_ctx_t *out) {
                 int can = 0;
                 cudaDeviceCanAccessPeer(&can, a.dev, b.dev);
                 if (can) {
+                    int atom = 0;
+                    if (cudaDeviceGetP2PAttribute(&atom, cudaDevP2PAttrNativeAtomicSupported, a.dev, b.dev) !=
+                            cudaSuccess || !atom) {
+                        cudaGetLastError();
+                        ctx->peer_atomics = false;
+                    }
                     DevGuard g(a.dev);
                     cudaError_t pe = cudaDeviceEnablePeerAccess(b.dev, 0);
                     if (pe == cudaErrorPeerAccessAlreadyEnabled) pe = cudaSuccess;
@@ -1988,7 +2045,7 @@ int skel_init_rank(int rank, int world, int cuda_device, const void *id, skel_ct
     ctx->rank_mode = true;
     ctx->rank = rank;
     int st = init_slot(ctx, rank, cuda_device);
-    if (st == SKEL_OK && world > 1) {
+    if (st == SKEL_OK) {  // a one-rank communicator too (the fused tail's rank path uses it)
         ncclUniqueId u;
         memcpy(&u, id, sizeof u);
         DevGuard g(cuda_device);
@@ -2556,18 +2613,21 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
     // reduce-scatter + Zip + all-gather, which moves data with copies)
     // SKEL_FORCE_MULTIMEM=1 (test hook): a one-device context takes the fused
     // multicast path too (a multicast object of one device), so the NVLS
-    // kernel and the binding can be exercised on a single GPU
+    // kernel and the binding can be exercised on a single GPU -- in rank mode a
+    // one-rank communicator's fused tail (with SKEL_NCCL_WINDOWS=1: real NCCL
+    // symmetric memory on the one GPU a test box has)
     static const bool force_mm = getenv("SKEL_FORCE_MULTIMEM") && atoi(getenv("SKEL_FORCE_MULTIMEM")) != 0;
-    const bool fused = ((D > 1 && D <= 16) || (force_mm && D == 1 && !ctx->rank_mode)) &&
+    const bool fused = ((D > 1 && D <= 16) || (force_mm && D == 1)) &&
                        (a->dist == SKEL_COPY || a->dist == SKEL_BLOCK || D == 1) &&
                        (out != a || a->dist == SKEL_COPY || D == 1) && !ctx->capturing &&
                        (ctx->rank_mode || ctx->peer_all);
-    if (!fused) {  // the same result as the unfused sequence
+    auto unfused = [&]() -> int {  // the same result as the fused kernel
         if (D > 1) TRY(set_distribution(b, SKEL_BLOCK, combine));
         if (a->dist != b->dist) TRY(set_distribution(a, b->dist, SKEL_COMBINE_NONE));
         TRY(run_ew(ctx, Kind::Zip, src, a, b, out, args, nargs));
         return D > 1 ? set_distribution(out, SKEL_COPY, SKEL_COMBINE_NONE) : SKEL_OK;
-    }
+    };
+    if (!fused) return unfused();
     Module *m = nullptr;
     TRY(get_module(ctx, Kind::Zip, src, &m));
     if (m->sig[4] != a->es || m->sig[5] != b->es)
@@ -2675,6 +2735,10 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
         const WinRec *wrb = win ? &ctx->wins[b->bufs[0].base] : nullptr;
         const WinRec *wro = win ? &ctx->wins[out->bufs[0].base] : nullptr;
         if (!win) {
+            // a buffer that moved into ncclMemAlloc memory for a window NCCL then
+            // declined has no CUDA IPC handle: the unfused sequence (every rank
+            // decides alike -- the window outcomes were agreed)
+            if (ctx->nccl_mem.count(b->bufs[0].base) || ctx->nccl_mem.count(out->bufs[0].base)) return unfused();
             TRY(ipc_peers(ctx, s, b->bufs[0]));
             TRY(ipc_peers(ctx, s, out->bufs[0]));
         }

@@ -270,6 +270,38 @@ template <class T> __device__ __forceinline__ void st_value(T *p, const T &v) {
 #pragma unroll
     for (int i = 0; i < W; ++i) st_relaxed_u32(q + i, a.w[i]);
 }
+// system scope: values and counters that other GPUs read or write over NVLink
+// (the cross-device single-pass Reduce, red.cuh skel_xdev_finish)
+__device__ __forceinline__ void fence_acq_rel_sys() { asm volatile("fence.acq_rel.sys;" ::: "memory"); }
+__device__ __forceinline__ unsigned atom_add_acq_rel_sys(unsigned *p, unsigned v) {
+    unsigned r;
+    asm volatile("atom.acq_rel.sys.global.add.u32 %0, [%1], %2;" : "=r"(r) : "l"(p), "r"(v) : "memory");
+    return r;
+}
+__device__ __forceinline__ void st_relaxed_sys_u32(unsigned *p, unsigned v) {
+    asm volatile("st.relaxed.sys.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+__device__ __forceinline__ unsigned ld_relaxed_sys_u32(const unsigned *p) {
+    unsigned v;
+    asm volatile("ld.relaxed.sys.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+    return v;
+}
+template <class T> __device__ __forceinline__ void st_value_sys(T *p, const T &v) {
+    constexpr int W = (int)((sizeof(T) + 3) / 4);
+    union U { T t; unsigned w[W]; U() {} } a;
+    a.t = v;
+    unsigned *q = reinterpret_cast<unsigned *>(p);
+#pragma unroll
+    for (int i = 0; i < W; ++i) st_relaxed_sys_u32(q + i, a.w[i]);
+}
+template <class T> __device__ __forceinline__ T ld_value_sys(const T *p) {
+    constexpr int W = (int)((sizeof(T) + 3) / 4);
+    union U { T t; unsigned w[W]; U() {} } a;
+    const unsigned *q = reinterpret_cast<const unsigned *>(p);
+#pragma unroll
+    for (int i = 0; i < W; ++i) a.w[i] = ld_relaxed_sys_u32(q + i);
+    return a.t;
+}
 template <class T> __device__ __forceinline__ T ld_value(const T *p) {
     constexpr int W = (int)((sizeof(T) + 3) / 4);
     union U { T t; unsigned w[W]; U() {} } a;

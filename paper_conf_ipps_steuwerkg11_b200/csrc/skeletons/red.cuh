@@ -432,9 +432,48 @@ __device__ __forceinline__ VT reduce_direct(const skel_T *__restrict__ in, skel_
     return r;
 }
 
+// ---- cross-device single pass --
+// A block-distributed Reduce over K in-process devices without a separate
+// exchange: the one thread that ends a device's Reduce publishes the device's
+// result into slot k of an array in logical device 0's memory (over NVLink
+// for another GPU), then takes a ticket from a counter there (release/acquire
+// at system scope).  The device that draws the last ticket folds the K
+// published values IN DEVICE ORDER (eq. (3) with a non-commutative operator
+// stays exact) and stores the result into every device's result slot, then
+// resets the counter.  Nobody waits for anybody -- the last arriver does the
+// fold -- so kernels of logical devices that share one GPU cannot deadlock.
+// It also copies the K device results to every device (a block-distributed
+// Scan seeds device k with results 0..k-1).  The host joins the devices' streams after the launches (every later use,
+// and the next Reduce's tickets, come after the last arriver's stores).
+#define SKEL_XMAX 16
+struct skel_xdev {
+    skel_S *slots;           // K published device results (logical device 0's memory)
+    unsigned *ticket;        // arrivals (logical device 0's memory)
+    skel_S *dst[SKEL_XMAX];  // result slot of every local device
+    skel_S *gat[SKEL_XMAX];  // every local device's copy of the K device results (the
+                             // cross-device Scan seeds device k from results 0..k-1)
+    int k, K, ndst;          // this device, devices holding data, local devices
+};
+template <class Tup> __device__ __forceinline__ void skel_xdev_finish(const skel_xdev &xd, const skel_T &v, Tup &tup) {
+    skel::st_value_sys(&xd.slots[xd.k], skel_S{v});
+    skel::fence_acq_rel_sys();  // the value before the ticket
+    const unsigned prev = skel::atom_add_acq_rel_sys(xd.ticket, 1u);
+    if (prev != (unsigned)(xd.K - 1)) return;
+    skel::fence_acq_rel_sys();  // every device's value after its ticket
+    skel_T acc = skel::ld_value_sys(&xd.slots[0]).v;
+    for (int j = 1; j < xd.K; ++j) acc = opf(acc, skel::ld_value_sys(&xd.slots[j]).v, tup);
+    for (int d = 0; d < xd.ndst; ++d) {
+        skel::st_value_sys(xd.dst[d], skel_S{acc});
+        if (xd.gat[d] != xd.slots)
+            for (int j = 0; j < xd.K; ++j) skel::st_value_sys(&xd.gat[d][j], skel::ld_value_sys(&xd.slots[j]));
+    }
+    skel::st_relaxed_sys_u32(xd.ticket, 0u);
+}
+
 extern "C" __global__ void __launch_bounds__(RB, SKEL_RED_MINB)
     skel_reduce_kernel(const __grid_constant__ skel_tmap tin, const skel_T *__restrict__ in, skel_u64 n, int use_tma,
-                       skel_S *partials, unsigned *pvalid, unsigned *counter, skel_S *result, const skel_Buf args) {
+                       skel_S *partials, unsigned *pvalid, unsigned *counter, skel_S *result,
+                       const __grid_constant__ skel_xdev xd, const skel_Buf args) {
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     __shared__ skel_u64 bars[STAGES];
     __shared__ VT wpart[NW];
@@ -554,6 +593,7 @@ extern "C" __global__ void __launch_bounds__(RB, SKEL_RED_MINB)
         if (t == 0) {
             result->v = r.v;
             *counter = 0;
+            if (xd.K) skel_xdev_finish(xd, r.v, tup);
         }
     }
 }
@@ -1301,7 +1341,8 @@ extern "C" __global__ void __launch_bounds__(RB)
 // one-CTA ordered fold of them (two short launches instead of the TMA ring
 // and the last-CTA handshake)
 extern "C" __global__ void __launch_bounds__(RB)
-    skel_fold_aggs_kernel(const skel_S *aggs, skel_u64 count, skel_S *out, const skel_Buf args) {
+    skel_fold_aggs_kernel(const skel_S *aggs, skel_u64 count, skel_S *out, const __grid_constant__ skel_xdev xd,
+                          const skel_Buf args) {
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     __shared__ VT wpart[NW];
     const int t = threadIdx.x;
@@ -1320,5 +1361,8 @@ extern "C" __global__ void __launch_bounds__(RB)
         for (int u = 0; u < 8; ++u) a = comb(a, e[u], tup);
     }
     const VT r = block_fold(a, wpart, tup);
-    if (t == 0) out->v = r.v;
+    if (t == 0) {
+        out->v = r.v;
+        if (xd.K) skel_xdev_finish(xd, r.v, tup);
+    }
 }

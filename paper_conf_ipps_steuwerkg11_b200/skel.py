@@ -48,7 +48,8 @@ class Stats(ctypes.Structure):
                 ("compile_disk_hits", ctypes.c_uint64), ("compile_misses", ctypes.c_uint64),
                 ("compile_ms", ctypes.c_double), ("disk_load_ms", ctypes.c_double),
                 ("scan_coop_fallbacks", ctypes.c_uint64), ("vmm_allocs", ctypes.c_uint64),
-                ("mc_binds", ctypes.c_uint64), ("multimem_launches", ctypes.c_uint64)]
+                ("mc_binds", ctypes.c_uint64), ("multimem_launches", ctypes.c_uint64),
+                ("xdev_reduces", ctypes.c_uint64)]
 
     def asdict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}

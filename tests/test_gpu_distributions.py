@@ -333,3 +333,73 @@ def test_user_combine_errors():
         with pytest.raises(skel.SkelError) as e:
             v.set_distribution(skel.BLOCK, "int f(int a, int b, int k){ return a + b + k; }")
         assert e.value.status == 3  # SKEL_ERR_TYPE
+
+
+@pytest.mark.parametrize("D", [2, 3, 8])
+def test_cross_device_reduce_single_pass(D):
+    """A block-distributed Reduce over in-process devices folds the device
+    results inside the Reduce kernels (the last device to finish folds them
+    in device order): counted by xdev_reduces, exact for a
+    non-commutative operator, its arrival counter reset for the next Reduce
+    (40 in a row, sizes on both the small and the TMA path) and across CUDA
+    graph replays of a reduce_to."""
+    src = """
+    struct A { unsigned m, c; };
+    A affine(A x, A y) { A r; r.m = x.m * y.m; r.c = x.c * y.m + y.c; return r; }"""
+    AF = np.dtype([("m", np.uint32), ("c", np.uint32)])
+    g = np.random.default_rng(D)
+    with skel.Context(D) as ctx:
+        x0 = ctx.stats()["xdev_reduces"]
+        for i in range(40):
+            n = [7, 1000, 300_007, 5_000_011][i % 4]
+            a = np.zeros(n, AF)
+            a["m"] = g.integers(0, 1 << 32, n, dtype=np.uint64).astype(np.uint32)
+            a["c"] = g.integers(0, 1 << 32, n, dtype=np.uint64).astype(np.uint32)
+            v = ctx.vector(a)
+            v.set_distribution(skel.BLOCK)
+            assert ctx.reduce(src, v).tobytes() == oracle.skel_reduce(src, a).tobytes(), (i, n)
+            v.destroy()
+        assert ctx.stats()["xdev_reduces"] - x0 == 40
+        x = si.uniform_int01(2_000_003, 77)
+        v = ctx.vector(x)
+        v.set_distribution(skel.BLOCK)
+        r = ctx.vector(n=1, dtype=np.int32)
+        ctx.reduce_to(SUM_I32, v, r)  # eager first: workspaces are sized outside the capture
+        ctx.sync()
+        gr = ctx.capture(lambda: ctx.reduce_to(SUM_I32, v, r))
+        for _ in range(20):
+            gr.launch()
+            ctx.sync()
+            r.mark_device_modified()
+            assert int(r.download()[0]) == int(x.sum())
+        gr.destroy()
+
+
+def test_cross_device_reduce_single_pass_matches_the_two_step_exchange():
+    """SKEL_XDEV_REDUCE=0 (gather of the device results + fold launches) and
+    the single pass give bit-identical integer and ordered results."""
+    import subprocess
+    import sys
+    from pathlib import Path
+    code = r'''
+import sys; sys.path.insert(0, ".")
+import numpy as np, skel_inputs as si
+from paper_conf_ipps_steuwerkg11_b200 import skel
+from paper_conf_ipps_steuwerkg11_b200.workloads import SUM_I32
+x = si.uniform_int01(1_000_003, 5)
+with skel.Context(4) as ctx:
+    v = ctx.vector(x); v.set_distribution(skel.BLOCK)
+    o = ctx.vector(n=x.size, dtype=np.int32)
+    ctx.scan(SUM_I32, v, o, np.int32(0))
+    print(int(ctx.reduce(SUM_I32, v)), int(o.download()[-1]), ctx.stats()["xdev_reduces"])
+'''
+    root = Path(__file__).resolve().parents[1]
+    outs = {}
+    for flag in ("0", "1"):
+        env = dict(__import__("os").environ, SKEL_XDEV_REDUCE=flag)
+        r = subprocess.run([sys.executable, "-c", code], capture_output=True, text=True, cwd=str(root), env=env,
+                           timeout=300)
+        assert r.returncode == 0, r.stderr[-2000:]
+        outs[flag] = r.stdout.split()
+    assert outs["0"][:2] == outs["1"][:2]
+    assert outs["0"][2] == "0" and int(outs["1"][2]) >= 2  # the Scan's device results come through it too

@@ -82,3 +82,33 @@ def test_rank_mode_nccl_windows_fall_back(fake_nccl):
     assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-3000:]
     oks = re.findall(r"rank (\d+)/\d+ device \d+: OK", r.stdout)
     assert sorted(map(int, oks)) == [0, 1], r.stdout[-2000:]
+
+
+def real_nccl_run(nproc, script_args, timeout=300, extra_env=None):
+    """torchrun WITHOUT the stand-in: the ranks load the real NCCL (the one
+    libskel links).  One GPU, so one rank: NCCL refuses two ranks on a device."""
+    env = dict(os.environ, SKEL_TEST_DEVICE="0", SKEL_BENCH_BACKEND="gloo")
+    env.pop("LD_PRELOAD", None)
+    env.update(extra_env or {})
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", "--nproc-per-node", str(nproc),
+           "--master-addr", "127.0.0.1", "--master-port", str(free_port()), *script_args]
+    return subprocess.run(cmd, capture_output=True, text=True, timeout=timeout, cwd=str(ROOT), env=env)
+
+
+@pytest.mark.parametrize("windows", ["0", "1"])
+def test_rank_mode_real_nccl_one_rank(windows):
+    """The rank path on the REAL NCCL library with a one-rank communicator
+    (ncclCommInitRank): the self-test's skeletons and transitions, and LM OSEM's
+    fused tail forced onto the rank path (SKEL_FORCE_MULTIMEM=1) -- its
+    ncclAllGather of the CUDA IPC handles and ncclAllReduce barriers, or with
+    SKEL_NCCL_WINDOWS=1 ncclMemAlloc + ncclCommWindowRegister(
+    NCCL_WIN_COLL_SYMMETRIC) + ncclDevCommCreate for the tail's vectors (or the
+    ranks' agreed fallback when NCCL declines) -- checked against the oracle."""
+    # SKEL_FORCE_MULTIMEM=1: a one-rank communicator takes the fused tail too
+    r = real_nccl_run(1, ["tools/rank_selftest.py"],
+                      extra_env={"SKEL_NCCL_WINDOWS": windows, "SKEL_LOG": "1", "SKEL_FORCE_MULTIMEM": "1"})
+    assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-3000:]
+    assert re.search(r"rank 0/1 device \d+: OK", r.stdout), r.stdout[-2000:] + r.stderr[-2000:]
+    if windows == "1":  # the outcome of the window set-up is logged either way
+        assert "NCCL symmetric window" in r.stderr, r.stderr[-2000:]
+        print([ln for ln in r.stderr.splitlines() if "NCCL symmetric window" in ln][:2])

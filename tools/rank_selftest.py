@@ -87,10 +87,16 @@ for dst in (skel.BLOCK, skel.SINGLE, skel.COPY):
     ctx.map("void mark(int i, int* c){ c[i] = (i * 7919) % 1000 - 500; }", idx, None, args=[c])
     c.mark_device_modified()
     c.set_distribution(dst, MX)
-    want = base.copy()
-    for d in range(world):
-        lo, hi = odist.part_range(n, world, d)
-        want[lo:hi] = np.maximum(base[lo:hi], ((np.arange(lo, hi) * 7919) % 1000 - 500).astype(np.int32))
+    # rank r's copy: base, with r's block of indices marked; the combine takes the
+    # maximum over the ranks' copies (a single rank: its copy, all marked)
+    marks = ((np.arange(n) * 7919) % 1000 - 500).astype(np.int32)
+    copies = []
+    for r in range(world):
+        cr = base.copy()
+        lo, hi = odist.part_range(n, world, r)
+        cr[lo:hi] = marks[lo:hi]
+        copies.append(cr)
+    want = np.max(np.stack(copies), axis=0)
     check(f"user combine->{dst}", np.array_equal(c.download(), want))
 # LM OSEM one subset, then two more with the fused peer-memory tail (CUDA IPC)
 ev = si.lmosem_events(20_000, subset=1)
