@@ -1742,6 +1742,29 @@ bool red_small(const Module *m, uint64_t cnt) {
 }
 
 // local reduce of the slot's data into dst
+// the second kernel of a two-launch small-vector Reduce / Scan as a
+// programmatic dependent of the first (it starts while the first finishes and
+// waits in griddepcontrol.wait for its results): hides one launch gap
+// (SKEL_PDL=0: plain launch)
+cudaError_t launch_dependent(const void *fn, dim3 grid, dim3 block, void **params, cudaStream_t st) {
+    static const bool pdl = [] {
+        const char *e = getenv("SKEL_PDL");
+        return !(e && atoi(e) == 0);
+    }();
+    if (!pdl) return cudaLaunchKernel(fn, grid, block, params, 0, st);
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = grid;
+    cfg.blockDim = block;
+    cfg.dynamicSmemBytes = 0;
+    cfg.stream = st;
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    at[0].val.programmaticStreamSerializationAllowed = 1;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    return cudaLaunchKernelExC(&cfg, fn, params);
+}
+
 // host mirror of red.cuh's skel_xdev (the cross-device single-pass Reduce);
 // K == 0: a device-local Reduce
 struct XDev {
@@ -1760,13 +1783,17 @@ int launch_reduce(skel_ctx_s *ctx, Module *m, Slot &s, const void *in, uint64_t 
         const uint64_t ST = red_small_tile(m, cnt);
         uint64_t nt = (cnt + ST - 1) / ST;
         void *aggs = s.ws + L.total;  // room reserved by reduce_core
-        void *pa[] = {&in, &cnt, &aggs, abuf.data()};
+        int early = 1;
+        const bool big = red_small_big_tiles(m, cnt);
+        void *pa_s[] = {&in, &cnt, &aggs, &early, abuf.data()};  // skel_scan_agg_kernel
+        void *pa_b[] = {&in, &cnt, &aggs, abuf.data()};          // skel_red_agg2_kernel
+        void **pa = big ? pa_b : pa_s;
         DevGuard g(s.dev);
-        const void *kagg = red_small_big_tiles(m, cnt) ? (const void *)m->k_red_agg2 : (const void *)m->k_scan_agg;
+        const void *kagg = big ? (const void *)m->k_red_agg2 : (const void *)m->k_scan_agg;
         CK(ctx, cudaLaunchKernel(kagg, dim3((unsigned)nt), dim3((unsigned)m->sig[9]), pa, 0, s.stream));
         const void *caggs = aggs;
         void *pf[] = {&caggs, &nt, &dst, const_cast<XDev *>(&xd), abuf.data()};
-        CK(ctx, cudaLaunchKernel((const void *)m->k_fold_aggs, dim3(1), dim3((unsigned)m->sig[9]), pf, 0, s.stream));
+        CK(ctx, launch_dependent((const void *)m->k_fold_aggs, dim3(1), dim3((unsigned)m->sig[9]), pf, s.stream));
         ctx->stats.kernel_launches += 2;
         return SKEL_OK;
     }
@@ -2995,12 +3022,12 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
         if (small && SM_TILE > 0) {
             const unsigned nt = (unsigned)((cnt + SM_TILE - 1) / SM_TILE);
             void *aggs = s.ws + L.total;
-            void *pa[] = {&pin, &cnt, &aggs, abuf.data()};
+            int early = 0;
+            void *pa[] = {&pin, &cnt, &aggs, &early, abuf.data()};
             CK(ctx, cudaLaunchKernel((const void *)m->k_scan_agg, dim3(nt), dim3((unsigned)m->sig[9]), pa, 0, s.stream));
             const void *caggs = aggs;
             void *ps[] = {&pin, &pout, &cnt, &caggs, idbuf.data(), &seed, abuf.data()};
-            CK(ctx, cudaLaunchKernel((const void *)m->k_scan_small, dim3(nt), dim3((unsigned)m->sig[9]), ps, 0,
-                                     s.stream));
+            CK(ctx, launch_dependent((const void *)m->k_scan_small, dim3(nt), dim3((unsigned)m->sig[9]), ps, s.stream));
             ctx->stats.kernel_launches += 2;
         } else if (small) {
             return fail(ctx, SKEL_ERR_CUDA, "persistent Scan grid cannot be co-resident and this module has no "

@@ -270,6 +270,13 @@ template <class T> __device__ __forceinline__ void st_value(T *p, const T &v) {
 #pragma unroll
     for (int i = 0; i < W; ++i) st_relaxed_u32(q + i, a.w[i]);
 }
+// programmatic dependent launch (the two-launch small-vector Reduce / Scan):
+// the second kernel is launched while the first one runs and waits here until
+// the first one has completed and its writes are visible; the first one lets
+// it be scheduled once every CTA has loaded its tile.  Both are no-ops for a
+// kernel launched without the programmatic attribute.
+__device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+__device__ __forceinline__ void pdl_trigger() { asm volatile("griddepcontrol.launch_dependents;" ::: "memory"); }
 // system scope: values and counters that other GPUs read or write over NVLink
 // (the cross-device single-pass Reduce, red.cuh skel_xdev_finish)
 __device__ __forceinline__ void fence_acq_rel_sys() { asm volatile("fence.acq_rel.sys;" ::: "memory"); }

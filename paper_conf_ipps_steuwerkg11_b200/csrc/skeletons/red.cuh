@@ -1249,10 +1249,15 @@ __device__ __forceinline__ int small_load(const skel_T *in, skel_u64 n, skel_u64
 
 // ordered fold of one tile of RB x PER elements into aggs[blockIdx.x]
 template <int PER, class Tup>
-__device__ __forceinline__ void tile_aggregate(const skel_T *in, skel_u64 n, skel_S *aggs, VT *wpart, Tup &tup) {
+__device__ __forceinline__ void tile_aggregate(const skel_T *in, skel_u64 n, skel_S *aggs, VT *wpart, Tup &tup,
+                                               bool EARLY_TRIGGER) {
     const int t = threadIdx.x;
     skel_T x[PER];
     const int m = small_load<PER>(in, n, blockIdx.x * ((skel_u64)RB * PER) + (skel_u64)t * PER, x);
+    // the dependent launch (it waits for our stores) may start: the Reduce's
+    // one-CTA fold as soon as the tiles are loaded; the tile Scan, whose CTAs
+    // would take SM slots from ours, only once every aggregate is out
+    if (EARLY_TRIGGER) skel::pdl_trigger();
     VT a;
     a.ok = false;
 #pragma unroll
@@ -1260,13 +1265,15 @@ __device__ __forceinline__ void tile_aggregate(const skel_T *in, skel_u64 n, ske
         if (k < m) a = comb(a, vt_make(x[k]), tup);
     const VT r = block_fold(a, wpart, tup);
     if (t == 0) aggs[blockIdx.x].v = r.v;  // every tile holds >= 1 element
+    if (!EARLY_TRIGGER) skel::pdl_trigger();
 }
 
+// (`early`: the dependent kernel is the Reduce's fold, else the tile Scan)
 extern "C" __global__ void __launch_bounds__(RB)
-    skel_scan_agg_kernel(const skel_T *__restrict__ in, skel_u64 n, skel_S *aggs, const skel_Buf args) {
+    skel_scan_agg_kernel(const skel_T *__restrict__ in, skel_u64 n, skel_S *aggs, int early, const skel_Buf args) {
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     __shared__ VT wpart[NW];
-    tile_aggregate<SPER>(in, n, aggs, wpart, tup);
+    tile_aggregate<SPER>(in, n, aggs, wpart, tup, early != 0);
 }
 // the same with tiles of twice the size: the small-vector Reduce above 2^21
 // 4-byte elements (more bytes in flight per thread)
@@ -1274,7 +1281,7 @@ extern "C" __global__ void __launch_bounds__(RB)
     skel_red_agg2_kernel(const skel_T *__restrict__ in, skel_u64 n, skel_S *aggs, const skel_Buf args) {
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     __shared__ VT wpart[NW];
-    tile_aggregate<2 * SPER>(in, n, aggs, wpart, tup);
+    tile_aggregate<2 * SPER>(in, n, aggs, wpart, tup, true);
 }
 
 extern "C" __global__ void __launch_bounds__(RB)
@@ -1288,6 +1295,7 @@ extern "C" __global__ void __launch_bounds__(RB)
     const skel_u64 b = blockIdx.x;
     skel_T x[SPER];  // loaded first: its latency overlaps the prefix fold
     const int m = small_load(in, n, b * SM_TILE + (skel_u64)t * SPER, x);
+    skel::pdl_wait();  // the tile aggregates (launched as a programmatic dependent of their kernel)
     // prefix of the tiles before this one, folded in order
     const skel_u64 per = (b + RB - 1) / RB;
     VT a;
@@ -1344,6 +1352,7 @@ extern "C" __global__ void __launch_bounds__(RB)
     skel_fold_aggs_kernel(const skel_S *aggs, skel_u64 count, skel_S *out, const __grid_constant__ skel_xdev xd,
                           const skel_Buf args) {
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
+    skel::pdl_wait();  // the tile aggregates (programmatic dependent launch)
     __shared__ VT wpart[NW];
     const int t = threadIdx.x;
     const skel_u64 per = (count + RB - 1) / RB;
