@@ -67,6 +67,9 @@ with skel.Context(1) as ctx:
                 "pairs_nrf_periodic": "#define MANDEL_NOREPLAY 1\n#define MANDEL_NR_FSETP 1\n" + MANDELBROT_PAIRS_PERIODIC,
                 "pairs_nrf_periodic_pb16": "#define MANDEL_NOREPLAY 1\n#define MANDEL_NR_FSETP 1\n#define MANDEL_PB 16\n" + MANDELBROT_PAIRS_PERIODIC,
                 "pairs_nrf_periodic_pb4": "#define MANDEL_NOREPLAY 1\n#define MANDEL_NR_FSETP 1\n#define MANDEL_PB 4\n" + MANDELBROT_PAIRS_PERIODIC,
+                "pairs_periodic_minb12": "#define SKEL_MINB 12\n" + MANDELBROT_PAIRS_PERIODIC,
+                "pairs_periodic_minb16": "#define SKEL_MINB 16\n" + MANDELBROT_PAIRS_PERIODIC,
+                "periodic_minb16": "#define SKEL_MINB 16\n" + MANDELBROT_PERIODIC,
                 "pairs_max": MX + MANDELBROT_PAIRS, "pairs_periodic_max": MX + MANDELBROT_PAIRS_PERIODIC})
     fns.update(extra)
     if os.environ.get("MANDEL_ONLY"):
