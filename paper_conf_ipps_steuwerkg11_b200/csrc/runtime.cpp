@@ -948,6 +948,35 @@ int set_distribution(skel_vec_s *v, skel_dist dist, skel_combine combine) {
 int ew_grid(const Slot &s, size_t chunks, int block, int per_thread = 1);
 int ensure_ws(skel_ctx_s *ctx, Slot &s, size_t bytes);
 
+// Kernel launches of the skeleton templates: as a programmatic dependent of
+// the previous kernel on the stream (cudaLaunchAttributeProgrammaticStreamSerialization).
+// Every such kernel starts with griddepcontrol.wait (prelude.cuh skel::pdl_wait:
+// it touches no memory before the previous kernel has completed and its writes
+// are visible) and then lets its own dependents be scheduled, so the next
+// kernel's CTAs are placed during this one's last wave and the launch gap
+// between consecutive skeletons disappears.  A non-kernel predecessor (copy,
+// event wait) or a kernel that never triggers keeps the ordinary ordering.
+// SKEL_PDL=0: plain launches.
+cudaError_t launch_dependent(const void *fn, dim3 grid, dim3 block, void **params, cudaStream_t st,
+                             size_t smem = 0) {
+    static const bool pdl = [] {
+        const char *e = getenv("SKEL_PDL");
+        return !(e && atoi(e) == 0);
+    }();
+    if (!pdl) return cudaLaunchKernel(fn, grid, block, params, smem, st);
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = grid;
+    cfg.blockDim = block;
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = st;
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    at[0].val.programmaticStreamSerializationAllowed = 1;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    return cudaLaunchKernelExC(&cfg, fn, params);
+}
+
 // one Zip launch out[i] = f(a[i], b[i]) on raw device pointers (out may alias a or b)
 int zip_raw(skel_ctx_s *ctx, Module *m, Slot &s, const void *pa, const void *pb, void *po, uint64_t cnt) {
     if (!cnt) return SKEL_OK;
@@ -959,7 +988,7 @@ int zip_raw(skel_ctx_s *ctx, Module *m, Slot &s, const void *pa, const void *pb,
     const int grid = ew_grid(s, chunks, block, vec_ok && E > 1 ? std::max<int>(1, (int)m->sig[10]) : 1);
     void *params[] = {&pa, &pb, &po, &cnt, &vec_ok, abuf.data()};
     DevGuard g(s.dev);
-    CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+    CK(ctx, launch_dependent((const void *)m->k_main, dim3(grid), dim3(block), params, s.stream));
     ctx->stats.kernel_launches++;
     return SKEL_OK;
 }
@@ -1419,7 +1448,7 @@ int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_
                                 : ew_grid(s, chunks, block, policy == 0 && vec_ok && E > 1 ? unroll : 1);
         void *params[] = {&pa, &pb, &po, &cnt, &vk, abuf.data()};
         const void *kf = policy >= 3 ? (const void *)m->k_main_u1 : (const void *)m->k_main;
-        CK(ctx, cudaLaunchKernel(kf, dim3(grid), dim3(block), params, 0, s.stream));
+        CK(ctx, launch_dependent(kf, dim3(grid), dim3(block), params, s.stream));
         ctx->stats.kernel_launches++;
     }
     if (rsz != 0) {
@@ -1742,29 +1771,6 @@ bool red_small(const Module *m, uint64_t cnt) {
 }
 
 // local reduce of the slot's data into dst
-// the second kernel of a two-launch small-vector Reduce / Scan as a
-// programmatic dependent of the first (it starts while the first finishes and
-// waits in griddepcontrol.wait for its results): hides one launch gap
-// (SKEL_PDL=0: plain launch)
-cudaError_t launch_dependent(const void *fn, dim3 grid, dim3 block, void **params, cudaStream_t st) {
-    static const bool pdl = [] {
-        const char *e = getenv("SKEL_PDL");
-        return !(e && atoi(e) == 0);
-    }();
-    if (!pdl) return cudaLaunchKernel(fn, grid, block, params, 0, st);
-    cudaLaunchConfig_t cfg = {};
-    cfg.gridDim = grid;
-    cfg.blockDim = block;
-    cfg.dynamicSmemBytes = 0;
-    cfg.stream = st;
-    cudaLaunchAttribute at[1];
-    at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
-    at[0].val.programmaticStreamSerializationAllowed = 1;
-    cfg.attrs = at;
-    cfg.numAttrs = 1;
-    return cudaLaunchKernelExC(&cfg, fn, params);
-}
-
 // host mirror of red.cuh's skel_xdev (the cross-device single-pass Reduce);
 // K == 0: a device-local Reduce
 struct XDev {
@@ -1810,8 +1816,8 @@ int launch_reduce(skel_ctx_s *ctx, Module *m, Slot &s, const void *in, uint64_t 
     void *params[] = {&tin, &in, &cnt, &use_tma, &partials, &pvalid, &counter, &result, const_cast<XDev *>(&xd),
                       abuf.data()};
     DevGuard g(s.dev);
-    CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3((unsigned)G), dim3((unsigned)RB), params,
-                             use_tma ? m->sig[11] : 0, s.stream));
+    CK(ctx, launch_dependent((const void *)m->k_main, dim3((unsigned)G), dim3((unsigned)RB), params, s.stream,
+                             use_tma ? m->sig[11] : 0));
     ctx->stats.kernel_launches++;
     return SKEL_OK;
 }
@@ -1898,7 +1904,7 @@ int reduce_core(skel_ctx_s *ctx, Module *m, skel_vec_s *in, const skel_arg *args
             void *outp = s.ws + L.o_fold;
             int k = K;
             void *params[] = {&vals, &k, &outp, abuf.data()};
-            CK(ctx, cudaLaunchKernel((const void *)m->k_fold, dim3(1), dim3(32), params, 0, s.stream));
+            CK(ctx, launch_dependent((const void *)m->k_fold, dim3(1), dim3(32), params, s.stream));
             ctx->stats.kernel_launches++;
         }
     }
@@ -2557,7 +2563,7 @@ int skel_map_index(skel_ctx_t ctx, const char *src, size_t n, skel_vec_t out, co
         int vk = policy == 2 ? 0 : vec_ok;
         const int grid = ew_grid(s, policy == 2 ? cnt : chunks, block, 1);
         void *params[] = {&po, &cnt, &base, &vk, abuf.data()};
-        CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+        CK(ctx, launch_dependent((const void *)m->k_main, dim3(grid), dim3(block), params, s.stream));
         ctx->stats.kernel_launches++;
     }
     if (rsz != 0) {
@@ -2604,7 +2610,7 @@ int skel_map_lanes(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t ou
         int ln = lanes;
         void *params[] = {&pa, &pb, &po, &cnt, &ln, abuf.data()};
         DevGuard g(s.dev);
-        CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
+        CK(ctx, launch_dependent((const void *)m->k_main, dim3(grid), dim3(block), params, s.stream));
         ctx->stats.kernel_launches++;
     }
     if (rsz != 0) {
@@ -2694,7 +2700,7 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
         int nsrc = D, ndst = D, op = (int)combine;
         void *params[] = {&pa, (void *)&bs, &nsrc, &bown, (void *)&os, &ndst, &cnt, &op, &vec_ok, abuf.data()};
         DevGuard g(s.dev);
-        CK(ctx, cudaLaunchKernel((const void *)m->k_zipcomb, dim3(grid), dim3(block), params, 0, s.stream));
+        CK(ctx, launch_dependent((const void *)m->k_zipcomb, dim3(grid), dim3(block), params, s.stream));
         ctx->stats.kernel_launches++;
         ctx->stats.d2d_bytes += (uint64_t)(D - 1) * cnt * (esb + eso);
         return SKEL_OK;
@@ -2726,7 +2732,7 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
             uint64_t ncall = cnt;
             void *params[] = {&pa, &mcb, &bown, &mco, &ncall, &vec_ok, abuf.data()};
             DevGuard g(s.dev);
-            CK(ctx, cudaLaunchKernel((const void *)m->k_zipcomb_mm, dim3(grid), dim3(block), params, 0, s.stream));
+            CK(ctx, launch_dependent((const void *)m->k_zipcomb_mm, dim3(grid), dim3(block), params, s.stream));
             ctx->stats.kernel_launches++;
             ctx->stats.multimem_launches++;
             ctx->stats.d2d_bytes += (uint64_t)cnt * (esb + eso);
@@ -2784,7 +2790,7 @@ int skel_zip_combine(skel_ctx_t ctx, const char *src, skel_vec_t a, skel_vec_t b
             uint64_t ncall = cnt;
             void *params[] = {&pa, &mcb, &bown, &mco, &ncall, &vec_ok, abuf.data()};
             DevGuard g(s.dev);
-            CK(ctx, cudaLaunchKernel((const void *)m->k_zipcomb_mm, dim3(grid), dim3(block), params, 0, s.stream));
+            CK(ctx, launch_dependent((const void *)m->k_zipcomb_mm, dim3(grid), dim3(block), params, s.stream));
             ctx->stats.kernel_launches++;
             ctx->stats.multimem_launches++;
         } else if (cnt) {
@@ -2971,7 +2977,7 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
             int k = s.d;
             void *seedp = s.ws + L.o_seed;
             void *params[] = {&aggs, &k, idbuf.data(), &seedp, abuf.data()};
-            CK(ctx, cudaLaunchKernel((const void *)m->k_seed, dim3(1), dim3(32), params, 0, s.stream));
+            CK(ctx, launch_dependent((const void *)m->k_seed, dim3(1), dim3(32), params, s.stream));
             ctx->stats.kernel_launches++;
             seed = seedp;
         }

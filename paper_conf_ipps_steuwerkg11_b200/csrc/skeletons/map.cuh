@@ -241,6 +241,8 @@ extern "C" __global__ void SKEL_EW_BOUNDS
     skel_ew_kernel(const skel_A *__restrict__ a, const skel_B *__restrict__ b, skel_O *__restrict__ out, skel_u64 n,
                    int lanes, const skel_Buf args) {
     (void)b;
+    skel::pdl_wait();  // launched as a programmatic dependent of the previous kernel (prelude.cuh)
+    skel::pdl_trigger();
     auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     const int lane = (int)(threadIdx.x & 31u);
     const int sub = lane & (lanes - 1);
@@ -287,6 +289,8 @@ __device__ __forceinline__ void skel_idx_one(skel_O *out, skel_u64 i, skel_u64 b
 }
 extern "C" __global__ void SKEL_EW_BOUNDS
     skel_ew_kernel(skel_O *__restrict__ out, skel_u64 n, skel_u64 base, int vec_ok, const skel_Buf args) {
+    skel::pdl_wait();
+    skel::pdl_trigger();
     auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
     const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;
@@ -302,6 +306,12 @@ extern "C" __global__ void SKEL_EW_BOUNDS
 template <int U>
 __device__ __forceinline__ void skel_ew_body(const skel_A *__restrict__ a, const skel_B *__restrict__ b,
                                              skel_O *__restrict__ out, skel_u64 n, int vec_ok, const skel_Buf &args) {
+    // every element-wise kernel is launched as a programmatic dependent of the
+    // previous kernel on its stream: it may be scheduled during that kernel's
+    // last wave and waits here for its completion (and memory) before touching
+    // anything; it lets the next launch be scheduled at once
+    skel::pdl_wait();
+    skel::pdl_trigger();
     auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
     const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;
@@ -458,6 +468,8 @@ __device__ __forceinline__ void skel_zipcomb_elem(const skel_A &xa, const skel_p
 extern "C" __global__ void SKEL_EW_BOUNDS
     skel_zipcomb_kernel(const skel_A *__restrict__ a, const skel_ptrs bsrc, int nsrc, skel_B *bown,
                         const skel_ptrs odst, int ndst, skel_u64 n, int op, int vec_ok, const skel_Buf args) {
+    skel::pdl_wait();
+    skel::pdl_trigger();
     auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
     const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;
@@ -546,6 +558,8 @@ __device__ __forceinline__ void skel_mm_one(const skel_A *a, const float *mcb, B
 extern "C" __global__ void SKEL_EW_BOUNDS
     skel_zipcomb_mm_kernel(const skel_A *__restrict__ a, const float *mcb, skel_B *bown, float *mco, skel_u64 n,
                            int vec_ok, const skel_Buf args) {
+    skel::pdl_wait();
+    skel::pdl_trigger();
     auto t = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     const skel_u64 tid = (skel_u64)blockIdx.x * blockDim.x + threadIdx.x;
     const skel_u64 stride = (skel_u64)gridDim.x * blockDim.x;

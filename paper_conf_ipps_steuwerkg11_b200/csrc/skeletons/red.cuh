@@ -474,6 +474,8 @@ extern "C" __global__ void __launch_bounds__(RB, SKEL_RED_MINB)
     skel_reduce_kernel(const __grid_constant__ skel_tmap tin, const skel_T *__restrict__ in, skel_u64 n, int use_tma,
                        skel_S *partials, unsigned *pvalid, unsigned *counter, skel_S *result,
                        const __grid_constant__ skel_xdev xd, const skel_Buf args) {
+    skel::pdl_wait();  // launched as a programmatic dependent (prelude.cuh)
+    skel::pdl_trigger();
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     __shared__ skel_u64 bars[STAGES];
     __shared__ VT wpart[NW];
@@ -600,6 +602,8 @@ extern "C" __global__ void __launch_bounds__(RB, SKEL_RED_MINB)
 
 // fold count >= 1 published values in order (cross-device Reduce)
 extern "C" __global__ void skel_fold_kernel(const skel_S *vals, int count, skel_S *out, const skel_Buf args) {
+    skel::pdl_wait();
+    skel::pdl_trigger();
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     if (threadIdx.x == 0 && blockIdx.x == 0) {
         skel_T acc = vals[0].v;
@@ -611,6 +615,8 @@ extern "C" __global__ void skel_fold_kernel(const skel_S *vals, int count, skel_
 // otherwise agg_0 (+) ... (+) agg_{k-1}
 extern "C" __global__ void skel_seed_kernel(const skel_S *aggs, int k, const skel_S identity, skel_S *out,
                                             const skel_Buf args) {
+    skel::pdl_wait();
+    skel::pdl_trigger();
     auto tup = skel::unpack<skel_Args, skel_Lay, skel_Seq>::run(args);
     if (threadIdx.x == 0 && blockIdx.x == 0) {
         if (k == 0) {
