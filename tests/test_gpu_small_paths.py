@@ -24,3 +24,17 @@ def test_reduce_and_scan_tests_on_each_path(small_max):
                         os.path.join(ROOT, "tests", "test_gpu_graphs.py")],
                        env=env, capture_output=True, text=True, timeout=1200, cwd=ROOT)
     assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-2000:]
+
+
+def test_skeletons_without_programmatic_dependent_launches():
+    """Every skeleton kernel is launched as a programmatic dependent of the
+    previous kernel on its stream and waits (griddepcontrol.wait) before
+    touching memory; with SKEL_PDL=0 the same kernels run with ordinary
+    launches.  The skeleton, graph and distribution suites pass both ways."""
+    env = dict(os.environ, SKEL_PDL="0")
+    r = subprocess.run([sys.executable, "-m", "pytest", "-q", "-x", "-m", "gpu",
+                        os.path.join(ROOT, "tests", "test_gpu_skeletons.py"),
+                        os.path.join(ROOT, "tests", "test_gpu_graphs.py"),
+                        os.path.join(ROOT, "tests", "test_gpu_distributions.py")],
+                       env=env, capture_output=True, text=True, timeout=1500, cwd=ROOT)
+    assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-2000:]
