@@ -15,6 +15,7 @@ timeout 900 ncu --set full --clock-control none --import-source on --nvtx --nvtx
     -o gpurun_out/${T}_prof_ew -f python bench.py --steps 1 --warmup 3 --e2e-steps 0 --no-cpu --no-extras > gpurun_out/${T}_prof_ew.log 2>&1
 timeout 900 ncu --set full --clock-control none --import-source on --nvtx --nvtx-include timed/ -k 'regex:skel_(reduce|scan)_kernel' -c 2 \
     -o gpurun_out/${T}_prof_rs -f python bench.py --steps 1 --warmup 3 --e2e-steps 0 --no-cpu --no-extras > gpurun_out/${T}_prof_rs.log 2>&1
+timeout 900 python tools/lmosem_scaling_proxy.py > gpurun_out/${T}_proxy.jsonl 2> gpurun_out/${T}_proxy.err
 for v in paper periodic pairs_periodic; do
   timeout 600 ncu --set full --clock-control none --import-source on -k regex:skel_ew -s 3 -c 1 \
       -o gpurun_out/${T}_mandel_$v -f python tools/mandel_one.py $v 128 > gpurun_out/${T}_mandel_$v.log 2>&1
