@@ -30,7 +30,7 @@ from __future__ import annotations
 import numpy as np
 
 from . import skel
-from .workloads import (LMOSEM_ERROR, LMOSEM_ERROR_PREPARED, LMOSEM_LANES, LMOSEM_LANES_PREPARED,
+from .workloads import (LMOSEM_ERROR, LMOSEM_ERROR_PREPARED, LMOSEM_LANES,
                         LMOSEM_ORDER_BUCKETS, LMOSEM_ORDER_HIST, LMOSEM_ORDER_SCATTER, LMOSEM_ORDER_SLOTS,
                         LMOSEM_UPDATE, SUM_I32)
 
@@ -39,13 +39,16 @@ DIMS = (150, 150, 280)
 # CTA size of every error-image Map (measured at 10^6/D events, D = 1..8,
 # tools/lm_lanes_probe.py: 128 is as fast or faster than 256 everywhere)
 MAP_BLOCK = 128
-# events per device from which the one-thread-per-event Map beats the lanes
-# Map on length-ordered events (measured crossover between 1.25e5 and 2.5e5)
-ORDERED_LANES_BELOW = 200_000
+# events per device from which the one-thread-per-event Map (16-byte forward
+# gathers) beats the 4-lane Map (scalar gathers) on length-ordered events
+# (round 2, graph replays: 10^6: 1.141 vs 1.147 ms; 5*10^5: 0.589 vs 0.582;
+# 2.5*10^5: 0.317 vs 0.300; 1.25*10^5: 0.179 vs 0.160)
+ORDERED_LANES_BELOW = 750_000
 # order="auto": events per device from which ordering them on the device pays
-# for itself (10^6: 0.076 ms ordering + 1.15 ms Map vs 1.29 ms lanes Map in
-# the given order; 1.25e5: 0.017 + 0.170 vs 0.178 ms)
-AUTO_ORDER_FROM = 400_000
+# for itself (ordering + ordered Map vs the 4-lane Map in the given order:
+# 10^6: 0.071 + 1.141 vs 1.287 ms; 2.5*10^5: 0.028 + 0.300 vs 0.335;
+# 1.25*10^5: 0.020 + 0.160 vs 0.177)
+AUTO_ORDER_FROM = 200_000
 
 
 class LMOSEM:
@@ -77,15 +80,16 @@ class LMOSEM:
         events.  Given order: 4 lanes per event at every measured part size
         (10^6/D events, D = 1..8: 1.29 / 0.655 / 0.337 / 0.179 ms against
         1.37 / 0.727 / 0.394 / 0.211 ms with one thread per event).
-        Length-ordered events: one thread per event down to ORDERED_LANES_BELOW,
-        4 lanes below it (D = 1: 1.14 vs 1.26 ms; D = 8: 0.169 vs 0.175 ms)."""
+        Length-ordered events: one thread per event with 16-byte forward
+        gathers from ORDERED_LANES_BELOW on, 4 lanes with scalar gathers below
+        it (the 16-byte gathers lose once a ray is split into pieces)."""
         ordered = self.ordered(per_device)
         lanes = self.lanes
         if lanes is None:
             lanes = 4 if (not ordered or per_device < ORDERED_LANES_BELOW) else 1
         if lanes == 1:
             return (LMOSEM_ERROR_PREPARED if ordered else LMOSEM_ERROR), 1
-        return (LMOSEM_LANES_PREPARED if ordered else LMOSEM_LANES), lanes
+        return LMOSEM_LANES, lanes
 
     def prepare(self):
         """Compile every function a subset may use (before timing or capturing)."""
@@ -93,7 +97,7 @@ class LMOSEM:
         ctx.set_block_size(MAP_BLOCK)
         for src in (LMOSEM_ERROR, LMOSEM_ERROR_PREPARED):
             ctx.prepare("map", src)
-        for src in (LMOSEM_LANES, LMOSEM_LANES_PREPARED):
+        for src in (LMOSEM_LANES,):
             ctx.prepare("lanes", src)
         ctx.set_block_size(0)
         ctx.prepare("zip", LMOSEM_UPDATE)
