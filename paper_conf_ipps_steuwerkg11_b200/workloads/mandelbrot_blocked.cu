@@ -36,6 +36,12 @@ struct Pos { float re, im; };
 #ifndef MANDEL_PERIODIC
 #define MANDEL_PERIODIC 0
 #endif
+// block index of the next save of the periodicity check: doubling is Brent's
+// schedule; any schedule whose gaps grow without bound finds every cycle (a
+// detection is exact either way: equal states repeat forever)
+#ifndef MANDEL_SAVE_NEXT
+#define MANDEL_SAVE_NEXT(s) ((s) << 1)
+#endif
 #if MANDEL_PERIODIC
 #ifndef __CUDA_ARCH__
 #include <cstring>
@@ -169,7 +175,7 @@ template <int B> static int mandel_blocked(Pos c, int cap) {
         if (++blk == next_save) {
             sx = mandel_bits(x);
             sy = mandel_bits(y);
-            next_save <<= 1;
+            next_save = MANDEL_SAVE_NEXT(next_save);
         }
 #endif
     }

@@ -86,6 +86,12 @@ static inline bool same_hi(mandel_f2 a, mandel_f2 b) { return std::memcmp(&a.hi,
 #ifndef MANDEL_PERIODIC
 #define MANDEL_PERIODIC 0
 #endif
+// block index of the next save of the periodicity check: doubling is Brent's
+// schedule; any schedule whose gaps grow without bound finds every cycle (a
+// detection is exact either way: equal states repeat forever)
+#ifndef MANDEL_SAVE_NEXT
+#define MANDEL_SAVE_NEXT(s) ((s) << 1)
+#endif
 
 // plain loop (eq. (5) as written) for at most `lim` updates from (x, y, n)
 static __forceinline__ int mandel_plain(float cr, float ci, float &x, float &y, int n, int lim) {
@@ -166,7 +172,7 @@ template <int B> static __forceinline__ int mandel_finish(float cr, float ci, fl
         if (++blk == next_save) {
             sx = mandel_bits(x);
             sy = mandel_bits(y);
-            next_save <<= 1;
+            next_save = MANDEL_SAVE_NEXT(next_save);
         }
 #endif
     }
@@ -266,7 +272,7 @@ static __forceinline__ Cnt2 mandel_pairs_nr(Pos2 c, int cap) {
         if (++blk == next_save) {
             SX = X;
             SY = Y;
-            next_save <<= 1;
+            next_save = MANDEL_SAVE_NEXT(next_save);
         }
 #endif
     }
@@ -337,7 +343,7 @@ Cnt2 mandelbrot_pairs(Pos2 c, int cap) {
             if (++blk == next_save) {
                 SX = X;
                 SY = Y;
-                next_save <<= 1;
+                next_save = MANDEL_SAVE_NEXT(next_save);
             }
 #endif
         }

@@ -70,6 +70,14 @@ with skel.Context(1) as ctx:
                 "pairs_periodic_minb12": "#define SKEL_MINB 12\n" + MANDELBROT_PAIRS_PERIODIC,
                 "pairs_periodic_minb16": "#define SKEL_MINB 16\n" + MANDELBROT_PAIRS_PERIODIC,
                 "periodic_minb16": "#define SKEL_MINB 16\n" + MANDELBROT_PERIODIC,
+                "periodic_g15": "#define MANDEL_SAVE_NEXT(s) ((s) + ((s) >> 1) + ((s) < 2))\n" + MANDELBROT_PERIODIC,
+                "periodic_g125": "#define MANDEL_SAVE_NEXT(s) ((s) + ((s) >> 2) + ((s) < 4))\n" + MANDELBROT_PERIODIC,
+                "pairs_periodic_g15": "#define MANDEL_SAVE_NEXT(s) ((s) + ((s) >> 1) + ((s) < 2))\n" + MANDELBROT_PAIRS_PERIODIC,
+                "pairs_periodic_g125": "#define MANDEL_SAVE_NEXT(s) ((s) + ((s) >> 2) + ((s) < 4))\n" + MANDELBROT_PAIRS_PERIODIC,
+                "periodic_g3": "#define MANDEL_SAVE_NEXT(s) ((s) * 3)\n" + MANDELBROT_PERIODIC,
+                "periodic_g4": "#define MANDEL_SAVE_NEXT(s) ((s) << 2)\n" + MANDELBROT_PERIODIC,
+                "pairs_periodic_g3": "#define MANDEL_SAVE_NEXT(s) ((s) * 3)\n" + MANDELBROT_PAIRS_PERIODIC,
+                "pairs_periodic_g4": "#define MANDEL_SAVE_NEXT(s) ((s) << 2)\n" + MANDELBROT_PAIRS_PERIODIC,
                 "pairs_max": MX + MANDELBROT_PAIRS, "pairs_periodic_max": MX + MANDELBROT_PAIRS_PERIODIC})
     fns.update(extra)
     if os.environ.get("MANDEL_ONLY"):
