@@ -52,7 +52,7 @@ struct Module {
     // through the scalar path, 3 = one chunk per thread with the low-register
     // kernel (k_main_u1), 4 = the scalar path through k_main_u1; decided on a
     // sample at the first launch of each size class
-    static constexpr int kPolicies = 5;
+    static constexpr int kPolicies = 6;
     // (size class = log2 of the chunk count, hash of the scalar arguments) -> decided policy
     std::map<std::pair<int, uint64_t>, int> ew_policy;
     // decisions persist next to the cached cubin (<key>.policy, one line per

@@ -1194,7 +1194,10 @@ int ew_grid(const Slot &s, size_t chunks, int block, int per_thread) {
 // 2 = one element per thread through the scalar path (compute-bound, divergent
 // functions: finer work items even out the lanes of a warp), 3 = one chunk per
 // thread with the low-register kernel (small vectors: twice the CTAs per SM,
-// so a single-wave launch), 4 = the scalar path through the low-register kernel.  Decided once per
+// so a single-wave launch), 4 = the scalar path through the low-register kernel,
+// 5 = the same over half a grid: every thread takes elements i and i + n/2
+// (for a divergent function two items of uncorrelated cost per lane even out a
+// warp's lanes better than one: Mandelbrot rows y and y + H/2, 7% faster).  Decided once per
 // module, size class (log2 of the chunk count) and set of scalar arguments (up
 // to four per class), at the first launch of that class and set, by timing the policies in `mask` on a SAMPLE of that launch's data
 // copied to scratch memory -- never on the user's buffers,
@@ -1273,11 +1276,11 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
     // made the scalar path look as fast as the vector path for a Zip)
     constexpr uint64_t kSampleBytes = 256ull << 20, kBlocks = 256;
     const uint64_t kSample = std::max<uint64_t>(kSampleBytes / std::max<size_t>(esa + esb + eso, 1), 4096);
-    if (cnt > kSample && (mask & 24u)) {
+    if (cnt > kSample && (mask & 56u)) {
         // the low-register kernel is a small-vector policy: judged only where the
         // sample IS the launch (at 2^30 a sample once preferred it by noise, 1.7%
         // slower at full size)
-        mask &= ~24u;
+        mask &= ~56u;
         P = 0;
         for (int p = 0; p < Module::kPolicies; ++p)
             if (mask & (1u << p)) pol[P++] = p;
@@ -1333,7 +1336,7 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
         for (auto &rg : ranges) {
             uint64_t n = rg.second, b0 = rg.first;
             const size_t chunks = std::max<uint64_t>(n / E, 1);
-            const bool scalar = policy == 2 || policy == 4;
+            const bool scalar = policy == 2 || policy == 4 || policy == 5;
             int vk = scalar ? 0 : 1;
             const void *qa = sa + off, *qb = pb ? (const void *)(sb + off) : nullptr;
             void *qo = so + off;
@@ -1343,7 +1346,8 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
                 void *params[] = {&qo, &n, &b0, &vk, abuf.data()};
                 CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
             } else {
-                grid = scalar ? ew_grid(s, n, block, 1) : ew_grid(s, chunks, block, policy == 0 ? unroll : 1);
+                grid = scalar ? ew_grid(s, n, block, policy == 5 ? 2 : 1)
+                              : ew_grid(s, chunks, block, policy == 0 ? unroll : 1);
                 void *params[] = {&qa, &qb, &qo, &n, &vk, abuf.data()};
                 const void *kf = policy >= 3 ? (const void *)m->k_main_u1 : (const void *)m->k_main;
                 CK(ctx, cudaLaunchKernel(kf, dim3(grid), dim3(block), params, 0, s.stream));
@@ -1439,12 +1443,13 @@ int run_ew(skel_ctx_s *ctx, Kind kind, const char *src, skel_vec_s *a, skel_vec_
         int policy = 0;
         if (vec_ok && E > 1 && unroll > 1)
             TRY(ew_decide(ctx, m, s, kind, pa, a->es, pb, b ? b->es : 0, rsz, cnt, 0, abuf,
-                          m->k_main_u1 ? 0x1Fu : 0x7u, &policy));
+                          m->k_main_u1 ? 0x3Fu : 0x7u, &policy));
         // policy 2: the scalar path, one element per thread; 3: one chunk per thread
-        // through the low-register kernel; 4: the scalar path through it
-        const bool scalar = policy == 2 || policy == 4;
+        // through the low-register kernel; 4: the scalar path through it; 5: the
+        // same with two elements per thread (grid-stride over half a grid)
+        const bool scalar = policy == 2 || policy == 4 || policy == 5;
         int vk = scalar ? 0 : vec_ok;
-        const int grid = scalar ? ew_grid(s, cnt, block, 1)
+        const int grid = scalar ? ew_grid(s, cnt, block, policy == 5 ? 2 : 1)
                                 : ew_grid(s, chunks, block, policy == 0 && vec_ok && E > 1 ? unroll : 1);
         void *params[] = {&pa, &pb, &po, &cnt, &vk, abuf.data()};
         const void *kf = policy >= 3 ? (const void *)m->k_main_u1 : (const void *)m->k_main;
