@@ -1342,7 +1342,7 @@ int ew_decide(skel_ctx_s *ctx, Module *m, Slot &s, Kind kind, const void *pa, si
             void *qo = so + off;
             int grid;
             if (kind == Kind::Idx) {
-                grid = ew_grid(s, scalar ? n : chunks, block, 1);
+                grid = ew_grid(s, scalar ? n : chunks, block, policy == 5 ? 2 : 1);
                 void *params[] = {&qo, &n, &b0, &vk, abuf.data()};
                 CK(ctx, cudaLaunchKernel((const void *)m->k_main, dim3(grid), dim3(block), params, 0, s.stream));
             } else {
@@ -2564,9 +2564,11 @@ int skel_map_index(skel_ctx_t ctx, const char *src, size_t n, skel_vec_t out, co
         // compute-bound function (Mandelbrot) balances better with the second
         int policy = 1;
         if (vec_ok && rsz != 0 && E > 1)
-            TRY(ew_decide(ctx, m, s, Kind::Idx, nullptr, 0, nullptr, 0, rsz, cnt, base, abuf, 0x6u, &policy));
-        int vk = policy == 2 ? 0 : vec_ok;
-        const int grid = ew_grid(s, policy == 2 ? cnt : chunks, block, 1);
+            TRY(ew_decide(ctx, m, s, Kind::Idx, nullptr, 0, nullptr, 0, rsz, cnt, base, abuf, 0x26u, &policy));
+        // (policy 5: the scalar path over half a grid, two indices per thread)
+        const bool scalar = policy == 2 || policy == 5;
+        int vk = scalar ? 0 : vec_ok;
+        const int grid = ew_grid(s, scalar ? cnt : chunks, block, policy == 5 ? 2 : 1);
         void *params[] = {&po, &cnt, &base, &vk, abuf.data()};
         CK(ctx, launch_dependent((const void *)m->k_main, dim3(grid), dim3(block), params, s.stream));
         ctx->stats.kernel_launches++;
