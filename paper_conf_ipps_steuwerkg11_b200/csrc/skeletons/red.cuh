@@ -27,6 +27,11 @@
 //    stage and written by TMA tensor stores (8 B/element).
 //  * Element types whose size is not 4, 8 or 16 bytes, unaligned views and
 //    the ragged last tile use direct (LDG/STG) loads with the same ordering.
+//  * A block-distributed Reduce over in-process devices ends inside these
+//    kernels: the last device to finish folds the device results in device
+//    order (skel_xdev_finish, system-scope ticket).
+//  * The kernels are launched as programmatic dependents of the previous
+//    kernel on the stream and wait for it first (griddepcontrol, prelude.cuh).
 
 // Reduce main loop: 1 = direct 128-bit loads, every warp folding its own
 // contiguous range (no barrier in the loop); 0 = TMA tiles through shared
