@@ -957,13 +957,16 @@ int ensure_ws(skel_ctx_s *ctx, Slot &s, size_t bytes);
 // between consecutive skeletons disappears.  A non-kernel predecessor (copy,
 // event wait) or a kernel that never triggers keeps the ordinary ordering.
 // SKEL_PDL=0: plain launches.
-cudaError_t launch_dependent(const void *fn, dim3 grid, dim3 block, void **params, cudaStream_t st,
-                             size_t smem = 0) {
+bool pdl_enabled() {
     static const bool pdl = [] {
         const char *e = getenv("SKEL_PDL");
         return !(e && atoi(e) == 0);
     }();
-    if (!pdl) return cudaLaunchKernel(fn, grid, block, params, smem, st);
+    return pdl;
+}
+cudaError_t launch_dependent(const void *fn, dim3 grid, dim3 block, void **params, cudaStream_t st,
+                             size_t smem = 0) {
+    if (!pdl_enabled()) return cudaLaunchKernel(fn, grid, block, params, smem, st);
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = grid;
     cfg.blockDim = block;
@@ -3015,12 +3018,19 @@ int skel_scan(skel_ctx_t ctx, const char *src, skel_vec_t in, skel_vec_t out, co
             cfg.blockDim = dim3((unsigned)m->sig[14]);
             cfg.dynamicSmemBytes = use_tma ? m->sig[12] : 0;
             cfg.stream = s.stream;
-            cudaLaunchAttribute attr[1];
+            cudaLaunchAttribute attr[2];
             attr[0].id = cudaLaunchAttributeCooperative;
             attr[0].val.cooperative = 1;
+            attr[1].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+            attr[1].val.programmaticStreamSerializationAllowed = 1;
             cfg.attrs = attr;
-            cfg.numAttrs = 1;
-            const cudaError_t le = cudaLaunchKernelExC(&cfg, (const void *)m->k_scan, params);
+            cfg.numAttrs = pdl_enabled() ? 2 : 1;
+            cudaError_t le = cudaLaunchKernelExC(&cfg, (const void *)m->k_scan, params);
+            if (le != cudaSuccess && le != cudaErrorCooperativeLaunchTooLarge && cfg.numAttrs == 2) {
+                cudaGetLastError();  // the driver declined the pair of attributes: cooperative only
+                cfg.numAttrs = 1;
+                le = cudaLaunchKernelExC(&cfg, (const void *)m->k_scan, params);
+            }
             if (le == cudaErrorCooperativeLaunchTooLarge) {
                 cudaGetLastError();  // fewer SMs than queried (MPS / green context): two short launches
                 ctx->stats.scan_coop_fallbacks++;

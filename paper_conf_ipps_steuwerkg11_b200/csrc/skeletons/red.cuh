@@ -956,6 +956,11 @@ extern "C" __global__ void __launch_bounds__(SCAN_THREADS, SKEL_SCAN_MINB)
                      skel_u64 *status, unsigned *flags, skel_S *aggv, skel_S *incv, unsigned *counters,
                      unsigned *epoch_ptr, skel_S *total, const skel_Buf args) {
     (void)incv;
+    // launched cooperatively AND as a programmatic dependent of the previous
+    // kernel: nothing is touched (and no CTA waits on another) before that
+    // kernel has completed, by which time the whole grid is resident
+    skel::pdl_wait();
+    skel::pdl_trigger();
     // the launch's epoch lives in device memory (graph replays must see a new
     // one): every CTA reads it before publishing anything; the last CTA to
     // finish advances it (all CTAs have read it by then)
