@@ -79,6 +79,9 @@ with skel.Context(1) as ctx:
                 "pairs_periodic_g3": "#define MANDEL_SAVE_NEXT(s) ((s) * 3)\n" + MANDELBROT_PAIRS_PERIODIC,
                 "pairs_periodic_g4": "#define MANDEL_SAVE_NEXT(s) ((s) << 2)\n" + MANDELBROT_PAIRS_PERIODIC,
                 "pairs_max": MX + MANDELBROT_PAIRS, "pairs_periodic_max": MX + MANDELBROT_PAIRS_PERIODIC})
+    rf = open(os.path.join(here, "mandel_refill_exp.cu")).read()
+    for P in (64, 128, 256, 512, 1024):
+        fns[f"refill_{P}"] = f"#define MR_P {P}\n" + rf
     fns.update(extra)
     if os.environ.get("MANDEL_ONLY"):
         keep = os.environ["MANDEL_ONLY"].split(",")
@@ -98,7 +101,18 @@ with skel.Context(1) as ctx:
             two = two or src.find("Pos2 c") >= 0
             v = vin2 if two else vin
             out = ctx.vector(n=v.n, dtype=si.CNT2_DTYPE if two else np.int32)
-            if name.startswith("dyn"):
+            if name.startswith("refill"):
+                P = int(name.split("_")[1]) if "_" in name else 256
+                npix = vin.n
+                nthr = -(-npix // P) * 32
+                img = ctx.vector(n=npix, dtype=np.int32)
+                rargs = [img, np.uint32(npix), np.int32(W), np.int32(H), np.int32(cap)]
+                srcr = src
+                ms = timed(lambda: ctx.map_index(srcr, nthr, None, args=rargs))
+                img.mark_device_modified()
+                out.upload(img.download())
+                img.destroy()
+            elif name.startswith("dyn"):
                 nthr = 148 * 2048
                 ctr = ctx.vector(np.zeros(2, np.uint32))
                 img = ctx.vector(n=vin.n, dtype=np.int32)
