@@ -18,7 +18,8 @@ for kv in os.environ.get("MANDEL_EXTRA", "").split(";"):
         k, v = kv.split("=", 1)
         extra[k] = open(v).read() if os.path.exists(v) else v
 
-W, H, cap = 4096, 3072, int(os.environ.get("MANDEL_CAP", "256"))
+W, H = int(os.environ.get("MANDEL_W", "4096")), int(os.environ.get("MANDEL_H", "3072"))
+cap = int(os.environ.get("MANDEL_CAP", "256"))
 peak = 148 * 128 * 1.965e9
 paper = si.mandelbrot_positions(W, H)
 members = np.zeros_like(paper)
